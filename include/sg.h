@@ -1,0 +1,238 @@
+/*
+ * sg.h -- C ABI of the B200-native synchronous-dataflow stream-graph executor.
+ *
+ * Follows the problem statement of Nguyen & Lee:
+ *   input  = a stream graph: filters (nodes) with firing rates, edges weighted
+ *            by their buffer size, composed by pipeline / split-join
+ *            (section 2.1.1; section 3.1),
+ *            plus the number of GPUs G and their topology (PAPER.md:494-502,
+ *            section 3.2.2);
+ *   output = partitions and a partition->GPU mapping minimising Tmax
+ *            (Eq. III.1-III.7), then generated kernels and
+ *            their pipelined execution.
+ *
+ * Conventions (all calls):
+ *   - Every call returns sg_status (0 = SG_OK, < 0 = error) unless noted.
+ *     No C++ exception crosses this boundary.  sg_last_error() returns a
+ *     thread-local message describing the last failure on the calling thread.
+ *   - Handles are opaque and owned by the caller; destroy them with the
+ *     matching *_destroy.  Distinct handles may be used from distinct threads;
+ *     one handle is not thread-safe.
+ *   - Streams are in NATURAL ORDER at the boundary: item i of the input stream
+ *     is input[i]; item i of the output stream is output[i].  Items are 4-byte
+ *     words of the graph's dtype.
+ *   - There is no CPU fallback: sg_run needs a CUDA device (sm_100a) and fails
+ *     with SG_E_CUDA otherwise.  Graph building, sg_plan (rates, partitioning,
+ *     ILP mapping, code generation and NVRTC compilation to sm_100a cubins) and
+ *     the size queries work without a GPU.
+ */
+#ifndef SG_H_
+#define SG_H_
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef enum {
+    SG_OK = 0,
+    SG_E_ARG = -1,          /* bad argument (NULL handle, negative size, bad kind params) */
+    SG_E_STRUCTURE = -2,    /* ill-formed hierarchy (unclosed split-join, empty graph, ...) */
+    SG_E_RATE = -3,         /* balance equations inconsistent */
+    SG_E_UNSUPPORTED = -4,  /* kind/dtype combination not supported */
+    SG_E_NOMEM = -5,        /* host or device allocation failed */
+    SG_E_CUDA = -6,         /* CUDA driver/runtime/NVRTC failure, or no device */
+    SG_E_COMM = -7,         /* inter-GPU transport failure */
+    SG_E_PLAN = -8,         /* partitioning / mapping failed (e.g. ILP infeasible) */
+    SG_E_SIZE = -9          /* a partition does not fit the device (shared memory) */
+} sg_status;
+
+typedef enum { SG_F32 = 0, SG_I32 = 1 } sg_dtype;
+
+/* Splitters: duplicate or weighted round-robin.  Joiners are always weighted
+ * round-robin (StreamIt `roundrobin`; default weight 1). */
+typedef enum { SG_SPLIT_DUPLICATE = 0, SG_SPLIT_ROUNDROBIN = 1 } sg_split_kind;
+
+/*
+ * Filter kinds.  PAPER.md defines no filter body; the semantics below are the
+ * readings of SURVEY.md 8(c)-3, repeated in DESIGN.md ("Readings").  x[i] is
+ * peek(i) (oldest first), y[j] the j-th pushed item.  FMA means one IEEE
+ * fused multiply-add; all other operations are single IEEE float operations.
+ *
+ *  kind                  p_i                p_f              peek / pop / push
+ *  SG_K_IDENTITY         -                  -                1 / 1 / 1
+ *  SG_K_FIR              {L, pop}           c[L]             max(L,pop)/pop/1: acc=0; acc=FMA(x[i],c[i],acc) i<L
+ *  SG_K_DELAY            {k}                -                prework pushes k zeros, then 1/1/1
+ *  SG_K_DECIMATE         {M}                -                M/M/1: y = x[0]
+ *  SG_K_EXPAND           {M}                -                1/1/M: x[0], then M-1 zeros
+ *  SG_K_COMPARE_EXCHANGE {up}               -                2/2/2: (min,max) if up else (max,min); signed
+ *  SG_K_FFT_REORDER      {n}                -                2n/2n/2n: even complex items, then odd
+ *  SG_K_COMBINE_DFT      {j}                -                2j/2j/2j: j/2 radix-2 butterflies, w=e^{-2 pi i k/j}
+ *  SG_K_FM_DEMOD         -                  {gain}           2/1/1: (float)(gain * atan((double)(x0*x1)))
+ *  SG_K_SUBTRACT         -                  -                2/2/1: x1 - x0
+ *  SG_K_AMPLIFY          -                  {k}              1/1/1: x0 * k
+ *  SG_K_ADD              {n}                -                n/n/1: s=0; s=s+x[i] in order (i32: wrapping)
+ *  SG_K_BEAM_FIR         {L, dec, frame}    wr[L], wi[L]     2F/2F/2F/dec: per-frame complex FIR, zero history
+ *  SG_K_BEAMFORM         {nch}              wr[nch], wi[nch] 2nch/2nch/2: complex weighted sum
+ *  SG_K_MAGNITUDE        -                  -                2/2/1: sqrt(FMA(a,a,b*b))
+ *
+ * dtype SG_I32 admits IDENTITY, DELAY, DECIMATE, EXPAND, COMPARE_EXCHANGE, ADD.
+ */
+typedef enum {
+    SG_K_IDENTITY = 0,
+    SG_K_FIR = 1,
+    SG_K_DELAY = 2,
+    SG_K_DECIMATE = 3,
+    SG_K_EXPAND = 4,
+    SG_K_COMPARE_EXCHANGE = 5,
+    SG_K_FFT_REORDER = 6,
+    SG_K_COMBINE_DFT = 7,
+    SG_K_FM_DEMOD = 8,
+    SG_K_SUBTRACT = 9,
+    SG_K_AMPLIFY = 10,
+    SG_K_ADD = 11,
+    SG_K_BEAM_FIR = 12,
+    SG_K_BEAMFORM = 13,
+    SG_K_MAGNITUDE = 14
+} sg_filter_kind;
+
+typedef struct {
+    sg_filter_kind kind;
+    int32_t n_i;
+    const int32_t* p_i; /* copied by sg_add_filter; caller keeps ownership */
+    int32_t n_f;
+    const float* p_f;   /* copied by sg_add_filter; caller keeps ownership */
+} sg_filter_desc;
+
+/* Handle type names carry a _t / _s suffix so that they do not collide with
+ * the function sg_plan() in C's ordinary identifier namespace. */
+typedef struct sg_graph sg_graph;
+typedef struct sg_plan_s sg_plan_t;
+
+/* Partitioner selection for sg_plan_opts.partitioner. */
+enum {
+    SG_PART_ALGORITHM1 = 0, /* the paper's Algorithm 1 with the B200 PEE */
+    SG_PART_SINGLE = 1,     /* one partition (SPSG baseline) */
+    SG_PART_PER_FILTER = 2, /* one partition per filter (splitters/joiners ride along) */
+    SG_PART_USER = 3        /* node_partition[] supplied by the caller */
+};
+
+/* Where boundary streams between GPUs travel (P2P). */
+enum {
+    SG_TRANSPORT_AUTO = 0,  /* P2P copy engine between devices; D2D copy for virtual GPUs */
+    SG_TRANSPORT_P2P = 1,   /* cudaMemcpyPeerAsync over NVLink */
+    SG_TRANSPORT_HOST = 2   /* host-staged D2H + H2D pair, as in [7] */
+};
+
+typedef struct sg_plan_opts {
+    int32_t partitioner;           /* SG_PART_*; default SG_PART_ALGORITHM1 */
+    const int32_t* node_partition; /* SG_PART_USER: partition id per node (flattened order) */
+    int32_t n_node_partition;
+    int32_t tile_iters;            /* iterations per CTA tile; 0 = chosen by the PEE */
+    int32_t threads;               /* threads per CTA; 0 = chosen by the PEE */
+    int64_t iters_per_fragment;    /* multi-GPU fragment size; 0 = auto */
+    int32_t transport;             /* SG_TRANSPORT_* */
+    int32_t virtual_gpus;          /* 1: map the G logical GPUs onto streams of one device */
+    const int32_t* devices;        /* physical device per logical GPU (NULL: 0..G-1) */
+    int32_t ilp_time_limit_ms;     /* exact branch-and-bound budget; 0 = 10000 */
+    int32_t codegen_mode;          /* 0 auto, 1 register (thread per iteration), 2 staged */
+    double link_gbps;              /* NVLink bandwidth per direction for the ILP; 0 = 770 */
+    double link_latency_us;        /* per-transfer latency Lat (Eq. III.3); 0 = 10 */
+    int32_t verbose;
+} sg_plan_opts;
+
+typedef struct sg_plan_info_s {
+    int32_t n_nodes;                 /* flattened nodes: filters, splitters, joiners */
+    int32_t n_edges;
+    int32_t n_partitions;
+    int32_t n_gpus;
+    int64_t in_per_iter;             /* input items consumed per steady-state iteration */
+    int64_t out_per_iter;            /* output items produced per steady-state iteration */
+    const int64_t* reps;             /* [n_nodes] repetition vector (gcd 1) */
+    const int64_t* init_firings;     /* [n_nodes] firings of the init schedule (may be < 0: lag) */
+    const int32_t* node_type;        /* [n_nodes] 0 filter, 1 dup splitter, 2 rr splitter, 3 joiner */
+    const int32_t* node_kind;        /* [n_nodes] sg_filter_kind or -1 */
+    const int32_t* node_partition;   /* [n_nodes] */
+    const int32_t* partition_gpu;    /* [n_partitions] */
+    const double* partition_time;    /* [n_partitions] PEE estimate T(p), ns per iteration */
+    const int32_t* partition_mode;   /* [n_partitions] 1 register, 2 staged */
+    double est_tmax;                 /* ILP objective, ns per iteration */
+    int32_t input_device;            /* device holding the caller's input */
+    int32_t output_device;           /* device holding the caller's output */
+    int64_t iters_per_fragment;
+    int32_t ilp_optimal;             /* 1 if the branch-and-bound proved optimality */
+} sg_plan_info_t;
+
+/* ---- graph construction (the top-level stream is an implicit pipeline) ---- */
+sg_status sg_graph_create(sg_dtype dtype, sg_graph** out);
+void sg_graph_destroy(sg_graph* g);
+
+/* Append a filter to the currently open pipeline.  Rates are derived from kind
+ * and parameters; parameters are validated and copied.  *elem_id (optional)
+ * receives the element's index in construction order. */
+sg_status sg_add_filter(sg_graph* g, const sg_filter_desc* desc, int32_t* elem_id);
+
+/* Append a split-join with n_branches branches to the currently open pipeline.
+ * split_w (ROUNDROBIN only) and join_w may be NULL (all weights 1); they are
+ * copied.  Each branch is then filled between sg_branch_begin / sg_branch_end,
+ * in any order; every branch must be filled (possibly empty = identity). */
+sg_status sg_add_splitjoin(sg_graph* g, sg_split_kind kind, const int32_t* split_w,
+                           const int32_t* join_w, int32_t n_branches, int32_t* sj_id);
+sg_status sg_branch_begin(sg_graph* g, int32_t sj_id, int32_t branch);
+sg_status sg_branch_end(sg_graph* g);
+
+/* ---- planning ---- */
+void sg_plan_opts_default(sg_plan_opts* o);
+
+/* Validate, flatten, solve the balance equations (SG_E_RATE), compute the init
+ * schedule, partition (Algorithm 1), build the PDG and solve the mapping ILP for
+ * n_gpus GPUs, generate one kernel per partition and compile it to sm_100a with
+ * NVRTC.  Does not need a GPU; device resources are created on first sg_run.
+ * The graph may be destroyed afterwards. */
+sg_status sg_plan(const sg_graph* g, int32_t n_gpus, const sg_plan_opts* opts, sg_plan_t** out);
+
+/* Minimal input prefix (items) needed for n_iters iterations; < 0 on error. */
+int64_t sg_input_items(const sg_plan_t* p, int64_t n_iters);
+/* Output items produced by n_iters iterations (n_iters * out_per_iter + any
+ * prework items of the output node); < 0 on error. */
+int64_t sg_output_items(const sg_plan_t* p, int64_t n_iters);
+
+/* Fills *out; pointers inside stay valid until sg_plan_destroy. */
+sg_status sg_plan_info(const sg_plan_t* p, sg_plan_info_t* out);
+
+/* Generated CUDA source of partition `part` (NUL-terminated, owned by the plan). */
+const char* sg_plan_source(const sg_plan_t* p, int32_t part);
+
+/* ---- execution ---- */
+/* Run n_iters steady-state iterations.
+ *   input  : device pointer on info.input_device holding >= sg_input_items(n_iters) items
+ *   output : device pointer on info.output_device with room for sg_output_items(n_iters) items
+ *   stream : cudaStream_t on input_device (NULL = legacy default stream); the call enqueues
+ *            work and returns; completion is ordered on `stream`.
+ * Inputs are not modified.  n_iters == 0 is a no-op.  Output is bit-identical
+ * for every plan of the same graph (Kahn determinism). */
+sg_status sg_run(sg_plan_t* p, const void* input, int64_t n_iters, void* output, void* stream);
+
+/* Same, with HOST buffers: copies in, runs, copies out, synchronises. */
+sg_status sg_run_host(sg_plan_t* p, const void* host_input, int64_t n_iters, void* host_output);
+
+/* Number of kernel launches the last sg_run enqueued (all devices). */
+int64_t sg_last_launch_count(const sg_plan_t* p);
+
+void sg_plan_destroy(sg_plan_t* p);
+
+/* Thread-local description of the last error on this thread ("" if none). */
+const char* sg_last_error(void);
+
+/* Library version string. */
+const char* sg_version(void);
+
+/* Benchmark hygiene: overwrite `bytes` of device scratch memory (> L2 size)
+ * with an nvcc-compiled sm_100a kernel enqueued on `stream`. */
+sg_status sg_flush_l2(void* scratch, int64_t bytes, void* stream);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* SG_H_ */

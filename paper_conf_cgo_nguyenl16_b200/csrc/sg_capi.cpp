@@ -1,0 +1,249 @@
+// sg_capi.cpp -- the extern "C" boundary declared in include/sg.h.
+// Every entry point catches all C++ exceptions and converts them to sg_status;
+// the message is kept in a thread-local buffer for sg_last_error().
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstring>
+#include <numeric>
+
+#include "sg_plan.h"
+#include "sg_runtime.h"
+
+struct sg_plan_s {
+    sg::Plan plan;
+};
+
+namespace {
+thread_local std::string t_err;
+
+sg_status fail(sg_status c, const std::string& m) {
+    t_err = m;
+    return c;
+}
+
+template <class F>
+sg_status guard(F&& f) {
+    try {
+        t_err.clear();
+        f();
+        return SG_OK;
+    } catch (const sg::Error& e) {
+        return fail(e.code, e.what());
+    } catch (const std::bad_alloc&) {
+        return fail(SG_E_NOMEM, "host allocation failed");
+    } catch (const std::exception& e) {
+        return fail(SG_E_ARG, e.what());
+    } catch (...) {
+        return fail(SG_E_ARG, "unknown error");
+    }
+}
+
+sg::Elem& current_pipe(sg_graph* g) { return g->elems[g->open.back()]; }
+}  // namespace
+
+extern "C" {
+
+const char* sg_last_error(void) { return t_err.c_str(); }
+const char* sg_version(void) { return "sg-b200 0.1 (sm_100a, NVRTC)"; }
+
+sg_status sg_graph_create(sg_dtype dtype, sg_graph** out) {
+    if (!out) return fail(SG_E_ARG, "out is NULL");
+    if (dtype != SG_F32 && dtype != SG_I32) return fail(SG_E_ARG, "bad dtype");
+    return guard([&] {
+        auto* g = new sg_graph();
+        g->dtype = dtype;
+        sg::Elem top;
+        top.type = sg::E_PIPE;
+        g->elems.push_back(top);
+        g->top = 0;
+        g->open.push_back(0);
+        *out = g;
+    });
+}
+
+void sg_graph_destroy(sg_graph* g) { delete g; }
+
+sg_status sg_add_filter(sg_graph* g, const sg_filter_desc* d, int32_t* elem_id) {
+    if (!g || !d) return fail(SG_E_ARG, "NULL argument");
+    if (d->n_i < 0 || d->n_f < 0 || (d->n_i && !d->p_i) || (d->n_f && !d->p_f)) return fail(SG_E_ARG, "bad parameter arrays");
+    return guard([&] {
+        sg::Elem e;
+        e.type = sg::E_FILTER;
+        e.kind = (int)d->kind;
+        e.iv.assign(d->p_i, d->p_i + d->n_i);
+        e.fv.assign(d->p_f, d->p_f + d->n_f);
+        sg::kind_rates(e.kind, e.iv, e.fv, g->dtype);  // validates (throws)
+        int id = (int)g->elems.size();
+        g->elems.push_back(std::move(e));
+        current_pipe(g).kids.push_back(id);
+        if (elem_id) *elem_id = id;
+    });
+}
+
+sg_status sg_add_splitjoin(sg_graph* g, sg_split_kind kind, const int32_t* split_w, const int32_t* join_w,
+                           int32_t nb, int32_t* sj_id) {
+    if (!g) return fail(SG_E_ARG, "NULL graph");
+    if (nb < 1) return fail(SG_E_ARG, "split-join needs >= 1 branch");
+    if (kind != SG_SPLIT_DUPLICATE && kind != SG_SPLIT_ROUNDROBIN) return fail(SG_E_ARG, "bad split kind");
+    return guard([&] {
+        sg::Elem e;
+        e.type = sg::E_SJ;
+        e.split_kind = kind == SG_SPLIT_DUPLICATE ? 0 : 1;
+        e.split_w.assign(nb, 1);
+        e.join_w.assign(nb, 1);
+        if (kind == SG_SPLIT_ROUNDROBIN && split_w) e.split_w.assign(split_w, split_w + nb);
+        if (join_w) e.join_w.assign(join_w, join_w + nb);
+        for (int b = 0; b < nb; b++)
+            if (e.split_w[b] < 1 || e.join_w[b] < 1) throw sg::Error(SG_E_ARG, "weights must be >= 1");
+        int id = (int)g->elems.size();
+        g->elems.push_back(e);
+        for (int b = 0; b < nb; b++) {
+            sg::Elem p;
+            p.type = sg::E_PIPE;
+            g->elems.push_back(p);
+            g->elems[id].branches.push_back((int)g->elems.size() - 1);
+        }
+        g->elems[id].branch_done.assign(nb, false);
+        current_pipe(g).kids.push_back(id);
+        if (sj_id) *sj_id = id;
+    });
+}
+
+sg_status sg_branch_begin(sg_graph* g, int32_t sj, int32_t b) {
+    if (!g) return fail(SG_E_ARG, "NULL graph");
+    if (sj < 0 || sj >= (int)g->elems.size() || g->elems[sj].type != sg::E_SJ) return fail(SG_E_ARG, "not a split-join id");
+    sg::Elem& e = g->elems[sj];
+    if (b < 0 || b >= (int)e.branches.size()) return fail(SG_E_ARG, "branch out of range");
+    if (e.branch_done[b]) return fail(SG_E_STRUCTURE, "branch already filled");
+    // the split-join must belong to the currently open pipeline
+    const auto& kids = current_pipe(g).kids;
+    if (std::find(kids.begin(), kids.end(), sj) == kids.end())
+        return fail(SG_E_STRUCTURE, "split-join is not in the currently open pipeline");
+    g->open.push_back(e.branches[b]);
+    g->open_branch.push_back({sj, b});
+    return SG_OK;
+}
+
+sg_status sg_branch_end(sg_graph* g) {
+    if (!g) return fail(SG_E_ARG, "NULL graph");
+    if (g->open.size() <= 1) return fail(SG_E_STRUCTURE, "no open branch");
+    auto sb = g->open_branch.back();
+    g->elems[sb.first].branch_done[sb.second] = true;
+    g->open.pop_back();
+    g->open_branch.pop_back();
+    return SG_OK;
+}
+
+void sg_plan_opts_default(sg_plan_opts* o) {
+    if (!o) return;
+    std::memset(o, 0, sizeof(*o));
+    o->partitioner = SG_PART_ALGORITHM1;
+    o->transport = SG_TRANSPORT_AUTO;
+}
+
+sg_status sg_plan(const sg_graph* g, int32_t n_gpus, const sg_plan_opts* opts, sg_plan_t** out) {
+    if (!g || !out) return fail(SG_E_ARG, "NULL argument");
+    if (n_gpus < 1 || n_gpus > 64) return fail(SG_E_ARG, "n_gpus must be in [1, 64]");
+    return guard([&] {
+        sg_plan_opts o;
+        sg_plan_opts_default(&o);
+        if (opts) o = *opts;
+        auto* p = new sg_plan_s();
+        try {
+            sg::build_plan(p->plan, *g, n_gpus, o);
+        } catch (...) {
+            delete p;
+            throw;
+        }
+        *out = p;
+    });
+}
+
+int64_t sg_input_items(const sg_plan_t* p, int64_t n) {
+    if (!p || n < 0) return -1;
+    return p->plan.flat.input_items(n);
+}
+int64_t sg_output_items(const sg_plan_t* p, int64_t n) {
+    if (!p || n < 0) return -1;
+    return p->plan.flat.output_items(n);
+}
+
+sg_status sg_plan_info(const sg_plan_t* pp, sg_plan_info_t* o) {
+    if (!pp || !o) return fail(SG_E_ARG, "NULL argument");
+    const sg::Plan& p = pp->plan;
+    std::memset(o, 0, sizeof(*o));
+    o->n_nodes = (int32_t)p.flat.nodes.size();
+    o->n_edges = (int32_t)p.flat.edges.size();
+    o->n_partitions = (int32_t)p.parts.size();
+    o->n_gpus = p.G;
+    o->in_per_iter = p.flat.in_per_iter;
+    o->out_per_iter = p.flat.out_per_iter;
+    o->reps = p.reps.data();
+    o->init_firings = p.ninit.data();
+    o->node_type = p.node_type.data();
+    o->node_kind = p.node_kind.data();
+    o->node_partition = p.node_part.data();
+    o->partition_gpu = p.part_gpu.data();
+    o->partition_time = p.part_time.data();
+    o->partition_mode = p.part_mode.data();
+    o->est_tmax = p.est_tmax;
+    o->input_device = p.devices[p.input_gpu];
+    o->output_device = p.devices[p.output_gpu];
+    o->iters_per_fragment = p.iters_per_fragment;
+    o->ilp_optimal = p.ilp_optimal ? 1 : 0;
+    return SG_OK;
+}
+
+const char* sg_plan_source(const sg_plan_t* p, int32_t part) {
+    if (!p || part < 0 || part >= (int)p->plan.kernels.size()) return nullptr;
+    return p->plan.kernels[part].ki.source.c_str();
+}
+
+sg_status sg_run(sg_plan_t* p, const void* input, int64_t n, void* output, void* stream) {
+    if (!p) return fail(SG_E_ARG, "NULL plan");
+    if (n < 0) return fail(SG_E_ARG, "negative n_iters");
+    if (n == 0) return SG_OK;
+    if (!input || !output) return fail(SG_E_ARG, "NULL buffer");
+    return guard([&] { p->plan.run(input, n, output, (cudaStream_t)stream); });
+}
+
+sg_status sg_run_host(sg_plan_t* p, const void* hin, int64_t n, void* hout) {
+    if (!p) return fail(SG_E_ARG, "NULL plan");
+    if (n < 0) return fail(SG_E_ARG, "negative n_iters");
+    if (n == 0) return SG_OK;
+    if (!hin || !hout) return fail(SG_E_ARG, "NULL buffer");
+    return guard([&] {
+        sg::Plan& pl = p->plan;
+        int64_t ni = pl.flat.input_items(n), no = pl.flat.output_items(n);
+        int din = pl.devices[pl.input_gpu], dout = pl.devices[pl.output_gpu];
+        void *din_p = nullptr, *dout_p = nullptr;
+        auto chk = [](cudaError_t e, const char* w) {
+            if (e != cudaSuccess) throw sg::Error(SG_E_CUDA, std::string(w) + ": " + cudaGetErrorString(e));
+        };
+        chk(cudaSetDevice(din), "cudaSetDevice");
+        chk(cudaMalloc(&din_p, (size_t)std::max<int64_t>(ni, 1) * 4), "cudaMalloc");
+        chk(cudaMemcpy(din_p, hin, (size_t)ni * 4, cudaMemcpyHostToDevice), "H2D");
+        chk(cudaSetDevice(dout), "cudaSetDevice");
+        chk(cudaMalloc(&dout_p, (size_t)std::max<int64_t>(no, 1) * 4), "cudaMalloc");
+        chk(cudaSetDevice(din), "cudaSetDevice");
+        try {
+            pl.run(din_p, n, dout_p, nullptr);
+            chk(cudaSetDevice(dout), "cudaSetDevice");
+            chk(cudaDeviceSynchronize(), "sync");
+            chk(cudaMemcpy(hout, dout_p, (size_t)no * 4, cudaMemcpyDeviceToHost), "D2H");
+        } catch (...) {
+            cudaFree(din_p);
+            cudaFree(dout_p);
+            throw;
+        }
+        cudaFree(din_p);
+        cudaFree(dout_p);
+    });
+}
+
+int64_t sg_last_launch_count(const sg_plan_t* p) { return p ? p->plan.last_launches : -1; }
+
+void sg_plan_destroy(sg_plan_t* p) { delete p; }
+
+}  // extern "C"

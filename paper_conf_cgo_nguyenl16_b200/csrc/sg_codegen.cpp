@@ -1,0 +1,1020 @@
+// sg_codegen.cpp -- one CUDA kernel per partition ("one partition corresponds
+// to one kernel"; code generator PAPER.md:274-277).
+//
+// Two emitters share one static view resolver:
+//
+//  * View resolution.  Splitters, joiners and the pure data-movement filters
+//    (IDENTITY, DELAY, DECIMATE, EXPAND, FFT_REORDER) never execute: a read of
+//    position p on their output is rewritten into a read of their input at a
+//    compile-time-resolved position (or a constant zero).  This is the paper's
+//    future-work "elimination of splitters and joiners ... re-adjust the index
+//    of input data of the follow-up filter" (Figs. 5.1/5.2),
+//    generalised to every filter that only rearranges data.  Positions are kept
+//    as affine forms of the runtime loop variables; a map whose divisor does
+//    not divide every coefficient falls back to a generated runtime reader.
+//
+//  * Register mode (thread per iteration).  When no node of the partition
+//    needs items of a neighbouring iteration (halo 0, peek == pop, aligned init
+//    offsets), each thread runs one whole steady-state iteration with every
+//    FIFO item an SSA register: the static schedule is flattened by symbolic
+//    execution; inputs are loaded lazily from a padded shared-memory row,
+//    outputs stored eagerly.  (BitonicSort, FFT.)
+//
+//  * Staged mode (tile of W iterations per CTA, the paper's one-kernel-per-
+//    partition model with FIFOs in shared memory).  Compute
+//    filters are grouped into dependence levels; all firings of one level run
+//    in parallel across the CTA, one barrier per level; buffers are placed by
+//    liveness (the shared-memory footprint of Fig. 3.2).
+//    Peek windows that reach into the previous tile are recomputed (halo), so
+//    tiles, fragments and GPUs never share state.  FIRs are register-blocked.
+//    (FMRadio, FilterBank, BeamFormer, any graph.)
+#include "sg_codegen.h"
+
+#include <algorithm>
+#include <cmath>
+#include <cstdio>
+#include <cstring>
+#include <functional>
+#include <map>
+#include <numeric>
+#include <set>
+#include <sstream>
+
+namespace sg {
+
+const char* kDeviceHeader =
+#include "sg_device_embed.inc"
+    ;
+
+static int64_t fdiv(int64_t a, int64_t b) {
+    int64_t q = a / b, r = a % b;
+    return (r != 0 && ((r < 0) != (b < 0))) ? q - 1 : q;
+}
+static int64_t fmodp(int64_t a, int64_t b) { return a - fdiv(a, b) * b; }
+
+bool is_view_kind(int k) {
+    return k == SG_K_IDENTITY || k == SG_K_DELAY || k == SG_K_DECIMATE || k == SG_K_EXPAND || k == SG_K_FFT_REORDER;
+}
+static bool is_view_node(const Node& n) { return n.type != N_FILTER || is_view_kind(n.kind); }
+
+void node_work(const Flat& f, int v, int64_t& flops, int64_t& intops, int64_t& dfma) {
+    const Node& n = f.nodes[v];
+    flops = intops = dfma = 0;
+    if (n.type != N_FILTER) return;
+    int64_t per = 0;
+    switch (n.kind) {
+    case SG_K_FIR: per = 2LL * n.iv[0]; break;
+    case SG_K_COMBINE_DFT: per = 10LL * (n.iv[0] / 2); break;
+    case SG_K_FM_DEMOD: per = 1; dfma = n.rep; break;
+    case SG_K_SUBTRACT: case SG_K_AMPLIFY: per = 1; break;
+    case SG_K_ADD: if (f.dtype == SG_F32) per = n.iv[0]; else intops = n.rep * n.iv[0]; break;
+    case SG_K_BEAM_FIR: per = 8LL * n.iv[0] * (n.iv[2] / n.iv[1]); break;
+    case SG_K_BEAMFORM: per = 8LL * n.iv[0]; break;
+    case SG_K_MAGNITUDE: per = 3; break;
+    case SG_K_COMPARE_EXCHANGE: intops = 2 * n.rep; break;
+    default: break;
+    }
+    flops = per * n.rep;
+}
+
+// ------------------------------------------------------------ affine forms
+struct Lin {
+    std::vector<std::pair<std::string, int64_t>> t;
+    int64_t c = 0;
+    static Lin k(int64_t c) { Lin l; l.c = c; return l; }
+    static Lin v(const std::string& name, int64_t a, int64_t c = 0) { Lin l; l.t.push_back({name, a}); l.c = c; return l; }
+    bool divisible(int64_t m) const {
+        for (auto& p : t) if (p.second % m) return false;
+        return true;
+    }
+    Lin divf(int64_t m) const {
+        Lin r;
+        for (auto& p : t) if (p.second / m) r.t.push_back({p.first, p.second / m});
+        r.c = fdiv(c, m);
+        return r;
+    }
+    int64_t modc(int64_t m) const { return fmodp(c, m); }
+    Lin scaled(int64_t s) const {
+        Lin r;
+        for (auto& p : t) if (p.second * s != 0) r.t.push_back({p.first, p.second * s});
+        r.c = c * s;
+        return r;
+    }
+    Lin plus(int64_t d) const { Lin r = *this; r.c += d; return r; }
+    bool is_const() const { return t.empty(); }
+    int64_t coef(const std::string& name) const {
+        for (auto& p : t) if (p.first == name) return p.second;
+        return 0;
+    }
+    std::string vars() const {  // "a*x + b*y" without constant, or ""
+        std::string s;
+        for (auto& p : t) {
+            if (!s.empty()) s += " + ";
+            if (p.second == 1) s += p.first;
+            else s += "(" + std::to_string(p.second) + ")*" + p.first;
+        }
+        return s;
+    }
+    std::string str() const {
+        std::string s = vars();
+        if (s.empty()) return std::to_string(c);
+        if (c) s += " + (" + std::to_string(c) + ")";
+        return "(" + s + ")";
+    }
+};
+
+struct Ref {
+    enum K { PHYS, ZERO, RUNTIME } k = PHYS;
+    int edge = -1;
+    Lin pos;
+};
+
+static std::string hexf(float x) {
+    if (!std::isfinite(x)) throw Error(SG_E_ARG, "non-finite filter parameter");
+    char b[64];
+    if (x == 0.0f) return std::signbit(x) ? "(-0.0f)" : "0.0f";
+    std::snprintf(b, sizeof b, "%af", (double)x);
+    return std::string("(") + b + ")";
+}
+
+void partition_boundary(const Flat& f, const std::vector<int>& nodes, std::vector<int>& ins, std::vector<int>& outs) {
+    std::vector<char> in(f.nodes.size(), 0);
+    for (int v : nodes) in[v] = 1;
+    ins.clear();
+    outs.clear();
+    for (int e = 0; e < (int)f.edges.size(); e++) {
+        const Edge& ed = f.edges[e];
+        bool s_in = ed.src >= 0 && in[ed.src], d_in = ed.dst >= 0 && in[ed.dst];
+        if (d_in && !s_in) ins.push_back(e);
+        if (s_in && !d_in) outs.push_back(e);
+    }
+}
+
+void edge_window(const Flat& f, int e, int64_t& lo, int64_t& extra) {
+    const Edge& ed = f.edges[e];
+    if (ed.dst < 0) {  // graph output: produced positions (prework items handled apart)
+        lo = ed.pre;
+        extra = 0;
+        return;
+    }
+    const Node& v = f.nodes[ed.dst];
+    lo = (v.ninit - v.halo) * ed.pop;
+    extra = v.halo * ed.pop + ed.peek - ed.pop;
+}
+
+// ---------------------------------------------------------------- resolver
+class Resolver {
+public:
+    Resolver(const Flat& f, const std::vector<int>& nodes) : f_(f), inpart_(f.nodes.size(), 0) {
+        for (int v : nodes) inpart_[v] = 1;
+    }
+    bool phys(int e) const {
+        const Edge& ed = f_.edges[e];
+        if (ed.src < 0 || !inpart_[ed.src]) return true;  // boundary input
+        return !is_view_node(f_.nodes[ed.src]);
+    }
+    Ref resolve(int e, Lin pos) const {
+        for (int guard = 0; guard < 100000; guard++) {
+            if (phys(e)) return {Ref::PHYS, e, pos};
+            const Edge& ed = f_.edges[e];
+            const Node& u = f_.nodes[ed.src];
+            switch (u.type) {
+            case N_SPLIT_DUP: e = u.in[0]; continue;
+            case N_SPLIT_RR: {
+                int b = ed.sport;
+                int64_t w = u.w[b], P = 0;
+                for (int i = 0; i < b; i++) P += u.w[i];
+                if (!pos.divisible(w)) return {Ref::RUNTIME, e, pos};
+                Lin q = pos.divf(w);
+                int64_t r = pos.modc(w);
+                pos = q.scaled(u.wsum).plus(P + r);
+                e = u.in[0];
+                continue;
+            }
+            case N_JOIN: {
+                int64_t S = u.wsum;
+                if (!pos.divisible(S)) return {Ref::RUNTIME, e, pos};
+                Lin q = pos.divf(S);
+                int64_t o = pos.modc(S), P = 0;
+                int b = 0;
+                while (o >= P + u.w[b]) { P += u.w[b]; b++; }
+                pos = q.scaled(u.w[b]).plus(o - P);
+                e = u.in[b];
+                continue;
+            }
+            case N_FILTER:
+                switch (u.kind) {
+                case SG_K_IDENTITY: e = u.in[0]; continue;
+                case SG_K_DELAY: pos = pos.plus(-(int64_t)u.iv[0]); e = u.in[0]; continue;
+                case SG_K_DECIMATE: pos = pos.scaled(u.iv[0]); e = u.in[0]; continue;
+                case SG_K_EXPAND: {
+                    int64_t M = u.iv[0];
+                    if (!pos.divisible(M)) return {Ref::RUNTIME, e, pos};
+                    if (pos.modc(M) != 0) return {Ref::ZERO, -1, Lin()};
+                    pos = pos.divf(M);
+                    e = u.in[0];
+                    continue;
+                }
+                case SG_K_FFT_REORDER: {
+                    int64_t n = u.iv[0], F = 2 * n;
+                    if (!pos.divisible(F)) return {Ref::RUNTIME, e, pos};
+                    Lin q = pos.divf(F);
+                    int64_t o = pos.modc(F), m = o / 2, r = o % 2;
+                    int64_t sc = m < n / 2 ? 2 * m : 2 * (m - n / 2) + 1;
+                    pos = q.scaled(F).plus(2 * sc + r);
+                    e = u.in[0];
+                    continue;
+                }
+                default: break;
+                }
+                break;
+            }
+            throw Error(SG_E_UNSUPPORTED, "internal: unresolvable view");
+        }
+        throw Error(SG_E_UNSUPPORTED, "internal: view chain too long");
+    }
+    // Physical edges reachable backwards from e through in-partition views.
+    void sources(int e, std::set<int>& out) const {
+        if (phys(e)) { out.insert(e); return; }
+        const Node& u = f_.nodes[f_.edges[e].src];
+        for (int i : u.in) sources(i, out);
+    }
+
+private:
+    const Flat& f_;
+    std::vector<char> inpart_;
+};
+
+bool register_mode_eligible(const Flat& f, const std::vector<int>& nodes, std::string* why) {
+    auto fail = [&](const std::string& s) { if (why) *why = s; return false; };
+    std::vector<int> ins, outs;
+    partition_boundary(f, nodes, ins, outs);
+    if (ins.size() != 1 || outs.size() != 1) return fail("needs exactly one boundary input and output");
+    std::vector<char> in(f.nodes.size(), 0);
+    for (int v : nodes) in[v] = 1;
+    int64_t live = 0;
+    for (int v : nodes) {
+        const Node& n = f.nodes[v];
+        if (n.halo != 0) return fail("node " + std::to_string(v) + " has a halo");
+        if (n.type == N_FILTER && n.kind == SG_K_BEAM_FIR) return fail("frame FIR");
+        if (n.type == N_FILTER && n.prework) return fail("prework");
+        if (n.type == N_FILTER && !is_view_kind(n.kind)) live = std::max(live, n.peek + n.push);
+        for (int e : n.in) {
+            const Edge& ed = f.edges[e];
+            if (ed.peek != ed.pop) return fail("peeking edge");
+            if (ed.src >= 0 && in[ed.src]) {
+                const Node& u = f.nodes[ed.src];
+                if (n.ninit * ed.pop != ed.pre + u.ninit * ed.push) return fail("misaligned init offsets");
+            }
+        }
+    }
+    const Edge& eo = f.edges[outs[0]];
+    if (eo.pre) return fail("output prework");
+    if (eo.dst >= 0) {
+        int64_t lo, ex;
+        edge_window(f, outs[0], lo, ex);
+        if (ex != 0 || lo != eo.pre + f.nodes[eo.src].ninit * eo.push) return fail("output window misaligned");
+    }
+    const Edge& ei = f.edges[ins[0]];
+    if (ei.per_iter > 256 || eo.per_iter > 256 || live > 512) return fail("iteration too large for registers");
+    return true;
+}
+
+// ---------------------------------------------------------------- common
+class GenBase {
+public:
+    GenBase(const Flat& f, const std::vector<int>& nodes, int part)
+        : f_(f), nodes_(nodes), part_(part), R_(f, nodes) {
+        T_ = f.dtype == SG_F32 ? "float" : "int";
+        partition_boundary(f, nodes, ins_, outs_);
+    }
+
+protected:
+    const Flat& f_;
+    std::vector<int> nodes_;
+    int part_;
+    Resolver R_;
+    std::string T_;
+    std::vector<int> ins_, outs_;
+    std::ostringstream consts_;
+    std::map<std::vector<float>, std::string> pool_;
+
+    std::string const_array(const std::vector<float>& v) {
+        auto it = pool_.find(v);
+        if (it != pool_.end()) return it->second;
+        std::string name = "SG_C" + std::to_string(pool_.size());
+        consts_ << "__constant__ float " << name << "[" << std::max<size_t>(1, v.size()) << "] = {";
+        for (size_t i = 0; i < v.size(); i++) consts_ << (i ? "," : "") << (i % 8 == 0 ? "\n  " : "") << hexf(v[i]);
+        if (v.empty()) consts_ << "0.0f";
+        consts_ << "};\n";
+        pool_[v] = name;
+        return name;
+    }
+    // Twiddles of CombineDFT(j): w_k = (cos(2 pi k / j), -sin(2 pi k / j)), double -> float.
+    std::pair<std::string, std::string> twiddles(int j) {
+        std::vector<float> wr(j / 2), wi(j / 2);
+        for (int k = 0; k < j / 2; k++) {
+            double a = 2.0 * M_PI * (double)k / (double)j;
+            wr[k] = (float)std::cos(a);
+            wi[k] = (float)(-std::sin(a));
+        }
+        return {const_array(wr), const_array(wi)};
+    }
+    // Work-function call for one firing of compute filter v: x_ -> y_.
+    std::string work_call(int v) {
+        const Node& n = f_.nodes[v];
+        const std::string& T = T_;
+        switch (n.kind) {
+        case SG_K_FIR: return "sg_work_fir<" + std::to_string(n.peek) + "," + std::to_string(n.iv[0]) + ">(x_, y_, " +
+                              const_array(n.fv) + ");";
+        case SG_K_COMPARE_EXCHANGE:
+            return "sg_work_compare_exchange<" + T + "," + (n.iv[0] ? "true" : "false") + ">(x_, y_);";
+        case SG_K_COMBINE_DFT: {
+            auto tw = twiddles(n.iv[0]);
+            return "sg_work_combine_dft<" + std::to_string(n.iv[0]) + ">(x_, y_, " + tw.first + ", " + tw.second + ");";
+        }
+        case SG_K_FM_DEMOD: return "sg_work_fm_demod(x_, y_, " + hexf(n.fv[0]) + ");";
+        case SG_K_SUBTRACT: return "sg_work_subtract(x_, y_);";
+        case SG_K_AMPLIFY: return "sg_work_amplify(x_, y_, " + hexf(n.fv[0]) + ");";
+        case SG_K_ADD: return "sg_work_add<" + std::to_string(n.iv[0]) + ">(x_, y_);";
+        case SG_K_BEAMFORM: {
+            std::vector<float> wr(n.fv.begin(), n.fv.begin() + n.iv[0]), wi(n.fv.begin() + n.iv[0], n.fv.end());
+            return "sg_work_beamform<" + std::to_string(n.iv[0]) + ">(x_, y_, " + const_array(wr) + ", " +
+                   const_array(wi) + ");";
+        }
+        case SG_K_MAGNITUDE: return "sg_work_magnitude(x_, y_);";
+        default: break;
+        }
+        throw Error(SG_E_UNSUPPORTED, std::string("no work function for ") + kind_name(n.kind));
+    }
+    std::string header(const char* mode) {
+        std::ostringstream h;
+        h << "// generated by sg_codegen.cpp: partition " << part_ << " (" << mode << " mode), " << nodes_.size()
+          << " nodes\n#include \"sg_device.cuh\"\n";
+        return h.str();
+    }
+    void fill_io(KernelInfo& ki) {
+        ki.in_edges = ins_;
+        ki.out_edges = outs_;
+        for (int e : ins_) {
+            int64_t lo, ex;
+            edge_window(f_, e, lo, ex);
+            ki.in_lo.push_back(lo);
+            ki.in_extra.push_back(ex);
+        }
+        for (int e : outs_) {
+            int64_t lo, ex;
+            edge_window(f_, e, lo, ex);
+            ki.out_lo.push_back(lo);
+            ki.out_extra.push_back(ex);
+        }
+        for (int v : nodes_) {
+            int64_t a, b, c;
+            node_work(f_, v, a, b, c);
+            ki.flops_per_iter += a;
+            ki.intops_per_iter += b;
+            ki.dfma_per_iter += c;
+        }
+    }
+    // kernel argument block: all 8-byte words
+    //   in ptr[NI], in_base[NI], in_limit[NI], out ptr[NO], out_base[NO], k_begin, k_end
+    std::string args_struct() {
+        size_t ni = ins_.size(), no = outs_.size();
+        std::ostringstream s;
+        s << "struct SgArgs { long long v[" << (3 * ni + 2 * no + 2) << "]; };\n";
+        s << "#define SG_IN(i) (reinterpret_cast<const " << T_ << "*>(a.v[(i)]))\n";
+        s << "#define SG_IN_BASE(i) (a.v[" << ni << " + (i)])\n";
+        s << "#define SG_IN_LIMIT(i) (a.v[" << 2 * ni << " + (i)])\n";
+        s << "#define SG_OUT(i) (reinterpret_cast<" << T_ << "*>(a.v[" << 3 * ni << " + (i)]))\n";
+        s << "#define SG_OUT_BASE(i) (a.v[" << 3 * ni + no << " + (i)])\n";
+        s << "#define SG_K_BEGIN (a.v[" << 3 * ni + 2 * no << "])\n";
+        s << "#define SG_K_END (a.v[" << 3 * ni + 2 * no + 1 << "])\n";
+        return s.str();
+    }
+};
+
+// ------------------------------------------------------------ register mode
+class RegGen : public GenBase {
+public:
+    using GenBase::GenBase;
+
+    KernelInfo run(const CodegenOpts& opt) {
+        KernelInfo ki;
+        ki.mode = 1;
+        ki.name = "sg_part" + std::to_string(part_);
+        fill_io(ki);
+        ein_ = ins_[0];
+        eout_ = outs_[0];
+        const Edge& ei = f_.edges[ein_];
+        const Edge& eo = f_.edges[eout_];
+        PIN_ = ei.per_iter;
+        POUT_ = eo.per_iter;
+        off_in_ = ki.in_lo[0];
+        off_out_ = ki.out_lo[0];
+        vin_ = PIN_ % 4 == 0;
+        vout_ = POUT_ % 4 == 0;
+        RIN_S_ = row_stride(PIN_);
+        ROUT_S_ = row_stride(POUT_);
+        body_.str("");
+        emit_body();
+        int bytes_per_thread = (int)((RIN_S_ + ROUT_S_) * 4);
+        int NT = opt.threads;
+        if (NT <= 0) {
+            NT = 256;
+            while (NT > 32 && (size_t)NT * bytes_per_thread > 72 * 1024) NT /= 2;
+        }
+        ki.threads = NT;
+        ki.tile = NT;
+        ki.smem = (size_t)NT * bytes_per_thread;
+        ki.min_blocks = std::max(1, std::min(8, (int)((200 * 1024) / std::max<size_t>(1, ki.smem))));
+        if (bytes_per_thread * NT > 200 * 1024) ki.min_blocks = 1;
+        std::ostringstream src;
+        src << header("register") << consts_.str() << args_struct();
+        src << "#define NT " << NT << "\n";
+        src << "extern \"C\" __global__ void __launch_bounds__(NT, " << ki.min_blocks << ") " << ki.name
+            << "(const SgArgs a) {\n"
+            << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
+            << "  " << T_ << "* s_in = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
+            << "  " << T_ << "* s_out = s_in + NT * " << RIN_S_ << ";\n"
+            << "  const " << T_ << "* gin = SG_IN(0);\n"
+            << "  " << T_ << "* gout = SG_OUT(0);\n"
+            << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * NT; t0 < SG_K_END; t0 += (long long)gridDim.x * NT) {\n"
+            << "    const int nt = (int)min((long long)NT, SG_K_END - t0);\n"
+            << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
+            << "    if (" << (vin_ ? "(reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0" : "false") << ")\n"
+            << "      sg_rows_g2s_v4<" << T_ << ", " << PIN_ << ", " << RIN_S_ << ", NT>(gsrc, s_in, nt);\n"
+            << "    else\n"
+            << "      sg_rows_g2s_v1<" << T_ << ", " << PIN_ << ", " << RIN_S_ << ", NT>(gsrc, s_in, nt);\n"
+            << "    __syncthreads();\n"
+            << "    if (threadIdx.x < nt) {\n"
+            << "      const " << T_ << "* xr = s_in + threadIdx.x * " << RIN_S_ << ";\n"
+            << "      " << T_ << "* yr = s_out + threadIdx.x * " << ROUT_S_ << ";\n"
+            << body_.str()
+            << "    }\n"
+            << "    __syncthreads();\n"
+            << "    " << T_ << "* gdst = gout + (t0 * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
+            << "    if (" << (vout_ ? "(reinterpret_cast<unsigned long long>(gdst) & 15ull) == 0" : "false") << ")\n"
+            << "      sg_rows_s2g_v4<" << T_ << ", " << POUT_ << ", " << ROUT_S_ << ", NT>(s_out, gdst, nt);\n"
+            << "    else\n"
+            << "      sg_rows_s2g_v1<" << T_ << ", " << POUT_ << ", " << ROUT_S_ << ", NT>(s_out, gdst, nt);\n"
+            << "  }\n}\n";
+        ki.source = src.str();
+        return ki;
+    }
+
+private:
+    int ein_ = -1, eout_ = -1;
+    int64_t PIN_ = 0, POUT_ = 0, off_in_ = 0, off_out_ = 0, RIN_S_ = 0, ROUT_S_ = 0;
+    bool vin_ = false, vout_ = false;
+    std::ostringstream body_;
+    std::map<std::pair<int, int64_t>, std::string> val_;  // (phys edge, local pos) -> SSA name
+    std::set<int64_t> loaded_;                            // input groups / items loaded
+    int nv_ = 0;
+
+    // Row stride (items) in shared memory: 128-bit row reads by 8 consecutive
+    // threads hit 8 distinct 16-byte bank groups iff stride/4 is odd; scalar
+    // rows use an odd stride.
+    static int64_t row_stride(int64_t P) {
+        if (P % 4 == 0) return (P / 4) % 2 == 1 ? P : P + 4;
+        return P % 2 == 1 ? P : P + 1;
+    }
+    std::string input_name(int64_t pos) {
+        int64_t r = pos - off_in_;
+        if (r < 0 || r >= PIN_) throw Error(SG_E_UNSUPPORTED, "internal: register-mode input out of row");
+        if (vin_) {
+            int64_t g = r / 4;
+            if (!loaded_.count(g)) {
+                loaded_.insert(g);
+                body_ << "      const " << (T_ == "float" ? "float4" : "int4") << " iq" << g << " = reinterpret_cast<const "
+                      << (T_ == "float" ? "float4" : "int4") << "*>(xr)[" << g << "];\n";
+            }
+            static const char* comp[4] = {"x", "y", "z", "w"};
+            return "iq" + std::to_string(g) + "." + comp[r % 4];
+        }
+        if (!loaded_.count(r)) {
+            loaded_.insert(r);
+            body_ << "      const " << T_ << " xi" << r << " = xr[" << r << "];\n";
+        }
+        return "xi" + std::to_string(r);
+    }
+    std::string value_of(const Ref& rf) {
+        if (rf.k == Ref::ZERO) return "(" + T_ + ")0";
+        if (rf.k != Ref::PHYS || !rf.pos.is_const()) throw Error(SG_E_UNSUPPORTED, "internal: dynamic ref in register mode");
+        if (rf.edge == ein_) return input_name(rf.pos.c);
+        auto it = val_.find({rf.edge, rf.pos.c});
+        if (it == val_.end()) throw Error(SG_E_UNSUPPORTED, "internal: value used before definition");
+        return it->second;
+    }
+    void emit_body() {
+        // output sources and readiness bookkeeping
+        std::vector<Ref> osrc(POUT_);
+        std::map<std::pair<int, int64_t>, std::vector<int64_t>> waiters;
+        int gs = vout_ ? 4 : 1;
+        std::vector<int> pending((POUT_ + gs - 1) / gs, 0);
+        for (int64_t p = 0; p < POUT_; p++) {
+            osrc[p] = R_.resolve(eout_, Lin::k(off_out_ + p));
+            if (osrc[p].k == Ref::PHYS && osrc[p].edge != ein_) {
+                waiters[{osrc[p].edge, osrc[p].pos.c}].push_back(p / gs);
+                pending[p / gs]++;
+            }
+        }
+        std::vector<char> stored(pending.size(), 0);
+        auto store_group = [&](int64_t g) {
+            if (stored[g]) return;
+            stored[g] = 1;
+            if (vout_) {
+                std::string v[4];
+                for (int i = 0; i < 4; i++) v[i] = value_of(osrc[4 * g + i]);
+                body_ << "      reinterpret_cast<" << (T_ == "float" ? "float4" : "int4") << "*>(yr)[" << g << "] = make_"
+                      << (T_ == "float" ? "float4" : "int4") << "(" << v[0] << ", " << v[1] << ", " << v[2] << ", " << v[3]
+                      << ");\n";
+            } else {
+                body_ << "      yr[" << g << "] = " << value_of(osrc[g]) << ";\n";
+            }
+        };
+        for (size_t g = 0; g < pending.size(); g++)
+            if (pending[g] == 0) store_group((int64_t)g);
+        for (int v : nodes_) {
+            const Node& n = f_.nodes[v];
+            if (is_view_node(n)) continue;
+            int ein = n.in[0], eo = n.out[0];
+            for (int64_t j = 0; j < n.rep; j++) {
+                int64_t lf = n.ninit + j;
+                std::vector<std::string> xs(n.peek);
+                for (int64_t i = 0; i < n.peek; i++) xs[i] = value_of(R_.resolve(ein, Lin::k(lf * n.pop + i)));
+                std::vector<std::string> ys(n.push);
+                body_ << "      " << T_ << " ";
+                for (int64_t jj = 0; jj < n.push; jj++) {
+                    ys[jj] = "v" + std::to_string(nv_++);
+                    body_ << (jj ? ", " : "") << ys[jj];
+                }
+                body_ << ";\n      { const " << T_ << " x_[" << n.peek << "] = {";
+                for (int64_t i = 0; i < n.peek; i++) body_ << (i ? ", " : "") << xs[i];
+                body_ << "}; " << T_ << " y_[" << n.push << "]; " << work_call(v);
+                for (int64_t jj = 0; jj < n.push; jj++) body_ << " " << ys[jj] << " = y_[" << jj << "];";
+                body_ << " }\n";
+                const Edge& oe = f_.edges[eo];
+                for (int64_t jj = 0; jj < n.push; jj++) {
+                    int64_t pos = oe.pre + lf * n.push + jj;
+                    val_[{eo, pos}] = ys[jj];
+                    auto w = waiters.find({eo, pos});
+                    if (w != waiters.end())
+                        for (int64_t g : w->second)
+                            if (--pending[g] == 0) store_group(g);
+                }
+            }
+        }
+        for (size_t g = 0; g < pending.size(); g++)
+            if (!stored[g]) throw Error(SG_E_UNSUPPORTED, "internal: output group never produced");
+    }
+};
+
+// -------------------------------------------------------------- staged mode
+class StageGen : public GenBase {
+public:
+    using GenBase::GenBase;
+
+    KernelInfo run(const CodegenOpts& opt) {
+        KernelInfo ki;
+        ki.mode = 2;
+        ki.name = "sg_part" + std::to_string(part_);
+        fill_io(ki);
+        compute_levels();
+        int NT = opt.threads > 0 ? opt.threads : 256;
+        // choose the tile: largest W whose shared-memory footprint fits the budget
+        size_t budget = opt.smem_budget > 0 ? (size_t)opt.smem_budget : (size_t)(100 * 1024);
+        int W = opt.tile;
+        if (W <= 0) {
+            int64_t per = 0;
+            for (int v : nodes_) per = std::max(per, f_.nodes[v].rep);
+            W = 1;
+            for (int cand : {1024, 512, 256, 128, 64, 32, 16, 8, 4, 2, 1}) {
+                layout(cand);
+                if (smem_bytes_ <= budget) { W = cand; break; }
+            }
+            layout(W);
+            if (smem_bytes_ > budget) {
+                layout(1);
+                W = 1;
+            }
+        }
+        layout(W);
+        if (smem_bytes_ > 227 * 1024)
+            throw Error(SG_E_SIZE, "partition " + std::to_string(part_) + " needs " + std::to_string(smem_bytes_) +
+                                       " B of shared memory for one iteration");
+        W_ = W;
+        NT_ = NT;
+        ki.threads = NT;
+        ki.tile = W;
+        ki.smem = smem_bytes_;
+        ki.min_blocks = std::max(1, std::min(4, (int)((220 * 1024) / std::max<size_t>(1024, smem_bytes_))));
+        ki.n_levels = nlev_;
+        std::ostringstream body;
+        emit_loads(body);
+        for (int L = 1; L <= nlev_; L++) {
+            body << "    // ---- level " << L << "\n";
+            int64_t rot = 0;
+            for (int v : nodes_) {
+                if (is_view_node(f_.nodes[v]) || level_[v] != L) continue;
+                emit_stage(body, v, rot);
+                rot += f_.nodes[v].halo + (int64_t)W * f_.nodes[v].rep;
+            }
+            body << "    __syncthreads();\n";
+        }
+        emit_stores(body);
+        std::ostringstream src;
+        src << header("staged") << consts_.str() << args_struct();
+        src << "#define NT " << NT << "\n#define W " << W << "\n";
+        src << readers_.str();
+        src << "extern \"C\" __global__ void __launch_bounds__(NT, " << ki.min_blocks << ") " << ki.name
+            << "(const SgArgs a) {\n"
+            << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
+            << "  " << T_ << "* sm = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
+            << "  const int tid = threadIdx.x;\n"
+            << "  for (long long k0 = SG_K_BEGIN + (long long)blockIdx.x * W; k0 < SG_K_END; k0 += (long long)gridDim.x * W) {\n"
+            << "    const int Wt = (int)min((long long)W, SG_K_END - k0);\n"
+            << body.str() << "  }\n}\n";
+        ki.source = src.str();
+        return ki;
+    }
+
+private:
+    std::map<int, int> level_;      // compute node -> level (1..)
+    int nlev_ = 0;
+    std::map<int, int64_t> off_;    // phys edge -> smem offset (items)
+    std::map<int, int64_t> wb_;     // phys edge -> window base (local position)
+    std::map<int, int64_t> size_;   // phys edge -> items at the chosen W
+    size_t smem_bytes_ = 0;
+    int W_ = 1, NT_ = 256;
+    std::ostringstream readers_;
+    std::set<int> reader_done_;
+
+    int producer_level(int e) {
+        const Edge& ed = f_.edges[e];
+        if (!R_.phys(e)) throw Error(SG_E_UNSUPPORTED, "internal");
+        if (ed.src < 0 || std::find(ins_.begin(), ins_.end(), e) != ins_.end()) return 0;
+        return level_.at(ed.src);
+    }
+    void compute_levels() {
+        nlev_ = 0;
+        for (int v : nodes_) {  // topological order
+            const Node& n = f_.nodes[v];
+            if (is_view_node(n)) continue;
+            std::set<int> src;
+            R_.sources(n.in[0], src);
+            int L = 0;
+            for (int e : src) L = std::max(L, producer_level(e));
+            level_[v] = L + 1;
+            nlev_ = std::max(nlev_, L + 1);
+        }
+    }
+    // buffers, windows and liveness-based placement for tile W
+    void layout(int W) {
+        off_.clear();
+        wb_.clear();
+        size_.clear();
+        struct Buf { int e; int64_t size; int birth, death; };
+        std::vector<Buf> bufs;
+        std::map<int, int> death;
+        auto note_reads = [&](int e_in, int lvl) {
+            std::set<int> src;
+            R_.sources(e_in, src);
+            for (int s : src) death[s] = std::max(death[s], lvl);
+        };
+        for (int v : nodes_) {
+            const Node& n = f_.nodes[v];
+            if (is_view_node(n)) continue;
+            note_reads(n.in[0], level_[v]);
+        }
+        for (int e : outs_) note_reads(e, nlev_ + 1);
+        for (size_t i = 0; i < ins_.size(); i++) {
+            int e = ins_[i];
+            int64_t lo, ex;
+            edge_window(f_, e, lo, ex);
+            int64_t sz = f_.edges[e].per_iter * W + ex;
+            wb_[e] = lo;
+            bufs.push_back({e, sz, 0, death.count(e) ? death[e] : 0});
+        }
+        for (int v : nodes_) {
+            const Node& n = f_.nodes[v];
+            if (is_view_node(n)) continue;
+            int e = n.out[0];
+            const Edge& ed = f_.edges[e];
+            wb_[e] = ed.pre + (n.ninit - n.halo) * n.push;
+            int64_t sz = (n.halo + (int64_t)W * n.rep) * n.push;
+            bufs.push_back({e, sz, level_[v], death.count(e) ? death[e] : level_[v]});
+        }
+        std::vector<int> order(bufs.size());
+        std::iota(order.begin(), order.end(), 0);
+        std::stable_sort(order.begin(), order.end(), [&](int a, int b) { return bufs[a].size > bufs[b].size; });
+        std::vector<int> placed;
+        int64_t top = 0;
+        for (int bi : order) {
+            Buf& b = bufs[bi];
+            int64_t sz = (b.size + 3) / 4 * 4;
+            // candidate offsets: 0 and the end of every live-overlapping placed buffer
+            std::vector<std::pair<int64_t, int64_t>> busy;
+            for (int pj : placed) {
+                Buf& q = bufs[pj];
+                bool overlap = !(q.death < b.birth || b.death < q.birth);
+                if (overlap) busy.push_back({off_[q.e], off_[q.e] + (q.size + 3) / 4 * 4});
+            }
+            std::sort(busy.begin(), busy.end());
+            int64_t o = 0;
+            for (auto& iv : busy) {
+                if (o + sz <= iv.first) break;
+                o = std::max(o, iv.second);
+            }
+            off_[b.e] = o;
+            size_[b.e] = b.size;
+            top = std::max(top, o + sz);
+            placed.push_back(bi);
+        }
+        smem_bytes_ = (size_t)std::max<int64_t>(top, 4) * 4;
+    }
+    std::string rd_name(int e) { return "sg_rd" + std::to_string(e); }
+    // runtime reader through views (fallback when static resolution fails)
+    void gen_reader(int e) {
+        if (reader_done_.count(e)) return;
+        reader_done_.insert(e);
+        std::ostringstream s;
+        s << "__device__ __forceinline__ " << T_ << " " << rd_name(e) << "(const " << T_ << "* sm, int lp) {\n";
+        if (R_.phys(e)) {
+            s << "  return sm[" << off_.at(e) - wb_.at(e) << " + lp];\n}\n";
+            readers_ << s.str();
+            return;
+        }
+        const Edge& ed = f_.edges[e];
+        const Node& u = f_.nodes[ed.src];
+        std::vector<int> deps;
+        switch (u.type) {
+        case N_SPLIT_DUP: s << "  return " << rd_name(u.in[0]) << "(sm, lp);\n"; deps.push_back(u.in[0]); break;
+        case N_SPLIT_RR: {
+            int64_t w = u.w[ed.sport], P = 0;
+            for (int i = 0; i < ed.sport; i++) P += u.w[i];
+            s << "  const int q = sg_fdiv32(lp, " << w << "), r = lp - q * " << w << ";\n";
+            s << "  return " << rd_name(u.in[0]) << "(sm, q * " << u.wsum << " + " << P << " + r);\n";
+            deps.push_back(u.in[0]);
+            break;
+        }
+        case N_JOIN: {
+            s << "  const int q = sg_fdiv32(lp, " << u.wsum << "), o = lp - q * " << u.wsum << ";\n";
+            int64_t P = 0;
+            for (size_t b = 0; b < u.w.size(); b++) {
+                s << "  if (o < " << P + u.w[b] << ") return " << rd_name(u.in[b]) << "(sm, q * " << u.w[b] << " + o - "
+                  << P << ");\n";
+                deps.push_back(u.in[b]);
+                P += u.w[b];
+            }
+            s << "  return (" << T_ << ")0;\n";
+            break;
+        }
+        case N_FILTER: {
+            int in = u.in[0];
+            deps.push_back(in);
+            switch (u.kind) {
+            case SG_K_IDENTITY: s << "  return " << rd_name(in) << "(sm, lp);\n"; break;
+            case SG_K_DELAY: s << "  return " << rd_name(in) << "(sm, lp - " << u.iv[0] << ");\n"; break;
+            case SG_K_DECIMATE: s << "  return " << rd_name(in) << "(sm, lp * " << u.iv[0] << ");\n"; break;
+            case SG_K_EXPAND:
+                s << "  const int q = sg_fdiv32(lp, " << u.iv[0] << ");\n  return (lp - q * " << u.iv[0] << ") == 0 ? "
+                  << rd_name(in) << "(sm, q) : (" << T_ << ")0;\n";
+                break;
+            case SG_K_FFT_REORDER: {
+                int64_t n = u.iv[0], F = 2 * n;
+                s << "  const int q = sg_fdiv32(lp, " << F << "), o = lp - q * " << F << ";\n"
+                  << "  const int m = o >> 1, r = o & 1;\n"
+                  << "  const int sc = m < " << n / 2 << " ? 2 * m : 2 * (m - " << n / 2 << ") + 1;\n"
+                  << "  return " << rd_name(in) << "(sm, q * " << F << " + 2 * sc + r);\n";
+                break;
+            }
+            default: throw Error(SG_E_UNSUPPORTED, "internal: reader for compute node");
+            }
+            break;
+        }
+        }
+        s << "}\n";
+        for (int d : deps) gen_reader(d);  // callees first
+        readers_ << s.str();
+    }
+    std::string read_expr(int e, const Lin& pos) {
+        Ref r = R_.resolve(e, pos);
+        if (r.k == Ref::ZERO) return "(" + T_ + ")0";
+        if (r.k == Ref::RUNTIME) {
+            gen_reader(r.edge);
+            return rd_name(r.edge) + "(sm, " + r.pos.str() + ")";
+        }
+        int64_t k = off_.at(r.edge) - wb_.at(r.edge);
+        return "sm[" + r.pos.plus(k).str() + "]";
+    }
+    void emit_loads(std::ostringstream& b) {
+        for (size_t i = 0; i < ins_.size(); i++) {
+            int e = ins_[i];
+            int64_t lo, ex;
+            edge_window(f_, e, lo, ex);
+            int64_t P = f_.edges[e].per_iter;
+            b << "    { // load boundary input " << i << " (edge " << e << ")\n"
+              << "      const " << T_ << "* g = SG_IN(" << i << ");\n"
+              << "      const long long gb = k0 * " << P << "LL + (" << lo << "LL) - SG_IN_BASE(" << i << ");\n"
+              << "      const long long lim = SG_IN_LIMIT(" << i << ");\n"
+              << "      const int n = Wt * " << P << " + " << ex << ";\n"
+              << "      " << T_ << "* s = sm + " << off_.at(e) << ";\n"
+              << "      for (int j = tid; j < n; j += NT) { const long long gi = gb + j; s[j] = (gi >= 0 && gi < lim) ? g[gi] : ("
+              << T_ << ")0; }\n"
+              << "    }\n";
+        }
+        b << "    __syncthreads();\n";
+    }
+    // choose a store period PER so that every position resolves statically
+    int store_period(int e, int64_t lo) {
+        for (int per : {1, 2, 4, 8, 16, 32, 64}) {
+            bool ok = true;
+            for (int c = 0; c < per && ok; c++) ok = R_.resolve(e, Lin::v("q", per, lo + c)).k != Ref::RUNTIME;
+            if (ok) return per;
+        }
+        return 1;
+    }
+    void emit_stores(std::ostringstream& b) {
+        for (size_t i = 0; i < outs_.size(); i++) {
+            int e = outs_[i];
+            int64_t lo, ex;
+            edge_window(f_, e, lo, ex);
+            int64_t P = f_.edges[e].per_iter;
+            int per = store_period(e, lo);
+            b << "    { // store boundary output " << i << " (edge " << e << ")\n"
+              << "      " << T_ << "* g = SG_OUT(" << i << ");\n"
+              << "      const long long gb = k0 * " << P << "LL + (" << lo << "LL) - SG_OUT_BASE(" << i << ");\n"
+              << "      const int n = Wt * " << P << " + " << ex << ";\n"
+              << "      const int nq = (n + " << per - 1 << ") / " << per << ";\n"
+              << "      for (int q = tid; q < nq; q += NT) {\n";
+            for (int c = 0; c < per; c++) {
+                std::string val = read_expr(e, Lin::v("q", per, lo + c));
+                b << "        if (" << per << " * q + " << c << " < n) g[gb + " << per << " * q + " << c << "] = " << val
+                  << ";\n";
+            }
+            b << "      }\n";
+            const Edge& ed = f_.edges[e];
+            if (ed.dst < 0 && ed.pre > 0)
+                b << "      if (k0 == 0) for (int j = tid; j < " << ed.pre << "; j += NT) g[j - SG_OUT_BASE(" << i
+                  << ")] = (" << T_ << ")0;\n";
+            b << "    }\n";
+        }
+    }
+    void emit_stage(std::ostringstream& b, int v, int64_t rot) {
+        const Node& n = f_.nodes[v];
+        int eo = n.out[0];
+        int64_t F0 = n.ninit - n.halo;
+        int64_t r = rot % NT_;
+        b << "    { // " << kind_name(n.kind) << " node " << v << "\n"
+          << "      const int nf = " << n.halo << " + Wt * " << n.rep << ";\n"
+          << "      const long long gf = k0 * " << n.rep << "LL;\n"
+          << "      " << T_ << "* o_ = sm + " << off_.at(eo) << ";\n";
+        if (n.kind == SG_K_BEAM_FIR) {
+            emit_beam_fir(b, v, F0, r);
+        } else if (n.kind == SG_K_FIR && n.iv[0] >= 4 && emit_fir_blocked(b, v, F0, r)) {
+        } else {
+            b << "      int j = tid - " << r << "; if (j < 0) j += NT;\n"
+              << "      for (; j < nf; j += NT) {\n"
+              << "        const int lf = " << F0 << " + j;\n";
+            emit_firing(b, v, "        ");
+            b << "      }\n";
+        }
+        b << "    }\n";
+    }
+    // one firing at local index `lf`, output slot j
+    void emit_firing(std::ostringstream& b, int v, const std::string& ind) {
+        const Node& n = f_.nodes[v];
+        b << ind << "if (gf + lf < 0) {";
+        for (int64_t jj = 0; jj < n.push; jj++) b << " o_[j * " << n.push << " + " << jj << "] = (" << T_ << ")0;";
+        b << " } else {\n";
+        b << ind << "  " << T_ << " x_[" << n.peek << "];\n";
+        for (int64_t i = 0; i < n.peek; i++)
+            b << ind << "  x_[" << i << "] = " << read_expr(n.in[0], Lin::v("lf", n.pop, i)) << ";\n";
+        b << ind << "  " << T_ << " y_[" << n.push << "]; " << work_call(v) << "\n";
+        for (int64_t jj = 0; jj < n.push; jj++)
+            b << ind << "  o_[j * " << n.push << " + " << jj << "] = y_[" << jj << "];\n";
+        b << ind << "}\n";
+    }
+    // Register-blocked FIR: a thread computes B consecutive firings from one
+    // window of (B-1)*pop + L inputs held in registers; per output the taps are
+    // accumulated in order i = 0..L-1 (the FIR semantics).
+    bool emit_fir_blocked(std::ostringstream& b, int v, int64_t F0, int64_t rot) {
+        const Node& n = f_.nodes[v];
+        int64_t L = n.iv[0], pop = n.pop;
+        // probe: positions lf0*pop + k must map to one physical buffer, affine in lf0 and k
+        Ref r0 = R_.resolve(n.in[0], Lin::v("lf0", pop, 0));
+        Ref r1 = R_.resolve(n.in[0], Lin::v("lf0", pop, 1));
+        if (r0.k != Ref::PHYS || r1.k != Ref::PHYS || r0.edge != r1.edge) return false;
+        int64_t a = r0.pos.coef("lf0"), s = r1.pos.c - r0.pos.c;
+        if (r0.pos.t.size() != (a ? 1u : 0u) || a != pop * s || s == 0) return false;
+        int B = 1;
+        for (int cand : {9, 7, 5, 3}) {
+            if ((cand - 1) * pop + L > 100) continue;
+            if (((cand * pop * s) & 1) == 0 && cand != 3) continue;
+            B = cand;
+            break;
+        }
+        if (B == 1) return false;
+        int64_t NW = (B - 1) * pop + L;
+        for (int64_t k = 0; k < NW; k++) {  // verify the whole window is affine
+            Ref rk = R_.resolve(n.in[0], Lin::v("lf0", pop, k));
+            if (rk.k != Ref::PHYS || rk.edge != r0.edge || rk.pos.coef("lf0") != a || rk.pos.c != r0.pos.c + s * k)
+                return false;
+        }
+        std::string C = const_array(n.fv);
+        int64_t base = off_.at(r0.edge) - wb_.at(r0.edge) + r0.pos.c;
+        b << "      const int nb = (nf + " << B - 1 << ") / " << B << ";\n"
+          << "      int jb = tid - " << rot % NT_ << "; if (jb < 0) jb += NT;\n"
+          << "      for (; jb < nb; jb += NT) {\n"
+          << "        const int j0 = jb * " << B << ";\n"
+          << "        const int lf0 = " << F0 << " + j0;\n"
+          << "        if (j0 + " << B << " <= nf && gf + lf0 >= 0) {\n"
+          << "          const " << T_ << "* w_ = sm + (" << base << " + " << a << " * lf0);\n"
+          << "          float w[" << NW << "];\n"
+          << "#pragma unroll\n"
+          << "          for (int k = 0; k < " << NW << "; k++) w[k] = w_[k * " << s << "];\n"
+          << "          float acc[" << B << "];\n"
+          << "#pragma unroll\n"
+          << "          for (int bb = 0; bb < " << B << "; bb++) acc[bb] = 0.0f;\n"
+          << "#pragma unroll\n"
+          << "          for (int i = 0; i < " << L << "; i++) {\n"
+          << "            const float c = " << C << "[i];\n"
+          << "#pragma unroll\n"
+          << "            for (int bb = 0; bb < " << B << "; bb++) acc[bb] = fmaf(w[bb * " << pop << " + i], c, acc[bb]);\n"
+          << "          }\n"
+          << "#pragma unroll\n"
+          << "          for (int bb = 0; bb < " << B << "; bb++) o_[j0 + bb] = acc[bb];\n"
+          << "        } else {\n"
+          << "          for (int j = j0; j < min(j0 + " << B << ", nf); j++) {\n"
+          << "            const int lf = " << F0 << " + j;\n";
+        emit_firing(b, v, "            ");
+        b << "          }\n        }\n      }\n";
+        return true;
+    }
+    // Frame-granular complex FIR: items = (firing, block of B outputs); taps in
+    // chunks of TC with the sample window in registers; x[s<0] = 0.
+    void emit_beam_fir(std::ostringstream& b, int v, int64_t F0, int64_t rot) {
+        const Node& n = f_.nodes[v];
+        int64_t L = n.iv[0], DEC = n.iv[1], FR = n.iv[2], OUT = FR / DEC;
+        int64_t B = 4, TC = 1;
+        for (int64_t c : {16, 8, 4, 2, 1})
+            if (L % c == 0) { TC = c; break; }
+        int64_t NB = (OUT + B - 1) / B, NWIN = (B - 1) * DEC + TC;
+        std::vector<float> wr(n.fv.begin(), n.fv.begin() + L), wi(n.fv.begin() + L, n.fv.end());
+        std::string WR = const_array(wr), WI = const_array(wi);
+        b << "      const int items = nf * " << NB << ";\n"
+          << "      int it = tid - " << rot % NT_ << "; if (it < 0) it += NT;\n"
+          << "      for (; it < items; it += NT) {\n"
+          << "        const int j = it / " << NB << ";\n"
+          << "        const int t0 = (it - j * " << NB << ") * " << B << ";\n"
+          << "        const int lf = " << F0 << " + j;\n"
+          << "        float re[" << B << "], im[" << B << "];\n"
+          << "#pragma unroll\n"
+          << "        for (int bb = 0; bb < " << B << "; bb++) { re[bb] = 0.0f; im[bb] = 0.0f; }\n"
+          << "        if (gf + lf >= 0) {\n"
+          << "#pragma unroll 1\n"
+          << "          for (int i0 = 0; i0 < " << L << "; i0 += " << TC << ") {\n"
+          << "            const int s0 = t0 * " << DEC << " - i0 - " << TC - 1 << ";\n"
+          << "            float xr[" << NWIN << "], xi[" << NWIN << "];\n";
+        for (int64_t k = 0; k < NWIN; k++) {
+            Lin pr = Lin::v("lf", n.pop, 2 * k);
+            pr.t.push_back({"s0", 2});
+            Lin pi = pr.plus(1);
+            b << "            { const int s = s0 + " << k << "; const bool ok = s >= 0 && s < " << FR << ";\n"
+              << "              xr[" << k << "] = ok ? " << read_expr(n.in[0], pr) << " : 0.0f;\n"
+              << "              xi[" << k << "] = ok ? " << read_expr(n.in[0], pi) << " : 0.0f; }\n";
+        }
+        b << "#pragma unroll\n"
+          << "            for (int ii = 0; ii < " << TC << "; ii++) {\n"
+          << "              const float cr = " << WR << "[i0 + ii], ci = " << WI << "[i0 + ii];\n"
+          << "#pragma unroll\n"
+          << "              for (int bb = 0; bb < " << B << "; bb++) {\n"
+          << "                const int k = bb * " << DEC << " - ii + " << TC - 1 << ";\n"
+          << "                sg_cmac(re[bb], im[bb], xr[k], xi[k], cr, ci);\n"
+          << "              }\n"
+          << "            }\n"
+          << "          }\n"
+          << "        }\n"
+          << "#pragma unroll\n"
+          << "        for (int bb = 0; bb < " << B << "; bb++)\n"
+          << "          if (t0 + bb < " << OUT << ") { o_[j * " << n.push << " + 2 * (t0 + bb)] = re[bb]; o_[j * " << n.push
+          << " + 2 * (t0 + bb) + 1] = im[bb]; }\n"
+          << "      }\n";
+    }
+};
+
+KernelInfo generate_kernel(const Flat& f, const std::vector<int>& nodes, int part_id, const CodegenOpts& opt) {
+    std::string why;
+    bool reg_ok = register_mode_eligible(f, nodes, &why);
+    int mode = opt.mode;
+    if (mode == 1 && !reg_ok) throw Error(SG_E_UNSUPPORTED, "register mode not possible: " + why);
+    if (mode == 0) mode = reg_ok ? 1 : 2;
+    if (mode == 1) {
+        RegGen g(f, nodes, part_id);
+        return g.run(opt);
+    }
+    StageGen g(f, nodes, part_id);
+    return g.run(opt);
+}
+
+}  // namespace sg

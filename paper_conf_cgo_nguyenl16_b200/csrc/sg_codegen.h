@@ -1,0 +1,54 @@
+// sg_codegen.h -- per-partition CUDA code generation.
+#pragma once
+#include <string>
+#include <vector>
+
+#include "sg_internal.h"
+
+namespace sg {
+
+struct CodegenOpts {
+    int mode = 0;        // 0 auto, 1 register, 2 staged
+    int threads = 0;     // 0 auto
+    int tile = 0;        // staged: iterations per tile (0 auto)
+    int smem_budget = 0; // bytes per CTA (0 = auto)
+};
+
+// What the runtime needs to launch a generated kernel.
+struct KernelInfo {
+    std::string name;
+    std::string source;       // full CUDA source (includes sg_device.cuh)
+    int mode = 0;             // 1 register (thread per iteration), 2 staged
+    int threads = 0;          // CTA size
+    int tile = 0;             // iterations per CTA tile
+    int min_blocks = 1;       // __launch_bounds__ second argument
+    size_t smem = 0;          // dynamic shared memory bytes
+    std::vector<int> in_edges, out_edges;   // boundary edges (flat edge ids), argument order
+    // per boundary edge: window of local positions needed/produced by one range
+    // of W iterations: [lo, lo + per_iter*W + extra)
+    std::vector<int64_t> in_lo, in_extra, out_lo, out_extra;
+    int64_t flops_per_iter = 0;     // algorithmic fp32 flops (FMA = 2), as written
+    int64_t intops_per_iter = 0;    // algorithmic integer ops (CE = 2 min/max)
+    int64_t dfma_per_iter = 0;
+    int n_levels = 0;
+};
+
+// Boundary input / output edges of a node set (sorted, deterministic).
+void partition_boundary(const Flat& f, const std::vector<int>& nodes, std::vector<int>& ins, std::vector<int>& outs);
+
+// Window [lo, lo + per_iter*W + extra) of local positions a range of W iterations
+// reads on edge e (its consumer's needs; graph output: the produced positions).
+void edge_window(const Flat& f, int e, int64_t& lo, int64_t& extra);
+
+bool register_mode_eligible(const Flat& f, const std::vector<int>& nodes, std::string* why);
+
+KernelInfo generate_kernel(const Flat& f, const std::vector<int>& nodes, int part_id, const CodegenOpts& opt);
+
+// Algorithmic work of one node per steady-state iteration (as written).
+void node_work(const Flat& f, int v, int64_t& flops, int64_t& intops, int64_t& dfma);
+
+bool is_view_kind(int kind);
+
+extern const char* kDeviceHeader;  // sg_device.cuh contents (embedded)
+
+}  // namespace sg

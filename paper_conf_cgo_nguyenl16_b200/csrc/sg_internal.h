@@ -1,0 +1,127 @@
+// sg_internal.h -- internal data structures of the stream-graph executor.
+//
+// Layers: graph IR + SDF analysis (sg_graph.cpp), planner
+// (sg_plan.cpp: PEE, Algorithm 1, PDG, ILP), code generator (sg_codegen.cpp),
+// runtime (sg_runtime.cpp: NVRTC, modules, launches, multi-GPU pipeline),
+// C ABI (sg_capi.cpp).
+#pragma once
+
+#include <cstdint>
+#include <map>
+#include <memory>
+#include <mutex>
+#include <stdexcept>
+#include <string>
+#include <vector>
+
+#include "../../include/sg.h"
+
+namespace sg {
+
+struct Error : std::runtime_error {
+    sg_status code;
+    Error(sg_status c, const std::string& m) : std::runtime_error(m), code(c) {}
+};
+
+// ------------------------------------------------------------------ builder
+enum ElemType { E_FILTER = 0, E_PIPE = 1, E_SJ = 2 };
+
+struct Elem {
+    ElemType type = E_FILTER;
+    // filter
+    int kind = -1;
+    std::vector<int32_t> iv;
+    std::vector<float> fv;
+    // pipeline
+    std::vector<int> kids;
+    // split-join
+    int split_kind = 0;  // 0 dup, 1 rr
+    std::vector<int32_t> split_w, join_w;
+    std::vector<int> branches;  // elem ids of branch pipelines
+    std::vector<bool> branch_done;
+};
+
+}  // namespace sg
+
+struct sg_graph {
+    sg_dtype dtype = SG_F32;
+    std::vector<sg::Elem> elems;
+    int top = 0;
+    std::vector<int> open;  // stack of open pipelines (elem ids); bottom = top
+    std::vector<std::pair<int, int>> open_branch;  // (sj, branch) matching open[1..]
+};
+
+namespace sg {
+
+// --------------------------------------------------------- flattened graph
+enum NodeType { N_FILTER = 0, N_SPLIT_DUP = 1, N_SPLIT_RR = 2, N_JOIN = 3 };
+
+struct Node {
+    NodeType type = N_FILTER;
+    int kind = -1;
+    std::vector<int32_t> iv;
+    std::vector<float> fv;
+    std::vector<int32_t> w;   // split / join weights
+    int64_t wsum = 0;
+    std::vector<int> in, out;  // edge ids, by port
+    // filter rates (splitters/joiners: per edge, see Edge)
+    int64_t pop = 0, push = 0, peek = 0, prework = 0;
+    // analysis
+    int64_t rep = 0;     // repetition vector entry
+    int64_t ninit = 0;   // init-schedule firings (signed: negative = lag)
+    int64_t halo = 0;    // extra firings before a range start (same for every start)
+    int elem = -1;       // builder element (filters)
+};
+
+struct Edge {
+    int src = -1, dst = -1;  // node ids (-1: graph input / output)
+    int sport = 0, dport = 0;
+    int64_t push = 0;  // items the producer pushes per firing onto this edge
+    int64_t pop = 0;   // items the consumer pops per firing from this edge
+    int64_t peek = 0;  // items the consumer reads per firing (>= pop)
+    int64_t pre = 0;   // prework items of the producer on this edge
+    int64_t per_iter = 0;  // items per steady-state iteration (= rep_src * push)
+};
+
+struct Flat {
+    sg_dtype dtype = SG_F32;
+    std::vector<Node> nodes;  // topological (construction) order
+    std::vector<Edge> edges;
+    int in_edge = -1, out_edge = -1;
+    int64_t in_per_iter = 0, out_per_iter = 0;
+    // Builds from the hierarchy; throws Error.
+    static Flat build(const sg_graph& g);
+    void solve_rates();       // balance equations -> rep
+    void solve_init();        // init schedule (signed) + halos
+    int64_t input_items(int64_t n) const;   // minimal input prefix for n iterations
+    int64_t output_items(int64_t n) const;
+    bool is_physical(int e) const { return edges[e].src < 0 || nodes[edges[e].src].type == N_FILTER; }
+};
+
+// kind metadata
+struct KindRates { int64_t peek, pop, push, prework; };
+KindRates kind_rates(int kind, const std::vector<int32_t>& iv, const std::vector<float>& fv, sg_dtype dt);
+const char* kind_name(int kind);
+
+// ------------------------------------------------------------------ planner
+struct Topology {
+    int G = 1;
+    int L = 0;
+    std::vector<uint8_t> dt;  // [L][G][G]: link l carries i->j
+    bool carries(int l, int i, int j) const { return dt[(size_t)l * G * G + (size_t)i * G + j] != 0; }
+    static Topology nvswitch(int G);
+    static Topology pcie_tree4();  // Fig. 3.3
+};
+
+struct PdgEdge { int src, dst; double bytes; };
+
+struct Partition {
+    std::vector<int> nodes;  // node ids (sorted, topological)
+    double t_est = 0;        // PEE estimate, ns per iteration
+    double t_comp = 0, t_dt = 0;
+    int mode = 0;            // 1 register, 2 staged
+    int gpu = 0;
+    int tile = 0, threads = 0;
+};
+
+}  // namespace sg

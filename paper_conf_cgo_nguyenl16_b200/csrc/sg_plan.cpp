@@ -1,0 +1,636 @@
+// sg_plan.cpp -- the mapping flow of Fig. 3.1:
+//   annotated graph -> partitioning (Algorithm 1, aided by the PEE)
+//   -> PDG -> ILP multi-GPU mapping over the GPU topology -> code generation.
+#include "sg_plan.h"
+
+#include <algorithm>
+#include <chrono>
+#include <cmath>
+#include <functional>
+#include <numeric>
+#include <set>
+
+#include "sg_codegen.h"
+
+namespace sg {
+
+// ============================================================ PEE (B200)
+// Section 3.3 of the paper predicts a partition's kernel time from per-node
+// work and the kernel parameters the code generator will choose ("the PEE
+// includes the same optimization done by the GPU code generator",
+// PAPER.md:579-581).  Here: the code generator's own mode decision
+// (register_mode_eligible) and its algorithmic work counts, priced with B200
+// throughputs:
+//   Tcomp = flops/(FP32 peak * eff) + int ops/INT peak + fp64 work + shared-memory bytes/SMEM bw
+//   Tdt   = boundary-stream bytes / HBM bandwidth
+//   T     = max(Tcomp, Tdt) + per-level barrier and per-fragment launch costs
+// (the max() of Eq. III.8 survives: compute and data movement overlap).
+namespace {
+constexpr double kClk = 1.9e9;
+constexpr double kSM = 148;
+constexpr double kFp32 = kSM * 128 * 2 * kClk;    // flop/s
+constexpr double kInt = kSM * 64 * kClk;          // int min/max per s
+constexpr double kFp64 = 37e12;                   // flop/s
+constexpr double kSmem = kSM * 128 * kClk;        // bytes/s
+constexpr double kHbm = 6.5536e12;                // bytes/s (MEASURED_PEAKS.json copy)
+constexpr double kLaunch = 4e-6;                  // s per kernel launch
+constexpr double kFragIters = 65536;              // iterations per fragment (estimate)
+constexpr int kTileEst = 64;
+}  // namespace
+
+PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
+    PeeEstimate est;
+    est.mode = register_mode_eligible(f, nodes, nullptr) ? 1 : 2;
+    std::vector<int> ins, outs;
+    partition_boundary(f, nodes, ins, outs);
+    double bytes = 0;
+    for (int e : ins) bytes += 4.0 * f.edges[e].per_iter;
+    for (int e : outs) bytes += 4.0 * f.edges[e].per_iter;
+    double flops = 0, intops = 0, dfma = 0, smem = 0;
+    int levels = 0;
+    for (int v : nodes) {
+        int64_t a, b, c;
+        node_work(f, v, a, b, c);
+        const Node& n = f.nodes[v];
+        double infl = est.mode == 2 ? (double)(n.halo + (int64_t)kTileEst * n.rep) / (double)(kTileEst * n.rep) : 1.0;
+        flops += a * infl;
+        intops += b * infl;
+        dfma += c * infl;
+        if (n.type == N_FILTER && !is_view_kind(n.kind)) {
+            levels++;
+            if (est.mode == 2) smem += 4.0 * n.rep * (n.peek + n.push) * infl;
+        }
+    }
+    if (est.mode == 1) smem = 0;
+    for (int e : ins) smem += 8.0 * f.edges[e].per_iter;
+    for (int e : outs) smem += 8.0 * f.edges[e].per_iter;
+    double eff = est.mode == 1 ? 0.8 : 0.5;
+    est.t_comp = flops / (kFp32 * eff) + intops / kInt + dfma * 80.0 / kFp64 + smem / kSmem;
+    est.t_dt = bytes / kHbm;
+    double bar = est.mode == 2 ? levels * 200.0 / kClk / (kTileEst * kSM * 2) : 0.0;
+    est.t = (std::max(est.t_comp, est.t_dt) + bar + kLaunch / kFragIters) * 1e9;  // ns per iteration
+    est.t_comp *= 1e9;
+    est.t_dt *= 1e9;
+    return est;
+}
+
+double paper_model(const std::vector<double>& t, const std::vector<double>& fr, int S, int W, int F, double D,
+                   double C1, double C2, double* tcomp, double* tdt, double* tdb) {
+    double tc = 0;  // Eq. III.9: Tcomp = sum_i t_i / min(f_i, S)
+    for (size_t i = 0; i < t.size(); i++) tc += t[i] / std::min(fr[i], (double)S);
+    double td = C1 * D / F;                 // Eq. III.10
+    double tb = C2 * D / (F + (double)W * S);  // Eq. III.11 (all threads swap WS and DB)
+    double texec = std::max(tc, td) + tb;   // Eq. III.8
+    if (tcomp) *tcomp = tc;
+    if (tdt) *tdt = td;
+    if (tdb) *tdb = tb;
+    return texec / W;                       // Eq. III.12
+}
+
+// ===================================================== partition structure
+// "A partition is convex if there is no path between two internal nodes that
+// goes through an external node" (footnote).
+bool is_convex(const Flat& f, const std::vector<char>& in) {
+    const int N = (int)f.nodes.size();
+    std::vector<char> seen(N, 0);
+    std::vector<int> st;
+    for (int v = 0; v < N; v++) {
+        if (!in[v]) continue;
+        for (int e : f.nodes[v].out) {
+            int w = f.edges[e].dst;
+            if (w >= 0 && !in[w] && !seen[w]) { seen[w] = 1; st.push_back(w); }
+        }
+    }
+    while (!st.empty()) {
+        int u = st.back();
+        st.pop_back();
+        for (int e : f.nodes[u].out) {
+            int w = f.edges[e].dst;
+            if (w < 0) continue;
+            if (in[w]) return false;
+            if (!seen[w]) { seen[w] = 1; st.push_back(w); }
+        }
+    }
+    return true;
+}
+
+namespace {
+struct PartState {
+    const Flat& f;
+    double cap;
+    std::vector<int> owner;                    // node -> partition id (-1 none)
+    std::vector<std::vector<int>> members;     // partition id -> nodes (empty = dead)
+    std::vector<double> T;
+    std::vector<char> io;                      // IO-bound flag
+    explicit PartState(const Flat& fl, double c) : f(fl), cap(c), owner(fl.nodes.size(), -1) {}
+
+    double cost(const std::vector<int>& nodes, bool* io_bound = nullptr) const {
+        PeeEstimate e = pee_estimate(f, nodes);
+        if (io_bound) *io_bound = e.io_bound();
+        return e.t;
+    }
+    int make(const std::vector<int>& nodes) {
+        int id = (int)members.size();
+        members.push_back(nodes);
+        bool iob = false;
+        T.push_back(cost(nodes, &iob));
+        io.push_back(iob);
+        for (int v : nodes) owner[v] = id;
+        return id;
+    }
+    bool connected(const std::vector<int>& a, const std::vector<int>& b) const {
+        std::vector<char> inb(f.nodes.size(), 0);
+        for (int v : b) inb[v] = 1;
+        for (int v : a) {
+            for (int e : f.nodes[v].out) if (f.edges[e].dst >= 0 && inb[f.edges[e].dst]) return true;
+            for (int e : f.nodes[v].in) if (f.edges[e].src >= 0 && inb[f.edges[e].src]) return true;
+        }
+        return false;
+    }
+    // Try-Merge: connected, convex, and T(merged) < T(a) + T(b).
+    bool try_merge_sets(const std::vector<std::vector<int>>& sets, const std::vector<double>& Ts,
+                        std::vector<int>& merged, double& tm) const {
+        merged.clear();
+        for (auto& s : sets) merged.insert(merged.end(), s.begin(), s.end());
+        std::sort(merged.begin(), merged.end());
+        std::vector<char> in(f.nodes.size(), 0);
+        for (int v : merged) in[v] = 1;
+        if (!is_convex(f, in)) return false;
+        tm = cost(merged);
+        double sum = std::accumulate(Ts.begin(), Ts.end(), 0.0);
+        if (!(tm < sum)) return false;
+        if (cap > 0 && tm > cap) return false;
+        return true;
+    }
+    bool try_merge(int a, int b) {
+        if (a == b || members[a].empty() || members[b].empty()) return false;
+        if (!connected(members[a], members[b])) return false;
+        std::vector<int> m;
+        double tm;
+        if (!try_merge_sets({members[a], members[b]}, {T[a], T[b]}, m, tm)) return false;
+        for (int v : members[b]) owner[v] = a;
+        members[a] = m;
+        members[b].clear();
+        T[a] = tm;
+        bool iob = false;
+        cost(m, &iob);
+        io[a] = iob;
+        return true;
+    }
+    std::vector<int> neighbours(int p) const {
+        std::set<int> s;
+        for (int v : members[p]) {
+            for (int e : f.nodes[v].out) { int w = f.edges[e].dst; if (w >= 0 && owner[w] >= 0 && owner[w] != p) s.insert(owner[w]); }
+            for (int e : f.nodes[v].in) { int w = f.edges[e].src; if (w >= 0 && owner[w] >= 0 && owner[w] != p) s.insert(owner[w]); }
+        }
+        return std::vector<int>(s.begin(), s.end());
+    }
+    std::vector<int> live() const {
+        std::vector<int> r;
+        for (int i = 0; i < (int)members.size(); i++) if (!members[i].empty()) r.push_back(i);
+        return r;
+    }
+};
+
+// innermost pipelines of the hierarchy, as node-id sequences (construction order)
+void innermost_pipelines(const sg_graph& g, std::vector<std::vector<int>>& out) {
+    int next = 0;
+    std::function<void(int)> walk = [&](int id) {
+        const Elem& e = g.elems[id];
+        if (e.type == E_FILTER) { next++; return; }
+        if (e.type == E_PIPE) {
+            bool inner = !e.kids.empty();
+            for (int k : e.kids) inner &= g.elems[k].type == E_FILTER;
+            if (inner) {
+                std::vector<int> seq;
+                for (size_t i = 0; i < e.kids.size(); i++) seq.push_back(next + (int)i);
+                next += (int)e.kids.size();
+                out.push_back(seq);
+                return;
+            }
+            for (int k : e.kids) walk(k);
+            return;
+        }
+        next++;  // splitter
+        for (int b : e.branches) walk(b);
+        next++;  // joiner
+    };
+    walk(g.top);
+}
+}  // namespace
+
+std::vector<std::vector<int>> algorithm1(const Flat& f, const sg_graph& g, double cap) {
+    PartState S(f, cap);
+    // ---- Phase 1: inside innermost pipelines (Alg. 1 lines 2-10)
+    std::vector<std::vector<int>> pipes;
+    innermost_pipelines(g, pipes);
+    for (auto& pipe : pipes) {
+        size_t i = 0;
+        while (i < pipe.size()) {
+            int p = S.make({pipe[i]});
+            size_t j = i + 1;
+            while (j < pipe.size()) {            // Try-Merge one neighbour node in pipe with p
+                int q = S.make({pipe[j]});
+                if (!S.try_merge(p, q)) {        // h <- last failed node
+                    S.members[q].clear();
+                    S.owner[pipe[j]] = -1;
+                    break;
+                }
+                j++;
+            }
+            i = j;
+        }
+    }
+    // ---- Phase 2: nodes outside partitions (lines 13-20)
+    for (int n = 0; n < (int)f.nodes.size(); n++) {
+        if (S.owner[n] >= 0) continue;
+        int p = S.make({n});
+        bool merged = true;
+        while (merged) {
+            merged = false;
+            std::set<int> cand;
+            for (int v : S.members[p]) {
+                for (int e : f.nodes[v].out) { int w = f.edges[e].dst; if (w >= 0 && S.owner[w] < 0) cand.insert(w); }
+                for (int e : f.nodes[v].in) { int w = f.edges[e].src; if (w >= 0 && S.owner[w] < 0) cand.insert(w); }
+            }
+            for (int k : cand) {
+                if (S.owner[k] >= 0) continue;
+                int q = S.make({k});
+                if (S.try_merge(p, q)) merged = true;
+                else { S.members[q].clear(); S.owner[k] = -1; }
+            }
+        }
+    }
+    // ---- Phase 3: IO-bound first, ascending T, three rounds (lines 23-31)
+    for (int round = 0; round < 3; round++) {
+        bool merged = true;
+        while (merged) {
+            merged = false;
+            std::vector<int> L1, L12 = S.live();
+            for (int p : L12) if (S.io[p]) L1.push_back(p);
+            std::vector<int>& outer = round == 2 ? L12 : L1;
+            std::sort(outer.begin(), outer.end(), [&](int a, int b) { return S.T[a] < S.T[b]; });
+            for (int p : outer) {
+                std::vector<int> nb = S.neighbours(p);
+                std::sort(nb.begin(), nb.end(), [&](int a, int b) { return S.T[a] < S.T[b]; });
+                for (int q : nb) {
+                    bool ok = round == 0 ? (bool)S.io[q] : true;
+                    if (!ok) continue;
+                    if (S.try_merge(p, q)) { merged = true; break; }
+                }
+                if (merged) break;
+            }
+        }
+    }
+    // ---- Phase 4 (lines 34-35): (1) two neighbours at once, (2) all nodes at once
+    bool merged = true;
+    while (merged) {
+        merged = false;
+        for (int p : S.live()) {
+            std::vector<int> nb = S.neighbours(p);
+            for (size_t a = 0; a < nb.size() && !merged; a++)
+                for (size_t b = a + 1; b < nb.size() && !merged; b++) {
+                    int q = nb[a], r = nb[b];
+                    std::vector<int> m;
+                    double tm;
+                    if (S.try_merge_sets({S.members[p], S.members[q], S.members[r]}, {S.T[p], S.T[q], S.T[r]}, m, tm)) {
+                        for (int v : S.members[q]) S.owner[v] = p;
+                        for (int v : S.members[r]) S.owner[v] = p;
+                        S.members[p] = m;
+                        S.members[q].clear();
+                        S.members[r].clear();
+                        S.T[p] = tm;
+                        bool iob;
+                        S.cost(m, &iob);
+                        S.io[p] = iob;
+                        merged = true;
+                    }
+                }
+            if (merged) break;
+        }
+    }
+    std::vector<std::vector<int>> parts;
+    for (int p : S.live()) parts.push_back(S.members[p]);
+    if (cap <= 0 && parts.size() > 1) {  // all nodes at once: never worse than single-partition
+        std::vector<int> all(f.nodes.size());
+        std::iota(all.begin(), all.end(), 0);
+        double sum = 0;
+        for (int p : S.live()) sum += S.T[p];
+        if (S.cost(all) < sum) parts = {all};
+    }
+    return parts;
+}
+
+// ========================================================= topology
+// NVSwitch (B200 HGX): every GPU k has an uplink k->switch and a downlink
+// switch->k; traffic i->j loads uplink i and downlink j.  The dtlist rule of
+// section 3.2.1 applied to this star.
+Topology Topology::nvswitch(int G) {
+    Topology t;
+    t.G = G;
+    t.L = 2 * G;
+    t.dt.assign((size_t)t.L * G * G, 0);
+    for (int i = 0; i < G; i++)
+        for (int j = 0; j < G; j++) {
+            if (i == j) continue;
+            t.dt[(size_t)i * G * G + (size_t)i * G + j] = 1;          // uplink of i
+            t.dt[(size_t)(G + j) * G * G + (size_t)i * G + j] = 1;    // downlink of j
+        }
+    return t;
+}
+
+// Fig. 3.3: Host - SW1 - {SW2: GPU1, GPU2}, {SW3: GPU3, GPU4}.
+// Links (each direction separately): GPUk<->its switch, SW2<->SW1, SW3<->SW1.
+// "the load of an uplink l is contributed by the data transfer from GPU i to
+// GPU j if and only if i is a child of l and j is not"; downlinks mirror it.
+Topology Topology::pcie_tree4() {
+    Topology t;
+    t.G = 4;
+    // links: 0-3 GPUk->SW (up), 4-7 SW->GPUk (down), 8 SW2->SW1, 9 SW1->SW2, 10 SW3->SW1, 11 SW1->SW3
+    t.L = 12;
+    t.dt.assign((size_t)t.L * 16, 0);
+    auto sw = [](int g) { return g < 2 ? 0 : 1; };  // 0 = SW2, 1 = SW3
+    for (int i = 0; i < 4; i++)
+        for (int j = 0; j < 4; j++) {
+            if (i == j) continue;
+            t.dt[(size_t)i * 16 + i * 4 + j] = 1;        // leaf uplink of i
+            t.dt[(size_t)(4 + j) * 16 + i * 4 + j] = 1;  // leaf downlink of j
+            if (sw(i) != sw(j)) {                        // crosses SW1
+                int up = sw(i) == 0 ? 8 : 10, down = sw(j) == 0 ? 9 : 11;
+                t.dt[(size_t)up * 16 + i * 4 + j] = 1;
+                t.dt[(size_t)down * 16 + i * 4 + j] = 1;
+            }
+        }
+    return t;
+}
+
+// ===================================================== ILP (Eq. III.1-III.7)
+double mapping_cost(const std::vector<double>& T, const std::vector<PdgEdge>& pdg, const Topology& topo, double lat,
+                    double bw, const std::vector<int>& a) {
+    std::vector<double> gl(topo.G, 0.0), ll(topo.L, 0.0);
+    for (size_t i = 0; i < T.size(); i++) gl[a[i]] += T[i];                       // III.4
+    for (auto& e : pdg) {                                                          // III.6-III.7
+        int k = a[e.src], h = a[e.dst];
+        if (k == h) continue;
+        for (int l = 0; l < topo.L; l++) if (topo.carries(l, k, h)) ll[l] += e.bytes;
+    }
+    double tmax = 0;
+    for (double x : gl) tmax = std::max(tmax, x);                                  // III.1
+    for (int l = 0; l < topo.L; l++) tmax = std::max(tmax, lat + ll[l] / bw);      // III.2-III.3
+    return tmax;
+}
+
+MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge>& pdg, const Topology& topo,
+                         double lat, double bw, int time_limit_ms, int method) {
+    const int P = (int)T.size(), G = topo.G;
+    MapResult best;
+    best.assign.assign(P, 0);
+    if (P == 0) { best.optimal = true; best.tmax = 0; return best; }
+    if (method == 1) {  // brute force over G^P
+        std::vector<int> a(P, 0);
+        best.tmax = mapping_cost(T, pdg, topo, lat, bw, a);
+        for (;;) {
+            int i = 0;
+            while (i < P && ++a[i] == G) a[i++] = 0;
+            if (i == P) break;
+            double c = mapping_cost(T, pdg, topo, lat, bw, a);
+            if (c < best.tmax - 1e-12) { best.tmax = c; best.assign = a; }
+        }
+        best.optimal = true;
+        return best;
+    }
+    // branch and bound: partitions by decreasing T; LPT incumbent
+    std::vector<int> ord(P);
+    std::iota(ord.begin(), ord.end(), 0);
+    std::stable_sort(ord.begin(), ord.end(), [&](int x, int y) { return T[x] > T[y]; });
+    {
+        std::vector<int> a(P, 0);
+        std::vector<double> gl(G, 0);
+        for (int i : ord) {
+            int g = (int)(std::min_element(gl.begin(), gl.end()) - gl.begin());
+            a[i] = g;
+            gl[g] += T[i];
+        }
+        best.assign = a;
+        best.tmax = mapping_cost(T, pdg, topo, lat, bw, a);
+        std::vector<int> z(P, 0);
+        double cz = mapping_cost(T, pdg, topo, lat, bw, z);
+        if (cz < best.tmax) { best.tmax = cz; best.assign = z; }
+    }
+    bool symmetric = true;  // all GPUs interchangeable (true for the NVSwitch star)
+    {
+        Topology s = Topology::nvswitch(G);
+        symmetric = s.L == topo.L && s.dt == topo.dt;
+    }
+    std::vector<std::vector<std::pair<int, double>>> adj(P);  // edges to earlier-ordered partitions
+    std::vector<int> rank(P);
+    for (int k = 0; k < P; k++) rank[ord[k]] = k;
+    for (auto& e : pdg) {
+        if (e.src == e.dst) continue;
+        int later = rank[e.src] > rank[e.dst] ? e.src : e.dst;
+        int other = later == e.src ? e.dst : e.src;
+        adj[later].push_back({other, later == e.src ? e.bytes : -e.bytes});  // sign: direction
+    }
+    std::vector<double> suffix(P + 1, 0.0);
+    for (int k = P - 1; k >= 0; k--) suffix[k] = suffix[k + 1] + T[ord[k]];
+    std::vector<int> a(P, -1);
+    std::vector<double> gl(G, 0.0), ll(topo.L, 0.0);
+    auto t0 = std::chrono::steady_clock::now();
+    bool timed_out = false;
+    long long nodes = 0;
+    double total = suffix[0];
+    std::function<void(int, int, double)> rec = [&](int k, int used, double cur) {
+        if (timed_out) return;
+        if ((++nodes & 4095) == 0) {
+            auto ms = std::chrono::duration_cast<std::chrono::milliseconds>(std::chrono::steady_clock::now() - t0).count();
+            if (ms > time_limit_ms) { timed_out = true; return; }
+        }
+        double lb = std::max(cur, total / G);
+        if (k < P) lb = std::max(lb, T[ord[k]]);
+        if (lb >= best.tmax - 1e-12) return;
+        if (k == P) {
+            best.tmax = cur;
+            for (int i = 0; i < P; i++) best.assign[i] = a[i];
+            return;
+        }
+        int i = ord[k];
+        int gmax = symmetric ? std::min(G - 1, used) : G - 1;
+        for (int g = 0; g <= gmax; g++) {
+            a[i] = g;
+            gl[g] += T[i];
+            double c = std::max(cur, gl[g]);
+            std::vector<std::pair<int, double>> touched;
+            for (auto& pr : adj[i]) {
+                int j = pr.first;
+                double D = std::fabs(pr.second);
+                int src = pr.second >= 0 ? g : a[j], dst = pr.second >= 0 ? a[j] : g;
+                if (src == dst) continue;
+                for (int l = 0; l < topo.L; l++)
+                    if (topo.carries(l, src, dst)) {
+                        ll[l] += D;
+                        touched.push_back({l, D});
+                        c = std::max(c, lat + ll[l] / bw);
+                    }
+            }
+            rec(k + 1, std::max(used, g + 1), c);
+            for (auto& t : touched) ll[t.first] -= t.second;
+            gl[g] -= T[i];
+            a[i] = -1;
+        }
+    };
+    rec(0, 0, lat);
+    best.optimal = !timed_out;
+    // recompute exactly
+    best.tmax = mapping_cost(T, pdg, topo, lat, bw, best.assign);
+    return best;
+}
+
+// ============================================================ plan assembly
+void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
+    p.flat = Flat::build(g);
+    p.G = G;
+    p.opts = o;
+    const Flat& f = p.flat;
+    const int N = (int)f.nodes.size();
+    // ---- partitions
+    std::vector<std::vector<int>> parts;
+    switch (o.partitioner) {
+    case SG_PART_SINGLE: {
+        std::vector<int> all(N);
+        std::iota(all.begin(), all.end(), 0);
+        parts.push_back(all);
+        break;
+    }
+    case SG_PART_PER_FILTER:
+        for (int v = 0; v < N; v++) parts.push_back({v});
+        break;
+    case SG_PART_USER: {
+        if (!o.node_partition || o.n_node_partition != N)
+            throw Error(SG_E_ARG, "SG_PART_USER needs node_partition[n_nodes] (n_nodes = " + std::to_string(N) + ")");
+        std::map<int, std::vector<int>> m;
+        for (int v = 0; v < N; v++) m[o.node_partition[v]].push_back(v);
+        for (auto& kv : m) parts.push_back(kv.second);
+        break;
+    }
+    case SG_PART_ALGORITHM1: {
+        double cap = 0;
+        if (G > 1) {
+            std::vector<int> all(N);
+            std::iota(all.begin(), all.end(), 0);
+            double sum = 0;
+            for (int v = 0; v < N; v++) sum += pee_estimate(f, {v}).t;
+            // G-aware cap: similar-sized partitions (goal 4)
+            cap = std::max(pee_estimate(f, all).t, sum / 4) / G * 1.25;
+        }
+        parts = algorithm1(f, g, cap);
+        break;
+    }
+    default: throw Error(SG_E_ARG, "unknown partitioner");
+    }
+    // validate: cover, convex; order topologically
+    std::vector<int> owner(N, -1);
+    for (size_t i = 0; i < parts.size(); i++) {
+        std::sort(parts[i].begin(), parts[i].end());
+        std::vector<char> in(N, 0);
+        for (int v : parts[i]) {
+            if (v < 0 || v >= N || owner[v] >= 0) throw Error(SG_E_PLAN, "partitions must cover each node exactly once");
+            owner[v] = (int)i;
+            in[v] = 1;
+        }
+        if (!is_convex(f, in)) throw Error(SG_E_PLAN, "partition " + std::to_string(i) + " is not convex");
+    }
+    for (int v = 0; v < N; v++) if (owner[v] < 0) throw Error(SG_E_PLAN, "node not covered by any partition");
+    const int P = (int)parts.size();
+    std::vector<std::set<int>> succ(P);
+    std::vector<int> indeg(P, 0);
+    for (auto& e : f.edges) {
+        if (e.src < 0 || e.dst < 0) continue;
+        int a = owner[e.src], b = owner[e.dst];
+        if (a != b && succ[a].insert(b).second) indeg[b]++;
+    }
+    std::vector<int> order;
+    std::vector<int> ready;
+    for (int i = 0; i < P; i++) if (!indeg[i]) ready.push_back(i);
+    while (!ready.empty()) {
+        std::sort(ready.begin(), ready.end(), std::greater<int>());
+        int x = ready.back();
+        ready.pop_back();
+        order.push_back(x);
+        for (int y : succ[x]) if (--indeg[y] == 0) ready.push_back(y);
+    }
+    if ((int)order.size() != P) throw Error(SG_E_PLAN, "partition graph is cyclic");
+    p.parts.assign(P, Partition());
+    p.part_order = order;
+    p.part_time.assign(P, 0.0);
+    p.part_mode.assign(P, 0);
+    std::vector<double> T(P);
+    for (int i = 0; i < P; i++) {
+        p.parts[i].nodes = parts[i];
+        PeeEstimate est = pee_estimate(f, parts[i]);
+        p.parts[i].t_est = T[i] = est.t;
+        p.parts[i].t_comp = est.t_comp;
+        p.parts[i].t_dt = est.t_dt;
+        p.part_time[i] = est.t;
+    }
+    // ---- PDG: D_ij = sum of the weights of crossing edges (bytes / iteration)
+    std::map<std::pair<int, int>, double> D;
+    for (auto& e : f.edges) {
+        if (e.src < 0 || e.dst < 0) continue;
+        int a = owner[e.src], b = owner[e.dst];
+        if (a != b) D[{a, b}] += 4.0 * e.per_iter;
+    }
+    p.pdg.clear();
+    for (auto& kv : D) p.pdg.push_back({kv.first.first, kv.first.second, kv.second});
+    // ---- mapping
+    p.part_gpu.assign(P, 0);
+    if (G > 1) {
+        Topology topo = Topology::nvswitch(G);
+        double bw = o.link_gbps > 0 ? o.link_gbps : 770.0;          // bytes per ns
+        double lat_us = o.link_latency_us > 0 ? o.link_latency_us : 10.0;
+        double lat = lat_us * 1e3 / 65536.0;                          // amortised per iteration (reading 12)
+        MapResult m = map_partitions(T, p.pdg, topo, lat, bw, o.ilp_time_limit_ms > 0 ? o.ilp_time_limit_ms : 10000, 0);
+        for (int i = 0; i < P; i++) p.part_gpu[i] = m.assign[i];
+        p.est_tmax = m.tmax;
+        p.ilp_optimal = m.optimal;
+    } else {
+        p.est_tmax = std::accumulate(T.begin(), T.end(), 0.0);
+        p.ilp_optimal = true;
+    }
+    // ---- devices
+    p.virtual_gpus = o.virtual_gpus != 0;
+    p.devices.assign(G, 0);
+    for (int gi = 0; gi < G; gi++) p.devices[gi] = o.devices ? o.devices[gi] : (p.virtual_gpus ? 0 : gi);
+    p.input_gpu = p.part_gpu[owner[f.edges[f.in_edge].dst]];
+    p.output_gpu = p.part_gpu[owner[f.edges[f.out_edge].src]];
+    p.iters_per_fragment = o.iters_per_fragment;
+    // ---- code generation + NVRTC (one kernel per partition)
+    p.kernels.resize(P);
+    CodegenOpts co;
+    co.mode = o.codegen_mode;
+    co.threads = o.threads;
+    co.tile = o.tile_iters;
+    for (int i = 0; i < P; i++) {
+        p.kernels[i].ki = generate_kernel(f, parts[i], i, co);
+        compile_kernel(p.kernels[i], o.verbose);
+        p.part_mode[i] = p.kernels[i].ki.mode;
+        p.parts[i].mode = p.kernels[i].ki.mode;
+        p.parts[i].gpu = p.part_gpu[i];
+        p.parts[i].tile = p.kernels[i].ki.tile;
+        p.parts[i].threads = p.kernels[i].ki.threads;
+    }
+    // ---- info arrays
+    p.reps.resize(N);
+    p.ninit.resize(N);
+    p.node_type.resize(N);
+    p.node_kind.resize(N);
+    p.node_part.resize(N);
+    for (int v = 0; v < N; v++) {
+        p.reps[v] = f.nodes[v].rep;
+        p.ninit[v] = f.nodes[v].ninit;
+        p.node_type[v] = (int32_t)f.nodes[v].type;
+        p.node_kind[v] = f.nodes[v].kind;
+        p.node_part[v] = owner[v];
+    }
+}
+
+}  // namespace sg

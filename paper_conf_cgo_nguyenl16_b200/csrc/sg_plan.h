@@ -1,0 +1,43 @@
+// sg_plan.h -- planner: PEE, Algorithm 1, PDG, ILP mapping, plan assembly.
+#pragma once
+#include <array>
+#include <vector>
+
+#include "sg_internal.h"
+#include "sg_runtime.h"
+
+namespace sg {
+
+// B200 performance-estimation engine (section 3.3, re-derived
+// for sm_100a): estimate of one partition, ns per steady-state iteration.
+struct PeeEstimate {
+    double t = 0, t_comp = 0, t_dt = 0;
+    int mode = 0;
+    bool io_bound() const { return t_dt >= t_comp; }
+};
+PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes);
+
+// The paper's analytic model Eq. III.8-III.12, kept as a
+// reference implementation for tests and reports (calibrated for M2090).
+double paper_model(const std::vector<double>& t, const std::vector<double>& fr, int S, int W, int F, double D,
+                   double C1, double C2, double* tcomp, double* tdt, double* tdb);
+
+bool is_convex(const Flat& f, const std::vector<char>& in_set);
+
+// Algorithm 1.  cap > 0 limits T(merged) (G-aware).
+std::vector<std::vector<int>> algorithm1(const Flat& f, const sg_graph& g, double cap);
+
+// ILP of Eq. III.1-III.7 solved exactly by branch and bound (or brute force).
+struct MapResult {
+    std::vector<int> assign;
+    double tmax = 0;
+    bool optimal = false;
+};
+MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge>& pdg, const Topology& topo,
+                         double lat, double bw, int time_limit_ms, int method);
+double mapping_cost(const std::vector<double>& T, const std::vector<PdgEdge>& pdg, const Topology& topo, double lat,
+                    double bw, const std::vector<int>& assign);
+
+void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o);
+
+}  // namespace sg

@@ -1,0 +1,507 @@
+// sg_runtime.cpp -- NVRTC compilation, module management and the pipelined
+// multi-GPU execution of a plan.
+//
+// Execution model (section 3.2.3, Fig. 3.5): the iteration
+// range is cut into fragments; "partitions mapped to the same GPU run
+// sequentially"; boundary streams of fragment n move to the consumer GPU while
+// the producer GPU already computes fragment n+1.  Transfers are peer-to-peer
+// -- over NVLink/NVSwitch on B200 -- on a dedicated copy
+// stream per GPU, double-buffered (ring of `ring_depth` slots per cut edge),
+// ordered by CUDA events only; the host never synchronises inside sg_run.
+//
+// Fragments never share state: every partition kernel recomputes the peek
+// halo of its first tile (sg_codegen.cpp), and each cut-edge slot holds the
+// whole window the consumer needs for the fragment (halo included).
+#include "sg_runtime.h"
+
+#include <dlfcn.h>
+#include <nvrtc.h>
+#include <sys/stat.h>
+
+#include <algorithm>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <fstream>
+#include <map>
+#include <mutex>
+#include <sstream>
+
+namespace sg {
+
+// ------------------------------------------------------- driver API shim
+// libsg.so does not link libcuda: driver entry points are resolved through
+// the runtime (cudaGetDriverEntryPoint) on first use, so the library loads on
+// machines without a driver (CPU build/plan checks) and fails loudly at run.
+namespace drv {
+typedef CUresult (*PFN_load)(CUmodule*, const void*);
+typedef CUresult (*PFN_getfn)(CUfunction*, CUmodule, const char*);
+typedef CUresult (*PFN_setattr)(CUfunction, CUfunction_attribute, int);
+typedef CUresult (*PFN_occ)(int*, CUfunction, int, size_t);
+typedef CUresult (*PFN_launch)(CUfunction, unsigned, unsigned, unsigned, unsigned, unsigned, unsigned, unsigned,
+                               CUstream, void**, void**);
+typedef CUresult (*PFN_unload)(CUmodule);
+typedef CUresult (*PFN_errstr)(CUresult, const char**);
+struct Api {
+    PFN_load load = nullptr;
+    PFN_getfn getfn = nullptr;
+    PFN_setattr setattr = nullptr;
+    PFN_occ occ = nullptr;
+    PFN_launch launch = nullptr;
+    PFN_unload unload = nullptr;
+    PFN_errstr errstr = nullptr;
+};
+static Api& api() {
+    static Api a;
+    static std::once_flag once;
+    static std::string err;
+    std::call_once(once, [] {
+        auto get = [](const char* name, void** fp) {
+            cudaDriverEntryPointQueryResult q;
+            cudaError_t e = cudaGetDriverEntryPoint(name, fp, cudaEnableDefault, &q);
+            if (e != cudaSuccess || q != cudaDriverEntryPointSuccess) { *fp = nullptr; cudaGetLastError(); }
+        };
+        get("cuModuleLoadData", (void**)&a.load);
+        get("cuModuleGetFunction", (void**)&a.getfn);
+        get("cuFuncSetAttribute", (void**)&a.setattr);
+        get("cuOccupancyMaxActiveBlocksPerMultiprocessor", (void**)&a.occ);
+        get("cuLaunchKernel", (void**)&a.launch);
+        get("cuModuleUnload", (void**)&a.unload);
+        get("cuGetErrorString", (void**)&a.errstr);
+    });
+    if (!a.load || !a.launch) throw Error(SG_E_CUDA, "CUDA driver not available (no GPU): the executor has no CPU fallback");
+    return a;
+}
+}  // namespace drv
+
+#define cuModuleLoadData drv::api().load
+#define cuModuleGetFunction drv::api().getfn
+#define cuFuncSetAttribute drv::api().setattr
+#define cuOccupancyMaxActiveBlocksPerMultiprocessor drv::api().occ
+#define cuLaunchKernel drv::api().launch
+#define cuModuleUnload drv::api().unload
+static const char* drv_errstr(CUresult r) {
+    const char* s = nullptr;
+    if (drv::api().errstr) drv::api().errstr(r, &s);
+    return s ? s : "?";
+}
+
+#define SG_CU(x)                                                                          \
+    do {                                                                                  \
+        CUresult r_ = (x);                                                                \
+        if (r_ != CUDA_SUCCESS) throw Error(SG_E_CUDA, std::string(#x) + ": " + drv_errstr(r_)); \
+    } while (0)
+#define SG_RT(x)                                                                          \
+    do {                                                                                  \
+        cudaError_t r_ = (x);                                                             \
+        if (r_ != cudaSuccess) throw Error(SG_E_CUDA, std::string(#x) + ": " + cudaGetErrorString(r_)); \
+    } while (0)
+
+// ------------------------------------------------------------------ NVRTC
+static std::mutex g_cache_mu;
+static std::map<uint64_t, std::string> g_cubin_cache;
+
+static uint64_t fnv1a(const std::string& s, uint64_t h = 1469598103934665603ULL) {
+    for (unsigned char c : s) { h ^= c; h *= 1099511628211ULL; }
+    return h;
+}
+
+std::string nvrtc_version() {
+    int maj = 0, min = 0;
+    nvrtcVersion(&maj, &min);
+    return std::to_string(maj) + "." + std::to_string(min);
+}
+
+static std::string cache_dir() {
+    const char* env = std::getenv("SG_CACHE_DIR");
+    if (env && *env) return env;
+    Dl_info info;
+    if (dladdr((void*)&cache_dir, &info) && info.dli_fname) {
+        std::string p = info.dli_fname;
+        size_t k = p.rfind('/');
+        if (k != std::string::npos) return p.substr(0, k) + "/.sg_cache";
+    }
+    return ".sg_cache";
+}
+
+static const char* kNvrtcOpts[] = {"--gpu-architecture=sm_100a", "--fmad=false",       "--std=c++17",
+                                   "-default-device",            "--generate-line-info", "--prec-div=true",
+                                   "--prec-sqrt=true",           "--ftz=false",         "-DSG_NVRTC=1"};
+
+void compile_kernel(CompiledKernel& ck, int verbose) {
+    std::string key_src = ck.ki.source + "\n//" + nvrtc_version();
+    for (const char* o : kNvrtcOpts) key_src += o;
+    key_src += kDeviceHeader;
+    uint64_t key = fnv1a(key_src);
+    {
+        std::lock_guard<std::mutex> lk(g_cache_mu);
+        auto it = g_cubin_cache.find(key);
+        if (it != g_cubin_cache.end()) { ck.cubin = it->second; return; }
+    }
+    char hex[32];
+    std::snprintf(hex, sizeof hex, "%016llx", (unsigned long long)key);
+    std::string dir = cache_dir();
+    std::string path = dir + "/" + hex + ".cubin";
+    {
+        std::ifstream in(path, std::ios::binary);
+        if (in) {
+            std::stringstream ss;
+            ss << in.rdbuf();
+            ck.cubin = ss.str();
+            if (!ck.cubin.empty()) {
+                std::lock_guard<std::mutex> lk(g_cache_mu);
+                g_cubin_cache[key] = ck.cubin;
+                return;
+            }
+        }
+    }
+    nvrtcProgram prog;
+    const char* hdrs[] = {kDeviceHeader};
+    const char* names[] = {"sg_device.cuh"};
+    if (nvrtcCreateProgram(&prog, ck.ki.source.c_str(), (ck.ki.name + ".cu").c_str(), 1, hdrs, names) != NVRTC_SUCCESS)
+        throw Error(SG_E_CUDA, "nvrtcCreateProgram failed");
+    std::vector<const char*> opts(std::begin(kNvrtcOpts), std::end(kNvrtcOpts));
+    if (verbose) opts.push_back("--ptxas-options=-v");
+    nvrtcResult rc = nvrtcCompileProgram(prog, (int)opts.size(), opts.data());
+    size_t logn = 0;
+    nvrtcGetProgramLogSize(prog, &logn);
+    std::string log(logn, '\0');
+    if (logn) nvrtcGetProgramLog(prog, &log[0]);
+    ck.log = log;
+    if (rc != NVRTC_SUCCESS) {
+        nvrtcDestroyProgram(&prog);
+        if (verbose) std::fprintf(stderr, "%s\n", ck.ki.source.c_str());
+        throw Error(SG_E_CUDA, "NVRTC failed for " + ck.ki.name + ":\n" + log.substr(0, 4000));
+    }
+    size_t n = 0;
+    nvrtcGetCUBINSize(prog, &n);
+    ck.cubin.assign(n, '\0');
+    nvrtcGetCUBIN(prog, &ck.cubin[0]);
+    nvrtcDestroyProgram(&prog);
+    if (verbose && !log.empty()) std::fprintf(stderr, "[sg] %s: %s\n", ck.ki.name.c_str(), log.c_str());
+    {
+        std::lock_guard<std::mutex> lk(g_cache_mu);
+        g_cubin_cache[key] = ck.cubin;
+    }
+    mkdir(dir.c_str(), 0755);
+    std::string tmp = path + ".tmp" + std::to_string((unsigned long long)(uintptr_t)&ck);
+    std::ofstream out(tmp, std::ios::binary);
+    if (out) {
+        out.write(ck.cubin.data(), (std::streamsize)ck.cubin.size());
+        out.close();
+        std::rename(tmp.c_str(), path.c_str());
+    }
+}
+
+// ---------------------------------------------------------------- helpers
+namespace {
+struct DevGuard {
+    int old = -1;
+    explicit DevGuard(int dev) {
+        if (cudaGetDevice(&old) != cudaSuccess) old = -1;
+        SG_RT(cudaSetDevice(dev));
+    }
+    ~DevGuard() {
+        if (old >= 0) cudaSetDevice(old);
+    }
+};
+
+void ensure_module(CompiledKernel& ck, int dev) {
+    if ((int)ck.fn.size() <= dev) {
+        ck.mod.resize(dev + 1, nullptr);
+        ck.fn.resize(dev + 1, nullptr);
+        ck.max_blocks_per_sm.resize(dev + 1, 0);
+    }
+    if (ck.fn[dev]) return;
+    SG_RT(cudaFree(nullptr));  // make the primary context current
+    SG_CU(cuModuleLoadData(&ck.mod[dev], ck.cubin.data()));
+    SG_CU(cuModuleGetFunction(&ck.fn[dev], ck.mod[dev], ck.ki.name.c_str()));
+    SG_CU(cuFuncSetAttribute(ck.fn[dev], CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)ck.ki.smem));
+    int nb = 0;
+    SG_CU(cuOccupancyMaxActiveBlocksPerMultiprocessor(&nb, ck.fn[dev], ck.ki.threads, ck.ki.smem));
+    if (nb <= 0)
+        throw Error(SG_E_SIZE, ck.ki.name + " cannot be resident (" + std::to_string(ck.ki.smem) + " B smem, " +
+                                   std::to_string(ck.ki.threads) + " threads)");
+    ck.max_blocks_per_sm[dev] = nb;
+}
+
+int sm_count(int dev) {
+    static std::map<int, int> cache;
+    static std::mutex mu;
+    std::lock_guard<std::mutex> lk(mu);
+    auto it = cache.find(dev);
+    if (it != cache.end()) return it->second;
+    int n = 0;
+    SG_RT(cudaDeviceGetAttribute(&n, cudaDevAttrMultiProcessorCount, dev));
+    cache[dev] = n;
+    return n;
+}
+
+struct IoBinding {
+    std::vector<const void*> in;
+    std::vector<int64_t> in_base, in_limit;
+    std::vector<void*> out;
+    std::vector<int64_t> out_base;
+};
+
+// Launch one partition kernel over iterations [kb, ke) on `stream`.
+int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int64_t ke, cudaStream_t stream) {
+    if (ke <= kb) return 0;
+    ensure_module(ck, dev);
+    std::vector<int64_t> v;
+    for (auto p : io.in) v.push_back((int64_t)(uintptr_t)p);
+    for (auto b : io.in_base) v.push_back(b);
+    for (auto l : io.in_limit) v.push_back(l);
+    for (auto p : io.out) v.push_back((int64_t)(uintptr_t)p);
+    for (auto b : io.out_base) v.push_back(b);
+    v.push_back(kb);
+    v.push_back(ke);
+    int64_t tiles = (ke - kb + ck.ki.tile - 1) / ck.ki.tile;
+    int64_t grid = std::min<int64_t>(tiles, (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev]);
+    void* params[] = {v.data()};
+    SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ck.ki.threads, 1, 1, (unsigned)ck.ki.smem,
+                         (CUstream)stream, params, nullptr));
+    return 1;
+}
+}  // namespace
+
+Plan::~Plan() {
+    for (auto& r : rings) {
+        for (size_t i = 0; i < r.src_slots.size(); i++) {
+            if (r.src_slots[i]) { cudaSetDevice(devices[r.src_gpu]); cudaFree(r.src_slots[i]); }
+            if (r.dst_slots.size() > i && r.dst_slots[i] && r.dst_slots[i] != r.src_slots[i]) {
+                cudaSetDevice(devices[r.dst_gpu]);
+                cudaFree(r.dst_slots[i]);
+            }
+        }
+        for (auto e : r.ev_copied) if (e) cudaEventDestroy(e);
+        for (auto e : r.ev_consumed) if (e) cudaEventDestroy(e);
+        for (auto e : r.ev_produced) if (e) cudaEventDestroy(e);
+    }
+    for (auto& g : gpus) {
+        cudaSetDevice(g.dev);
+        if (g.compute) cudaStreamDestroy(g.compute);
+        if (g.copy) cudaStreamDestroy(g.copy);
+        if (g.ev_start) cudaEventDestroy(g.ev_start);
+        if (g.ev_done) cudaEventDestroy(g.ev_done);
+    }
+    if (user_ev) cudaEventDestroy(user_ev);
+    for (auto& ck : kernels)
+        for (size_t d = 0; d < ck.mod.size(); d++)
+            if (ck.mod[d]) { cudaSetDevice((int)d); drv::api().unload(ck.mod[d]); }
+}
+
+void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
+    if (n <= 0) return;
+    int ndev = 0;
+    if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0) {
+        cudaGetLastError();
+        throw Error(SG_E_CUDA, "no CUDA device: the executor has no CPU fallback");
+    }
+    for (int d : devices)
+        if (d >= ndev) throw Error(SG_E_CUDA, "plan maps a GPU to device " + std::to_string(d) + " but only " +
+                                                  std::to_string(ndev) + " are visible");
+    last_launches = 0;
+    const int64_t n_in = flat.input_items(n);
+    // ---- fast path: one partition on one GPU, launched on the caller's stream
+    if (parts.size() == 1) {
+        CompiledKernel& ck = kernels[0];
+        DevGuard dg(devices[0]);
+        IoBinding io;
+        io.in = {in};
+        io.in_base = {0};
+        io.in_limit = {n_in};
+        io.out = {out};
+        io.out_base = {0};
+        last_launches += launch(ck, devices[0], io, 0, n, stream);
+        return;
+    }
+    // ---- general path: fragments pipelined over partitions and GPUs
+    int64_t F = iters_per_fragment;
+    if (F <= 0) {  // auto: >= 2 full waves per kernel, ~8 fragments per GPU for pipelining
+        int64_t wave = 1;
+        for (auto& ck : kernels) wave = std::max<int64_t>(wave, (int64_t)ck.ki.tile * 148 * 2);
+        F = std::max<int64_t>(wave, (n + 8 * G - 1) / (8 * G));
+        int64_t ring_bytes_per_iter = 0;
+        for (auto& e : flat.edges)
+            if (e.src >= 0 && e.dst >= 0 && node_part[e.src] != node_part[e.dst]) ring_bytes_per_iter += 4 * e.per_iter;
+        if (ring_bytes_per_iter > 0) F = std::min<int64_t>(F, std::max<int64_t>(wave, ((int64_t)1 << 30) / ring_bytes_per_iter));
+    }
+    F = std::min(F, n);
+    if (rt_ready && rt_fragment >= F) F = std::min(rt_fragment, n);
+    if (!rt_ready || rt_fragment < F) {
+        // (re)allocate rings for fragment size F
+        for (auto& r : rings) {
+            for (size_t i = 0; i < r.src_slots.size(); i++) {
+                cudaSetDevice(devices[r.src_gpu]);
+                if (r.src_slots[i]) cudaFree(r.src_slots[i]);
+                if (r.dst_slots[i] && r.dst_slots[i] != r.src_slots[i]) {
+                    cudaSetDevice(devices[r.dst_gpu]);
+                    cudaFree(r.dst_slots[i]);
+                }
+            }
+            for (auto e : r.ev_copied) cudaEventDestroy(e);
+            for (auto e : r.ev_consumed) cudaEventDestroy(e);
+            for (auto e : r.ev_produced) cudaEventDestroy(e);
+        }
+        rings.clear();
+        if (gpus.empty()) {
+            gpus.resize(G);
+            for (int g = 0; g < G; g++) {
+                gpus[g].dev = devices[g];
+                DevGuard dg(devices[g]);
+                SG_RT(cudaStreamCreateWithFlags(&gpus[g].compute, cudaStreamNonBlocking));
+                SG_RT(cudaStreamCreateWithFlags(&gpus[g].copy, cudaStreamNonBlocking));
+                SG_RT(cudaEventCreateWithFlags(&gpus[g].ev_start, cudaEventDisableTiming));
+                SG_RT(cudaEventCreateWithFlags(&gpus[g].ev_done, cudaEventDisableTiming));
+            }
+            // enable peer access between distinct physical devices
+            for (int a = 0; a < G; a++)
+                for (int b = 0; b < G; b++) {
+                    if (devices[a] == devices[b]) continue;
+                    int ok = 0;
+                    cudaDeviceCanAccessPeer(&ok, devices[a], devices[b]);
+                    if (ok) {
+                        DevGuard dg(devices[a]);
+                        cudaError_t e = cudaDeviceEnablePeerAccess(devices[b], 0);
+                        if (e != cudaSuccess && e != cudaErrorPeerAccessAlreadyEnabled)
+                            throw Error(SG_E_COMM, std::string("peer access: ") + cudaGetErrorString(e));
+                        cudaGetLastError();
+                    }
+                }
+        }
+        // cut edges between partitions
+        for (size_t ei = 0; ei < flat.edges.size(); ei++) {
+            const Edge& ed = flat.edges[ei];
+            if (ed.src < 0 || ed.dst < 0) continue;
+            int ps = node_part[ed.src], pd = node_part[ed.dst];
+            if (ps == pd) continue;
+            CutRing r;
+            r.edge = (int)ei;
+            r.src_part = ps;
+            r.dst_part = pd;
+            r.src_gpu = part_gpu[ps];
+            r.dst_gpu = part_gpu[pd];
+            edge_window(flat, (int)ei, r.lo, r.extra);
+            r.per_iter = ed.per_iter;
+            r.slot_items = r.per_iter * F + r.extra;
+            for (int s = 0; s < ring_depth; s++) {
+                void* p = nullptr;
+                {
+                    DevGuard dg(devices[r.src_gpu]);
+                    SG_RT(cudaMalloc(&p, (size_t)r.slot_items * 4));
+                }
+                r.src_slots.push_back(p);
+                void* q = p;
+                if (r.dst_gpu != r.src_gpu) {
+                    DevGuard dg(devices[r.dst_gpu]);
+                    SG_RT(cudaMalloc(&q, (size_t)r.slot_items * 4));
+                }
+                r.dst_slots.push_back(q);
+                cudaEvent_t e1, e2, e3;
+                {
+                    DevGuard dg(devices[r.dst_gpu]);
+                    SG_RT(cudaEventCreateWithFlags(&e2, cudaEventDisableTiming));
+                }
+                {
+                    DevGuard dg(devices[r.src_gpu]);
+                    SG_RT(cudaEventCreateWithFlags(&e1, cudaEventDisableTiming));
+                    SG_RT(cudaEventCreateWithFlags(&e3, cudaEventDisableTiming));
+                }
+                r.ev_copied.push_back(e1);
+                r.ev_consumed.push_back(e2);
+                r.ev_produced.push_back(e3);
+            }
+            rings.push_back(std::move(r));
+        }
+        if (!user_ev) SG_RT(cudaEventCreateWithFlags(&user_ev, cudaEventDisableTiming));
+        rt_fragment = F;
+        rt_ready = true;
+    }
+    // per partition: which rings feed it / leave it
+    std::vector<std::vector<int>> ring_in(parts.size()), ring_out(parts.size());
+    for (size_t ri = 0; ri < rings.size(); ri++) {
+        ring_in[rings[ri].dst_part].push_back((int)ri);
+        ring_out[rings[ri].src_part].push_back((int)ri);
+    }
+    // order every GPU after the caller's stream
+    SG_RT(cudaEventRecord(user_ev, stream));
+    for (auto& g : gpus) {
+        DevGuard dg(g.dev);
+        SG_RT(cudaStreamWaitEvent(g.compute, user_ev, 0));
+        SG_RT(cudaStreamWaitEvent(g.copy, user_ev, 0));
+    }
+    const int64_t nfrag = (n + F - 1) / F;
+    for (int64_t fi = 0; fi < nfrag; fi++) {
+        const int64_t ka = fi * F, kb = std::min(n, ka + F);
+        const int slot = (int)(fi % ring_depth);
+        for (int p : part_order) {
+            CompiledKernel& ck = kernels[p];
+            const int g = part_gpu[p];
+            GpuCtx& gc = gpus[g];
+            DevGuard dg(gc.dev);
+            IoBinding io;
+            for (int e : ck.ki.in_edges) {
+                if (flat.edges[e].src < 0) {  // graph input (resident on this GPU: input_gpu)
+                    io.in.push_back(in);
+                    io.in_base.push_back(0);
+                    io.in_limit.push_back(n_in);
+                    continue;
+                }
+                int ri = -1;
+                for (int r : ring_in[p]) if (rings[r].edge == e) ri = r;
+                CutRing& r = rings[ri];
+                if (r.src_gpu != r.dst_gpu) SG_RT(cudaStreamWaitEvent(gc.compute, r.ev_copied[slot], 0));
+                io.in.push_back(r.dst_slots[slot]);
+                io.in_base.push_back(ka * r.per_iter + r.lo);
+                io.in_limit.push_back(r.slot_items);
+            }
+            for (int e : ck.ki.out_edges) {
+                if (flat.edges[e].dst < 0) {
+                    io.out.push_back(out);
+                    io.out_base.push_back(0);
+                    continue;
+                }
+                int ri = -1;
+                for (int r : ring_out[p]) if (rings[r].edge == e) ri = r;
+                CutRing& r = rings[ri];
+                // slot reuse: the copy (or the same-GPU consumer) of fragment fi - depth must be done
+                if (fi >= ring_depth) {
+                    if (r.src_gpu != r.dst_gpu) SG_RT(cudaStreamWaitEvent(gc.compute, r.ev_copied[slot], 0));
+                    else SG_RT(cudaStreamWaitEvent(gc.compute, r.ev_consumed[slot], 0));
+                }
+                io.out.push_back(r.src_slots[slot]);
+                io.out_base.push_back(ka * r.per_iter + r.lo);
+            }
+            last_launches += launch(ck, gc.dev, io, ka, kb, gc.compute);
+            // consumed slots of incoming rings are free again
+            for (int ri : ring_in[p]) SG_RT(cudaEventRecord(rings[ri].ev_consumed[slot], gc.compute));
+            // ship outgoing boundary streams to other GPUs (copy engine, P2P)
+            for (int ri : ring_out[p]) {
+                CutRing& r = rings[ri];
+                if (r.src_gpu == r.dst_gpu) continue;
+                SG_RT(cudaEventRecord(r.ev_produced[slot], gc.compute));
+                SG_RT(cudaStreamWaitEvent(gc.copy, r.ev_produced[slot], 0));
+                if (fi >= ring_depth) SG_RT(cudaStreamWaitEvent(gc.copy, r.ev_consumed[slot], 0));
+                int64_t items = r.per_iter * (kb - ka) + r.extra;
+                if (devices[r.src_gpu] == devices[r.dst_gpu])
+                    SG_RT(cudaMemcpyAsync(r.dst_slots[slot], r.src_slots[slot], (size_t)items * 4,
+                                          cudaMemcpyDeviceToDevice, gc.copy));
+                else
+                    SG_RT(cudaMemcpyPeerAsync(r.dst_slots[slot], devices[r.dst_gpu], r.src_slots[slot],
+                                              devices[r.src_gpu], (size_t)items * 4, gc.copy));
+                SG_RT(cudaEventRecord(r.ev_copied[slot], gc.copy));
+            }
+        }
+    }
+    // join everything back onto the caller's stream
+    for (auto& g : gpus) {
+        DevGuard dg(g.dev);
+        SG_RT(cudaEventRecord(g.ev_done, g.compute));
+        SG_RT(cudaStreamWaitEvent(stream, g.ev_done, 0));
+        SG_RT(cudaEventRecord(g.ev_start, g.copy));
+        SG_RT(cudaStreamWaitEvent(stream, g.ev_start, 0));
+    }
+}
+
+}  // namespace sg

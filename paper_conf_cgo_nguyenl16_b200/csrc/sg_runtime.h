@@ -1,0 +1,75 @@
+// sg_runtime.h -- plan object and runtime of the stream-graph executor.
+#pragma once
+#include <cuda.h>
+#include <cuda_runtime.h>
+
+#include <string>
+#include <vector>
+
+#include "sg_codegen.h"
+#include "sg_internal.h"
+
+namespace sg {
+
+struct CompiledKernel {
+    KernelInfo ki;
+    std::string cubin;
+    std::string log;
+    // per physical device (index = device ordinal)
+    std::vector<CUmodule> mod;
+    std::vector<CUfunction> fn;
+    std::vector<int> max_blocks_per_sm;
+};
+
+struct CutRing {          // one boundary stream between partitions (a PDG edge member)
+    int edge = -1;
+    int src_part = -1, dst_part = -1;  // -1: graph input / output
+    int src_gpu = 0, dst_gpu = 0;
+    int64_t lo = 0, extra = 0, per_iter = 0;
+    int64_t slot_items = 0;
+    std::vector<void*> src_slots, dst_slots;  // device buffers (dst == src when same GPU)
+    std::vector<cudaEvent_t> ev_copied, ev_consumed, ev_produced;
+};
+
+struct GpuCtx {
+    int dev = 0;
+    cudaStream_t compute = nullptr, copy = nullptr;
+    cudaEvent_t ev_start = nullptr, ev_done = nullptr;
+};
+
+struct Plan {
+    Flat flat;
+    int G = 1;
+    sg_plan_opts opts{};
+    std::vector<Partition> parts;
+    std::vector<int> part_order;           // topological order of partitions
+    std::vector<CompiledKernel> kernels;   // one per partition
+    std::vector<int> devices;              // logical gpu -> physical device
+    bool virtual_gpus = false;
+    double est_tmax = 0;
+    bool ilp_optimal = false;
+    std::vector<PdgEdge> pdg;
+    // info arrays
+    std::vector<int64_t> reps, ninit;
+    std::vector<int32_t> node_type, node_kind, node_part, part_gpu, part_mode;
+    std::vector<double> part_time;
+    int input_gpu = 0, output_gpu = 0;
+    int64_t iters_per_fragment = 0;
+    // runtime state (created lazily)
+    bool rt_ready = false;
+    std::vector<GpuCtx> gpus;
+    std::vector<CutRing> rings;
+    int64_t rt_fragment = 0;
+    int ring_depth = 2;
+    int64_t last_launches = 0;
+    cudaEvent_t user_ev = nullptr;
+
+    ~Plan();
+    void run(const void* in, int64_t n, void* out, cudaStream_t stream);
+};
+
+// NVRTC -> sm_100a cubin (cached by content hash in memory and on disk).
+void compile_kernel(CompiledKernel& ck, int verbose);
+std::string nvrtc_version();
+
+}  // namespace sg

@@ -1,0 +1,294 @@
+"""Thin ctypes binding of libsg.so (include/sg.h).  Argument marshalling only:
+every step of the stream-graph path (rates, planning, code generation, kernels,
+transfers) runs in the native library.  There is no CPU fallback: sg_run on a
+machine without a CUDA device fails with SG_E_CUDA.
+
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    with sg.plan(program, n_gpus=1) as p:          # program: workloads.spec.Program or sg.Graph
+        p.run(x_cuda, n_iters, y_cuda)             # device tensors, current torch stream
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+from typing import Optional, Sequence
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+_LIB_PATH = os.path.join(_HERE, "libsg.so")
+_lib = None
+
+SG_OK, SG_E_ARG, SG_E_STRUCTURE, SG_E_RATE, SG_E_UNSUPPORTED = 0, -1, -2, -3, -4
+SG_E_NOMEM, SG_E_CUDA, SG_E_COMM, SG_E_PLAN, SG_E_SIZE = -5, -6, -7, -8, -9
+SG_F32, SG_I32 = 0, 1
+SG_PART_ALGORITHM1, SG_PART_SINGLE, SG_PART_PER_FILTER, SG_PART_USER = 0, 1, 2, 3
+
+KINDS = {"IDENTITY": 0, "FIR": 1, "DELAY": 2, "DECIMATE": 3, "EXPAND": 4, "COMPARE_EXCHANGE": 5,
+         "FFT_REORDER": 6, "COMBINE_DFT": 7, "FM_DEMOD": 8, "SUBTRACT": 9, "AMPLIFY": 10, "ADD": 11,
+         "BEAM_FIR": 12, "BEAMFORM": 13, "MAGNITUDE": 14}
+
+EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_splitjoin", "sg_branch_begin",
+           "sg_branch_end", "sg_plan_opts_default", "sg_plan", "sg_input_items", "sg_output_items",
+           "sg_plan_info", "sg_plan_source", "sg_run", "sg_run_host", "sg_last_launch_count",
+           "sg_plan_destroy", "sg_last_error", "sg_version", "sg_flush_l2"]
+
+
+class SgError(RuntimeError):
+    def __init__(self, code: int, msg: str):
+        super().__init__(f"[sg status {code}] {msg}")
+        self.code = code
+
+
+class FilterDesc(ctypes.Structure):
+    _fields_ = [("kind", ctypes.c_int), ("n_i", ctypes.c_int32), ("p_i", ctypes.POINTER(ctypes.c_int32)),
+                ("n_f", ctypes.c_int32), ("p_f", ctypes.POINTER(ctypes.c_float))]
+
+
+class PlanOpts(ctypes.Structure):
+    _fields_ = [("partitioner", ctypes.c_int32), ("node_partition", ctypes.POINTER(ctypes.c_int32)),
+                ("n_node_partition", ctypes.c_int32), ("tile_iters", ctypes.c_int32), ("threads", ctypes.c_int32),
+                ("iters_per_fragment", ctypes.c_int64), ("transport", ctypes.c_int32),
+                ("virtual_gpus", ctypes.c_int32), ("devices", ctypes.POINTER(ctypes.c_int32)),
+                ("ilp_time_limit_ms", ctypes.c_int32), ("codegen_mode", ctypes.c_int32),
+                ("link_gbps", ctypes.c_double), ("link_latency_us", ctypes.c_double), ("verbose", ctypes.c_int32)]
+
+
+class PlanInfo(ctypes.Structure):
+    _fields_ = [("n_nodes", ctypes.c_int32), ("n_edges", ctypes.c_int32), ("n_partitions", ctypes.c_int32),
+                ("n_gpus", ctypes.c_int32), ("in_per_iter", ctypes.c_int64), ("out_per_iter", ctypes.c_int64),
+                ("reps", ctypes.POINTER(ctypes.c_int64)), ("init_firings", ctypes.POINTER(ctypes.c_int64)),
+                ("node_type", ctypes.POINTER(ctypes.c_int32)), ("node_kind", ctypes.POINTER(ctypes.c_int32)),
+                ("node_partition", ctypes.POINTER(ctypes.c_int32)), ("partition_gpu", ctypes.POINTER(ctypes.c_int32)),
+                ("partition_time", ctypes.POINTER(ctypes.c_double)),
+                ("partition_mode", ctypes.POINTER(ctypes.c_int32)), ("est_tmax", ctypes.c_double),
+                ("input_device", ctypes.c_int32), ("output_device", ctypes.c_int32),
+                ("iters_per_fragment", ctypes.c_int64), ("ilp_optimal", ctypes.c_int32)]
+
+
+def lib():
+    """Load libsg.so (building it in-tree with nvcc if it is not there yet)."""
+    global _lib
+    if _lib is not None:
+        return _lib
+    if not os.path.exists(_LIB_PATH):
+        from . import build as _b
+        _b.build()
+    L = ctypes.CDLL(_LIB_PATH)
+    vp, i32, i64 = ctypes.c_void_p, ctypes.c_int32, ctypes.c_int64
+    sig = {
+        "sg_graph_create": ([ctypes.c_int, ctypes.POINTER(vp)], ctypes.c_int),
+        "sg_graph_destroy": ([vp], None),
+        "sg_add_filter": ([vp, ctypes.POINTER(FilterDesc), ctypes.POINTER(i32)], ctypes.c_int),
+        "sg_add_splitjoin": ([vp, ctypes.c_int, ctypes.POINTER(i32), ctypes.POINTER(i32), i32, ctypes.POINTER(i32)],
+                             ctypes.c_int),
+        "sg_branch_begin": ([vp, i32, i32], ctypes.c_int),
+        "sg_branch_end": ([vp], ctypes.c_int),
+        "sg_plan_opts_default": ([ctypes.POINTER(PlanOpts)], None),
+        "sg_plan": ([vp, i32, ctypes.POINTER(PlanOpts), ctypes.POINTER(vp)], ctypes.c_int),
+        "sg_input_items": ([vp, i64], i64),
+        "sg_output_items": ([vp, i64], i64),
+        "sg_plan_info": ([vp, ctypes.POINTER(PlanInfo)], ctypes.c_int),
+        "sg_plan_source": ([vp, i32], ctypes.c_char_p),
+        "sg_run": ([vp, vp, i64, vp, vp], ctypes.c_int),
+        "sg_run_host": ([vp, vp, i64, vp], ctypes.c_int),
+        "sg_last_launch_count": ([vp], i64),
+        "sg_plan_destroy": ([vp], None),
+        "sg_last_error": ([], ctypes.c_char_p),
+        "sg_version": ([], ctypes.c_char_p),
+        "sg_flush_l2": ([vp, i64, vp], ctypes.c_int),
+    }
+    for name, (args, res) in sig.items():
+        fn = getattr(L, name)
+        fn.argtypes = args
+        fn.restype = res
+    _lib = L
+    return L
+
+
+def _check(rc: int):
+    if rc != SG_OK:
+        raise SgError(rc, lib().sg_last_error().decode())
+
+
+def _i32arr(v: Sequence[int]):
+    return (ctypes.c_int32 * max(1, len(v)))(*v)
+
+
+class Graph:
+    """sg_graph handle.  Build with add_filter / splitjoin, or from a workloads Program."""
+
+    def __init__(self, dtype: str = "f32"):
+        self._h = ctypes.c_void_p()
+        self.dtype = dtype
+        _check(lib().sg_graph_create(SG_F32 if dtype == "f32" else SG_I32, ctypes.byref(self._h)))
+
+    def add_filter(self, kind, ints=(), floats=()) -> int:
+        k = KINDS[kind] if isinstance(kind, str) else int(kind)
+        iv = _i32arr(list(ints))
+        fv = (ctypes.c_float * max(1, len(floats)))(*floats)
+        d = FilterDesc(k, len(ints), iv, len(floats), fv)
+        eid = ctypes.c_int32(-1)
+        _check(lib().sg_add_filter(self._h, ctypes.byref(d), ctypes.byref(eid)))
+        return eid.value
+
+    def add_splitjoin(self, dup: bool, n_branches: int, split_w=None, join_w=None) -> int:
+        sj = ctypes.c_int32(-1)
+        sw = _i32arr(split_w) if split_w is not None else None
+        jw = _i32arr(join_w) if join_w is not None else None
+        _check(lib().sg_add_splitjoin(self._h, 0 if dup else 1, sw, jw, n_branches, ctypes.byref(sj)))
+        return sj.value
+
+    def branch_begin(self, sj: int, b: int):
+        _check(lib().sg_branch_begin(self._h, sj, b))
+
+    def branch_end(self):
+        _check(lib().sg_branch_end(self._h))
+
+    def close(self):
+        if self._h:
+            lib().sg_graph_destroy(self._h)
+            self._h = ctypes.c_void_p()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def graph_from_program(prog) -> Graph:
+    """Marshal a neutral workloads.spec.Program into C-ABI builder calls."""
+    from workloads.spec import Filter, Pipeline  # neutral description, no arithmetic
+    g = Graph(prog.dtype)
+
+    def emit(s):
+        if isinstance(s, Filter):
+            g.add_filter(s.kind, s.ints, s.floats)
+        elif isinstance(s, Pipeline):
+            for c in s.children:
+                emit(c)
+        else:
+            sj = g.add_splitjoin(s.split == "dup", len(s.branches), s.split_w, s.join_w)
+            for b, br in enumerate(s.branches):
+                g.branch_begin(sj, b)
+                emit(br)
+                g.branch_end()
+
+    emit(prog.top)
+    return g
+
+
+class Plan:
+    def __init__(self, graph, n_gpus: int = 1, **kw):
+        own = False
+        if not isinstance(graph, Graph):
+            graph, own = graph_from_program(graph), True
+        o = PlanOpts()
+        lib().sg_plan_opts_default(ctypes.byref(o))
+        self._keep = []
+        for k, v in kw.items():
+            if k == "node_partition":
+                arr = _i32arr(v)
+                self._keep.append(arr)
+                o.node_partition = arr
+                o.n_node_partition = len(v)
+                o.partitioner = SG_PART_USER
+            elif k == "devices":
+                arr = _i32arr(v)
+                self._keep.append(arr)
+                o.devices = arr
+            elif k == "partitioner" and isinstance(v, str):
+                o.partitioner = {"algorithm1": 0, "single": 1, "per_filter": 2}[v]
+            else:
+                setattr(o, k, v)
+        self._h = ctypes.c_void_p()
+        try:
+            _check(lib().sg_plan(graph._h, n_gpus, ctypes.byref(o), ctypes.byref(self._h)))
+        finally:
+            if own:
+                graph.close()
+        self.dtype = graph.dtype
+
+    def info(self) -> dict:
+        i = PlanInfo()
+        _check(lib().sg_plan_info(self._h, ctypes.byref(i)))
+        n, P = i.n_nodes, i.n_partitions
+        return {
+            "n_nodes": n, "n_edges": i.n_edges, "n_partitions": P, "n_gpus": i.n_gpus,
+            "in_per_iter": i.in_per_iter, "out_per_iter": i.out_per_iter,
+            "reps": [i.reps[k] for k in range(n)], "init_firings": [i.init_firings[k] for k in range(n)],
+            "node_type": [i.node_type[k] for k in range(n)], "node_kind": [i.node_kind[k] for k in range(n)],
+            "node_partition": [i.node_partition[k] for k in range(n)],
+            "partition_gpu": [i.partition_gpu[k] for k in range(P)],
+            "partition_time": [i.partition_time[k] for k in range(P)],
+            "partition_mode": [i.partition_mode[k] for k in range(P)],
+            "est_tmax": i.est_tmax, "input_device": i.input_device, "output_device": i.output_device,
+            "iters_per_fragment": i.iters_per_fragment, "ilp_optimal": bool(i.ilp_optimal),
+        }
+
+    def input_items(self, n: int) -> int:
+        v = lib().sg_input_items(self._h, n)
+        if v < 0:
+            _check(SG_E_ARG)
+        return v
+
+    def output_items(self, n: int) -> int:
+        v = lib().sg_output_items(self._h, n)
+        if v < 0:
+            _check(SG_E_ARG)
+        return v
+
+    def source(self, part: int = 0) -> str:
+        s = lib().sg_plan_source(self._h, part)
+        return s.decode() if s else ""
+
+    def run(self, x, n_iters: int, y, stream=None):
+        """x, y: CUDA tensors (or raw device pointers); enqueued on `stream` (default: torch current stream)."""
+        xp = x.data_ptr() if hasattr(x, "data_ptr") else int(x)
+        yp = y.data_ptr() if hasattr(y, "data_ptr") else int(y)
+        if stream is None:
+            import torch
+            stream = torch.cuda.current_stream().cuda_stream
+        elif hasattr(stream, "cuda_stream"):
+            stream = stream.cuda_stream
+        _check(lib().sg_run(self._h, ctypes.c_void_p(xp), n_iters, ctypes.c_void_p(yp), ctypes.c_void_p(stream)))
+
+    def run_host(self, x, n_iters: int, y):
+        """x, y: contiguous host numpy arrays (4-byte items); copies in, runs, copies out, synchronises."""
+        _check(lib().sg_run_host(self._h, ctypes.c_void_p(x.ctypes.data), n_iters, ctypes.c_void_p(y.ctypes.data)))
+
+    def last_launch_count(self) -> int:
+        return lib().sg_last_launch_count(self._h)
+
+    def close(self):
+        if getattr(self, "_h", None):
+            lib().sg_plan_destroy(self._h)
+            self._h = ctypes.c_void_p()
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.close()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def plan(program_or_graph, n_gpus: int = 1, **kw) -> Plan:
+    return Plan(program_or_graph, n_gpus, **kw)
+
+
+def flush_l2(scratch, stream=None):
+    """Overwrite a device scratch tensor (> L2) with the nvcc-built sg_flush_l2 kernel."""
+    if stream is None:
+        import torch
+        stream = torch.cuda.current_stream().cuda_stream
+    _check(lib().sg_flush_l2(ctypes.c_void_p(scratch.data_ptr()), scratch.numel() * scratch.element_size(),
+                             ctypes.c_void_p(stream)))
+
+
+def version() -> str:
+    return lib().sg_version().decode()

@@ -1,0 +1,105 @@
+"""GPU parity: the CUDA path (through the C ABI) against the oracle, element by element.
+
+Bar (BASELINE.json north_star): integer graphs bit-exact; fp32 graphs every
+element |err| <= 1e-5 * max(1, |ref|).  Sizes span several CTA tiles plus a
+ragged tail.  Inputs are seeded (workloads.inputs); input lengths come from the
+oracle's own in_items (never from the CUDA path).
+"""
+import numpy as np
+import pytest
+
+from workloads import apps, inputs
+
+pytestmark = pytest.mark.gpu
+
+TOL = 1e-5
+
+
+def _torch():
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    return torch
+
+
+def run_gpu(prog, x, n, **plan_kw):
+    torch = _torch()
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    with sg.plan(prog, plan_kw.pop("n_gpus", 1), **plan_kw) as p:
+        xd = torch.from_numpy(x).cuda()
+        dt = torch.int32 if prog.dtype == "i32" else torch.float32
+        yd = torch.full((max(1, p.output_items(n)),), -7, dtype=dt, device="cuda")
+        p.run(xd, n, yd)
+        torch.cuda.synchronize()
+        launches = p.last_launch_count()
+        return yd[: p.output_items(n)].cpu().numpy(), p.info(), launches
+
+
+def assert_parity(prog, y, ref):
+    assert y.shape == ref.shape, (y.shape, ref.shape)
+    if prog.dtype == "i32":
+        bad = np.nonzero(y != ref)[0]
+        assert bad.size == 0, f"{bad.size} mismatches, first at {bad[:5]}: {y[bad[:5]]} vs {ref[bad[:5]]}"
+        return
+    err = np.abs(y.astype(np.float64) - ref.astype(np.float64))
+    lim = TOL * np.maximum(1.0, np.abs(ref.astype(np.float64)))
+    bad = np.nonzero(~(err <= lim))[0]
+    assert bad.size == 0, f"{bad.size} elements out of tolerance, first at {bad[:5]}: {y[bad[:5]]} vs {ref[bad[:5]]}"
+
+
+SMALL = {"bitonic32": 3 * 256 + 17, "fft64": 300, "fmradio10": 1500, "filterbank64": 100, "beamformer12x4": 3}
+
+
+@pytest.mark.parametrize("name", list(apps.CONFIGS))
+def test_parity_small(oracle_lib, name):
+    prog = apps.CONFIGS[name]()
+    n = SMALL[name]
+    x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), inputs.SEEDS[name])
+    ref = oracle_lib.run(prog, x, n)
+    y, info, launches = run_gpu(prog, x, n)
+    assert launches >= 1
+    assert_parity(prog, y, ref)
+
+
+@pytest.mark.parametrize("variant", ["ties", "sorted", "reversed"])
+def test_parity_bitonic_variants(oracle_lib, variant):
+    prog = apps.bitonic(32)
+    n = 1000
+    x = inputs.make_input("i32", 32 * n, 5, variant=variant)
+    y, _, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+@pytest.mark.parametrize("variant", ["impulse", "dc"])
+def test_parity_fft_variants(oracle_lib, variant):
+    prog = apps.fft(64)
+    n = 64
+    x = inputs.make_input("f32", 256 * n, 0, variant=variant, block=64)
+    y, _, _ = run_gpu(prog, x, n)
+    assert_parity(prog, y, oracle_lib.run(prog, x, n))
+
+
+def test_parity_filterbank_exact_integers(oracle_lib):
+    prog = apps.filterbank(64, small_int=True)
+    n = 77
+    x = inputs.make_input("f32", 8 * n, 3, variant="smallint")
+    y, _, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+def test_zero_iterations_is_noop():
+    torch = _torch()
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    with sg.plan(apps.bitonic(32), 1) as p:
+        y = torch.full((4,), 5, dtype=torch.int32, device="cuda")
+        p.run(torch.zeros(4, dtype=torch.int32, device="cuda"), 0, y)
+        torch.cuda.synchronize()
+        assert y.tolist() == [5, 5, 5, 5]
+
+
+@pytest.mark.parametrize("n", [1, 2, 255, 256, 257])
+def test_parity_bitonic_edge_sizes(oracle_lib, n):
+    prog = apps.bitonic(32)
+    x = inputs.make_input("i32", 32 * n, n)
+    y, _, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, oracle_lib.run(prog, x, n))
