@@ -1,0 +1,328 @@
+#!/usr/bin/env python
+"""Benchmark of the steady-state stream-graph path (BASELINE.json metric).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--config NAME] [--impl sg|reference]
+
+One step = one sg_run() over the whole workload (all of SURVEY.md 8(a)'s timed
+rows: tile loads, filter execution, stores; plus boundary streams when the plan
+has several partitions/GPUs).  Default workload: BASELINE.json configs[1],
+BitonicSort 32-key int32, 2^20 iterations, one GPU.  Inputs resident in HBM;
+L2 flushed (256 MiB overwrite with our sg_flush_l2 kernel) before every timed
+step, outside the per-step CUDA-event window.  Under torchrun (N > 1) every rank
+runs an independent replica on its own GPU ("replicas only" for this HBM-bound
+graph); value = all ranks' iterations / max-over-ranks time.
+
+--impl reference times the oracle (the plain sequential CPU interpreter in
+oracle/, as it stands) on the host cores, on a bounded sample of the workload.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "steady-state iters/s (output items/s) at 1/2/4/8 B200; % of roofline"
+
+# workload table: iterations per step, roofline class, algorithmic bytes / ops per iteration
+WORKLOADS = {
+    "bitonic32": dict(n=1 << 20, bound="hbm", desc="BitonicSort 32-key int32, 1M iterations"),
+    "fft64": dict(n=1 << 20, bound="hbm", desc="StreamIt FFT2 N=64 fp32 (2 x 64-pt complex FFT per iteration)"),
+    "fmradio10": dict(n=1 << 24, bound="alu", desc="FMRadio + 10-band equalizer fp32"),
+    "beamformer12x4": dict(n=4096, bound="alu", desc="BeamFormer 12 channels x 4 beams fp32, 1024-sample frames"),
+    "filterbank64": dict(n=1 << 20, bound="alu", desc="FilterBank 64 branches fp32 (M=8, L=32)"),
+}
+
+
+def measured_peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            return json.load(f), "measured"
+    except Exception:
+        return {"hbm_gbs": 6650.0, "sm_max_mhz": 1965.0}, "fallback"
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons, sampled in the background during the timed region."""
+
+    FIELDS = ["clocks.sm", "clocks.max.sm", "clocks_event_reasons.active",
+              "clocks_event_reasons.hw_slowdown", "clocks_event_reasons.hw_thermal_slowdown",
+              "clocks_event_reasons.sw_thermal_slowdown", "clocks_event_reasons.sw_power_cap"]
+
+    def __init__(self, gpu_index: int):
+        self.idx = gpu_index
+        self.rows = []
+        self.proc = None
+        self.t = None
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", f"--id={self.idx}", "--query-gpu=" + ",".join(self.FIELDS),
+                 "--format=csv,noheader,nounits", "-lms", "50"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+        except Exception:
+            self.proc = None
+            return
+        self.t = threading.Thread(target=self._read, daemon=True)
+        self.t.start()
+
+    def _read(self):
+        for line in self.proc.stdout:
+            parts = [p.strip() for p in line.split(",")]
+            if len(parts) == len(self.FIELDS):
+                self.rows.append(parts)
+
+    def stop(self):
+        if self.proc is None:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"], "samples": 0}
+        time.sleep(0.12)
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=2)
+        except Exception:
+            self.proc.kill()
+        if self.t:
+            self.t.join(timeout=2)
+        sm = [float(r[0]) for r in self.rows if r[0].replace(".", "").isdigit()]
+        mx = [float(r[1]) for r in self.rows if r[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = set()
+        for r in self.rows:
+            for k, nm in enumerate(names):
+                if r[3 + k].lower().startswith("active"):
+                    reasons.add(nm)
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": sorted(reasons), "samples": len(self.rows)}
+
+
+def cpu_baseline(prog, name, target_s=10.0):
+    """The oracle as it stands, on a bounded sample of the workload, one host core."""
+    from oracle import oracle as O
+    from workloads import inputs
+    n_total = WORKLOADS[name]["n"]
+    n0 = 16 if name == "beamformer12x4" else 4096
+    x = inputs.make_input(prog.dtype, O.in_items(prog, n0), inputs.SEEDS[name])
+    t = time.perf_counter()
+    O.run(prog, x, n0)
+    rate = n0 / max(1e-6, time.perf_counter() - t)
+    n = int(min(n_total, max(n0, rate * target_s)))
+    x = inputs.make_input(prog.dtype, O.in_items(prog, n), inputs.SEEDS[name])
+    t = time.perf_counter()
+    O.run(prog, x, n)
+    dt = time.perf_counter() - t
+    return {"value": n / dt, "unit": "iters/s", "cores": 1, "kind": "oracle",
+            "sample": f"first {n} of {n_total} iterations of {name} (seeded input), sequential C interpreter, "
+                      f"{dt:.1f} s, gcc -O2 -ffp-contract=off"}
+
+
+def run_reference(args):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return 0
+    from workloads import apps
+    name = args.config
+    prog = apps.CONFIGS[name]()
+    vals = []
+    cb = None
+    for _ in range(max(1, args.warmup)):
+        pass  # the oracle has no warm state worth excluding beyond the first call below
+    for k in range(args.steps if args.steps <= 3 else 3):
+        cb = cpu_baseline(prog, name, target_s=5.0)
+        vals.append(cb["value"])
+    v = statistics.median(vals)
+    cb["value"] = v
+    line = {"impl": "reference", "metric": METRIC, "value": v, "unit": "iters/s", "n_gpus": args.gpus,
+            "steps": len(vals), "warmup": args.warmup, "ms_per_step": None, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "i32" if prog.dtype == "i32" else "f32",
+            "data": "synthetic", "config": {"workload": name, "desc": WORKLOADS[name]["desc"],
+                                             "iters": WORKLOADS[name]["n"], "sample": cb["sample"]},
+            "cpu_baseline": cb, "e2e": {"value": v, "unit": "iters/s", "h2d_bytes_per_step": 0,
+                                        "d2h_bytes_per_step": 0}}
+    print(json.dumps(line))
+    return 0
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=3000)
+    ap.add_argument("--warmup", type=int, default=20)
+    ap.add_argument("--config", default="bitonic32", choices=list(WORKLOADS))
+    ap.add_argument("--impl", default="sg", choices=["sg", "reference"])
+    ap.add_argument("--iters", type=int, default=0, help="override iterations per step")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-flush", action="store_true")
+    args = ap.parse_args()
+    if args.warmup < 3:
+        args.warmup = 3
+    if args.impl == "reference":
+        return run_reference(args)
+
+    import torch
+    import torch.distributed as dist
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    from workloads import apps, inputs
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    torch.cuda.set_device(local)
+    name = args.config
+    W = WORKLOADS[name]
+    n = args.iters or W["n"]
+    prog = apps.CONFIGS[name]()
+    plan = sg.plan(prog, 1, devices=[local])
+    info = plan.info()
+    nin, nout = plan.input_items(n), plan.output_items(n)
+    dt = torch.int32 if prog.dtype == "i32" else torch.float32
+    x_host = torch.from_numpy(inputs.make_input(prog.dtype, nin, inputs.SEEDS[name] + rank))
+    x = x_host.to(f"cuda:{local}")
+    y = torch.empty(nout, dtype=dt, device=f"cuda:{local}")
+    flush = torch.empty(256 << 20, dtype=torch.uint8, device=f"cuda:{local}")
+    stream = torch.cuda.current_stream()
+
+    for _ in range(args.warmup):
+        plan.run(x, n, y, stream)
+    launches_per_step = plan.last_launch_count()
+    torch.cuda.synchronize()
+
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    sampler = ClockSampler(local)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    sampler.start()
+    time.sleep(0.15)
+    wall0 = time.perf_counter()
+    for k in range(args.steps):
+        if not args.no_flush:
+            sg.flush_l2(flush, stream.cuda_stream)
+        ev[k][0].record(stream)
+        plan.run(x, n, y, stream)
+        ev[k][1].record(stream)
+    torch.cuda.synchronize()
+    wall = time.perf_counter() - wall0
+    if world > 1:
+        dist.barrier()
+    clocks = sampler.stop()
+    step_ms = [a.elapsed_time(b) for a, b in ev]
+    total_ms = sum(step_ms)
+    if world > 1:
+        t = torch.tensor([total_ms], dtype=torch.float64, device=f"cuda:{local}")
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        total_ms = float(t.item())
+    ms_per_step = total_ms / args.steps
+    value = world * n * args.steps / (total_ms / 1e3)
+
+    # roofline of the dominant kernel (single partition: one launch per step)
+    peaks, peak_src = measured_peaks()
+    # kernel duration: CUDA events around the launch on its stream (one kernel per step here)
+    kern_ms = statistics.median(step_ms) if launches_per_step == 1 else None
+    ki_bytes = (info["in_per_iter"] + info["out_per_iter"]) * 4 * n
+    roof = None
+    if W["bound"] == "hbm":
+        if kern_ms:
+            ach = ki_bytes / (kern_ms / 1e3) / 1e9
+            roof = {"bound": "hbm", "achieved": ach, "peak": peaks["hbm_gbs"], "unit": "GB/s",
+                    "frac": ach / peaks["hbm_gbs"], "traffic": None,
+                    "algorithmic_bytes_per_launch": ki_bytes, "peak_source": peak_src + " copy bandwidth"}
+    else:
+        fl = _flops_per_iter(prog, info["reps"])
+        if kern_ms:
+            ach = fl * n / (kern_ms / 1e3) / 1e12
+            pk = 148 * 128 * 2 * peaks.get("sm_max_mhz", 1965.0) * 1e6 / 1e12
+            roof = {"bound": "alu", "achieved": ach, "peak": pk, "unit": "TFLOP/s", "frac": ach / pk,
+                    "traffic": None, "algorithmic_flops_per_launch": fl * n,
+                    "peak_source": "derived: 148 SMs x 128 FP32 lanes x 2 x sm_max_mhz (FFMA)"}
+    prof = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    if roof is not None and os.path.exists(prof):
+        try:
+            tr = json.load(open(prof)).get(name)
+            if tr:
+                roof["traffic"] = tr["dram_bytes_per_launch"]
+        except Exception:
+            pass
+
+    # end to end through the public C ABI with HOST buffers (pinned), copies inside the timed region
+    e2e = None
+    if rank == 0 or world > 1:
+        xh = x_host.pin_memory()
+        yh = torch.empty(nout, dtype=dt).pin_memory()
+        xnp, ynp = xh.numpy(), yh.numpy()
+        plan.run_host(xnp, n, ynp)
+        k2 = max(3, min(20, args.steps))
+        t0 = time.perf_counter()
+        for _ in range(k2):
+            plan.run_host(xnp, n, ynp)
+        e2e_s = (time.perf_counter() - t0) / k2
+        e2e = {"value": world * n / e2e_s, "unit": "iters/s", "h2d_bytes_per_step": nin * 4,
+               "d2h_bytes_per_step": nout * 4, "steps": k2, "timing": "host wall clock around sg_run_host"}
+
+    cb = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        cb = cpu_baseline(prog, name)
+
+    if rank == 0:
+        line = {
+            "metric": METRIC, "value": value, "unit": "iters/s", "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": "i32" if prog.dtype == "i32" else "f32", "data": "synthetic",
+            "config": {"workload": name, "desc": W["desc"], "iters_per_step": n,
+                       "items_per_s_out": value * info["out_per_iter"],
+                       "l2": "flushed before every step (256 MiB sg_flush_l2), outside the event window"
+                       if not args.no_flush else "not flushed",
+                       "parallelism": f"replicas x{world}" if world > 1 else "1 GPU, 1 partition",
+                       "partitions": info["n_partitions"], "partition_mode": info["partition_mode"],
+                       "wall_s": wall},
+            "roofline": roof, "cpu_baseline": cb, "e2e": e2e,
+            "gpu_launches": args.steps * (launches_per_step + (0 if args.no_flush else 1)),
+            "clocks": clocks,
+        }
+        print(json.dumps(line))
+    plan.close()
+    if world > 1:
+        dist.destroy_process_group()
+    return 0
+
+
+def _flops_per_iter(prog, reps):
+    """Algorithmic fp32 flops per iteration as written (FMA = 2): program text x repetition vector."""
+    from workloads.spec import Filter, Pipeline
+    k = [0]
+    tot = [0]
+
+    def walk(s):
+        if isinstance(s, Filter):
+            rep = reps[k[0]]
+            k[0] += 1
+            iv = s.ints
+            per = {"FIR": 2 * iv[0] if iv else 0, "COMBINE_DFT": 10 * (iv[0] // 2) if iv else 0, "FM_DEMOD": 1,
+                   "SUBTRACT": 1, "AMPLIFY": 1, "ADD": iv[0] if iv else 0,
+                   "BEAM_FIR": 8 * iv[0] * (iv[2] // iv[1]) if len(iv) >= 3 else 0,
+                   "BEAMFORM": 8 * iv[0] if iv else 0, "MAGNITUDE": 3}.get(s.kind, 0)
+            tot[0] += per * rep
+        elif isinstance(s, Pipeline):
+            for c in s.children:
+                walk(c)
+        else:
+            k[0] += 1
+            for b in s.branches:
+                walk(b)
+            k[0] += 1
+
+    walk(prog.top)
+    return tot[0]
+
+
+if __name__ == "__main__":
+    sys.exit(main())

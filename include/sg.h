@@ -194,8 +194,9 @@ sg_status sg_plan(const sg_graph* g, int32_t n_gpus, const sg_plan_opts* opts, s
 
 /* Minimal input prefix (items) needed for n_iters iterations; < 0 on error. */
 int64_t sg_input_items(const sg_plan_t* p, int64_t n_iters);
-/* Output items produced by n_iters iterations (n_iters * out_per_iter + any
- * prework items of the output node); < 0 on error. */
+/* Output items of n_iters iterations: n_iters * out_per_iter, i.e. the first
+ * that many items of the graph's output stream (prework items of the output
+ * node included); < 0 on error. */
 int64_t sg_output_items(const sg_plan_t* p, int64_t n_iters);
 
 /* Fills *out; pointers inside stay valid until sg_plan_destroy. */
@@ -227,6 +228,30 @@ const char* sg_last_error(void);
 
 /* Library version string. */
 const char* sg_version(void);
+
+/* ---- planner building blocks (PAPER.md sections 3.2-3.3), for tests and tools ----
+ * Topology kinds: 0 = NVSwitch star of n_gpus GPUs (uplink k and downlink k per GPU,
+ * L = 2G), 1 = the 4-GPU PCIe tree of Fig. 3.3 (n_gpus must be 4). */
+int32_t sg_topology_links(int32_t kind, int32_t n_gpus); /* L, or < 0 on error */
+/* dtlist as a dense [L][G][G] 0/1 array:
+ * dtlist[l*G*G + i*G + j] = 1 iff traffic GPU i -> GPU j loads link l.  Caller-owned. */
+sg_status sg_topology_dtlist(int32_t kind, int32_t n_gpus, uint8_t* dtlist);
+/* The mapping ILP of Eq. III.1-III.7 on P partitions with
+ * times T[P] and PDG edges (e_src, e_dst, e_bytes)[n_e]: minimise Tmax =
+ * max(max_j sum_i n_ij T_i, max_l Lat + D_l / bw).  method 0 = exact branch and
+ * bound (time limit in ms; *optimal = 0 if it hit the limit), 1 = brute force
+ * over G^P.  assign[P] receives the GPU of each partition. */
+sg_status sg_map_ilp(int32_t P, const double* T, int32_t n_e, const int32_t* e_src, const int32_t* e_dst,
+                     const double* e_bytes, int32_t topo_kind, int32_t n_gpus, double lat, double bw,
+                     int32_t time_limit_ms, int32_t method, int32_t* assign, double* tmax, int32_t* optimal);
+/* The paper's kernel model, Eq. III.8-III.12: returns T = Texec / W with
+ * Tcomp = sum_i t_i / min(f_i, S), Tdt = C1 D / F, Tdb = C2 D / (F + W S),
+ * Texec = max(Tcomp, Tdt) + Tdb.  Outputs may be NULL. */
+double sg_paper_model(int32_t n, const double* t, const double* f, int32_t S, int32_t W, int32_t F, double D,
+                      double C1, double C2, double* tcomp, double* tdt, double* tdb);
+/* PDG of a plan: fills up to `cap` edges (partition src, dst,
+ * bytes per iteration); returns the number of edges. */
+int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst, double* bytes);
 
 /* Benchmark hygiene: overwrite `bytes` of device scratch memory (> L2 size)
  * with an nvcc-compiled sm_100a kernel enqueued on `stream`. */

@@ -213,33 +213,59 @@ sg_status sg_run_host(sg_plan_t* p, const void* hin, int64_t n, void* hout) {
     if (n < 0) return fail(SG_E_ARG, "negative n_iters");
     if (n == 0) return SG_OK;
     if (!hin || !hout) return fail(SG_E_ARG, "NULL buffer");
+    return guard([&] { p->plan.run_host(hin, n, hout); });
+}
+
+int32_t sg_topology_links(int32_t kind, int32_t G) {
+    if (kind == 0 && G >= 1 && G <= 64) return 2 * G;
+    if (kind == 1 && G == 4) return 12;
+    return -1;
+}
+
+sg_status sg_topology_dtlist(int32_t kind, int32_t G, uint8_t* dt) {
+    if (!dt || sg_topology_links(kind, G) < 0) return fail(SG_E_ARG, "bad topology kind / size");
+    sg::Topology t = kind == 0 ? sg::Topology::nvswitch(G) : sg::Topology::pcie_tree4();
+    std::memcpy(dt, t.dt.data(), t.dt.size());
+    return SG_OK;
+}
+
+sg_status sg_map_ilp(int32_t P, const double* T, int32_t ne, const int32_t* es, const int32_t* ed, const double* eb,
+                     int32_t topo_kind, int32_t G, double lat, double bw, int32_t ms, int32_t method, int32_t* assign,
+                     double* tmax, int32_t* optimal) {
+    if (P < 0 || (P && (!T || !assign)) || ne < 0 || (ne && (!es || !ed || !eb)) || bw <= 0)
+        return fail(SG_E_ARG, "bad ILP arguments");
+    if (sg_topology_links(topo_kind, G) < 0) return fail(SG_E_ARG, "bad topology");
     return guard([&] {
-        sg::Plan& pl = p->plan;
-        int64_t ni = pl.flat.input_items(n), no = pl.flat.output_items(n);
-        int din = pl.devices[pl.input_gpu], dout = pl.devices[pl.output_gpu];
-        void *din_p = nullptr, *dout_p = nullptr;
-        auto chk = [](cudaError_t e, const char* w) {
-            if (e != cudaSuccess) throw sg::Error(SG_E_CUDA, std::string(w) + ": " + cudaGetErrorString(e));
-        };
-        chk(cudaSetDevice(din), "cudaSetDevice");
-        chk(cudaMalloc(&din_p, (size_t)std::max<int64_t>(ni, 1) * 4), "cudaMalloc");
-        chk(cudaMemcpy(din_p, hin, (size_t)ni * 4, cudaMemcpyHostToDevice), "H2D");
-        chk(cudaSetDevice(dout), "cudaSetDevice");
-        chk(cudaMalloc(&dout_p, (size_t)std::max<int64_t>(no, 1) * 4), "cudaMalloc");
-        chk(cudaSetDevice(din), "cudaSetDevice");
-        try {
-            pl.run(din_p, n, dout_p, nullptr);
-            chk(cudaSetDevice(dout), "cudaSetDevice");
-            chk(cudaDeviceSynchronize(), "sync");
-            chk(cudaMemcpy(hout, dout_p, (size_t)no * 4, cudaMemcpyDeviceToHost), "D2H");
-        } catch (...) {
-            cudaFree(din_p);
-            cudaFree(dout_p);
-            throw;
+        std::vector<double> Tv(T, T + P);
+        std::vector<sg::PdgEdge> pdg;
+        for (int i = 0; i < ne; i++) {
+            if (es[i] < 0 || es[i] >= P || ed[i] < 0 || ed[i] >= P) throw sg::Error(SG_E_ARG, "PDG edge out of range");
+            pdg.push_back({es[i], ed[i], eb[i]});
         }
-        cudaFree(din_p);
-        cudaFree(dout_p);
+        sg::Topology t = topo_kind == 0 ? sg::Topology::nvswitch(G) : sg::Topology::pcie_tree4();
+        sg::MapResult m = sg::map_partitions(Tv, pdg, t, lat, bw, ms > 0 ? ms : 10000, method);
+        for (int i = 0; i < P; i++) assign[i] = m.assign[i];
+        if (tmax) *tmax = m.tmax;
+        if (optimal) *optimal = m.optimal ? 1 : 0;
     });
+}
+
+double sg_paper_model(int32_t n, const double* t, const double* f, int32_t S, int32_t W, int32_t F, double D,
+                      double C1, double C2, double* tcomp, double* tdt, double* tdb) {
+    if (n < 0 || (n && (!t || !f)) || S < 1 || W < 1 || F < 1) return -1.0;
+    std::vector<double> tv(t, t + n), fv(f, f + n);
+    return sg::paper_model(tv, fv, S, W, F, D, C1, C2, tcomp, tdt, tdb);
+}
+
+int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst, double* bytes) {
+    if (!p) return -1;
+    const auto& e = p->plan.pdg;
+    for (int i = 0; i < (int)e.size() && i < cap; i++) {
+        if (src) src[i] = e[i].src;
+        if (dst) dst[i] = e[i].dst;
+        if (bytes) bytes[i] = e[i].bytes;
+    }
+    return (int32_t)e.size();
 }
 
 int64_t sg_last_launch_count(const sg_plan_t* p) { return p ? p->plan.last_launches : -1; }

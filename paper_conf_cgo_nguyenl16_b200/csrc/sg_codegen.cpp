@@ -152,8 +152,8 @@ void partition_boundary(const Flat& f, const std::vector<int>& nodes, std::vecto
 
 void edge_window(const Flat& f, int e, int64_t& lo, int64_t& extra) {
     const Edge& ed = f.edges[e];
-    if (ed.dst < 0) {  // graph output: produced positions (prework items handled apart)
-        lo = ed.pre;
+    if (ed.dst < 0) {  // graph output: iteration k owns positions [k*P, (k+1)*P)
+        lo = ed.pre + f.nodes[ed.src].ninit * ed.push;
         extra = 0;
         return;
     }
@@ -402,6 +402,7 @@ public:
         KernelInfo ki;
         ki.mode = 1;
         ki.name = "sg_part" + std::to_string(part_);
+        ki.name_sync = ki.name + "_sync";
         fill_io(ki);
         ein_ = ins_[0];
         eout_ = outs_[0];
@@ -417,22 +418,28 @@ public:
         ROUT_S_ = row_stride(POUT_);
         body_.str("");
         emit_body();
+        const std::string VT4 = T_ == "float" ? "float4" : "int4";
+        std::ostringstream src;
+        src << header("register") << consts_.str() << args_struct();
+        // ---------------- variant 1: synchronous tiles (any alignment / row size)
         int bytes_per_thread = (int)((RIN_S_ + ROUT_S_) * 4);
         int NT = opt.threads;
         if (NT <= 0) {
             NT = 256;
             while (NT > 32 && (size_t)NT * bytes_per_thread > 72 * 1024) NT /= 2;
         }
-        ki.threads = NT;
-        ki.tile = NT;
-        ki.smem = (size_t)NT * bytes_per_thread;
-        ki.min_blocks = std::max(1, std::min(8, (int)((200 * 1024) / std::max<size_t>(1, ki.smem))));
-        if (bytes_per_thread * NT > 200 * 1024) ki.min_blocks = 1;
-        std::ostringstream src;
-        src << header("register") << consts_.str() << args_struct();
-        src << "#define NT " << NT << "\n";
-        src << "extern \"C\" __global__ void __launch_bounds__(NT, " << ki.min_blocks << ") " << ki.name
+        ki.threads_sync = NT;
+        ki.tile_sync = NT;
+        ki.smem_sync = (size_t)NT * bytes_per_thread;
+        int minb = std::max(1, std::min(8, (int)((200 * 1024) / std::max<size_t>(1, ki.smem_sync))));
+        if (bytes_per_thread * NT > 200 * 1024) minb = 1;
+        src << "#define SG_LD4(g) (reinterpret_cast<const " << VT4 << "*>(xr)[g])\n"
+            << "#define SG_LD1(r) (xr[r])\n"
+            << "#define SG_ST4(g, v) (reinterpret_cast<" << VT4 << "*>(yr)[g] = (v))\n"
+            << "#define SG_ST1(g, v) (yr[g] = (v))\n";
+        src << "extern \"C\" __global__ void __launch_bounds__(" << NT << ", " << minb << ") " << ki.name_sync
             << "(const SgArgs a) {\n"
+            << "  constexpr int NT = " << NT << ";\n"
             << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
             << "  " << T_ << "* s_in = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
             << "  " << T_ << "* s_out = s_in + NT * " << RIN_S_ << ";\n"
@@ -441,9 +448,9 @@ public:
             << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * NT; t0 < SG_K_END; t0 += (long long)gridDim.x * NT) {\n"
             << "    const int nt = (int)min((long long)NT, SG_K_END - t0);\n"
             << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
-            << "    if (" << (vin_ ? "(reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0" : "false") << ")\n"
-            << "      sg_rows_g2s_v4<" << T_ << ", " << PIN_ << ", " << RIN_S_ << ", NT>(gsrc, s_in, nt);\n"
-            << "    else\n"
+            << (vin_ ? std::string("    if ((reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0)\n      sg_rows_g2s_v4<") +
+                           T_ + ", " + std::to_string(PIN_) + ", " + std::to_string(RIN_S_) + ", NT>(gsrc, s_in, nt);\n    else\n"
+                     : std::string())
             << "      sg_rows_g2s_v1<" << T_ << ", " << PIN_ << ", " << RIN_S_ << ", NT>(gsrc, s_in, nt);\n"
             << "    __syncthreads();\n"
             << "    if (threadIdx.x < nt) {\n"
@@ -453,11 +460,156 @@ public:
             << "    }\n"
             << "    __syncthreads();\n"
             << "    " << T_ << "* gdst = gout + (t0 * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
-            << "    if (" << (vout_ ? "(reinterpret_cast<unsigned long long>(gdst) & 15ull) == 0" : "false") << ")\n"
-            << "      sg_rows_s2g_v4<" << T_ << ", " << POUT_ << ", " << ROUT_S_ << ", NT>(s_out, gdst, nt);\n"
-            << "    else\n"
+            << (vout_ ? std::string("    if ((reinterpret_cast<unsigned long long>(gdst) & 15ull) == 0)\n      sg_rows_s2g_v4<") +
+                            T_ + ", " + std::to_string(POUT_) + ", " + std::to_string(ROUT_S_) + ", NT>(s_out, gdst, nt);\n    else\n"
+                      : std::string())
             << "      sg_rows_s2g_v1<" << T_ << ", " << POUT_ << ", " << ROUT_S_ << ", NT>(s_out, gdst, nt);\n"
-            << "  }\n}\n";
+            << "  }\n}\n"
+            << "#undef SG_LD4\n#undef SG_LD1\n#undef SG_ST4\n#undef SG_ST1\n";
+        // ---------------- variant 2: warp-specialised TMA pipeline (PAPER.md:220-228's
+        // data-transfer threads become one producer warp driving the TMA engine)
+        // layout 1: 128-byte rows, 2-D tensor map with 128B swizzle (one TMA per tile / slab)
+        // layout 2: 16-byte-multiple rows, one bulk copy per row into padded shared rows
+        ki.tma_in = PIN_ * 4 == 128 ? 1 : (PIN_ % 4 == 0 ? 2 : 0);
+        ki.tma_out = POUT_ * 4 == 128 ? 1 : (POUT_ % 4 == 0 ? 2 : 0);
+        ki.pin = PIN_;
+        ki.pout = POUT_;
+        ki.off_in = off_in_;
+        ki.off_out = off_out_;
+        if (ki.tma_in && ki.tma_out && opt.mode != -1) {
+            auto stage_bytes = [&](int lay, int64_t P, int64_t RS, int rows) -> int64_t {
+                int64_t b = lay == 1 ? rows * 128 : rows * RS * 4;
+                return (b + 1023) / 1024 * 1024;
+            };
+            int nt = 0, nsi = 0, nso = 0;
+            for (int budget : {110 * 1024, 220 * 1024}) {
+                for (int cand : {128, 64, 32}) {
+                    if (opt.threads > 0 && cand != opt.threads) continue;
+                    for (int si : {4, 3, 2}) {
+                        for (int so : {2, 1}) {
+                            int64_t tot = si * stage_bytes(ki.tma_in, PIN_, RIN_S_, cand) +
+                                          so * stage_bytes(ki.tma_out, POUT_, ROUT_S_, cand) + 1024;
+                            if (tot <= budget && !nt) { nt = cand; nsi = si; nso = so; }
+                        }
+                    }
+                }
+                if (nt) break;
+            }
+            if (nt) {
+                const int64_t inb = stage_bytes(ki.tma_in, PIN_, RIN_S_, nt);
+                const int64_t outb = stage_bytes(ki.tma_out, POUT_, ROUT_S_, nt);
+                ki.threads = nt + 32;
+                ki.tile = nt;
+                ki.smem = (size_t)(nsi * inb + nso * outb + 1024 + 1024);  // + barriers + alignment slack
+                ki.has_tma = true;
+                const int nwc = nt / 32;
+                src << "// ---- TMA pipeline: " << nt << " rows per tile, " << nsi << " input stages, " << nso
+                    << " output stages\n";
+                if (ki.tma_in == 1)
+                    src << "#define SG_LD4(g) (*reinterpret_cast<const " << VT4 << "*>(xb + ((((g) ^ swz)) << 4)))\n"
+                        << "#define SG_LD1(r) (reinterpret_cast<const " << T_ << "*>(xb + ((((r) >> 2) ^ swz) << 4))[(r) & 3])\n";
+                else
+                    src << "#define SG_LD4(g) (*reinterpret_cast<const " << VT4 << "*>(xb + ((g) << 4)))\n"
+                        << "#define SG_LD1(r) (reinterpret_cast<const " << T_ << "*>(xb)[r])\n";
+                if (ki.tma_out == 1)
+                    src << "#define SG_ST4(g, v) (*reinterpret_cast<" << VT4 << "*>(yb + ((((g) ^ swz)) << 4)) = (v))\n"
+                        << "#define SG_ST1(g, v) (reinterpret_cast<" << T_ << "*>(yb + ((((g) >> 2) ^ swz) << 4))[(g) & 3] = (v))\n";
+                else
+                    src << "#define SG_ST4(g, v) (*reinterpret_cast<" << VT4 << "*>(yb + ((g) << 4)) = (v))\n"
+                        << "#define SG_ST1(g, v) (reinterpret_cast<" << T_ << "*>(yb)[g] = (v))\n";
+                src << "extern \"C\" __global__ void __launch_bounds__(" << nt + 32 << ", 1) " << ki.name
+                    << "(const SgArgs a, const __grid_constant__ SgTmap tin, const __grid_constant__ SgTmap tout) {\n"
+                    << "  constexpr int NT = " << nt << ", NWC = " << nwc << ", NSI = " << nsi << ", NSO = " << nso << ";\n"
+                    << "  constexpr int INB = " << inb << ", OUTB = " << outb << ";\n"
+                    << "  extern __shared__ __align__(1024) unsigned char sg_smem_raw[];\n"
+                    << "  unsigned char* sg_smem = reinterpret_cast<unsigned char*>((reinterpret_cast<unsigned long long>(sg_smem_raw) + 1023ull) & ~1023ull);\n"
+                    << "  unsigned char* in_st = sg_smem;\n"
+                    << "  unsigned char* out_st = sg_smem + NSI * INB;\n"
+                    << "  unsigned long long* full = reinterpret_cast<unsigned long long*>(out_st + NSO * OUTB);\n"
+                    << "  unsigned long long* empty = full + NSI;\n"
+                    << "  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;\n"
+                    << "  const long long nrows = SG_K_END - SG_K_BEGIN;\n"
+                    << "  const long long ntiles = (nrows + NT - 1) / NT;\n"
+                    << "  if (threadIdx.x == 0) {\n"
+                    << "    for (int s = 0; s < NSI; s++) { sg_mbar_init(&full[s], 1); sg_mbar_init(&empty[s], NWC); }\n"
+                    << "    sg_fence_barrier_init();\n"
+                    << "  }\n"
+                    << "  __syncthreads();\n"
+                    << "  if (warp == NWC) {  // ---- producer warp\n";
+                if (ki.tma_in == 1) {
+                    src << "    if (lane == 0) {\n"
+                        << "      sg_prefetch_tmap(&tin);\n"
+                        << "      int i = 0;\n"
+                        << "      for (long long t = blockIdx.x; t < ntiles; t += gridDim.x, i++) {\n"
+                        << "        const int s = i % NSI;\n"
+                        << "        sg_mbar_wait(&empty[s], ((i / NSI) & 1) ^ 1);\n"
+                        << "        sg_mbar_arrive_expect_tx(&full[s], NT * 128);\n"
+                        << "        sg_tma_load_2d(in_st + s * INB, &tin, 0, (int)(t * NT), &full[s]);\n"
+                        << "      }\n"
+                        << "    }\n";
+                } else {
+                    src << "    const " << T_ << "* gin = SG_IN(0) + (SG_K_BEGIN * " << PIN_ << "LL + (" << off_in_
+                        << "LL) - SG_IN_BASE(0));\n"
+                        << "    int i = 0;\n"
+                        << "    for (long long t = blockIdx.x; t < ntiles; t += gridDim.x, i++) {\n"
+                        << "      const int s = i % NSI;\n"
+                        << "      const int nt = (int)min((long long)NT, nrows - t * NT);\n"
+                        << "      sg_mbar_wait(&empty[s], ((i / NSI) & 1) ^ 1);\n"
+                        << "      if (lane == 0) sg_mbar_arrive_expect_tx(&full[s], (unsigned)(nt * " << PIN_ * 4 << "));\n"
+                        << "      __syncwarp();\n"
+                        << "      for (int r = lane; r < nt; r += 32)\n"
+                        << "        sg_bulk_g2s(in_st + s * INB + r * " << RIN_S_ * 4 << ", gin + (t * NT + r) * " << PIN_
+                        << "LL, " << PIN_ * 4 << ", &full[s]);\n"
+                        << "    }\n";
+                }
+                src << "    return;\n"
+                    << "  }\n"
+                    << "  // ---- consumer warps: one iteration per thread, registers only\n"
+                    << "  " << T_ << "* gout = SG_OUT(0) + (SG_K_BEGIN * " << POUT_ << "LL + (" << off_out_
+                    << "LL) - SG_OUT_BASE(0));\n"
+                    << "  int i = 0;\n"
+                    << "  for (long long t = blockIdx.x; t < ntiles; t += gridDim.x, i++) {\n"
+                    << "    const int s = i % NSI, so = i % NSO;\n"
+                    << "    const int nt = (int)min((long long)NT, nrows - t * NT);\n"
+                    << "    sg_mbar_wait(&full[s], (i / NSI) & 1);\n";
+                if (ki.tma_out == 1) src << "    if (lane == 0) sg_bulk_wait_read<NSO - 1>();\n";
+                else src << "    sg_bulk_wait_read<NSO - 1>();\n";
+                src << "    __syncwarp();\n"
+                    << "    const int row = threadIdx.x;\n"
+                    << "    const int swz = row & 7;\n"
+                    << "    const unsigned char* xb = in_st + s * INB + row * "
+                    << (ki.tma_in == 1 ? 128 : RIN_S_ * 4) << ";\n"
+                    << "    unsigned char* yb = out_st + so * OUTB + row * " << (ki.tma_out == 1 ? 128 : ROUT_S_ * 4) << ";\n"
+                    << "    (void)swz;\n"
+                    << "    if (row < nt) {\n"
+                    << body_.str()
+                    << "    }\n"
+                    << "    __syncwarp();\n"
+                    << "    if (lane == 0) sg_mbar_arrive(&empty[s]);\n"
+                    << "    sg_fence_proxy_async();\n"
+                    << "    __syncwarp();\n";
+                if (ki.tma_out == 1) {
+                    src << "    if (lane == 0 && warp * 32 < nt) {\n"
+                        << "      sg_tma_store_2d(&tout, 0, (int)(t * NT + warp * 32), out_st + so * OUTB + warp * 32 * 128);\n"
+                        << "      sg_bulk_commit();\n"
+                        << "    }\n";
+                } else {
+                    src << "    if (row < nt) {\n"
+                        << "      sg_bulk_s2g(gout + (t * NT + row) * " << POUT_ << "LL, yb, " << POUT_ * 4 << ");\n"
+                        << "      sg_bulk_commit();\n"
+                        << "    }\n";
+                }
+                src << "  }\n"
+                    << "  sg_bulk_wait<0>();\n"
+                    << "}\n";
+            }
+        }
+        if (!ki.has_tma) {
+            ki.threads = ki.threads_sync;
+            ki.tile = ki.tile_sync;
+            ki.smem = ki.smem_sync;
+        }
+        ki.min_blocks = 1;
         ki.source = src.str();
         return ki;
     }
@@ -485,15 +637,14 @@ private:
             int64_t g = r / 4;
             if (!loaded_.count(g)) {
                 loaded_.insert(g);
-                body_ << "      const " << (T_ == "float" ? "float4" : "int4") << " iq" << g << " = reinterpret_cast<const "
-                      << (T_ == "float" ? "float4" : "int4") << "*>(xr)[" << g << "];\n";
+                body_ << "      const " << (T_ == "float" ? "float4" : "int4") << " iq" << g << " = SG_LD4(" << g << ");\n";
             }
             static const char* comp[4] = {"x", "y", "z", "w"};
             return "iq" + std::to_string(g) + "." + comp[r % 4];
         }
         if (!loaded_.count(r)) {
             loaded_.insert(r);
-            body_ << "      const " << T_ << " xi" << r << " = xr[" << r << "];\n";
+            body_ << "      const " << T_ << " xi" << r << " = SG_LD1(" << r << ");\n";
         }
         return "xi" + std::to_string(r);
     }
@@ -525,11 +676,11 @@ private:
             if (vout_) {
                 std::string v[4];
                 for (int i = 0; i < 4; i++) v[i] = value_of(osrc[4 * g + i]);
-                body_ << "      reinterpret_cast<" << (T_ == "float" ? "float4" : "int4") << "*>(yr)[" << g << "] = make_"
-                      << (T_ == "float" ? "float4" : "int4") << "(" << v[0] << ", " << v[1] << ", " << v[2] << ", " << v[3]
-                      << ");\n";
+                body_ << "      SG_ST4(" << g << ", make_" << (T_ == "float" ? "float4" : "int4") << "(" << v[0] << ", "
+                      << v[1] << ", " << v[2] << ", " << v[3] << "));\n";
             } else {
-                body_ << "      yr[" << g << "] = " << value_of(osrc[g]) << ";\n";
+                std::string v0 = value_of(osrc[g]);
+                body_ << "      SG_ST1(" << g << ", " << v0 << ");\n";
             }
         };
         for (size_t g = 0; g < pending.size(); g++)
@@ -853,10 +1004,6 @@ private:
                   << ";\n";
             }
             b << "      }\n";
-            const Edge& ed = f_.edges[e];
-            if (ed.dst < 0 && ed.pre > 0)
-                b << "      if (k0 == 0) for (int j = tid; j < " << ed.pre << "; j += NT) g[j - SG_OUT_BASE(" << i
-                  << ")] = (" << T_ << ")0;\n";
             b << "    }\n";
         }
     }

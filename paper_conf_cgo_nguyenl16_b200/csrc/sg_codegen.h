@@ -31,6 +31,13 @@ struct KernelInfo {
     int64_t intops_per_iter = 0;    // algorithmic integer ops (CE = 2 min/max)
     int64_t dfma_per_iter = 0;
     int n_levels = 0;
+    // register mode: the TMA-pipelined variant (name) and the synchronous fallback (name_sync)
+    std::string name_sync;
+    bool has_tma = false;
+    int tma_in = 0, tma_out = 0;     // 1: 2-D tensor map + 128B swizzle, 2: per-row bulk copies
+    int64_t pin = 0, pout = 0, off_in = 0, off_out = 0;
+    int threads_sync = 0, tile_sync = 0;
+    size_t smem_sync = 0;
 };
 
 // Boundary input / output edges of a node set (sorted, deterministic).

@@ -219,6 +219,15 @@ SG_DEV void sg_tma_store_2d(const void* tmap, int c0, int c1, const void* ssrc) 
     asm volatile("cp.async.bulk.tensor.2d.global.shared::cta.tile.bulk_group [%0, {%1, %2}], [%3];"
                  :: "l"(tmap), "r"(c0), "r"(c1), "r"(sg_smem_addr(ssrc)) : "memory");
 }
+// 1-D bulk copies (cp.async.bulk): 16-byte aligned addresses, size multiple of 16.
+SG_DEV void sg_bulk_g2s(void* sdst, const void* gsrc, sg_u32 bytes, unsigned long long* bar) {
+    asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];"
+                 :: "r"(sg_smem_addr(sdst)), "l"(gsrc), "r"(bytes), "r"(sg_smem_addr(bar)) : "memory");
+}
+SG_DEV void sg_bulk_s2g(void* gdst, const void* ssrc, sg_u32 bytes) {
+    asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;"
+                 :: "l"(gdst), "r"(sg_smem_addr(ssrc)), "r"(bytes) : "memory");
+}
 SG_DEV void sg_bulk_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
 template <int N>
 SG_DEV void sg_bulk_wait_read() { asm volatile("cp.async.bulk.wait_group.read %0;" :: "n"(N) : "memory"); }
@@ -227,6 +236,9 @@ SG_DEV void sg_bulk_wait() { asm volatile("cp.async.bulk.wait_group %0;" :: "n"(
 SG_DEV void sg_prefetch_tmap(const void* tmap) {
     asm volatile("prefetch.tensormap [%0];" :: "l"(tmap) : "memory");
 }
+
+// Tensor-map kernel parameter (CUtensorMap is 128 bytes, 64-byte aligned).
+struct __align__(64) SgTmap { unsigned long long v[16]; };
 
 // 128B-swizzle address of 16-byte chunk `c` (0..7) of row `r` in a [rows][128 B] tile
 // written by TMA with CU_TENSOR_MAP_SWIZZLE_128B (tile base 1024-byte aligned).

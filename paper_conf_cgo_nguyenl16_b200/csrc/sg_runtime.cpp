@@ -42,6 +42,9 @@ typedef CUresult (*PFN_launch)(CUfunction, unsigned, unsigned, unsigned, unsigne
                                CUstream, void**, void**);
 typedef CUresult (*PFN_unload)(CUmodule);
 typedef CUresult (*PFN_errstr)(CUresult, const char**);
+typedef CUresult (*PFN_tmap)(CUtensorMap*, CUtensorMapDataType, cuuint32_t, void*, const cuuint64_t*, const cuuint64_t*,
+                             const cuuint32_t*, const cuuint32_t*, CUtensorMapInterleave, CUtensorMapSwizzle,
+                             CUtensorMapL2promotion, CUtensorMapFloatOOBfill);
 struct Api {
     PFN_load load = nullptr;
     PFN_getfn getfn = nullptr;
@@ -50,6 +53,7 @@ struct Api {
     PFN_launch launch = nullptr;
     PFN_unload unload = nullptr;
     PFN_errstr errstr = nullptr;
+    PFN_tmap tmap = nullptr;
 };
 static Api& api() {
     static Api a;
@@ -68,6 +72,7 @@ static Api& api() {
         get("cuLaunchKernel", (void**)&a.launch);
         get("cuModuleUnload", (void**)&a.unload);
         get("cuGetErrorString", (void**)&a.errstr);
+        get("cuTensorMapEncodeTiled", (void**)&a.tmap);
     });
     if (!a.load || !a.launch) throw Error(SG_E_CUDA, "CUDA driver not available (no GPU): the executor has no CPU fallback");
     return a;
@@ -210,19 +215,37 @@ void ensure_module(CompiledKernel& ck, int dev) {
     if ((int)ck.fn.size() <= dev) {
         ck.mod.resize(dev + 1, nullptr);
         ck.fn.resize(dev + 1, nullptr);
+        ck.fn_sync.resize(dev + 1, nullptr);
         ck.max_blocks_per_sm.resize(dev + 1, 0);
+        ck.max_blocks_sync.resize(dev + 1, 0);
     }
     if (ck.fn[dev]) return;
     SG_RT(cudaFree(nullptr));  // make the primary context current
     SG_CU(cuModuleLoadData(&ck.mod[dev], ck.cubin.data()));
-    SG_CU(cuModuleGetFunction(&ck.fn[dev], ck.mod[dev], ck.ki.name.c_str()));
-    SG_CU(cuFuncSetAttribute(ck.fn[dev], CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)ck.ki.smem));
-    int nb = 0;
-    SG_CU(cuOccupancyMaxActiveBlocksPerMultiprocessor(&nb, ck.fn[dev], ck.ki.threads, ck.ki.smem));
-    if (nb <= 0)
-        throw Error(SG_E_SIZE, ck.ki.name + " cannot be resident (" + std::to_string(ck.ki.smem) + " B smem, " +
-                                   std::to_string(ck.ki.threads) + " threads)");
-    ck.max_blocks_per_sm[dev] = nb;
+    auto setup = [&](const std::string& name, int threads, size_t smem, CUfunction& f, int& nb) {
+        SG_CU(cuModuleGetFunction(&f, ck.mod[dev], name.c_str()));
+        SG_CU(cuFuncSetAttribute(f, CU_FUNC_ATTRIBUTE_MAX_DYNAMIC_SHARED_SIZE_BYTES, (int)smem));
+        SG_CU(cuOccupancyMaxActiveBlocksPerMultiprocessor(&nb, f, threads, smem));
+        if (nb <= 0)
+            throw Error(SG_E_SIZE, name + " cannot be resident (" + std::to_string(smem) + " B smem, " +
+                                       std::to_string(threads) + " threads)");
+    };
+    setup(ck.ki.name, ck.ki.threads, ck.ki.smem, ck.fn[dev], ck.max_blocks_per_sm[dev]);
+    if (ck.ki.mode == 1 && ck.ki.has_tma)
+        setup(ck.ki.name_sync, ck.ki.threads_sync, ck.ki.smem_sync, ck.fn_sync[dev], ck.max_blocks_sync[dev]);
+}
+
+// 2-D row tensor map: dims {P items, rows}, box {P, box_rows}, 128B swizzle.
+void encode_rows_map(CUtensorMap* m, bool is_f32, const void* base, int64_t P, int64_t rows, int box_rows) {
+    if (!drv::api().tmap) throw Error(SG_E_CUDA, "cuTensorMapEncodeTiled unavailable");
+    cuuint64_t dims[2] = {(cuuint64_t)P, (cuuint64_t)rows};
+    cuuint64_t strides[1] = {(cuuint64_t)P * 4};
+    cuuint32_t box[2] = {(cuuint32_t)P, (cuuint32_t)box_rows};
+    cuuint32_t estr[2] = {1, 1};
+    SG_CU(drv::api().tmap(m, is_f32 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_INT32, 2,
+                          const_cast<void*>(base), dims, strides, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
+                          CU_TENSOR_MAP_SWIZZLE_128B, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                          CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE));
 }
 
 int sm_count(int dev) {
@@ -245,7 +268,8 @@ struct IoBinding {
 };
 
 // Launch one partition kernel over iterations [kb, ke) on `stream`.
-int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int64_t ke, cudaStream_t stream) {
+int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int64_t ke, cudaStream_t stream,
+               bool is_f32) {
     if (ke <= kb) return 0;
     ensure_module(ck, dev);
     std::vector<int64_t> v;
@@ -256,10 +280,35 @@ int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int
     for (auto b : io.out_base) v.push_back(b);
     v.push_back(kb);
     v.push_back(ke);
-    int64_t tiles = (ke - kb + ck.ki.tile - 1) / ck.ki.tile;
+    const KernelInfo& ki = ck.ki;
+    if (ki.mode == 1 && ki.has_tma) {
+        const char* in_row0 = (const char*)io.in[0] + (kb * ki.pin + ki.off_in - io.in_base[0]) * 4;
+        char* out_row0 = (char*)io.out[0] + (kb * ki.pout + ki.off_out - io.out_base[0]) * 4;
+        bool aligned = ((uintptr_t)in_row0 % 16 == 0) && ((uintptr_t)out_row0 % 16 == 0) && (ke - kb) < (1LL << 31);
+        if (aligned) {
+            alignas(64) CUtensorMap tin, tout;
+            std::memset(&tin, 0, sizeof tin);
+            std::memset(&tout, 0, sizeof tout);
+            if (ki.tma_in == 1) encode_rows_map(&tin, is_f32, in_row0, ki.pin, ke - kb, ki.tile);
+            if (ki.tma_out == 1) encode_rows_map(&tout, is_f32, out_row0, ki.pout, ke - kb, 32);
+            int64_t tiles = (ke - kb + ki.tile - 1) / ki.tile;
+            int64_t grid = std::min<int64_t>(tiles, (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev]);
+            void* params[] = {v.data(), &tin, &tout};
+            SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
+                                 (CUstream)stream, params, nullptr));
+            return 1;
+        }
+        int64_t tiles = (ke - kb + ki.tile_sync - 1) / ki.tile_sync;
+        int64_t grid = std::min<int64_t>(tiles, (int64_t)sm_count(dev) * ck.max_blocks_sync[dev]);
+        void* params[] = {v.data()};
+        SG_CU(cuLaunchKernel(ck.fn_sync[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads_sync, 1, 1,
+                             (unsigned)ki.smem_sync, (CUstream)stream, params, nullptr));
+        return 1;
+    }
+    int64_t tiles = (ke - kb + ki.tile - 1) / ki.tile;
     int64_t grid = std::min<int64_t>(tiles, (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev]);
     void* params[] = {v.data()};
-    SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ck.ki.threads, 1, 1, (unsigned)ck.ki.smem,
+    SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
                          (CUstream)stream, params, nullptr));
     return 1;
 }
@@ -286,6 +335,9 @@ Plan::~Plan() {
         if (g.ev_done) cudaEventDestroy(g.ev_done);
     }
     if (user_ev) cudaEventDestroy(user_ev);
+    if (host_in_dev) { cudaSetDevice(devices[input_gpu]); cudaFree(host_in_dev); }
+    if (host_out_dev) { cudaSetDevice(devices[output_gpu]); cudaFree(host_out_dev); }
+    if (host_stream) { cudaSetDevice(devices[input_gpu]); cudaStreamDestroy(host_stream); }
     for (auto& ck : kernels)
         for (size_t d = 0; d < ck.mod.size(); d++)
             if (ck.mod[d]) { cudaSetDevice((int)d); drv::api().unload(ck.mod[d]); }
@@ -313,7 +365,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
         io.in_limit = {n_in};
         io.out = {out};
         io.out_base = {0};
-        last_launches += launch(ck, devices[0], io, 0, n, stream);
+        last_launches += launch(ck, devices[0], io, 0, n, stream, flat.dtype == SG_F32);
         return;
     }
     // ---- general path: fragments pipelined over partitions and GPUs
@@ -473,7 +525,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                 io.out.push_back(r.src_slots[slot]);
                 io.out_base.push_back(ka * r.per_iter + r.lo);
             }
-            last_launches += launch(ck, gc.dev, io, ka, kb, gc.compute);
+            last_launches += launch(ck, gc.dev, io, ka, kb, gc.compute, flat.dtype == SG_F32);
             // consumed slots of incoming rings are free again
             for (int ri : ring_in[p]) SG_RT(cudaEventRecord(rings[ri].ev_consumed[slot], gc.compute));
             // ship outgoing boundary streams to other GPUs (copy engine, P2P)
@@ -502,6 +554,38 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
         SG_RT(cudaEventRecord(g.ev_start, g.copy));
         SG_RT(cudaStreamWaitEvent(stream, g.ev_start, 0));
     }
+}
+
+// HOST buffers in and out: H2D copy, run, D2H copy, synchronise (the end-to-end
+// path a user without device memory takes).  Staging buffers are kept.
+void Plan::run_host(const void* hin, int64_t n, void* hout) {
+    if (n <= 0) return;
+    int ndev = 0;
+    if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0) {
+        cudaGetLastError();
+        throw Error(SG_E_CUDA, "no CUDA device: the executor has no CPU fallback");
+    }
+    const size_t bi = (size_t)flat.input_items(n) * 4, bo = (size_t)flat.output_items(n) * 4;
+    const int din = devices[input_gpu], dout = devices[output_gpu];
+    DevGuard dg(din);
+    if (!host_stream) SG_RT(cudaStreamCreateWithFlags(&host_stream, cudaStreamNonBlocking));
+    if (host_in_cap < bi) {
+        if (host_in_dev) cudaFree(host_in_dev);
+        host_in_dev = nullptr;
+        SG_RT(cudaMalloc(&host_in_dev, bi));
+        host_in_cap = bi;
+    }
+    if (host_out_cap < bo) {
+        DevGuard d2(dout);
+        if (host_out_dev) cudaFree(host_out_dev);
+        host_out_dev = nullptr;
+        SG_RT(cudaMalloc(&host_out_dev, bo));
+        host_out_cap = bo;
+    }
+    SG_RT(cudaMemcpyAsync(host_in_dev, hin, bi, cudaMemcpyHostToDevice, host_stream));
+    run(host_in_dev, n, host_out_dev, host_stream);
+    SG_RT(cudaMemcpyAsync(hout, host_out_dev, bo, cudaMemcpyDeviceToHost, host_stream));
+    SG_RT(cudaStreamSynchronize(host_stream));
 }
 
 }  // namespace sg

@@ -17,8 +17,10 @@ struct CompiledKernel {
     std::string log;
     // per physical device (index = device ordinal)
     std::vector<CUmodule> mod;
-    std::vector<CUfunction> fn;
+    std::vector<CUfunction> fn;            // main variant (TMA pipeline when ki.has_tma)
+    std::vector<CUfunction> fn_sync;       // register mode: synchronous fallback
     std::vector<int> max_blocks_per_sm;
+    std::vector<int> max_blocks_sync;
 };
 
 struct CutRing {          // one boundary stream between partitions (a PDG edge member)
@@ -64,8 +66,15 @@ struct Plan {
     int64_t last_launches = 0;
     cudaEvent_t user_ev = nullptr;
 
+    // sg_run_host staging (device buffers reused across calls)
+    void* host_in_dev = nullptr;
+    void* host_out_dev = nullptr;
+    size_t host_in_cap = 0, host_out_cap = 0;
+    cudaStream_t host_stream = nullptr;
+
     ~Plan();
     void run(const void* in, int64_t n, void* out, cudaStream_t stream);
+    void run_host(const void* hin, int64_t n, void* hout);
 };
 
 // NVRTC -> sm_100a cubin (cached by content hash in memory and on disk).

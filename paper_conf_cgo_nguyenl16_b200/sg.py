@@ -29,7 +29,8 @@ KINDS = {"IDENTITY": 0, "FIR": 1, "DELAY": 2, "DECIMATE": 3, "EXPAND": 4, "COMPA
 EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_splitjoin", "sg_branch_begin",
            "sg_branch_end", "sg_plan_opts_default", "sg_plan", "sg_input_items", "sg_output_items",
            "sg_plan_info", "sg_plan_source", "sg_run", "sg_run_host", "sg_last_launch_count",
-           "sg_plan_destroy", "sg_last_error", "sg_version", "sg_flush_l2"]
+           "sg_plan_destroy", "sg_last_error", "sg_version", "sg_flush_l2", "sg_topology_links",
+           "sg_topology_dtlist", "sg_map_ilp", "sg_paper_model", "sg_plan_pdg"]
 
 
 class SgError(RuntimeError):
@@ -95,6 +96,15 @@ def lib():
         "sg_last_error": ([], ctypes.c_char_p),
         "sg_version": ([], ctypes.c_char_p),
         "sg_flush_l2": ([vp, i64, vp], ctypes.c_int),
+        "sg_topology_links": ([i32, i32], i32),
+        "sg_topology_dtlist": ([i32, i32, ctypes.POINTER(ctypes.c_uint8)], ctypes.c_int),
+        "sg_map_ilp": ([i32, ctypes.POINTER(ctypes.c_double), i32, ctypes.POINTER(i32), ctypes.POINTER(i32),
+                        ctypes.POINTER(ctypes.c_double), i32, i32, ctypes.c_double, ctypes.c_double, i32, i32,
+                        ctypes.POINTER(i32), ctypes.POINTER(ctypes.c_double), ctypes.POINTER(i32)], ctypes.c_int),
+        "sg_paper_model": ([i32, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ctypes.c_double), i32, i32, i32,
+                            ctypes.c_double, ctypes.c_double, ctypes.c_double, ctypes.POINTER(ctypes.c_double),
+                            ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ctypes.c_double)], ctypes.c_double),
+        "sg_plan_pdg": ([vp, i32, ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(ctypes.c_double)], i32),
     }
     for name, (args, res) in sig.items():
         fn = getattr(L, name)
@@ -256,6 +266,13 @@ class Plan:
         """x, y: contiguous host numpy arrays (4-byte items); copies in, runs, copies out, synchronises."""
         _check(lib().sg_run_host(self._h, ctypes.c_void_p(x.ctypes.data), n_iters, ctypes.c_void_p(y.ctypes.data)))
 
+    def pdg(self):
+        n = lib().sg_plan_pdg(self._h, 0, None, None, None)
+        a, b = (ctypes.c_int32 * max(1, n))(), (ctypes.c_int32 * max(1, n))()
+        c = (ctypes.c_double * max(1, n))()
+        lib().sg_plan_pdg(self._h, n, a, b, c)
+        return [(a[i], b[i], c[i]) for i in range(n)]
+
     def last_launch_count(self) -> int:
         return lib().sg_last_launch_count(self._h)
 
@@ -288,6 +305,43 @@ def flush_l2(scratch, stream=None):
         stream = torch.cuda.current_stream().cuda_stream
     _check(lib().sg_flush_l2(ctypes.c_void_p(scratch.data_ptr()), scratch.numel() * scratch.element_size(),
                              ctypes.c_void_p(stream)))
+
+
+def topology_dtlist(kind: int, n_gpus: int):
+    """dtlist[l][i][j] as nested lists (kind 0 NVSwitch star, 1 = PCIe tree of Fig. 3.3)."""
+    L = lib().sg_topology_links(kind, n_gpus)
+    if L < 0:
+        raise SgError(SG_E_ARG, "bad topology")
+    buf = (ctypes.c_uint8 * (L * n_gpus * n_gpus))()
+    _check(lib().sg_topology_dtlist(kind, n_gpus, buf))
+    G = n_gpus
+    return [[[buf[l * G * G + i * G + j] for j in range(G)] for i in range(G)] for l in range(L)]
+
+
+def map_ilp(T, edges, n_gpus, topo_kind=0, lat=0.0, bw=1.0, method=0, time_limit_ms=10000):
+    """Solve Eq. III.1-III.7; edges = [(src, dst, bytes)].  Returns (assign, tmax, optimal)."""
+    P = len(T)
+    Ta = (ctypes.c_double * max(1, P))(*T)
+    ne = len(edges)
+    es = (ctypes.c_int32 * max(1, ne))(*[e[0] for e in edges])
+    ed = (ctypes.c_int32 * max(1, ne))(*[e[1] for e in edges])
+    eb = (ctypes.c_double * max(1, ne))(*[e[2] for e in edges])
+    asg = (ctypes.c_int32 * max(1, P))()
+    tm = ctypes.c_double(0)
+    opt = ctypes.c_int32(0)
+    _check(lib().sg_map_ilp(P, Ta, ne, es, ed, eb, topo_kind, n_gpus, lat, bw, time_limit_ms, method, asg,
+                            ctypes.byref(tm), ctypes.byref(opt)))
+    return [asg[i] for i in range(P)], tm.value, bool(opt.value)
+
+
+def paper_model(t, f, S, W, F, D, C1=38.4, C2=11.2):
+    """Eq. III.8-III.12; returns (T, Tcomp, Tdt, Tdb)."""
+    n = len(t)
+    ta = (ctypes.c_double * max(1, n))(*t)
+    fa = (ctypes.c_double * max(1, n))(*f)
+    a, b, c = ctypes.c_double(), ctypes.c_double(), ctypes.c_double()
+    T = lib().sg_paper_model(n, ta, fa, S, W, F, D, C1, C2, ctypes.byref(a), ctypes.byref(b), ctypes.byref(c))
+    return T, a.value, b.value, c.value
 
 
 def version() -> str:

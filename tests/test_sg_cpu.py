@@ -1,0 +1,357 @@
+"""CPU tests of the product library (no GPU): the C ABI loads and exports every
+symbol include/sg.h declares; the SDF analysis agrees with the oracle's
+independent solver; error codes; the planner (topology dtlist of Fig. 3.3,
+ILP exactness against brute force and HiGHS, Algorithm 1 invariants, the
+paper's Eq. III.8-III.12); code generation + NVRTC sm_100a compilation of the
+benchmark programs and of random graphs.
+"""
+import os
+import re
+
+import numpy as np
+import pytest
+
+from workloads import apps
+from workloads.spec import Filter, Pipeline, Program, SplitJoin
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.fixture(scope="module")
+def sg():
+    from paper_conf_cgo_nguyenl16_b200 import build, sg as s
+    build.build()
+    s.lib()
+    return s
+
+
+def test_library_exports_every_declared_symbol(sg):
+    hdr = open(os.path.join(ROOT, "include", "sg.h")).read()
+    hdr = re.sub(r"/\*.*?\*/", "", hdr, flags=re.S)
+    declared = set(re.findall(r"\b(sg_[a-z0-9_]+)\s*\(", hdr))
+    assert len(declared) >= 20
+    L = sg.lib()
+    for name in sorted(declared):
+        assert hasattr(L, name), f"libsg.so does not export {name}"
+    assert set(sg.EXPORTS) == declared
+
+
+def test_library_is_sm100a(sg):
+    import subprocess
+    so = os.path.join(ROOT, "paper_conf_cgo_nguyenl16_b200", "libsg.so")
+    out = subprocess.run(["cuobjdump", "--list-elf", so], capture_output=True, text=True).stdout
+    assert "sm_100a" in out
+
+
+# ------------------------------------------------------- SDF analysis vs oracle
+@pytest.mark.parametrize("name", list(apps.CONFIGS))
+def test_rates_match_oracle(sg, oracle_lib, name):
+    prog = apps.CONFIGS[name]()
+    r = oracle_lib.rates(prog)
+    with sg.plan(prog, 1, partitioner="single") as p:
+        i = p.info()
+        assert i["reps"] == r["reps"]
+        assert i["in_per_iter"] == r["in_per_iter"] and i["out_per_iter"] == r["out_per_iter"]
+        for n in (1, 2, 5):
+            assert p.input_items(n) == oracle_lib.in_items(prog, n)
+            assert p.output_items(n) == n * r["out_per_iter"]
+        assert p.input_items(0) == 0 and p.output_items(0) == 0
+
+
+@pytest.mark.parametrize("seed", range(24))
+def test_random_graph_rates_and_in_items_match_oracle(sg, oracle_lib, seed):
+    prog = apps.random_program(seed, "f32" if seed % 2 else "i32")
+    r = oracle_lib.rates(prog)
+    with sg.plan(prog, 1, partitioner="single") as p:
+        i = p.info()
+        assert i["reps"] == r["reps"]
+        for n in (1, 3):
+            assert p.input_items(n) == oracle_lib.in_items(prog, n), n
+            got = p.output_items(n)
+            # output items of n iterations = what the oracle emits on in_items(n) inputs
+            x = np.zeros(oracle_lib.in_items(prog, n), np.int32 if prog.dtype == "i32" else np.float32)
+            assert oracle_lib.run_items(prog, x, 10 ** 9).size >= got
+
+
+def test_delay_prework_counts_in_output(sg, oracle_lib):
+    prog = Program("d", "f32", Pipeline([Filter("FIR", [3, 1], [1.0, 2.0, 3.0]), Filter("DELAY", [5])]))
+    with sg.plan(prog, 1) as p:
+        assert p.output_items(4) == 4                       # first 4 stream items: prework zeros
+        assert p.input_items(4) == oracle_lib.in_items(prog, 4) == 0
+        assert p.output_items(9) == 9
+        assert p.input_items(9) == oracle_lib.in_items(prog, 9) == 6
+
+
+# ------------------------------------------------------------------ errors
+def test_inconsistent_rates_rejected(sg):
+    bad = Program("bad", "f32", Pipeline([SplitJoin("dup", [Filter("IDENTITY"), Filter("DECIMATE", [2])])]))
+    with pytest.raises(sg.SgError) as e:
+        sg.plan(bad, 1)
+    assert e.value.code == sg.SG_E_RATE
+
+
+def test_structure_errors(sg):
+    g = sg.Graph("f32")
+    sj = g.add_splitjoin(True, 2)
+    g.branch_begin(sj, 0)
+    g.add_filter("IDENTITY")
+    g.branch_end()
+    with pytest.raises(sg.SgError) as e:          # branch 1 never filled
+        sg.Plan(g, 1)
+    assert e.value.code == sg.SG_E_STRUCTURE
+    with pytest.raises(sg.SgError):
+        g.branch_end()                            # nothing open
+    empty = sg.Graph("f32")
+    with pytest.raises(sg.SgError) as e:
+        sg.Plan(empty, 1)
+    assert e.value.code == sg.SG_E_STRUCTURE
+
+
+def test_bad_parameters_rejected(sg):
+    g = sg.Graph("f32")
+    with pytest.raises(sg.SgError) as e:
+        g.add_filter("FIR", [4, 1], [1.0, 2.0])   # 4 taps, 2 coefficients
+    assert e.value.code == sg.SG_E_ARG
+    gi = sg.Graph("i32")
+    with pytest.raises(sg.SgError) as e:
+        gi.add_filter("FIR", [1, 1], [1.0])        # float kind on an int graph
+    assert e.value.code == sg.SG_E_UNSUPPORTED
+    with pytest.raises(sg.SgError):
+        sg.plan(apps.bitonic(8), 0)
+
+
+def test_run_without_gpu_fails_loudly(sg):
+    import torch
+    if torch.cuda.is_available():
+        pytest.skip("GPU present")
+    with sg.plan(apps.bitonic(8), 1) as p:
+        x = np.zeros(8 * 4, np.int32)
+        y = np.zeros(8 * 4, np.int32)
+        with pytest.raises(sg.SgError) as e:
+            p.run_host(x, 4, y)
+        assert e.value.code == sg.SG_E_CUDA
+
+
+# ---------------------------------------------------------------- topology
+def test_pcie_tree_dtlist_matches_fig_3_3(sg):
+    """PAPER.md:468-490 (section 3.2.1, Fig. 3.3): GPU1->GPU2 uses two links,
+    GPU2->GPU3 uses four, and link SW2->SW1 carries exactly (1,3),(1,4),(2,3),(2,4)."""
+    import json
+    gold = json.load(open(os.path.join(ROOT, "tests", "golden", "fig3_3_pcie_tree.json")))
+    dt = np.array(sg.topology_dtlist(1, 4))
+    assert dt.shape == (12, 4, 4)
+    for src, dst, n in gold["links_used"]:
+        assert int(dt[:, src - 1, dst - 1].sum()) == n
+    up_sw2 = 8  # link index of SW2 -> SW1 in sg_topology_dtlist(1, 4)
+    pairs = sorted((i + 1, j + 1) for i in range(4) for j in range(4) if dt[up_sw2, i, j])
+    assert pairs == sorted(tuple(p) for p in gold["sw2_to_sw1_pairs"])
+    # the uplink rule: uplink l carries i->j iff i is under l and j is not
+    for l in range(12):
+        assert not any(dt[l, i, i] for i in range(4))
+
+
+def test_nvswitch_star(sg):
+    G = 8
+    dt = np.array(sg.topology_dtlist(0, G))
+    assert dt.shape == (2 * G, G, G)
+    for i in range(G):
+        for j in range(G):
+            used = set(np.nonzero(dt[:, i, j])[0])
+            assert used == (set() if i == j else {i, G + j})
+
+
+# --------------------------------------------------------------------- ILP
+def _rand_instance(seed, P, G):
+    rng = np.random.default_rng(seed)
+    T = list(rng.uniform(1, 10, P))
+    edges = []
+    for i in range(P - 1):
+        edges.append((i, i + 1, float(rng.uniform(0, 40))))
+    for _ in range(P // 2):
+        a, b = sorted(rng.choice(P, 2, replace=False))
+        edges.append((int(a), int(b), float(rng.uniform(0, 20))))
+    return T, edges
+
+
+@pytest.mark.parametrize("seed", range(12))
+@pytest.mark.parametrize("G,topo", [(2, 0), (3, 0), (4, 0), (4, 1)])
+def test_ilp_branch_and_bound_equals_brute_force(sg, seed, G, topo):
+    P = 6 if G < 4 else 5
+    T, edges = _rand_instance(seed, P, G)
+    lat, bw = 0.3, 10.0
+    a1, t1, opt1 = sg.map_ilp(T, edges, G, topo, lat, bw, method=0)
+    a2, t2, opt2 = sg.map_ilp(T, edges, G, topo, lat, bw, method=1)
+    assert opt1 and opt2
+    assert abs(t1 - t2) <= 1e-9 * max(1, t2)
+
+
+def _milp_tmax(T, edges, G, dt, lat, bw):
+    """The same model, Eq. III.1-III.7 linearised, solved by HiGHS."""
+    from scipy.optimize import LinearConstraint, milp, Bounds
+    P, E, L = len(T), len(edges), dt.shape[0]
+    nv = P * G + E * G * G + 1
+    idx_n = lambda i, j: i * G + j
+    idx_e = lambda e, k, h: P * G + e * G * G + k * G + h
+    it = nv - 1
+    c = np.zeros(nv)
+    c[it] = 1
+    A, lo, hi = [], [], []
+
+    def row():
+        return np.zeros(nv)
+
+    for i in range(P):                                   # III.5
+        r = row()
+        for j in range(G):
+            r[idx_n(i, j)] = 1
+        A.append(r); lo.append(1); hi.append(1)
+    for j in range(G):                                   # III.1 + III.4
+        r = row()
+        for i in range(P):
+            r[idx_n(i, j)] = T[i]
+        r[it] = -1
+        A.append(r); lo.append(-np.inf); hi.append(0)
+    for e, (s, d, D) in enumerate(edges):                # III.6 linearised
+        for k in range(G):
+            for h in range(G):
+                r = row(); r[idx_e(e, k, h)] = 1; r[idx_n(s, k)] = -1
+                A.append(r); lo.append(-np.inf); hi.append(0)
+                r = row(); r[idx_e(e, k, h)] = 1; r[idx_n(d, h)] = -1
+                A.append(r); lo.append(-np.inf); hi.append(0)
+                r = row(); r[idx_e(e, k, h)] = 1; r[idx_n(s, k)] = -1; r[idx_n(d, h)] = -1
+                A.append(r); lo.append(-1); hi.append(np.inf)
+    for l in range(L):                                   # III.2 + III.3 + III.7
+        r = row()
+        for e, (s, d, D) in enumerate(edges):
+            for k in range(G):
+                for h in range(G):
+                    if dt[l, k, h]:
+                        r[idx_e(e, k, h)] = D / bw
+        r[it] = -1
+        A.append(r); lo.append(-np.inf); hi.append(-lat)
+    integrality = np.ones(nv)
+    integrality[it] = 0
+    bounds = Bounds(np.zeros(nv), np.concatenate([np.ones(nv - 1), [np.inf]]))
+    res = milp(c, constraints=LinearConstraint(np.array(A), lo, hi), integrality=integrality, bounds=bounds)
+    assert res.success
+    return res.fun
+
+
+@pytest.mark.parametrize("seed", range(6))
+@pytest.mark.parametrize("G,topo", [(2, 0), (4, 0), (4, 1)])
+def test_ilp_matches_highs(sg, seed, G, topo):
+    P = 7
+    T, edges = _rand_instance(100 + seed, P, G)
+    lat, bw = 0.2, 8.0
+    dt = np.array(sg.topology_dtlist(topo, G))
+    _, tmax, opt = sg.map_ilp(T, edges, G, topo, lat, bw)
+    assert opt
+    ref = _milp_tmax(T, edges, G, dt, lat, bw)
+    assert abs(tmax - ref) <= 1e-6 * max(1.0, ref)
+
+
+def test_ilp_single_gpu_and_no_edges(sg):
+    a, t, opt = sg.map_ilp([3.0, 4.0, 5.0], [], 1, 0, 0.0, 1.0)
+    assert a == [0, 0, 0] and abs(t - 12.0) < 1e-12 and opt
+    a, t, opt = sg.map_ilp([3.0, 4.0, 5.0], [], 3, 0, 0.0, 1.0)
+    assert sorted(a) == [0, 1, 2] and abs(t - 5.0) < 1e-12
+
+
+# ------------------------------------------------------------- paper model
+def test_paper_model_closed_form(sg):
+    """Eq. III.8-III.12 with the paper's constants C1 = 38.4, C2 = 11.2."""
+    t, f = [10.0, 4.0, 6.0], [1.0, 8.0, 3.0]
+    S, W, F, D = 4, 16, 32, 1000.0
+    T, tc, tdt, tdb = sg.paper_model(t, f, S, W, F, D)
+    assert tc == pytest.approx(10 / 1 + 4 / 4 + 6 / 3)
+    assert tdt == pytest.approx(38.4 * 1000 / 32)
+    assert tdb == pytest.approx(11.2 * 1000 / (32 + 16 * 4))
+    assert T == pytest.approx((max(tc, tdt) + tdb) / W)
+
+
+# ------------------------------------------------------------ Algorithm 1
+def _edges(prog):
+    from test_oracle import _edge_list
+    return [(u, v) for (u, _, v, _) in _edge_list(prog)]
+
+
+def _convex(n, edges, part):
+    succ = [[] for _ in range(n)]
+    for u, v in edges:
+        succ[u].append(v)
+    inside = set(part)
+    seen, st = set(), [w for u in part for w in succ[u] if w not in inside]
+    while st:
+        x = st.pop()
+        if x in seen:
+            continue
+        seen.add(x)
+        for w in succ[x]:
+            if w in inside:
+                return False
+            st.append(w)
+    return True
+
+
+@pytest.mark.parametrize("name,G", [("fmradio10", 1), ("fmradio10", 2), ("filterbank64", 4), ("bitonic32", 2),
+                                    ("beamformer12x4", 2), ("fft64", 1)])
+def test_algorithm1_invariants(sg, name, G):
+    prog = apps.CONFIGS[name]()
+    with sg.plan(prog, G) as p:
+        i = p.info()
+        n = i["n_nodes"]
+        parts = {}
+        for v, q in enumerate(i["node_partition"]):
+            parts.setdefault(q, []).append(v)
+        assert sorted(parts) == list(range(i["n_partitions"]))       # every node in exactly one partition
+        E = _edges(prog)
+        for q, nodes in parts.items():
+            assert _convex(n, E, nodes), f"partition {q} not convex"
+        assert all(0 <= g < G for g in i["partition_gpu"])
+        loads = [0.0] * G
+        for q, g in enumerate(i["partition_gpu"]):
+            loads[g] += i["partition_time"][q]
+        assert i["est_tmax"] >= max(loads) - 1e-9
+        pdg = p.pdg()
+        for (a, b, D) in pdg:
+            assert a != b and D > 0
+        if G == 1:
+            assert i["n_partitions"] == 1    # phase 4(2): never worse than the single partition
+
+
+def test_user_and_per_filter_partitions(sg):
+    prog = apps.fmradio(3)
+    with sg.plan(prog, 1, partitioner="per_filter") as p:
+        assert p.info()["n_partitions"] == p.info()["n_nodes"]
+    n = 0
+    with sg.plan(prog, 1, partitioner="single") as p:
+        n = p.info()["n_nodes"]
+    with pytest.raises(sg.SgError) as e:    # non-convex: nodes 0 and 2 without 1
+        sg.plan(prog, 1, node_partition=[0, 1, 0] + [2] * (n - 3))
+    assert e.value.code == sg.SG_E_PLAN
+
+
+# ------------------------------------------------------------- codegen/NVRTC
+@pytest.mark.parametrize("seed", range(10))
+def test_random_graph_compiles(sg, seed):
+    prog = apps.random_program(1000 + seed, "f32" if seed % 2 else "i32")
+    with sg.plan(prog, 1, partitioner="single") as p:
+        src = p.source(0)
+        assert "extern \"C\" __global__" in src
+    with sg.plan(prog, 1, partitioner="per_filter") as p:
+        assert p.info()["n_partitions"] >= 1
+
+
+def test_benchmark_kernels_are_blackwell_native(sg):
+    """The register-mode BitonicSort kernel streams with TMA (UTMALDG/UTMASTG)."""
+    import glob
+    import subprocess
+    with sg.plan(apps.bitonic(32), 1) as p:
+        assert "sg_tma_load_2d" in p.source(0)
+    cubins = glob.glob(os.path.join(ROOT, "paper_conf_cgo_nguyenl16_b200", ".sg_cache", "*.cubin"))
+    found = False
+    for c in cubins:
+        sass = subprocess.run(["cuobjdump", "-sass", c], capture_output=True, text=True).stdout
+        if "UTMALDG" in sass and "UTMASTG" in sass:
+            found = True
+    assert found
