@@ -605,6 +605,7 @@ public:
             }
         }
         if (!ki.has_tma) {
+            ki.name = ki.name_sync;
             ki.threads = ki.threads_sync;
             ki.tile = ki.tile_sync;
             ki.smem = ki.smem_sync;
@@ -773,6 +774,7 @@ public:
             body << "    __syncthreads();\n";
         }
         emit_stores(body);
+        body << "    __syncthreads();  // stores of this tile read buffers the next tile's loads may reuse\n";
         std::ostringstream src;
         src << header("staged") << consts_.str() << args_struct();
         src << "#define NT " << NT << "\n#define W " << W << "\n";

@@ -355,3 +355,13 @@ def test_benchmark_kernels_are_blackwell_native(sg):
         if "UTMALDG" in sass and "UTMASTG" in sass:
             found = True
     assert found
+
+
+@pytest.mark.parametrize("name", ["bitonic32", "fmradio10"])
+@pytest.mark.parametrize("part", ["single", "per_filter"])
+def test_kernel_entry_points_exist(sg, name, part):
+    prog = apps.CONFIGS[name]() if name != "fmradio10" else apps.fmradio(3)
+    with sg.plan(prog, 1, partitioner=part) as p:
+        for q in range(p.info()["n_partitions"]):
+            src = p.source(q)
+            assert re.search(r'__global__ void __launch_bounds__\([^)]*\) sg_part%d(_sync)?\(' % q, src), q
