@@ -227,7 +227,8 @@ def main():
     # roofline of the dominant kernel (single partition: one launch per step)
     peaks, peak_src = measured_peaks()
     # kernel duration: CUDA events around the launch on its stream (one kernel per step here)
-    kern_ms = statistics.median(step_ms) if launches_per_step == 1 else None
+    # one partition => every launch of the step is this partition's kernel (main + stream-start variant)
+    kern_ms = statistics.median(step_ms) if info["n_partitions"] == 1 else None
     ki_bytes = (info["in_per_iter"] + info["out_per_iter"]) * 4 * n
     roof = None
     if W["bound"] == "hbm":
@@ -237,12 +238,16 @@ def main():
                     "frac": ach / peaks["hbm_gbs"], "traffic": None,
                     "algorithmic_bytes_per_launch": ki_bytes, "peak_source": peak_src + " copy bandwidth"}
     else:
-        fl = _flops_per_iter(prog, info["reps"])
+        fl_written = _flops_per_iter(prog, info["reps"])
+        fl = min(fl_written, info["flops_per_iter_pruned"]) if info["flops_per_iter_pruned"] > 0 else fl_written
         if kern_ms:
             ach = fl * n / (kern_ms / 1e3) / 1e12
             pk = 148 * 128 * 2 * peaks.get("sm_max_mhz", 1965.0) * 1e6 / 1e12
             roof = {"bound": "alu", "achieved": ach, "peak": pk, "unit": "TFLOP/s", "frac": ach / pk,
                     "traffic": None, "algorithmic_flops_per_launch": fl * n,
+                    "flops_per_iter": fl, "flops_per_iter_as_written": fl_written,
+                    "flops_counting": "as written" if fl == fl_written else
+                    "pruned (dead firings and zero taps eliminated by the code generator)",
                     "peak_source": "derived: 148 SMs x 128 FP32 lanes x 2 x sm_max_mhz (FFMA)"}
     prof = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     if roof is not None and os.path.exists(prof):

@@ -136,7 +136,7 @@ typedef struct sg_plan_opts {
     int32_t virtual_gpus;          /* 1: map the G logical GPUs onto streams of one device */
     const int32_t* devices;        /* physical device per logical GPU (NULL: 0..G-1) */
     int32_t ilp_time_limit_ms;     /* exact branch-and-bound budget; 0 = 10000 */
-    int32_t codegen_mode;          /* 0 auto, 1 register (thread per iteration), 2 staged */
+    int32_t codegen_mode;          /* 0 auto, 1 register (thread per iteration), 2 staged, 3 staged general path only */
     double link_gbps;              /* NVLink bandwidth per direction for the ILP; 0 = 770 */
     double link_latency_us;        /* per-transfer latency Lat (Eq. III.3); 0 = 10 */
     int32_t verbose;
@@ -162,6 +162,9 @@ typedef struct sg_plan_info_s {
     int32_t output_device;           /* device holding the caller's output */
     int64_t iters_per_fragment;
     int32_t ilp_optimal;             /* 1 if the branch-and-bound proved optimality */
+    double flops_per_iter_written;   /* algorithmic fp32 flops per iteration as written (FMA = 2) */
+    double flops_per_iter_pruned;    /* same after dead-firing / zero-tap elimination (<= written) */
+    int64_t intops_per_iter;         /* algorithmic integer ops per iteration (min/max, adds) */
 } sg_plan_info_t;
 
 /* ---- graph construction (the top-level stream is an implicit pipeline) ---- */

@@ -192,6 +192,18 @@ sg_status sg_plan_info(const sg_plan_t* pp, sg_plan_info_t* o) {
     o->output_device = p.devices[p.output_gpu];
     o->iters_per_fragment = p.iters_per_fragment;
     o->ilp_optimal = p.ilp_optimal ? 1 : 0;
+    double written = 0, pruned = 0;
+    int64_t intops = 0;
+    for (const auto& ck : p.kernels) {
+        written += (double)ck.ki.flops_per_iter;
+        pruned += ck.ki.flops_exec_per_iter >= 0 ? std::min<double>((double)ck.ki.flops_exec_per_iter,
+                                                                    (double)ck.ki.flops_per_iter)
+                                                 : (double)ck.ki.flops_per_iter;
+        intops += ck.ki.intops_per_iter;
+    }
+    o->flops_per_iter_written = written;
+    o->flops_per_iter_pruned = pruned;
+    o->intops_per_iter = intops;
     return SG_OK;
 }
 

@@ -733,60 +733,112 @@ public:
         fill_io(ki);
         compute_levels();
         int NT = opt.threads > 0 ? opt.threads : 256;
-        // choose the tile: largest W whose shared-memory footprint fits the budget
+        NT_ = NT;
+        // ---------------- fused fast path (full tiles without stream-start firings)
+        std::string fast, fast_start;
+        int WF = 0;
+        size_t smem_fast = 0;
+        if (opt.mode != -2) {
+            try {
+                fused_ = true;
+                fused_analyze();
+                size_t fb = opt.smem_budget > 0 ? (size_t)opt.smem_budget : (size_t)(110 * 1024);
+                for (int cand : {4096, 2048, 1024, 512, 256, 128, 64, 32, 16, 8, 4, 2, 1}) {
+                    if (opt.tile > 0 && cand != opt.tile) continue;
+                    fused_layout(cand);
+                    if (smem_bytes_ <= fb) { WF = cand; break; }
+                }
+                if (WF == 0) {
+                    fused_layout(1);
+                    if (smem_bytes_ <= 227 * 1024) WF = 1;
+                }
+                if (WF > 0) {
+                    fused_layout(WF);
+                    smem_fast = smem_bytes_;
+                    fast = fused_emit(WF, false);
+                    fast_start = fused_emit(WF, true);
+                    ki.flops_exec_per_iter = fused_flops_per_iter();
+                }
+            } catch (const FusedFail&) {
+                WF = 0;
+                fast.clear();
+            }
+            fused_ = false;
+        }
+        // ---------------- slow (general) path: every compute filter materialised
         size_t budget = opt.smem_budget > 0 ? (size_t)opt.smem_budget : (size_t)(100 * 1024);
         int W = opt.tile;
         if (W <= 0) {
-            int64_t per = 0;
-            for (int v : nodes_) per = std::max(per, f_.nodes[v].rep);
             W = 1;
             for (int cand : {1024, 512, 256, 128, 64, 32, 16, 8, 4, 2, 1}) {
                 layout(cand);
                 if (smem_bytes_ <= budget) { W = cand; break; }
             }
-            layout(W);
-            if (smem_bytes_ > budget) {
-                layout(1);
-                W = 1;
-            }
         }
         layout(W);
-        if (smem_bytes_ > 227 * 1024)
+        if (WF == 0 && smem_bytes_ > 227 * 1024)
             throw Error(SG_E_SIZE, "partition " + std::to_string(part_) + " needs " + std::to_string(smem_bytes_) +
                                        " B of shared memory for one iteration");
         W_ = W;
-        NT_ = NT;
-        ki.threads = NT;
-        ki.tile = W;
-        ki.smem = smem_bytes_;
-        ki.min_blocks = std::max(1, std::min(4, (int)((220 * 1024) / std::max<size_t>(1024, smem_bytes_))));
-        ki.n_levels = nlev_;
-        std::ostringstream body;
-        emit_loads(body);
+        std::ostringstream slow;
+        if (WF == 0) {
+        emit_loads(slow);
         for (int L = 1; L <= nlev_; L++) {
-            body << "    // ---- level " << L << "\n";
+            slow << "    // ---- level " << L << "\n";
             int64_t rot = 0;
             for (int v : nodes_) {
                 if (is_view_node(f_.nodes[v]) || level_[v] != L) continue;
-                emit_stage(body, v, rot);
+                emit_stage(slow, v, rot);
                 rot += f_.nodes[v].halo + (int64_t)W * f_.nodes[v].rep;
             }
-            body << "    __syncthreads();\n";
+            slow << "    __syncthreads();\n";
         }
-        emit_stores(body);
-        body << "    __syncthreads();  // stores of this tile read buffers the next tile's loads may reuse\n";
+        emit_stores(slow);
+        slow << "    __syncthreads();  // stores of this tile read buffers the next tile's loads may reuse\n";
+        }
+        size_t smem_slow = smem_bytes_;
+        ki.n_levels = nlev_;
+        int64_t ksafe = 0;
+        for (int v : nodes_) {
+            const Node& n = f_.nodes[v];
+            int64_t F0 = n.ninit - n.halo;
+            if (F0 < 0) ksafe = std::max(ksafe, (-F0 + n.rep - 1) / n.rep);
+        }
+        const int WT = WF > 0 ? WF : W;
+        ki.threads = NT;
+        ki.tile = WT;
+        ki.smem = WF > 0 ? smem_fast : smem_slow;
+        ki.min_blocks = std::max(1, std::min(2, (int)((220 * 1024) / std::max<size_t>(1024, ki.smem))));
+        ki.fused = WF > 0;
+        ki.ksafe = ksafe;
         std::ostringstream src;
         src << header("staged") << consts_.str() << args_struct();
-        src << "#define NT " << NT << "\n#define W " << W << "\n";
+        src << "#define NT " << NT << "\n";
         src << readers_.str();
-        src << "extern \"C\" __global__ void __launch_bounds__(NT, " << ki.min_blocks << ") " << ki.name
-            << "(const SgArgs a) {\n"
-            << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
-            << "  " << T_ << "* sm = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
-            << "  const int tid = threadIdx.x;\n"
-            << "  for (long long k0 = SG_K_BEGIN + (long long)blockIdx.x * W; k0 < SG_K_END; k0 += (long long)gridDim.x * W) {\n"
-            << "    const int Wt = (int)min((long long)W, SG_K_END - k0);\n"
-            << body.str() << "  }\n}\n";
+        auto kernel = [&](const std::string& name, const std::string& body, bool fusedk) {
+            src << "extern \"C\" __global__ void __launch_bounds__(NT, " << ki.min_blocks << ") " << name
+                << "(const SgArgs a) {\n"
+                << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
+                << "  " << T_ << "* sm = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
+                << "  const int tid = threadIdx.x;\n"
+                << "  for (long long kt = SG_K_BEGIN + (long long)blockIdx.x * " << WT << "; kt < SG_K_END; kt += (long long)gridDim.x * "
+                << WT << ") {\n"
+                << "    const int Wtt = (int)min((long long)" << WT << ", SG_K_END - kt);\n";
+            if (fusedk)
+                src << "    const long long k0 = kt;\n    const int Wt = Wtt;\n" << body << "  }\n}\n";
+            else
+                src << "    for (long long k0 = kt; k0 < kt + Wtt; k0 += " << W << ") {\n"
+                    << "      const int Wt = (int)min((long long)" << W << ", kt + Wtt - k0);\n"
+                    << body << "    }\n  }\n}\n";
+        };
+        if (WF > 0) {
+            // steady state: tiles with kt >= ksafe; stream start (firings g < 0 emit zeros): the rest
+            kernel(ki.name, fast, true);
+            ki.name_start = ki.name + "_start";
+            kernel(ki.name_start, fast_start, true);
+        } else {
+            kernel(ki.name, slow.str(), false);
+        }
         ki.source = src.str();
         return ki;
     }
@@ -802,6 +854,502 @@ private:
     std::ostringstream readers_;
     std::set<int> reader_done_;
 
+    // ======================================================= fused fast path
+    // Compute filters whose every output item is read once by a single consumer
+    // are inlined into it (SSA registers, no buffer); the rest ("roots") are
+    // materialised in shared memory, compacted to their live firings (dead-firing
+    // elimination, e.g. FIR outputs dropped by a decimator).  Sibling roots that
+    // read the same buffers form one group and share one register window;
+    // reductions (ADD, FIR) are emitted transposed across a block of B firings.
+    bool fused_ = false;
+    std::map<int, int64_t> cs_;    // phys edge -> compaction stride (live firings of the producer)
+    std::map<int, int64_t> cf0_;   // phys edge -> first live local firing of the producer
+    std::set<int> inl_;            // inlined compute nodes
+    struct FGroup {
+        std::vector<int> roots;
+        bool special = false;
+        int B = 1;
+        int level = 0;
+        std::set<int> srcs;
+        int64_t NB = 0;
+    };
+    std::vector<FGroup> fg_;
+    int flev_ = 0;
+    std::map<int, std::vector<Lin>> patterns_;   // materialised edge -> positions read (forms in "jb")
+    std::set<int> full_read_;                    // edges read densely (stores, frame FIRs)
+    std::map<int, int64_t> NL_;                  // root -> live firings per fast tile
+    std::vector<char> inpart_v_;
+
+    struct Sym {
+        bool dry = true;
+        std::ostringstream* os = nullptr;
+        std::map<std::string, std::string> loads;
+        std::map<std::string, std::vector<std::string>> firings;
+        std::map<int, std::set<std::string>> touched;
+        std::map<int, std::vector<Lin>> reads;
+        int64_t nloads = 0, flops = 0;
+        bool runtime = false;
+        int* nv = nullptr;
+        std::string ind = "        ";
+        bool guarded = false;                      // stream-start variant: firings g < 0 emit zeros
+        std::map<int, int64_t> node_flops, node_firings;
+    };
+    int nvar_ = 0;
+
+    bool in_part(int v) const { return v >= 0 && inpart_v_[v]; }
+    bool compute_node(int v) const { return in_part(v) && !is_view_node(f_.nodes[v]); }
+    bool special(int v) const { return f_.nodes[v].type == N_FILTER && f_.nodes[v].kind == SG_K_BEAM_FIR; }
+    // edge whose producer is not inlined: a shared-memory buffer in the fused layout
+    bool materialised(int e) const {
+        if (!R_.phys(e)) return false;
+        int s = f_.edges[e].src;
+        return s < 0 || !in_part(s) || !inl_.count(s);
+    }
+    void consumers_of(int e, std::set<int>& comp, bool& boundary) const {
+        const Edge& ed = f_.edges[e];
+        if (ed.dst < 0 || !in_part(ed.dst)) { boundary = true; return; }
+        const Node& w = f_.nodes[ed.dst];
+        if (is_view_node(w)) { for (int o : w.out) consumers_of(o, comp, boundary); return; }
+        comp.insert(ed.dst);
+    }
+    void sources_of(int e, std::set<int>& out) const {
+        if (R_.phys(e)) {
+            if (materialised(e)) { out.insert(e); return; }
+            sources_of(f_.nodes[f_.edges[e].src].in[0], out);
+            return;
+        }
+        for (int i : f_.nodes[f_.edges[e].src].in) sources_of(i, out);
+    }
+    std::string zero() const { return "(" + T_ + ")0"; }
+    static bool is_zero(const std::string& x) { return x == "0"; }
+
+    std::string sym_value(Sym& c, int e, const Lin& pos) {
+        Ref r = R_.resolve(e, pos);
+        if (r.k == Ref::ZERO) return "0";
+        if (r.k == Ref::RUNTIME) { c.runtime = true; return "0"; }
+        int pe = r.edge;
+        const Edge& ed = f_.edges[pe];
+        if (materialised(pe)) {
+            c.reads[pe].push_back(r.pos);
+            std::string key = std::to_string(pe) + "@" + r.pos.str();
+            auto it = c.loads.find(key);
+            if (it != c.loads.end()) return it->second;
+            c.nloads++;
+            std::string name = "l" + std::to_string((*c.nv)++);
+            if (!c.dry) *c.os << c.ind << "const " << T_ << " " << name << " = sm[" << buf_index(pe, r.pos).str() << "];\n";
+            c.loads[key] = name;
+            return name;
+        }
+        const Node& w = f_.nodes[ed.src];
+        Lin q = r.pos.plus(-ed.pre);
+        if (!q.divisible(w.push)) { c.runtime = true; return "0"; }
+        Lin fw = q.divf(w.push);
+        int64_t j = q.modc(w.push);
+        auto outs = sym_firing(c, ed.src, fw);
+        return outs[j];
+    }
+    std::vector<std::string> sym_firing(Sym& c, int v, const Lin& lf) {
+        std::string key = std::to_string(v) + ":" + lf.str();
+        auto it = c.firings.find(key);
+        if (it != c.firings.end()) return it->second;
+        c.touched[v].insert(key);
+        const Node& n = f_.nodes[v];
+        std::vector<std::string> x(n.peek);
+        int64_t use = n.kind == SG_K_FIR ? n.iv[0] : n.peek;
+        for (int64_t i = 0; i < use; i++) x[i] = sym_value(c, n.in[0], lf.scaled(n.pop).plus(i));
+        for (int64_t i = use; i < n.peek; i++) x[i] = "0";
+        std::vector<std::string> y(n.push);
+        for (auto& s : y) s = "y" + std::to_string((*c.nv)++);
+        std::ostringstream& o = *c.os;
+        const int64_t flops_before = c.flops;
+        c.node_firings[v]++;
+        if (n.kind == SG_K_FIR) {
+            int64_t nz = 0;
+            for (int64_t i = 0; i < n.iv[0]; i++) if (!is_zero(x[i])) nz++;
+            c.flops += 2 * nz;
+            if (nz == 0) { y[0] = "0"; }
+            else if (!c.dry) {
+                o << c.ind << "float " << y[0] << " = 0.0f;\n";
+                for (int64_t i = 0; i < n.iv[0]; i++)
+                    if (!is_zero(x[i])) o << c.ind << y[0] << " = fmaf(" << x[i] << ", " << hexf(n.fv[i]) << ", " << y[0] << ");\n";
+            }
+        } else if (n.kind == SG_K_ADD) {
+            c.flops += n.iv[0];
+            if (!c.dry) {
+                o << c.ind << T_ << " " << y[0] << " = " << zero() << ";\n";
+                for (int64_t i = 0; i < n.iv[0]; i++) {
+                    if (is_zero(x[i])) continue;
+                    if (T_ == "float") o << c.ind << y[0] << " = " << y[0] << " + " << x[i] << ";\n";
+                    else o << c.ind << y[0] << " = (int)((unsigned)" << y[0] << " + (unsigned)" << x[i] << ");\n";
+                }
+            }
+        } else {
+            int64_t a, b2, d;
+            node_work(f_, v, a, b2, d);
+            c.flops += n.rep ? a / n.rep : 0;
+            if (!c.dry) {
+                o << c.ind << T_ << " ";
+                for (size_t jj = 0; jj < y.size(); jj++) o << (jj ? ", " : "") << y[jj];
+                o << ";\n" << c.ind << "{ const " << T_ << " x_[" << n.peek << "] = {";
+                for (int64_t i = 0; i < n.peek; i++) o << (i ? ", " : "") << (is_zero(x[i]) ? zero() : x[i]);
+                o << "}; " << T_ << " y_[" << n.push << "]; " << work_call(v);
+                for (size_t jj = 0; jj < y.size(); jj++) o << " " << y[jj] << " = y_[" << jj << "];";
+                o << " }\n";
+            }
+        }
+        c.node_flops[v] += c.flops - flops_before;
+        if (c.guarded && !c.dry)
+            for (auto& yy : y)
+                if (!is_zero(yy))
+                    o << c.ind << yy << " = (k0 * " << n.rep << "LL + " << lf.str() << " < 0) ? " << zero() << " : " << yy << ";\n";
+        c.firings[key] = y;
+        return y;
+    }
+    int64_t root_S(int r) const { auto it = cs_.find(f_.nodes[r].out[0]); return it == cs_.end() ? 1 : it->second; }
+    int64_t root_F0L(int r) const {
+        int e = f_.nodes[r].out[0];
+        auto it = cf0_.find(e);
+        return it == cf0_.end() ? f_.nodes[r].ninit - f_.nodes[r].halo : it->second;
+    }
+    // One block of a group: roots' live firings F0L + S*(jb*B + beta), beta < B.
+    void sym_block(Sym& c, const FGroup& g, bool emit_stores) {
+        std::ostringstream& o = *c.os;
+        for (int r : g.roots) {
+            const Node& n = f_.nodes[r];
+            const int64_t S = root_S(r), F0L = root_F0L(r), B = g.B;
+            std::vector<Lin> lf(B);
+            for (int64_t be = 0; be < B; be++) lf[be] = Lin::v("jb", S * B, F0L + S * be);
+            std::vector<std::vector<std::string>> outs(B);
+            if (n.kind == SG_K_FIR || (n.kind == SG_K_ADD && T_ == "float")) {
+                const bool fir = n.kind == SG_K_FIR;
+                const int64_t terms = fir ? n.iv[0] : n.iv[0];
+                std::vector<std::string> acc(B);
+                for (int64_t be = 0; be < B; be++) {
+                    acc[be] = "a" + std::to_string((*c.nv)++);
+                    if (!c.dry) o << c.ind << "float " << acc[be] << " = 0.0f;\n";
+                }
+                c.node_firings[r] += B;
+                for (int64_t i = 0; i < terms; i++)
+                    for (int64_t be = 0; be < B; be++) {
+                        std::string x = sym_value(c, n.in[0], lf[be].scaled(n.pop).plus(i));
+                        if (is_zero(x)) continue;
+                        c.flops += fir ? 2 : 1;
+                        c.node_flops[r] += fir ? 2 : 1;
+                        if (c.dry) continue;
+                        if (fir) o << c.ind << acc[be] << " = fmaf(" << x << ", " << hexf(n.fv[i]) << ", " << acc[be] << ");\n";
+                        else o << c.ind << acc[be] << " = " << acc[be] << " + " << x << ";\n";
+                    }
+                for (int64_t be = 0; be < B; be++) outs[be] = {acc[be]};
+            } else {
+                for (int64_t be = 0; be < B; be++) outs[be] = sym_firing(c, r, lf[be]);
+            }
+            if (c.dry || !emit_stores) continue;
+            const int e = n.out[0];
+            for (int64_t be = 0; be < B; be++)
+                for (int64_t j = 0; j < n.push; j++) {
+                    std::string val = is_zero(outs[be][j]) ? zero() : outs[be][j];
+                    if (c.guarded && !is_zero(outs[be][j]))
+                        val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[be].str() + " < 0) ? " + zero() + " : " + val + ")";
+                    o << c.ind << "if (jb * " << B << " + " << be << " < NL" << r << ") sm[" << off_.at(e) << " + (jb * " << B
+                      << " + " << be << ") * " << n.push << " + " << j << "] = " << val << ";\n";
+                }
+        }
+    }
+    bool dry_ok(const FGroup& g, Sym& c) {
+        c = Sym();
+        c.dry = true;
+        std::ostringstream sink;
+        c.os = &sink;
+        c.nv = &nvar_;
+        sym_block(c, g, false);
+        return !c.runtime;
+    }
+    void fused_analyze() {
+        inpart_v_.assign(f_.nodes.size(), 0);
+        for (int v : nodes_) inpart_v_[v] = 1;
+        inl_.clear();
+        cs_.clear();
+        cf0_.clear();
+        patterns_.clear();
+        full_read_.clear();
+        fg_.clear();
+        // ---- inline decisions, consumers first
+        for (auto it = nodes_.rbegin(); it != nodes_.rend(); ++it) {
+            int u = *it;
+            if (!compute_node(u) || special(u)) continue;
+            std::set<int> comp;
+            bool boundary = false;
+            consumers_of(f_.nodes[u].out[0], comp, boundary);
+            if (boundary || comp.size() != 1) continue;
+            int v = *comp.begin();
+            if (special(v)) continue;
+            inl_.insert(u);
+            FGroup g;
+            g.roots = {v};
+            bool ok = false;
+            int Bn = 0;
+            Sym c;
+            for (int B : {1, 2, 4, 8, 16, 32, 64}) {
+                g.B = B;
+                if (dry_ok(g, c)) { Bn = B; ok = true; break; }
+            }
+            if (!ok) { inl_.erase(u); continue; }
+            g.B = std::max(Bn, 8);
+            if (!dry_ok(g, c)) g.B = Bn, dry_ok(g, c);
+            int64_t c1 = c.touched[u].size();
+            g.B *= 16;
+            if (!dry_ok(g, c)) { inl_.erase(u); continue; }
+            int64_t cK = c.touched[u].size();
+            if (!(c1 * 16 <= 1.25 * cK)) inl_.erase(u);
+        }
+        // ---- roots, their sources and levels
+        std::vector<int> roots;
+        for (int v : nodes_) if (compute_node(v) && !inl_.count(v)) roots.push_back(v);
+        std::map<int, int> lvl;
+        std::map<int, std::set<int>> srcs;
+        flev_ = 0;
+        for (int r : roots) {
+            sources_of(f_.nodes[r].in[0], srcs[r]);
+            int L = 0;
+            for (int e : srcs[r]) {
+                int sp = f_.edges[e].src;
+                if (sp >= 0 && in_part(sp)) L = std::max(L, lvl.at(sp));
+            }
+            lvl[r] = L + 1;
+            flev_ = std::max(flev_, L + 1);
+        }
+        // stores and frame FIRs read densely
+        for (int e : outs_) {
+            std::set<int> s2;
+            if (R_.phys(e)) s2.insert(e); else sources_of(e, s2);
+            if (!R_.phys(e)) {
+                // views between the buffer and the store: positions may be strided; keep dense
+            }
+            for (int x : s2) full_read_.insert(x);
+        }
+        for (int r : roots) if (special(r)) for (int e : srcs[r]) full_read_.insert(e);
+        // ---- levels from the top: live strides, groups, block sizes, read patterns
+        for (int L = flev_; L >= 1; L--) {
+            std::vector<int> here;
+            for (int r : roots) if (lvl[r] == L) here.push_back(r);
+            for (int r : here) {
+                const Node& n = f_.nodes[r];
+                const int e = n.out[0];
+                const Edge& ed = f_.edges[e];
+                int64_t S = 1, rho = 0;
+                auto pit = patterns_.find(e);
+                if (!special(r) && n.push == 1 && !full_read_.count(e) && pit != patterns_.end() && !pit->second.empty()) {
+                    int64_t g = 0, c0 = pit->second[0].c;
+                    for (auto& lp : pit->second) {
+                        for (auto& t : lp.t) g = std::gcd(g, std::llabs(t.second));
+                        g = std::gcd(g, std::llabs(lp.c - c0));
+                    }
+                    if (g > 1 && n.rep % g == 0) { S = g; rho = fmodp(c0 - ed.pre, S); }
+                }
+                const int64_t F0 = n.ninit - n.halo;
+                cs_[e] = S;
+                cf0_[e] = F0 + fmodp(rho - F0, S);
+            }
+            // group siblings: same rep, stride, sources (non-special)
+            std::map<std::string, FGroup> bysig;
+            std::vector<FGroup> singles;
+            for (int r : here) {
+                FGroup g;
+                g.roots = {r};
+                g.level = L;
+                g.srcs = srcs[r];
+                if (special(r)) { g.special = true; singles.push_back(g); continue; }
+                std::ostringstream sig;
+                sig << f_.nodes[r].rep << "/" << root_S(r) << "/" << f_.nodes[r].push << "/" << f_.nodes[r].halo << "/"
+                    << f_.nodes[r].ninit << ":";
+                for (int e : srcs[r]) sig << e << ",";
+                auto it = bysig.find(sig.str());
+                if (it == bysig.end()) bysig[sig.str()] = g;
+                else it->second.roots.push_back(r);
+            }
+            for (auto& kv : bysig) singles.push_back(kv.second);
+            for (auto& g : singles) {
+                if (!g.special) {
+                    Sym c;
+                    int B0 = 0;
+                    for (int B : {1, 2, 4, 8, 16, 32, 64}) {
+                        g.B = B;
+                        if (dry_ok(g, c)) { B0 = B; break; }
+                    }
+                    if (!B0) throw FusedFail();
+                    g.B = B0;
+                    dry_ok(g, c);
+                    while (g.B * 2 <= 16) {
+                        FGroup h = g;
+                        h.B = g.B * 2;
+                        Sym c2;
+                        if (!dry_ok(h, c2) || c2.flops > 2048 || c2.nloads > 96) break;
+                        g.B = h.B;
+                        c = c2;
+                    }
+                    dry_ok(g, c);
+                    for (auto& kv : c.reads) for (auto& lp : kv.second) patterns_[kv.first].push_back(lp);
+                }
+                fg_.push_back(g);
+            }
+        }
+        std::stable_sort(fg_.begin(), fg_.end(), [](const FGroup& a, const FGroup& b) { return a.level < b.level; });
+    }
+    void fused_layout(int W) {
+        off_.clear();
+        wb_.clear();
+        size_.clear();
+        NL_.clear();
+        struct Buf { int e; int64_t size; int birth, death; };
+        std::map<int, Buf> bufs;
+        auto note = [&](int e, int64_t size, int birth) {
+            if (!bufs.count(e)) bufs[e] = {e, size, birth, birth};
+        };
+        for (size_t i = 0; i < ins_.size(); i++) {
+            int e = ins_[i];
+            int64_t lo, ex;
+            edge_window(f_, e, lo, ex);
+            wb_[e] = lo;
+            note(e, f_.edges[e].per_iter * W + ex, 0);
+        }
+        for (auto& g : fg_) {
+            for (int r : g.roots) {
+                const Node& n = f_.nodes[r];
+                const int e = n.out[0];
+                const int64_t S = root_S(r), F0 = n.ninit - n.halo, F0L = root_F0L(r);
+                const int64_t end = F0 + n.halo + (int64_t)W * n.rep;  // exclusive
+                const int64_t NL = end > F0L ? (end - 1 - F0L) / S + 1 : 0;
+                NL_[r] = NL;
+                wb_[e] = f_.edges[e].pre + F0L * n.push;
+                note(e, NL * n.push, g.level);
+            }
+        }
+        for (auto& g : fg_) {
+            int64_t nb = 0;
+            for (int r : g.roots) nb = std::max(nb, (NL_[r] + g.B - 1) / g.B);
+            g.NB = g.special ? 0 : nb;
+        }
+        // extents read by the first and last block of every group; liveness
+        for (auto& g : fg_) {
+            for (int e : g.srcs) if (bufs.count(e)) bufs[e].death = std::max(bufs[e].death, g.level);
+            if (g.special || g.NB == 0) continue;
+            Sym c;
+            dry_ok(g, c);
+            for (auto& kv : c.reads) {
+                int e = kv.first;
+                if (!bufs.count(e)) continue;
+                for (auto& lp : kv.second)
+                    for (int64_t jb : {(int64_t)0, g.NB - 1}) {
+                        int64_t pos = lp.c + lp.coef("jb") * jb;
+                        int64_t idx;
+                        auto it = cs_.find(e);
+                        if (it != cs_.end() && it->second > 1) {
+                            int64_t q = pos - f_.edges[e].pre - cf0_.at(e);
+                            if (fmodp(q, it->second) != 0) throw FusedFail();
+                            idx = fdiv(q, it->second);
+                        } else {
+                            idx = pos - wb_.at(e);
+                        }
+                        if (idx < 0) throw FusedFail();
+                        bufs[e].size = std::max(bufs[e].size, idx + 1);
+                    }
+            }
+        }
+        for (int e : outs_) {
+            std::set<int> s2;
+            if (R_.phys(e)) s2.insert(e); else sources_of(e, s2);
+            for (int x : s2) if (bufs.count(x)) bufs[x].death = flev_ + 1;
+        }
+        std::vector<Buf> list;
+        for (auto& kv : bufs) list.push_back(kv.second);
+        std::stable_sort(list.begin(), list.end(), [](const Buf& a, const Buf& b) { return a.size > b.size; });
+        std::vector<Buf> placed;
+        int64_t top = 0;
+        for (auto& b : list) {
+            int64_t sz = (b.size + 3) / 4 * 4;
+            std::vector<std::pair<int64_t, int64_t>> busy;
+            for (auto& q : placed)
+                if (!(q.death < b.birth || b.death < q.birth))
+                    busy.push_back({off_[q.e], off_[q.e] + (q.size + 3) / 4 * 4});
+            std::sort(busy.begin(), busy.end());
+            int64_t o = 0;
+            for (auto& iv : busy) {
+                if (o + sz <= iv.first) break;
+                o = std::max(o, iv.second);
+            }
+            off_[b.e] = o;
+            size_[b.e] = b.size;
+            top = std::max(top, o + sz);
+            placed.push_back(b);
+        }
+        smem_bytes_ = (size_t)std::max<int64_t>(top, 4) * 4;
+    }
+    // Fused tile body for a runtime Wt <= W.  guarded: the stream-start variant.
+    std::string fused_emit(int W, bool guarded) {
+        std::ostringstream b;
+        emit_loads(b);
+        for (int L = 1; L <= flev_; L++) {
+            b << "    // ---- fused level " << L << "\n";
+            int64_t rot = 0;
+            for (auto& g : fg_) {
+                if (g.level != L) continue;
+                if (g.special) {
+                    for (int r : g.roots) {
+                        emit_stage(b, r, rot);
+                        rot += f_.nodes[r].halo + (int64_t)W * f_.nodes[r].rep;
+                    }
+                    continue;
+                }
+                b << "    { // group of " << g.roots.size() << " root(s) [" << kind_name(f_.nodes[g.roots[0]].kind)
+                  << "], B = " << g.B << ", blocks per full tile = " << g.NB << "\n";
+                b << "      int NBg = 0;\n";
+                for (int r : g.roots) {
+                    const Node& n = f_.nodes[r];
+                    const int64_t S = root_S(r), F0 = n.ninit - n.halo, F0L = root_F0L(r);
+                    b << "      const int NL" << r << " = (" << F0 + n.halo - 1 - F0L << " + Wt * " << n.rep << ") / " << S
+                      << " + 1;\n"
+                      << "      NBg = max(NBg, (NL" << r << " + " << g.B - 1 << ") / " << g.B << ");\n";
+                }
+                b << "      int jb = tid - " << rot % NT_ << "; if (jb < 0) jb += NT;\n"
+                  << "      for (; jb < NBg; jb += NT) {\n";
+                Sym c;
+                c.dry = false;
+                c.os = &b;
+                c.nv = &nvar_;
+                c.guarded = guarded;
+                sym_block(c, g, true);
+                if (c.runtime) throw FusedFail();
+                b << "      }\n    }\n";
+                rot += g.NB;
+            }
+            b << "    __syncthreads();\n";
+        }
+        emit_stores(b);
+        b << "    __syncthreads();\n";
+        return b.str();
+    }
+    // Algorithmic fp32 work per iteration of the fused plan: dead firings and zero
+    // taps removed, recomputed (halo / inlining overlap) firings not counted.
+    int64_t fused_flops_per_iter() {
+        double tot = 0;
+        for (auto& g : fg_) {
+            if (g.special) {
+                for (int r : g.roots) { int64_t a, b2, d; node_work(f_, r, a, b2, d); tot += a; }
+                continue;
+            }
+            Sym c;
+            dry_ok(g, c);
+            for (auto& kv : c.node_flops) {
+                int v = kv.first;
+                int64_t nf = c.node_firings[v];
+                if (nf <= 0) continue;
+                const Node& n = f_.nodes[v];
+                int64_t S = inl_.count(v) ? 1 : root_S(v);
+                tot += (double)kv.second / nf * (double)n.rep / S;
+            }
+        }
+        return (int64_t)(tot + 0.5);
+    }
     int producer_level(int e) {
         const Edge& ed = f_.edges[e];
         if (!R_.phys(e)) throw Error(SG_E_UNSUPPORTED, "internal");
@@ -950,15 +1498,27 @@ private:
         for (int d : deps) gen_reader(d);  // callees first
         readers_ << s.str();
     }
+    struct FusedFail {};
+    // shared-memory index of position `pos` of physical edge e in the current layout
+    Lin buf_index(int e, const Lin& pos) {
+        auto it = cs_.find(e);
+        if (fused_ && it != cs_.end() && it->second > 1) {
+            const Edge& ed = f_.edges[e];
+            Lin q = pos.plus(-(ed.pre + cf0_.at(e)));
+            if (!q.divisible(it->second) || q.modc(it->second) != 0) throw FusedFail();
+            return q.divf(it->second).plus(off_.at(e));
+        }
+        return pos.plus(off_.at(e) - wb_.at(e));
+    }
     std::string read_expr(int e, const Lin& pos) {
         Ref r = R_.resolve(e, pos);
         if (r.k == Ref::ZERO) return "(" + T_ + ")0";
         if (r.k == Ref::RUNTIME) {
+            if (fused_) throw FusedFail();
             gen_reader(r.edge);
             return rd_name(r.edge) + "(sm, " + r.pos.str() + ")";
         }
-        int64_t k = off_.at(r.edge) - wb_.at(r.edge);
-        return "sm[" + r.pos.plus(k).str() + "]";
+        return "sm[" + buf_index(r.edge, r.pos).str() + "]";
     }
     void emit_loads(std::ostringstream& b) {
         for (size_t i = 0; i < ins_.size(); i++) {
@@ -1163,7 +1723,9 @@ KernelInfo generate_kernel(const Flat& f, const std::vector<int>& nodes, int par
         return g.run(opt);
     }
     StageGen g(f, nodes, part_id);
-    return g.run(opt);
+    CodegenOpts o2 = opt;
+    if (mode == 3) o2.mode = -2;  // staged without the fused fast path (general path only)
+    return g.run(o2);
 }
 
 }  // namespace sg

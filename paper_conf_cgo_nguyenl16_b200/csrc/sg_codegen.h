@@ -38,6 +38,10 @@ struct KernelInfo {
     int64_t pin = 0, pout = 0, off_in = 0, off_out = 0;
     int threads_sync = 0, tile_sync = 0;
     size_t smem_sync = 0;
+    bool fused = false;              // staged mode: fused fast path present
+    int64_t flops_exec_per_iter = -1;  // fused: algorithmic flops after dead/zero pruning (no recompute)
+    std::string name_start;          // staged fused: stream-start variant (tiles with k0 < ksafe)
+    int64_t ksafe = 0;
 };
 
 // Boundary input / output edges of a node set (sorted, deterministic).

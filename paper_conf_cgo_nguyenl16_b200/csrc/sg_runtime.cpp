@@ -233,6 +233,8 @@ void ensure_module(CompiledKernel& ck, int dev) {
     setup(ck.ki.name, ck.ki.threads, ck.ki.smem, ck.fn[dev], ck.max_blocks_per_sm[dev]);
     if (ck.ki.mode == 1 && ck.ki.has_tma)
         setup(ck.ki.name_sync, ck.ki.threads_sync, ck.ki.smem_sync, ck.fn_sync[dev], ck.max_blocks_sync[dev]);
+    if (ck.ki.mode == 2 && !ck.ki.name_start.empty())
+        setup(ck.ki.name_start, ck.ki.threads, ck.ki.smem, ck.fn_sync[dev], ck.max_blocks_sync[dev]);
 }
 
 // 2-D row tensor map: dims {P items, rows}, box {P, box_rows}, 128B swizzle.
@@ -305,12 +307,27 @@ int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int
                              (unsigned)ki.smem_sync, (CUstream)stream, params, nullptr));
         return 1;
     }
+    int64_t launches = 0;
+    if (ki.mode == 2 && !ki.name_start.empty() && kb < ki.ksafe) {
+        // stream-start tiles (firings g < 0 must emit zeros): the guarded variant
+        int64_t ks = std::min(ke, kb + ((ki.ksafe - kb + ki.tile - 1) / ki.tile) * ki.tile);
+        std::vector<int64_t> v2 = v;
+        v2[v2.size() - 1] = ks;
+        int64_t tiles = (ks - kb + ki.tile - 1) / ki.tile;
+        void* params[] = {v2.data()};
+        SG_CU(cuLaunchKernel(ck.fn_sync[dev], (unsigned)tiles, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
+                             (CUstream)stream, params, nullptr));
+        launches++;
+        kb = ks;
+        v[v.size() - 2] = kb;
+        if (ke <= kb) return launches;
+    }
     int64_t tiles = (ke - kb + ki.tile - 1) / ki.tile;
     int64_t grid = std::min<int64_t>(tiles, (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev]);
     void* params[] = {v.data()};
     SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
                          (CUstream)stream, params, nullptr));
-    return 1;
+    return launches + 1;
 }
 }  // namespace
 

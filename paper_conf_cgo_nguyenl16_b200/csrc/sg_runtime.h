@@ -18,7 +18,7 @@ struct CompiledKernel {
     // per physical device (index = device ordinal)
     std::vector<CUmodule> mod;
     std::vector<CUfunction> fn;            // main variant (TMA pipeline when ki.has_tma)
-    std::vector<CUfunction> fn_sync;       // register mode: synchronous fallback
+    std::vector<CUfunction> fn_sync;       // register mode: synchronous fallback; staged: stream-start variant
     std::vector<int> max_blocks_per_sm;
     std::vector<int> max_blocks_sync;
 };

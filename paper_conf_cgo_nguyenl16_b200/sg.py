@@ -62,7 +62,9 @@ class PlanInfo(ctypes.Structure):
                 ("partition_time", ctypes.POINTER(ctypes.c_double)),
                 ("partition_mode", ctypes.POINTER(ctypes.c_int32)), ("est_tmax", ctypes.c_double),
                 ("input_device", ctypes.c_int32), ("output_device", ctypes.c_int32),
-                ("iters_per_fragment", ctypes.c_int64), ("ilp_optimal", ctypes.c_int32)]
+                ("iters_per_fragment", ctypes.c_int64), ("ilp_optimal", ctypes.c_int32),
+                ("flops_per_iter_written", ctypes.c_double), ("flops_per_iter_pruned", ctypes.c_double),
+                ("intops_per_iter", ctypes.c_int64)]
 
 
 def lib():
@@ -206,6 +208,8 @@ class Plan:
                 arr = _i32arr(v)
                 self._keep.append(arr)
                 o.devices = arr
+            elif k == "codegen_mode" and isinstance(v, str):
+                o.codegen_mode = {"auto": 0, "register": 1, "staged": 2, "general": 3}[v]
             elif k == "partitioner" and isinstance(v, str):
                 o.partitioner = {"algorithm1": 0, "single": 1, "per_filter": 2}[v]
             else:
@@ -233,6 +237,8 @@ class Plan:
             "partition_mode": [i.partition_mode[k] for k in range(P)],
             "est_tmax": i.est_tmax, "input_device": i.input_device, "output_device": i.output_device,
             "iters_per_fragment": i.iters_per_fragment, "ilp_optimal": bool(i.ilp_optimal),
+            "flops_per_iter_written": i.flops_per_iter_written, "flops_per_iter_pruned": i.flops_per_iter_pruned,
+            "intops_per_iter": i.intops_per_iter,
         }
 
     def input_items(self, n: int) -> int:
