@@ -3,12 +3,12 @@
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--config NAME] [--impl sg|reference]
 
-One step = one sg_run() over the whole workload (all of SURVEY.md 8(a)'s timed
+One step = one sg_run() over the whole workload (replayed as a CUDA graph) (all of SURVEY.md 8(a)'s timed
 rows: tile loads, filter execution, stores; plus boundary streams when the plan
 has several partitions/GPUs).  Default workload: BASELINE.json configs[1],
 BitonicSort 32-key int32, 2^20 iterations, one GPU.  Inputs resident in HBM;
-L2 flushed (256 MiB overwrite with our sg_flush_l2 kernel) before every timed
-step, outside the per-step CUDA-event window.  Under torchrun (N > 1) every rank
+L2 flushed (256 MiB write + read-back with our sg_flush_l2 kernels) before every
+timed step, outside the per-step CUDA-event window.  Under torchrun (N > 1) every rank
 runs an independent replica on its own GPU ("replicas only" for this HBM-bound
 graph); value = all ranks' iterations / max-over-ranks time.
 
@@ -160,6 +160,7 @@ def main():
     ap.add_argument("--iters", type=int, default=0, help="override iterations per step")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-flush", action="store_true")
+    ap.add_argument("--eager", action="store_true", help="launch sg_run every step instead of replaying a CUDA graph")
     args = ap.parse_args()
     if args.warmup < 3:
         args.warmup = 3
@@ -195,6 +196,29 @@ def main():
         plan.run(x, n, y, stream)
     launches_per_step = plan.last_launch_count()
     torch.cuda.synchronize()
+    # CUDA graph of one sg_run (the C ABI call enqueues only kernels and events on the
+    # capturing stream); replaying it removes host launch gaps from the timed window.
+    graph = None
+    if not args.eager:
+        try:
+            gs = torch.cuda.Stream()
+            graph = torch.cuda.CUDAGraph()
+            with torch.cuda.graph(graph, stream=gs):
+                plan.run(x, n, y, torch.cuda.current_stream())
+            torch.cuda.synchronize()
+            for _ in range(args.warmup):
+                graph.replay()
+            torch.cuda.synchronize()
+        except Exception as exc:  # capture not possible (e.g. multi-GPU plan): eager launches
+            print(f"[bench] CUDA graph capture failed ({exc}); eager launches", file=sys.stderr)
+            graph = None
+            torch.cuda.synchronize()
+
+    def step():
+        if graph is not None:
+            graph.replay()
+        else:
+            plan.run(x, n, y, stream)
 
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
     sampler = ClockSampler(local)
@@ -208,7 +232,7 @@ def main():
         if not args.no_flush:
             sg.flush_l2(flush, stream.cuda_stream)
         ev[k][0].record(stream)
-        plan.run(x, n, y, stream)
+        step()
         ev[k][1].record(stream)
     torch.cuda.synchronize()
     wall = time.perf_counter() - wall0
@@ -284,13 +308,14 @@ def main():
             "vs_baseline": None, "dtype": "i32" if prog.dtype == "i32" else "f32", "data": "synthetic",
             "config": {"workload": name, "desc": W["desc"], "iters_per_step": n,
                        "items_per_s_out": value * info["out_per_iter"],
-                       "l2": "flushed before every step (256 MiB sg_flush_l2), outside the event window"
+                       "l2": "flushed before every step (256 MiB sg_flush_l2: write + read back), outside the event window"
                        if not args.no_flush else "not flushed",
                        "parallelism": f"replicas x{world}" if world > 1 else "1 GPU, 1 partition",
                        "partitions": info["n_partitions"], "partition_mode": info["partition_mode"],
+                       "launch": "CUDA graph replay of one sg_run" if graph is not None else "eager sg_run",
                        "wall_s": wall},
             "roofline": roof, "cpu_baseline": cb, "e2e": e2e,
-            "gpu_launches": args.steps * (launches_per_step + (0 if args.no_flush else 1)),
+            "gpu_launches": args.steps * (launches_per_step + (0 if args.no_flush else 2)),
             "clocks": clocks,
         }
         print(json.dumps(line))

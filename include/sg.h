@@ -256,8 +256,9 @@ double sg_paper_model(int32_t n, const double* t, const double* f, int32_t S, in
  * bytes per iteration); returns the number of edges. */
 int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst, double* bytes);
 
-/* Benchmark hygiene: overwrite `bytes` of device scratch memory (> L2 size)
- * with an nvcc-compiled sm_100a kernel enqueued on `stream`. */
+/* Benchmark hygiene: evict L2 by overwriting `bytes` of device scratch memory
+ * (> L2 size) and reading it back (dirty lines written back before the next
+ * kernel), with nvcc-compiled sm_100a kernels enqueued on `stream`. */
 sg_status sg_flush_l2(void* scratch, int64_t bytes, void* stream);
 
 #ifdef __cplusplus

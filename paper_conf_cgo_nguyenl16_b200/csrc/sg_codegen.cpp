@@ -743,8 +743,7 @@ public:
                 fused_ = true;
                 fused_analyze();
                 size_t fb = opt.smem_budget > 0 ? (size_t)opt.smem_budget : (size_t)(110 * 1024);
-                for (int cand : {4096, 2048, 1024, 512, 256, 128, 64, 32, 16, 8, 4, 2, 1}) {
-                    if (opt.tile > 0 && cand != opt.tile) continue;
+                for (int cand : fused_tile_candidates(opt.tile)) {
                     fused_layout(cand);
                     if (smem_bytes_ <= fb) { WF = cand; break; }
                 }
@@ -862,6 +861,7 @@ private:
     // read the same buffers form one group and share one register window;
     // reductions (ADD, FIR) are emitted transposed across a block of B firings.
     bool fused_ = false;
+    std::map<int, int64_t> plP_, plQ_;  // phys edge -> planar layout: period P, row length Q (odd)
     std::map<int, int64_t> cs_;    // phys edge -> compaction stride (live firings of the producer)
     std::map<int, int64_t> cf0_;   // phys edge -> first live local firing of the producer
     std::set<int> inl_;            // inlined compute nodes
@@ -872,6 +872,7 @@ private:
         int level = 0;
         std::set<int> srcs;
         int64_t NB = 0;
+        int64_t flops_block = 0;   // dry-run work of one block (cost model)
     };
     std::vector<FGroup> fg_;
     int flev_ = 0;
@@ -1014,6 +1015,51 @@ private:
     // One block of a group: roots' live firings F0L + S*(jb*B + beta), beta < B.
     void sym_block(Sym& c, const FGroup& g, bool emit_stores) {
         std::ostringstream& o = *c.os;
+        bool all_fir = g.roots.size() > 1;
+        for (int r : g.roots) all_fir = all_fir && f_.nodes[r].kind == SG_K_FIR;
+        if (all_fir) {  // sibling FIRs: taps outer, roots and block inner -> independent chains, window loaded once
+            const int64_t B = g.B;
+            int64_t maxL = 0;
+            std::vector<std::vector<Lin>> lf(g.roots.size(), std::vector<Lin>(B));
+            std::vector<std::vector<std::string>> acc(g.roots.size(), std::vector<std::string>(B));
+            for (size_t k = 0; k < g.roots.size(); k++) {
+                int r = g.roots[k];
+                const int64_t S = root_S(r), F0L = root_F0L(r);
+                maxL = std::max<int64_t>(maxL, f_.nodes[r].iv[0]);
+                c.node_firings[r] += B;
+                for (int64_t be = 0; be < B; be++) {
+                    lf[k][be] = Lin::v("jb", S * B, F0L + S * be);
+                    acc[k][be] = "a" + std::to_string((*c.nv)++);
+                    if (!c.dry) o << c.ind << "float " << acc[k][be] << " = 0.0f;\n";
+                }
+            }
+            for (int64_t i = 0; i < maxL; i++)
+                for (size_t k = 0; k < g.roots.size(); k++) {
+                    const Node& n = f_.nodes[g.roots[k]];
+                    if (i >= n.iv[0]) continue;
+                    for (int64_t be = 0; be < B; be++) {
+                        std::string x = sym_value(c, n.in[0], lf[k][be].scaled(n.pop).plus(i));
+                        if (is_zero(x)) continue;
+                        c.flops += 2;
+                        c.node_flops[g.roots[k]] += 2;
+                        if (!c.dry) o << c.ind << acc[k][be] << " = fmaf(" << x << ", " << hexf(n.fv[i]) << ", " << acc[k][be] << ");\n";
+                    }
+                }
+            if (c.dry || !emit_stores) return;
+            for (size_t k = 0; k < g.roots.size(); k++) {
+                const Node& n = f_.nodes[g.roots[k]];
+                const int r = g.roots[k];
+                for (int64_t be = 0; be < B; be++) {
+                    std::string val = acc[k][be];
+                    if (c.guarded)
+                        val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[k][be].str() + " < 0) ? " + zero() + " : " + val + ")";
+                    Lin pos = lf[k][be].scaled(n.push).plus(f_.edges[n.out[0]].pre);
+                    o << c.ind << "if (jb * " << B << " + " << be << " < NL" << r << ") sm["
+                      << buf_index(n.out[0], pos).str() << "] = " << val << ";\n";
+                }
+            }
+            return;
+        }
         for (int r : g.roots) {
             const Node& n = f_.nodes[r];
             const int64_t S = root_S(r), F0L = root_F0L(r), B = g.B;
@@ -1050,8 +1096,9 @@ private:
                     std::string val = is_zero(outs[be][j]) ? zero() : outs[be][j];
                     if (c.guarded && !is_zero(outs[be][j]))
                         val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[be].str() + " < 0) ? " + zero() + " : " + val + ")";
-                    o << c.ind << "if (jb * " << B << " + " << be << " < NL" << r << ") sm[" << off_.at(e) << " + (jb * " << B
-                      << " + " << be << ") * " << n.push << " + " << j << "] = " << val << ";\n";
+                    Lin pos = lf[be].scaled(n.push).plus(f_.edges[e].pre + j);
+                    o << c.ind << "if (jb * " << B << " + " << be << " < NL" << r << ") sm[" << buf_index(e, pos).str()
+                      << "] = " << val << ";\n";
                 }
         }
     }
@@ -1188,12 +1235,46 @@ private:
                         c = c2;
                     }
                     dry_ok(g, c);
+                    g.flops_block = c.flops + c.nloads;
                     for (auto& kv : c.reads) for (auto& lp : kv.second) patterns_[kv.first].push_back(lp);
                 }
                 fg_.push_back(g);
             }
         }
         std::stable_sort(fg_.begin(), fg_.end(), [](const FGroup& a, const FGroup& b) { return a.level < b.level; });
+        // planar layouts for buffers read by frame FIRs: period P = gcd of every reader's and
+        // writer's position strides, so that per-thread blocks of odd length hit distinct banks
+        plP_.clear();
+        std::map<int, int64_t> gP;
+        std::set<int> special_read;
+        auto acc = [&](int e, int64_t a) { gP[e] = std::gcd(gP[e], std::llabs(a)); };
+        for (auto& g : fg_) {
+            if (!g.special) continue;
+            for (int r : g.roots) {
+                const Node& n = f_.nodes[r];
+                Lin pr = Lin::v("lf", n.pop, 0);
+                pr.t.push_back({"s0", 2});
+                for (int k = 0; k < 2; k++) {
+                    Ref rf = R_.resolve(n.in[0], pr.plus(k));
+                    if (rf.k != Ref::PHYS || !materialised(rf.edge)) continue;
+                    special_read.insert(rf.edge);
+                    for (auto& t : rf.pos.t) acc(rf.edge, t.second);
+                }
+                acc(n.out[0], n.push);   // its own output: positions j*push + 2*t
+                acc(n.out[0], 2);
+            }
+        }
+        for (auto& kv : patterns_)
+            for (auto& lp : kv.second)
+                for (auto& t : lp.t) acc(kv.first, t.second);
+        for (auto& g : fg_) {
+            if (g.special) continue;
+            for (int r : g.roots) acc(f_.nodes[r].out[0], f_.nodes[r].push * root_S(r) * g.B);
+        }
+        for (int e : special_read) {
+            int64_t P = gP[e];
+            if (P > 1 && P <= 64 && (!cs_.count(e) || cs_[e] == 1)) plP_[e] = P;
+        }
     }
     void fused_layout(int W) {
         off_.clear();
@@ -1260,6 +1341,15 @@ private:
             if (R_.phys(e)) s2.insert(e); else sources_of(e, s2);
             for (int x : s2) if (bufs.count(x)) bufs[x].death = flev_ + 1;
         }
+        plQ_.clear();
+        for (auto& kv : bufs) {
+            auto it = plP_.find(kv.first);
+            if (it == plP_.end()) continue;
+            int64_t P = it->second, Q = (kv.second.size + P - 1) / P;
+            if (Q % 2 == 0) Q++;
+            plQ_[kv.first] = Q;
+            kv.second.size = P * Q;
+        }
         std::vector<Buf> list;
         for (auto& kv : bufs) list.push_back(kv.second);
         std::stable_sort(list.begin(), list.end(), [](const Buf& a, const Buf& b) { return a.size > b.size; });
@@ -1283,6 +1373,63 @@ private:
             placed.push_back(b);
         }
         smem_bytes_ = (size_t)std::max<int64_t>(top, 4) * 4;
+    }
+    // live root firings in a tile of W iterations
+    int64_t nl_of(int r, int64_t W) const {
+        const Node& n = f_.nodes[r];
+        const int64_t S = root_S(r), F0 = n.ninit - n.halo, F0L = root_F0L(r);
+        return (F0 + n.halo - 1 - F0L + W * n.rep) / S + 1;
+    }
+    // Tile sizes ordered by a cost model: per level, ceil(blocks / NT) rounds of
+    // the heaviest block, summed, per iteration; candidates include the sizes that
+    // make a group's block count a multiple of NT (no straggler round).
+    std::vector<int> fused_tile_candidates(int forced) {
+        if (forced > 0) return {forced};
+        std::set<int64_t> cand;
+        for (int64_t w = 1; w <= 4096; w *= 2) cand.insert(w);
+        for (auto& g : fg_) {
+            if (g.special) continue;
+            for (int64_t k = 1; k <= 16; k++) {
+                int64_t lo = 1, hi = 8192;  // largest W with NB_g(W) <= k*NT
+                if ((nl_of(g.roots[0], 1) + g.B - 1) / g.B > k * NT_) continue;
+                while (lo < hi) {
+                    int64_t mid = (lo + hi + 1) / 2;
+                    int64_t nb = 0;
+                    for (int r : g.roots) nb = std::max(nb, (nl_of(r, mid) + g.B - 1) / g.B);
+                    if (nb <= k * NT_) lo = mid; else hi = mid - 1;
+                }
+                if (lo >= 1 && lo <= 8192) cand.insert(lo);
+            }
+        }
+        std::vector<std::pair<double, int>> scored;
+        for (int64_t W : cand) {
+            double tile = 0;
+            for (int L = 1; L <= flev_; L++) {
+                int64_t items = 0, worst = 1;
+                for (auto& g : fg_) {
+                    if (g.level != L) continue;
+                    if (g.special) {
+                        for (int r : g.roots) {
+                            const Node& n = f_.nodes[r];
+                            int64_t per = (n.iv[2] / n.iv[1] + 3) / 4;
+                            items += (n.halo + W * n.rep) * per;
+                            worst = std::max<int64_t>(worst, 32LL * n.iv[0]);
+                        }
+                        continue;
+                    }
+                    int64_t nb = 0;
+                    for (int r : g.roots) nb = std::max(nb, (nl_of(r, W) + g.B - 1) / g.B);
+                    items += nb;
+                    worst = std::max(worst, g.flops_block);
+                }
+                tile += (double)((items + NT_ - 1) / NT_) * (double)worst + 200.0;
+            }
+            scored.push_back({tile / (double)W, (int)W});
+        }
+        std::sort(scored.begin(), scored.end());
+        std::vector<int> out;
+        for (auto& p : scored) out.push_back(p.second);
+        return out;
     }
     // Fused tile body for a runtime Wt <= W.  guarded: the stream-start variant.
     std::string fused_emit(int W, bool guarded) {
@@ -1501,6 +1648,13 @@ private:
     struct FusedFail {};
     // shared-memory index of position `pos` of physical edge e in the current layout
     Lin buf_index(int e, const Lin& pos) {
+        auto pit = plP_.find(e);
+        if (fused_ && pit != plP_.end() && pit->second > 1) {  // planar: [P][Q], Q odd
+            const int64_t P = pit->second, Q = plQ_.at(e);
+            Lin j = pos.plus(-wb_.at(e));
+            if (!j.divisible(P)) throw FusedFail();
+            return j.divf(P).plus(j.modc(P) * Q + off_.at(e));
+        }
         auto it = cs_.find(e);
         if (fused_ && it != cs_.end() && it->second > 1) {
             const Edge& ed = f_.edges[e];
@@ -1531,9 +1685,14 @@ private:
               << "      const long long gb = k0 * " << P << "LL + (" << lo << "LL) - SG_IN_BASE(" << i << ");\n"
               << "      const long long lim = SG_IN_LIMIT(" << i << ");\n"
               << "      const int n = Wt * " << P << " + " << ex << ";\n"
-              << "      " << T_ << "* s = sm + " << off_.at(e) << ";\n"
-              << "      for (int j = tid; j < n; j += NT) { const long long gi = gb + j; s[j] = (gi >= 0 && gi < lim) ? g[gi] : ("
-              << T_ << ")0; }\n"
+              << "      " << T_ << "* s = sm + " << off_.at(e) << ";\n";
+            auto pit = plP_.find(e);
+            std::string dst = "s[j]";
+            if (fused_ && pit != plP_.end())
+                dst = "s[(j % " + std::to_string(pit->second) + ") * " + std::to_string(plQ_.at(e)) + " + j / " +
+                      std::to_string(pit->second) + "]";
+            b << "      for (int j = tid; j < n; j += NT) { const long long gi = gb + j; " << dst
+              << " = (gi >= 0 && gi < lim) ? g[gi] : (" << T_ << ")0; }\n"
               << "    }\n";
         }
         b << "    __syncthreads();\n";
@@ -1542,7 +1701,13 @@ private:
     int store_period(int e, int64_t lo) {
         for (int per : {1, 2, 4, 8, 16, 32, 64}) {
             bool ok = true;
-            for (int c = 0; c < per && ok; c++) ok = R_.resolve(e, Lin::v("q", per, lo + c)).k != Ref::RUNTIME;
+            for (int c = 0; c < per && ok; c++) {
+                Ref r = R_.resolve(e, Lin::v("q", per, lo + c));
+                ok = r.k != Ref::RUNTIME;
+                if (ok && r.k == Ref::PHYS && fused_) {
+                    try { buf_index(r.edge, r.pos); } catch (const FusedFail&) { ok = false; }
+                }
+            }
             if (ok) return per;
         }
         return 1;
@@ -1665,7 +1830,7 @@ private:
     void emit_beam_fir(std::ostringstream& b, int v, int64_t F0, int64_t rot) {
         const Node& n = f_.nodes[v];
         int64_t L = n.iv[0], DEC = n.iv[1], FR = n.iv[2], OUT = FR / DEC;
-        int64_t B = 4, TC = 1;
+        int64_t B = 3, TC = 1;  // odd block: lanes 3*DEC samples apart -> distinct banks in planar buffers
         for (int64_t c : {16, 8, 4, 2, 1})
             if (L % c == 0) { TC = c; break; }
         int64_t NB = (OUT + B - 1) / B, NWIN = (B - 1) * DEC + TC;
@@ -1706,8 +1871,15 @@ private:
           << "        }\n"
           << "#pragma unroll\n"
           << "        for (int bb = 0; bb < " << B << "; bb++)\n"
-          << "          if (t0 + bb < " << OUT << ") { o_[j * " << n.push << " + 2 * (t0 + bb)] = re[bb]; o_[j * " << n.push
-          << " + 2 * (t0 + bb) + 1] = im[bb]; }\n"
+          << "          if (t0 + bb < " << OUT << ") {\n";
+        {
+            const int eo = n.out[0];
+            Lin pos = Lin::v("j", n.push, f_.edges[eo].pre + F0 * n.push);
+            pos.t.push_back({"(t0 + bb)", 2});
+            b << "            sm[" << buf_index(eo, pos).str() << "] = re[bb];\n"
+              << "            sm[" << buf_index(eo, pos.plus(1)).str() << "] = im[bb];\n";
+        }
+        b << "          }\n"
           << "      }\n";
     }
 };
