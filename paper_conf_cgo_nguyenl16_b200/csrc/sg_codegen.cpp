@@ -476,7 +476,9 @@ public:
         ki.pout = POUT_;
         ki.off_in = off_in_;
         ki.off_out = off_out_;
-        if (ki.tma_in && ki.tma_out && opt.mode != -1) {
+        if (opt.mode != -1 && try_inplace(ki, src, VT4)) {
+            // in-place component kernel generated
+        } else if (ki.tma_in && ki.tma_out && opt.mode != -1) {
             auto stage_bytes = [&](int lay, int64_t P, int64_t RS, int rows) -> int64_t {
                 int64_t b = lay == 1 ? rows * 128 : rows * RS * 4;
                 return (b + 1023) / 1024 * 1024;
@@ -616,6 +618,207 @@ public:
     }
 
 private:
+    // ---------------------------------------------------------------------
+    // In-place component variant.  Outputs whose dependence cones share no
+    // input item form independent components (FFT: its two branches); each
+    // component runs on its own warps (warp-uniform), loads its inputs
+    // eagerly, computes, writes its outputs back into the same shared-memory
+    // row slots (they are read by no other component) and bulk-stores its
+    // contiguous output chunk.  One stage buffer serves as input and output.
+    typedef std::vector<uint64_t> Bits;
+    std::map<std::pair<int, int64_t>, Bits> cone_memo_;
+    Bits cone_of(int e, int64_t pos) {
+        Bits b((PIN_ + 63) / 64, 0);
+        Ref r = R_.resolve(e, Lin::k(pos));
+        if (r.k == Ref::ZERO) return b;
+        if (r.edge == ein_) {
+            int64_t q = r.pos.c - off_in_;
+            if (q < 0 || q >= PIN_) throw Error(SG_E_UNSUPPORTED, "internal: cone out of row");
+            b[q / 64] |= 1ull << (q % 64);
+            return b;
+        }
+        const Edge& ed = f_.edges[r.edge];
+        const Node& u = f_.nodes[ed.src];
+        int64_t g = (r.pos.c - ed.pre) / u.push;
+        auto key = std::make_pair(ed.src, g);
+        auto it = cone_memo_.find(key);
+        if (it != cone_memo_.end()) return it->second;
+        for (int64_t i = 0; i < u.peek; i++) {
+            Bits c = cone_of(u.in[0], g * u.pop + i);
+            for (size_t w = 0; w < b.size(); w++) b[w] |= c[w];
+        }
+        cone_memo_[key] = b;
+        return b;
+    }
+    std::map<std::pair<int, int64_t>, std::vector<std::string>> dmemo_;
+    std::string dval(std::ostringstream& o, int e, int64_t pos) {
+        Ref r = R_.resolve(e, Lin::k(pos));
+        if (r.k == Ref::ZERO) return "(" + T_ + ")0";
+        if (r.edge == ein_) {
+            int64_t q = r.pos.c - off_in_;
+            static const char* comp[4] = {"x", "y", "z", "w"};
+            return "iq" + std::to_string(q / 4) + "." + comp[q % 4];
+        }
+        const Edge& ed = f_.edges[r.edge];
+        int u = ed.src;
+        const Node& n = f_.nodes[u];
+        int64_t q = r.pos.c - ed.pre, g = q / n.push, j = q % n.push;
+        auto key = std::make_pair(u, g);
+        auto it = dmemo_.find(key);
+        if (it != dmemo_.end()) return it->second[j];
+        std::vector<std::string> xs(n.peek);
+        for (int64_t i = 0; i < n.peek; i++) xs[i] = dval(o, n.in[0], g * n.pop + i);
+        std::vector<std::string> ys(n.push);
+        o << "      " << T_ << " ";
+        for (int64_t jj = 0; jj < n.push; jj++) {
+            ys[jj] = "v" + std::to_string(nv_++);
+            o << (jj ? ", " : "") << ys[jj];
+        }
+        o << ";\n      { const " << T_ << " x_[" << n.peek << "] = {";
+        for (int64_t i = 0; i < n.peek; i++) o << (i ? ", " : "") << xs[i];
+        o << "}; " << T_ << " y_[" << n.push << "]; " << work_call(u);
+        for (int64_t jj = 0; jj < n.push; jj++) o << " " << ys[jj] << " = y_[" << jj << "];";
+        o << " }\n";
+        dmemo_[key] = ys;
+        return ys[j];
+    }
+    bool try_inplace(KernelInfo& ki, std::ostringstream& src, const std::string& VT4) {
+        if (PIN_ != POUT_ || PIN_ % 4 != 0 || PIN_ * 4 == 128 || RIN_S_ != ROUT_S_) return false;
+        // components: union-find over output positions sharing an input item
+        std::vector<Bits> oc(POUT_);
+        for (int64_t p = 0; p < POUT_; p++) oc[p] = cone_of(eout_, off_out_ + p);
+        std::vector<int> par(POUT_);
+        std::iota(par.begin(), par.end(), 0);
+        std::function<int(int)> find = [&](int x) { return par[x] == x ? x : par[x] = find(par[x]); };
+        for (int64_t q = 0; q < PIN_; q++) {
+            int first = -1;
+            for (int64_t p = 0; p < POUT_; p++)
+                if (oc[p][q / 64] >> (q % 64) & 1) {
+                    if (first < 0) first = (int)p;
+                    else par[find((int)p)] = find(first);
+                }
+        }
+        std::map<int, std::vector<int64_t>> comps;
+        for (int64_t p = 0; p < POUT_; p++) comps[find((int)p)].push_back(p);
+        const int C = (int)comps.size();
+        if (C < 2 || C > 8) return false;
+        struct Comp { int64_t lo, hi; Bits in; };
+        std::vector<Comp> cs;
+        for (auto& kv : comps) {
+            Comp c;
+            c.lo = kv.second.front();
+            c.hi = kv.second.back() + 1;
+            if ((int64_t)kv.second.size() != c.hi - c.lo || c.lo % 4 || c.hi % 4) return false;
+            c.in = Bits((PIN_ + 63) / 64, 0);
+            for (int64_t p : kv.second) for (size_t w = 0; w < c.in.size(); w++) c.in[w] |= oc[p][w];
+            cs.push_back(c);
+        }
+        // in place: output slot p must not be an input of another component
+        for (size_t a = 0; a < cs.size(); a++)
+            for (size_t b2 = 0; b2 < cs.size(); b2++) {
+                if (a == b2) continue;
+                for (int64_t p = cs[a].lo; p < cs[a].hi; p++)
+                    if (cs[b2].in[p / 64] >> (p % 64) & 1) return false;
+            }
+        // tile rows R and stages NS
+        const int64_t rowb = RIN_S_ * 4;
+        int R = 0, NS = 0;
+        for (int r : {128, 96, 64, 32})
+            for (int ns : {4, 3, 2})
+                if ((int64_t)ns * ((r * rowb + 1023) / 1024 * 1024) + 2048 <= 220 * 1024 && r * (ns - 1) > R * (NS - 1)) {
+                    R = r;  // score: rows in flight beyond the tile being computed
+                    NS = ns;
+                }
+        if (!R) return false;
+        const int64_t STB = (R * rowb + 1023) / 1024 * 1024;
+        const int NWC = (R / 32) * C;
+        // bodies
+        std::ostringstream bodies;
+        for (int c = 0; c < C; c++) {
+            dmemo_.clear();
+            std::ostringstream o;
+            for (int64_t g = 0; g < PIN_ / 4; g++) {
+                bool need = false;
+                for (int i = 0; i < 4; i++) { int64_t q = 4 * g + i; need |= (cs[c].in[q / 64] >> (q % 64)) & 1; }
+                if (need) o << "      const " << VT4 << " iq" << g << " = SG_LD4(" << g << ");\n";
+            }
+            std::ostringstream st;
+            for (int64_t g = cs[c].lo / 4; g < cs[c].hi / 4; g++) {
+                std::string v[4];
+                for (int i = 0; i < 4; i++) v[i] = dval(o, eout_, off_out_ + 4 * g + i);
+                st << "      SG_ST4(" << g << ", make_" << VT4 << "(" << v[0] << ", " << v[1] << ", " << v[2] << ", " << v[3] << "));\n";
+            }
+            bodies << "    " << (c ? "} else if" : "if") << " (comp == " << c << ") {\n" << o.str() << st.str()
+                   << "      lo = " << cs[c].lo << "; len = " << cs[c].hi - cs[c].lo << ";\n";
+        }
+        bodies << "    }\n";
+        ki.has_tma = true;
+        ki.tma_in = ki.tma_out = 2;
+        ki.threads = NWC * 32 + 32;
+        ki.tile = R;
+        ki.smem = (size_t)(NS * STB + 2048);
+        src << "// ---- in-place component pipeline: " << C << " components, " << R << " rows per tile, " << NS
+            << " stages\n"
+            << "#define SG_LD4(g) (*reinterpret_cast<const " << VT4 << "*>(xb + ((g) << 4)))\n"
+            << "#define SG_ST4(g, v) (*reinterpret_cast<" << VT4 << "*>(xb + ((g) << 4)) = (v))\n"
+            << "extern \"C\" __global__ void __launch_bounds__(" << NWC * 32 + 32 << ", 1) " << ki.name
+            << "(const SgArgs a, const __grid_constant__ SgTmap tin, const __grid_constant__ SgTmap tout) {\n"
+            << "  constexpr int R = " << R << ", NWC = " << NWC << ", NS = " << NS << ", C = " << C << ";\n"
+            << "  constexpr int STB = " << STB << ";\n"
+            << "  extern __shared__ __align__(1024) unsigned char sg_smem_raw[];\n"
+            << "  unsigned char* st = reinterpret_cast<unsigned char*>((reinterpret_cast<unsigned long long>(sg_smem_raw) + 1023ull) & ~1023ull);\n"
+            << "  unsigned long long* full = reinterpret_cast<unsigned long long*>(st + NS * STB);\n"
+            << "  unsigned long long* empty = full + NS;\n"
+            << "  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;\n"
+            << "  const long long nrows = SG_K_END - SG_K_BEGIN;\n"
+            << "  const long long ntiles = (nrows + R - 1) / R;\n"
+            << "  if (threadIdx.x == 0) {\n"
+            << "    for (int s = 0; s < NS; s++) { sg_mbar_init(&full[s], 1); sg_mbar_init(&empty[s], NWC); }\n"
+            << "    sg_fence_barrier_init();\n"
+            << "  }\n"
+            << "  __syncthreads();\n"
+            << "  if (warp == NWC) {  // ---- producer warp: one bulk copy per row\n"
+            << "    const " << T_ << "* gin = SG_IN(0) + (SG_K_BEGIN * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
+            << "    int i = 0;\n"
+            << "    for (long long t = blockIdx.x; t < ntiles; t += gridDim.x, i++) {\n"
+            << "      const int s = i % NS;\n"
+            << "      const int nt = (int)min((long long)R, nrows - t * R);\n"
+            << "      sg_mbar_wait(&empty[s], ((i / NS) & 1) ^ 1);\n"
+            << "      if (lane == 0) sg_mbar_arrive_expect_tx(&full[s], (unsigned)(nt * " << PIN_ * 4 << "));\n"
+            << "      __syncwarp();\n"
+            << "      for (int r = lane; r < nt; r += 32)\n"
+            << "        sg_bulk_g2s(st + s * STB + r * " << rowb << ", gin + (t * R + r) * " << PIN_ << "LL, " << PIN_ * 4
+            << ", &full[s]);\n"
+            << "    }\n"
+            << "    return;\n"
+            << "  }\n"
+            << "  // ---- consumer warps: warp w runs component w % C on rows (w / C) * 32 + lane\n"
+            << "  " << T_ << "* gout = SG_OUT(0) + (SG_K_BEGIN * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
+            << "  const int comp = warp % C;\n"
+            << "  const int row = (warp / C) * 32 + lane;\n"
+            << "  int i = 0;\n"
+            << "  for (long long t = blockIdx.x; t < ntiles; t += gridDim.x, i++) {\n"
+            << "    const int s = i % NS;\n"
+            << "    const int nt = (int)min((long long)R, nrows - t * R);\n"
+            << "    sg_mbar_wait(&full[s], (i / NS) & 1);\n"
+            << "    unsigned char* xb = st + s * STB + row * " << rowb << ";\n"
+            << "    int lo = 0, len = 0;\n"
+            << "    if (row < nt) {\n"
+            << bodies.str()
+            << "      sg_fence_proxy_async();\n"
+            << "      sg_bulk_s2g(gout + (t * R + row) * " << POUT_ << "LL + lo, xb + lo * 4, (unsigned)(len * 4));\n"
+            << "      sg_bulk_commit();\n"
+            << "      sg_bulk_wait_read<0>();\n"
+            << "    }\n"
+            << "    __syncwarp();\n"
+            << "    if (lane == 0) sg_mbar_arrive(&empty[s]);\n"
+            << "  }\n"
+            << "  sg_bulk_wait<0>();\n"
+            << "}\n"
+            << "#undef SG_LD4\n#undef SG_ST4\n";
+        return true;
+    }
+
     int ein_ = -1, eout_ = -1;
     int64_t PIN_ = 0, POUT_ = 0, off_in_ = 0, off_out_ = 0, RIN_S_ = 0, ROUT_S_ = 0;
     bool vin_ = false, vout_ = false;
