@@ -655,7 +655,7 @@ private:
         Ref r = R_.resolve(e, Lin::k(pos));
         if (r.k == Ref::ZERO) return "(" + T_ + ")0";
         if (r.edge == ein_) {
-            int64_t q = r.pos.c - off_in_;
+            int64_t q = r.pos.c - off_in_ - rel_ilo_;
             static const char* comp[4] = {"x", "y", "z", "w"};
             return "iq" + std::to_string(q / 4) + "." + comp[q % 4];
         }
@@ -682,6 +682,12 @@ private:
         dmemo_[key] = ys;
         return ys[j];
     }
+    // dval with input names relative to a component's input chunk (group index - ilo/4)
+    std::string dval_rel(std::ostringstream& o, int e, int64_t pos, int64_t ilo) {
+        rel_ilo_ = ilo;
+        return dval(o, e, pos);
+    }
+    int64_t rel_ilo_ = 0;
     bool try_inplace(KernelInfo& ki, std::ostringstream& src, const std::string& VT4) {
         if (PIN_ != POUT_ || PIN_ % 4 != 0 || PIN_ * 4 == 128 || RIN_S_ != ROUT_S_) return false;
         // components: union-find over output positions sharing an input item
@@ -732,26 +738,50 @@ private:
         if (!R) return false;
         const int64_t STB = (R * rowb + 1023) / 1024 * 1024;
         const int NWC = (R / 32) * C;
-        // bodies
-        std::ostringstream bodies;
+        // bodies (component-relative: loads from its input chunk base, stores to its output base)
+        std::vector<std::string> btext(C);
+        std::vector<int64_t> ilo(C, 0);
         for (int c = 0; c < C; c++) {
+            int64_t first = -1;
+            for (int64_t q = 0; q < PIN_ && first < 0; q++) if (cs[c].in[q / 64] >> (q % 64) & 1) first = q;
+            ilo[c] = first < 0 ? 0 : first / 4 * 4;
             dmemo_.clear();
+            nv_ = 0;
             std::ostringstream o;
             for (int64_t g = 0; g < PIN_ / 4; g++) {
                 bool need = false;
                 for (int i = 0; i < 4; i++) { int64_t q = 4 * g + i; need |= (cs[c].in[q / 64] >> (q % 64)) & 1; }
-                if (need) o << "      const " << VT4 << " iq" << g << " = SG_LD4(" << g << ");\n";
+                if (need) o << "      const " << VT4 << " iq" << g - ilo[c] / 4 << " = SG_LD4I(" << g - ilo[c] / 4 << ");\n";
             }
             std::ostringstream st;
             for (int64_t g = cs[c].lo / 4; g < cs[c].hi / 4; g++) {
                 std::string v[4];
-                for (int i = 0; i < 4; i++) v[i] = dval(o, eout_, off_out_ + 4 * g + i);
-                st << "      SG_ST4(" << g << ", make_" << VT4 << "(" << v[0] << ", " << v[1] << ", " << v[2] << ", " << v[3] << "));\n";
+                for (int i = 0; i < 4; i++) v[i] = dval_rel(o, eout_, off_out_ + 4 * g + i, ilo[c]);
+                st << "      SG_ST4O(" << g - cs[c].lo / 4 << ", make_" << VT4 << "(" << v[0] << ", " << v[1] << ", " << v[2]
+                   << ", " << v[3] << "));\n";
             }
-            bodies << "    " << (c ? "} else if" : "if") << " (comp == " << c << ") {\n" << o.str() << st.str()
-                   << "      lo = " << cs[c].lo << "; len = " << cs[c].hi - cs[c].lo << ";\n";
+            btext[c] = o.str() + st.str();
         }
-        bodies << "    }\n";
+        bool shared = true;
+        for (int c = 1; c < C; c++) shared = shared && btext[c] == btext[0] && cs[c].hi - cs[c].lo == cs[0].hi - cs[0].lo;
+        std::ostringstream bodies;
+        std::string ibx = "0", obx = "0";
+        for (int c = C - 1; c >= 0; c--) {
+            ibx = c == C - 1 ? std::to_string(ilo[c] / 4) : "(comp == " + std::to_string(c) + " ? " + std::to_string(ilo[c] / 4) + " : " + ibx + ")";
+            obx = c == C - 1 ? std::to_string(cs[c].lo / 4) : "(comp == " + std::to_string(c) + " ? " + std::to_string(cs[c].lo / 4) + " : " + obx + ")";
+        }
+        bodies << "    const int ib = " << ibx << ", ob = " << obx << ";\n"
+               << "    const unsigned char* xi = xb + ib * 16;\n"
+               << "    unsigned char* xo = xb + ob * 16;\n";
+        if (shared) {
+            bodies << "    {  // one body shared by all " << C << " structurally identical components\n" << btext[0]
+                   << "      lo = ob * 4; len = " << cs[0].hi - cs[0].lo << ";\n    }\n";
+        } else {
+            for (int c = 0; c < C; c++)
+                bodies << "    " << (c ? "} else if" : "if") << " (comp == " << c << ") {\n" << btext[c]
+                       << "      lo = " << cs[c].lo << "; len = " << cs[c].hi - cs[c].lo << ";\n";
+            bodies << "    }\n";
+        }
         ki.has_tma = true;
         ki.tma_in = ki.tma_out = 2;
         ki.threads = NWC * 32 + 32;
@@ -759,8 +789,8 @@ private:
         ki.smem = (size_t)(NS * STB + 2048);
         src << "// ---- in-place component pipeline: " << C << " components, " << R << " rows per tile, " << NS
             << " stages\n"
-            << "#define SG_LD4(g) (*reinterpret_cast<const " << VT4 << "*>(xb + ((g) << 4)))\n"
-            << "#define SG_ST4(g, v) (*reinterpret_cast<" << VT4 << "*>(xb + ((g) << 4)) = (v))\n"
+            << "#define SG_LD4I(g) (*reinterpret_cast<const " << VT4 << "*>(xi + ((g) << 4)))\n"
+            << "#define SG_ST4O(g, v) (*reinterpret_cast<" << VT4 << "*>(xo + ((g) << 4)) = (v))\n"
             << "extern \"C\" __global__ void __launch_bounds__(" << NWC * 32 + 32 << ", 1) " << ki.name
             << "(const SgArgs a, const __grid_constant__ SgTmap tin, const __grid_constant__ SgTmap tout) {\n"
             << "  constexpr int R = " << R << ", NWC = " << NWC << ", NS = " << NS << ", C = " << C << ";\n"
@@ -815,7 +845,7 @@ private:
             << "  }\n"
             << "  sg_bulk_wait<0>();\n"
             << "}\n"
-            << "#undef SG_LD4\n#undef SG_ST4\n";
+            << "#undef SG_LD4I\n#undef SG_ST4O\n";
         return true;
     }
 
@@ -1480,6 +1510,8 @@ private:
         }
     }
     void fused_layout(int W) {
+        W_ = W;
+        beam_B_.clear();
         off_.clear();
         wb_.clear();
         size_.clear();
@@ -1641,15 +1673,10 @@ private:
         for (int L = 1; L <= flev_; L++) {
             b << "    // ---- fused level " << L << "\n";
             int64_t rot = 0;
+            emit_specials(b, L, rot);
             for (auto& g : fg_) {
                 if (g.level != L) continue;
-                if (g.special) {
-                    for (int r : g.roots) {
-                        emit_stage(b, r, rot);
-                        rot += f_.nodes[r].halo + (int64_t)W * f_.nodes[r].rep;
-                    }
-                    continue;
-                }
+                if (g.special) continue;
                 b << "    { // group of " << g.roots.size() << " root(s) [" << kind_name(f_.nodes[g.roots[0]].kind)
                   << "], B = " << g.B << ", blocks per full tile = " << g.NB << "\n";
                 b << "      int NBg = 0;\n";
@@ -1677,6 +1704,39 @@ private:
         emit_stores(b);
         b << "    __syncthreads();\n";
         return b.str();
+    }
+    // frame-FIR stages of one level, peers sharing one body where possible
+    void emit_specials(std::ostringstream& b, int L, int64_t& rot) {
+        std::vector<int> sp;
+        for (auto& g : fg_)
+            if (g.special && g.level == L)
+                for (int r : g.roots) sp.push_back(r);
+        std::vector<char> done(sp.size(), 0);
+        for (size_t a = 0; a < sp.size(); a++) {
+            if (done[a]) continue;
+            std::vector<int> peers{sp[a]};
+            done[a] = 1;
+            for (size_t c = a + 1; c < sp.size(); c++)
+                if (!done[c] && f_.nodes[sp[c]].iv == f_.nodes[sp[a]].iv && f_.nodes[sp[c]].fv == f_.nodes[sp[a]].fv) {
+                    peers.push_back(sp[c]);
+                    done[c] = 1;
+                }
+            std::vector<int64_t> din, dout;
+            if (peers.size() > 1 && beam_peer_offsets(peers, din, dout)) {
+                const Node& n = f_.nodes[peers[0]];
+                b << "    { // " << peers.size() << " peer frame FIRs (shared body)\n"
+                  << "      const int nf = " << n.halo << " + Wt * " << n.rep << ";\n"
+                  << "      const long long gf = k0 * " << n.rep << "LL;\n";
+                emit_beam_fir(b, peers[0], n.ninit - n.halo, rot, peers, din, dout);
+                b << "    }\n";
+                rot += (int64_t)peers.size() * (n.halo + (int64_t)W_ * n.rep);
+            } else {
+                for (int r : peers) {
+                    emit_stage(b, r, rot);
+                    rot += f_.nodes[r].halo + (int64_t)W_ * f_.nodes[r].rep;
+                }
+            }
+        }
     }
     // Algorithmic fp32 work per iteration of the fused plan: dead firings and zero
     // taps removed, recomputed (halo / inlining overlap) firings not counted.
@@ -2030,48 +2090,168 @@ private:
     }
     // Frame-granular complex FIR: items = (firing, block of B outputs); taps in
     // chunks of TC with the sample window in registers; x[s<0] = 0.
-    void emit_beam_fir(std::ostringstream& b, int v, int64_t F0, int64_t rot) {
+    // Frame-granular complex FIR: items = (firing, block of B consecutive outputs);
+    // taps in chunks of TC with the sample window in registers; x[s<0] = 0.
+    // B odd (lanes 3/5/7.. samples apart hit distinct banks of planar buffers),
+    // chosen with the other frame FIRs of the same level to avoid straggler
+    // rounds; interior chunks skip the boundary checks; short filters are fully
+    // unrolled so coefficients become immediates.
+    std::map<int, int64_t> beam_B_;
+    int64_t beam_block(int v, int64_t W) {
+        auto it = beam_B_.find(v);
+        if (it != beam_B_.end()) return it->second;
+        // all frame FIRs of v's level (same L/dec/frame/rep) share the choice
         const Node& n = f_.nodes[v];
+        int64_t peers = 0;
+        for (int u : nodes_)
+            if (compute_node(u) && special(u) && f_.nodes[u].iv == n.iv && level_of_special(u) == level_of_special(v)) peers++;
+        int64_t best = 3;
+        double bestc = 1e300;
+        const int64_t OUT = n.iv[2] / n.iv[1], L = n.iv[0], DEC = n.iv[1];
+        for (int64_t B : {3, 5, 7, 9}) {
+            int64_t items = peers * (n.halo + W * n.rep) * ((OUT + B - 1) / B);
+            int64_t rounds = (items + NT_ - 1) / NT_;
+            double per_item = (double)B * L * 4 + ((B - 1) * DEC + 16) * 2.0 * L / 16.0;
+            double cost = rounds * per_item;
+            if (cost < bestc - 1e-9) { bestc = cost; best = B; }
+        }
+        beam_B_[v] = best;
+        return best;
+    }
+    std::map<int, int> special_level_;
+    int level_of_special(int v) {
+        auto it = special_level_.find(v);
+        if (it != special_level_.end()) return it->second;
+        int L = level_.count(v) ? level_.at(v) : 0;
+        for (auto& g : fg_)
+            for (int r : g.roots)
+                if (r == v) L = g.level;
+        special_level_[v] = L;
+        return L;
+    }
+    // peers: frame FIRs with identical parameters whose reads/writes differ only by a
+    // constant offset; one body serves all of them (item -> peer, firing, block).
+    bool beam_peer_offsets(const std::vector<int>& peers, std::vector<int64_t>& din, std::vector<int64_t>& dout) {
+        const Node& n0 = f_.nodes[peers[0]];
+        const int64_t L = n0.iv[0], DEC = n0.iv[1], TC = 16, B = 9;
+        const int64_t NWIN = (B - 1) * DEC + TC;
+        din.assign(peers.size(), 0);
+        dout.assign(peers.size(), 0);
+        for (size_t q = 0; q < peers.size(); q++) {
+            const Node& n = f_.nodes[peers[q]];
+            if (n.iv != n0.iv || n.fv != n0.fv || n.halo != n0.halo || n.ninit != n0.ninit || n.rep != n0.rep) return false;
+            for (int64_t k = 0; k < NWIN; k += NWIN - 1)
+                for (int r = 0; r < 2; r++) {
+                    Lin pr = Lin::v("lf", n.pop, 2 * k + r);
+                    pr.t.push_back({"s0", 2});
+                    Lin p0 = pr;
+                    Ref a = R_.resolve(n0.in[0], p0), c = R_.resolve(n.in[0], pr);
+                    if (a.k != Ref::PHYS || c.k != Ref::PHYS) return false;
+                    Lin ia = buf_index(a.edge, a.pos), ic = buf_index(c.edge, c.pos);
+                    if (ia.vars() != ic.vars()) return false;
+                    int64_t d = ic.c - ia.c;
+                    if (k == 0 && r == 0) din[q] = d;
+                    else if (d != din[q]) return false;
+                }
+            Lin pos = Lin::v("j", n.push, f_.edges[n.out[0]].pre + (n.ninit - n.halo) * n.push);
+            pos.t.push_back({"(t0 + bb)", 2});
+            Lin oa = buf_index(n0.out[0], pos), oc = buf_index(n.out[0], pos);
+            Lin oa1 = buf_index(n0.out[0], pos.plus(1)), oc1 = buf_index(n.out[0], pos.plus(1));
+            if (oa.vars() != oc.vars() || oc.c - oa.c != oc1.c - oa1.c) return false;
+            dout[q] = oc.c - oa.c;
+            (void)L;
+        }
+        return true;
+    }
+    void emit_beam_fir(std::ostringstream& b, int v, int64_t F0, int64_t rot, const std::vector<int>& peers = {},
+                       const std::vector<int64_t>& din = {}, const std::vector<int64_t>& dout = {}) {
+        const Node& n = f_.nodes[v];
+        const int64_t NP = peers.empty() ? 1 : (int64_t)peers.size();
         int64_t L = n.iv[0], DEC = n.iv[1], FR = n.iv[2], OUT = FR / DEC;
-        int64_t B = 3, TC = 1;  // odd block: lanes 3*DEC samples apart -> distinct banks in planar buffers
+        int64_t TC = 1;
         for (int64_t c : {16, 8, 4, 2, 1})
             if (L % c == 0) { TC = c; break; }
+        const int64_t B = beam_block(v, W_);
         int64_t NB = (OUT + B - 1) / B, NWIN = (B - 1) * DEC + TC;
+        const bool unroll = L <= 64;
         std::vector<float> wr(n.fv.begin(), n.fv.begin() + L), wi(n.fv.begin() + L, n.fv.end());
-        std::string WR = const_array(wr), WI = const_array(wi);
-        b << "      const int items = nf * " << NB << ";\n"
+        std::string WR = unroll ? "" : const_array(wr), WI = unroll ? "" : const_array(wi);
+        std::string DINT, DOUTT;
+        if (NP > 1) {
+            DINT = "SG_DIN" + std::to_string(v) + "_" + std::to_string(nvar_++);
+            DOUTT = "SG_DOUT" + std::to_string(v) + "_" + std::to_string(nvar_++);
+            consts_ << "__constant__ int " << DINT << "[" << NP << "] = {";
+            for (int64_t q = 0; q < NP; q++) consts_ << (q ? ", " : "") << din[q];
+            consts_ << "};\n__constant__ int " << DOUTT << "[" << NP << "] = {";
+            for (int64_t q = 0; q < NP; q++) consts_ << (q ? ", " : "") << dout[q];
+            consts_ << "};\n";
+        }
+        b << "      const int items = nf * " << NB * NP << ";\n"
           << "      int it = tid - " << rot % NT_ << "; if (it < 0) it += NT;\n"
           << "      for (; it < items; it += NT) {\n"
-          << "        const int j = it / " << NB << ";\n"
-          << "        const int t0 = (it - j * " << NB << ") * " << B << ";\n"
+          << "        const int pq = it / (nf * " << NB << ");\n"
+          << "        const int itp = it - pq * (nf * " << NB << ");\n"
+          << "        const int j = itp / " << NB << ";\n"
+          << "        const int t0 = (itp - j * " << NB << ") * " << B << ";\n"
           << "        const int lf = " << F0 << " + j;\n"
+          << "        " << T_ << "* smi = sm + " << (NP > 1 ? DINT + "[pq]" : std::string("0")) << ";\n"
+          << "        " << T_ << "* smo = sm + " << (NP > 1 ? DOUTT + "[pq]" : std::string("0")) << ";\n"
+          << "        (void)pq; (void)smi; (void)smo;\n"
           << "        float re[" << B << "], im[" << B << "];\n"
           << "#pragma unroll\n"
           << "        for (int bb = 0; bb < " << B << "; bb++) { re[bb] = 0.0f; im[bb] = 0.0f; }\n"
-          << "        if (gf + lf >= 0) {\n"
-          << "#pragma unroll 1\n"
-          << "          for (int i0 = 0; i0 < " << L << "; i0 += " << TC << ") {\n"
-          << "            const int s0 = t0 * " << DEC << " - i0 - " << TC - 1 << ";\n"
-          << "            float xr[" << NWIN << "], xi[" << NWIN << "];\n";
-        for (int64_t k = 0; k < NWIN; k++) {
-            Lin pr = Lin::v("lf", n.pop, 2 * k);
-            pr.t.push_back({"s0", 2});
-            Lin pi = pr.plus(1);
-            b << "            { const int s = s0 + " << k << "; const bool ok = s >= 0 && s < " << FR << ";\n"
-              << "              xr[" << k << "] = ok ? " << read_expr(n.in[0], pr) << " : 0.0f;\n"
-              << "              xi[" << k << "] = ok ? " << read_expr(n.in[0], pi) << " : 0.0f; }\n";
+          << "        if (gf + lf >= 0) {\n";
+        auto chunk = [&](const std::string& i0expr, bool checked, const std::string& cr_of, const std::string& ci_of) {
+            b << "          {\n"
+              << "            const int s0 = t0 * " << DEC << " - (" << i0expr << ") - " << TC - 1 << ";\n"
+              << "            float xr[" << NWIN << "], xi[" << NWIN << "];\n";
+            for (int64_t k = 0; k < NWIN; k++) {
+                Lin pr = Lin::v("lf", n.pop, 2 * k);
+                pr.t.push_back({"s0", 2});
+                Lin pi = pr.plus(1);
+                std::string er = "smi" + read_expr(n.in[0], pr).substr(2), ei = "smi" + read_expr(n.in[0], pi).substr(2);
+                if (checked)
+                    b << "            { const int s = s0 + " << k << "; const bool ok = s >= 0 && s < " << FR << ";\n"
+                      << "              xr[" << k << "] = ok ? " << er << " : 0.0f;\n"
+                      << "              xi[" << k << "] = ok ? " << ei << " : 0.0f; }\n";
+                else
+                    b << "            xr[" << k << "] = " << er << "; xi[" << k << "] = " << ei << ";\n";
+            }
+            b << "#pragma unroll\n"
+              << "            for (int ii = 0; ii < " << TC << "; ii++) {\n"
+              << "              const float cr = " << cr_of << ", ci = " << ci_of << ";\n"
+              << "#pragma unroll\n"
+              << "              for (int bb = 0; bb < " << B << "; bb++) {\n"
+              << "                const int k = bb * " << DEC << " - ii + " << TC - 1 << ";\n"
+              << "                sg_cmac(re[bb], im[bb], xr[k], xi[k], cr, ci);\n"
+              << "              }\n"
+              << "            }\n"
+              << "          }\n";
+        };
+        if (unroll) {
+            for (int64_t i0 = 0; i0 < L; i0 += TC) {
+                // immediates: a switch-free table via a constexpr lambda index is not available in NVRTC C++17
+                // device code, so emit the chunk's TC coefficients as an initialised local array
+                std::string cr = const_array(std::vector<float>(wr.begin() + i0, wr.begin() + i0 + TC));
+                std::string ci = const_array(std::vector<float>(wi.begin() + i0, wi.begin() + i0 + TC));
+                b << "          if (t0 * " << DEC << " - " << i0 + TC - 1 << " >= 0 && t0 * " << DEC << " + " << (B - 1) * DEC
+                  << " - " << i0 << " < " << FR << ") {\n";
+                chunk(std::to_string(i0), false, cr + "[ii]", ci + "[ii]");
+                b << "          } else {\n";
+                chunk(std::to_string(i0), true, cr + "[ii]", ci + "[ii]");
+                b << "          }\n";
+            }
+        } else {
+            b << "#pragma unroll 1\n"
+              << "          for (int i0 = 0; i0 < " << L << "; i0 += " << TC << ") {\n"
+              << "            if (t0 * " << DEC << " - i0 - " << TC - 1 << " >= 0 && t0 * " << DEC << " + " << (B - 1) * DEC
+              << " - i0 < " << FR << ") {\n";
+            chunk("i0", false, WR + "[i0 + ii]", WI + "[i0 + ii]");
+            b << "            } else {\n";
+            chunk("i0", true, WR + "[i0 + ii]", WI + "[i0 + ii]");
+            b << "            }\n          }\n";
         }
-        b << "#pragma unroll\n"
-          << "            for (int ii = 0; ii < " << TC << "; ii++) {\n"
-          << "              const float cr = " << WR << "[i0 + ii], ci = " << WI << "[i0 + ii];\n"
-          << "#pragma unroll\n"
-          << "              for (int bb = 0; bb < " << B << "; bb++) {\n"
-          << "                const int k = bb * " << DEC << " - ii + " << TC - 1 << ";\n"
-          << "                sg_cmac(re[bb], im[bb], xr[k], xi[k], cr, ci);\n"
-          << "              }\n"
-          << "            }\n"
-          << "          }\n"
-          << "        }\n"
+        b << "        }\n"
           << "#pragma unroll\n"
           << "        for (int bb = 0; bb < " << B << "; bb++)\n"
           << "          if (t0 + bb < " << OUT << ") {\n";
@@ -2079,8 +2259,8 @@ private:
             const int eo = n.out[0];
             Lin pos = Lin::v("j", n.push, f_.edges[eo].pre + F0 * n.push);
             pos.t.push_back({"(t0 + bb)", 2});
-            b << "            sm[" << buf_index(eo, pos).str() << "] = re[bb];\n"
-              << "            sm[" << buf_index(eo, pos.plus(1)).str() << "] = im[bb];\n";
+            b << "            smo[" << buf_index(eo, pos).str() << "] = re[bb];\n"
+              << "            smo[" << buf_index(eo, pos.plus(1)).str() << "] = im[bb];\n";
         }
         b << "          }\n"
           << "      }\n";
