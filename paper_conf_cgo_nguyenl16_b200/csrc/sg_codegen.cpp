@@ -33,6 +33,7 @@
 #include <algorithm>
 #include <cmath>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <functional>
 #include <map>
@@ -984,6 +985,18 @@ public:
                     fused_layout(1);
                     if (smem_bytes_ <= 227 * 1024) WF = 1;
                 }
+                if (WF > 0 && opt.threads <= 0) {
+                    fused_layout(WF);
+                    if (smem_bytes_ > 113 * 1024) {  // one CTA per SM: give it 16 warps
+                        NT_ = NT = 512;
+                        int W2 = 0;
+                        for (int cand : fused_tile_candidates(opt.tile)) {
+                            fused_layout(cand);
+                            if (smem_bytes_ <= 227 * 1024) { W2 = cand; break; }
+                        }
+                        if (W2 > 0) WF = W2;
+                    }
+                }
                 if (WF > 0) {
                     fused_layout(WF);
                     smem_fast = smem_bytes_;
@@ -1041,6 +1054,7 @@ public:
         ki.tile = WT;
         ki.smem = WF > 0 ? smem_fast : smem_slow;
         ki.min_blocks = std::max(1, std::min(2, (int)((220 * 1024) / std::max<size_t>(1024, ki.smem))));
+        if (const char* mb = std::getenv("SG_MINB")) ki.min_blocks = std::max(1, std::atoi(mb));
         ki.fused = WF > 0;
         ki.ksafe = ksafe;
         std::ostringstream src;
@@ -1248,7 +1262,8 @@ private:
     // One block of a group: roots' live firings F0L + S*(jb*B + beta), beta < B.
     void sym_block(Sym& c, const FGroup& g, bool emit_stores) {
         std::ostringstream& o = *c.os;
-        bool all_fir = g.roots.size() > 1;
+        static const bool interleave = std::getenv("SG_INTERLEAVE") != nullptr;  // measured slower by default
+        bool all_fir = g.roots.size() > 1 && interleave;
         for (int r : g.roots) all_fir = all_fir && f_.nodes[r].kind == SG_K_FIR;
         if (all_fir) {  // sibling FIRs: taps outer, roots and block inner -> independent chains, window loaded once
             const int64_t B = g.B;
@@ -1458,8 +1473,9 @@ private:
                     }
                     if (!B0) throw FusedFail();
                     g.B = B0;
+                    static const int bmax = std::getenv("SG_FUSED_BMAX") ? std::atoi(std::getenv("SG_FUSED_BMAX")) : 16;
                     dry_ok(g, c);
-                    while (g.B * 2 <= 16) {
+                    while (g.B * 2 <= bmax) {
                         FGroup h = g;
                         h.B = g.B * 2;
                         Sym c2;
@@ -2173,7 +2189,7 @@ private:
             if (L % c == 0) { TC = c; break; }
         const int64_t B = beam_block(v, W_);
         int64_t NB = (OUT + B - 1) / B, NWIN = (B - 1) * DEC + TC;
-        const bool unroll = L <= 64;
+        const bool unroll = false;  // rolled tap loop: small code (I-cache) beats immediates here
         std::vector<float> wr(n.fv.begin(), n.fv.begin() + L), wi(n.fv.begin() + L, n.fv.end());
         std::string WR = unroll ? "" : const_array(wr), WI = unroll ? "" : const_array(wi);
         std::string DINT, DOUTT;
