@@ -161,6 +161,9 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-flush", action="store_true")
     ap.add_argument("--eager", action="store_true", help="launch sg_run every step instead of replaying a CUDA graph")
+    ap.add_argument("--mode", default="replicas", choices=["replicas", "pipeline"],
+                    help="N>1: independent replicas (default; the headline graph is HBM-bound) or the paper's "
+                         "pipelined partition mapping, one process per GPU, NCCL boundary streams")
     args = ap.parse_args()
     if args.warmup < 3:
         args.warmup = 3
@@ -182,24 +185,30 @@ def main():
     W = WORKLOADS[name]
     n = args.iters or W["n"]
     prog = apps.CONFIGS[name]()
-    plan = sg.plan(prog, 1, devices=[local])
+    pipeline = args.mode == "pipeline" and world > 1
+    if pipeline:
+        from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan
+        plan = pipeline_plan(prog)
+    else:
+        plan = sg.plan(prog, 1, devices=[local])
     info = plan.info()
     nin, nout = plan.input_items(n), plan.output_items(n)
     dt = torch.int32 if prog.dtype == "i32" else torch.float32
-    x_host = torch.from_numpy(inputs.make_input(prog.dtype, nin, inputs.SEEDS[name] + rank))
+    x_host = torch.from_numpy(inputs.make_input(prog.dtype, nin, inputs.SEEDS[name] + (0 if pipeline else rank)))
     x = x_host.to(f"cuda:{local}")
     y = torch.empty(nout, dtype=dt, device=f"cuda:{local}")
     flush = torch.empty(256 << 20, dtype=torch.uint8, device=f"cuda:{local}")
     stream = torch.cuda.current_stream()
 
+    run_step = (lambda: plan.run_rank(x, n, y, stream)) if pipeline else (lambda: plan.run(x, n, y, stream))
     for _ in range(args.warmup):
-        plan.run(x, n, y, stream)
+        run_step()
     launches_per_step = plan.last_launch_count()
     torch.cuda.synchronize()
     # CUDA graph of one sg_run (the C ABI call enqueues only kernels and events on the
     # capturing stream); replaying it removes host launch gaps from the timed window.
     graph = None
-    if not args.eager:
+    if not args.eager and not pipeline:
         try:
             gs = torch.cuda.Stream()
             graph = torch.cuda.CUDAGraph()
@@ -218,7 +227,7 @@ def main():
         if graph is not None:
             graph.replay()
         else:
-            plan.run(x, n, y, stream)
+            run_step()
 
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
     sampler = ClockSampler(local)
@@ -246,7 +255,7 @@ def main():
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
         total_ms = float(t.item())
     ms_per_step = total_ms / args.steps
-    value = world * n * args.steps / (total_ms / 1e3)
+    value = (1 if pipeline else world) * n * args.steps / (total_ms / 1e3)
 
     # roofline of the dominant kernel (single partition: one launch per step)
     peaks, peak_src = measured_peaks()
@@ -284,7 +293,7 @@ def main():
 
     # end to end through the public C ABI with HOST buffers (pinned), copies inside the timed region
     e2e = None
-    if rank == 0 or world > 1:
+    if not pipeline:
         xh = x_host.pin_memory()
         yh = torch.empty(nout, dtype=dt).pin_memory()
         xnp, ynp = xh.numpy(), yh.numpy()
@@ -304,13 +313,15 @@ def main():
     if rank == 0:
         line = {
             "metric": METRIC, "value": value, "unit": "iters/s", "n_gpus": world, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "weak",
+            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True,
+            "scaling": "strong" if pipeline else "weak",
             "vs_baseline": None, "dtype": "i32" if prog.dtype == "i32" else "f32", "data": "synthetic",
             "config": {"workload": name, "desc": W["desc"], "iters_per_step": n,
                        "items_per_s_out": value * info["out_per_iter"],
                        "l2": "flushed before every step (256 MiB sg_flush_l2: write + read back), outside the event window"
                        if not args.no_flush else "not flushed",
-                       "parallelism": f"replicas x{world}" if world > 1 else "1 GPU, 1 partition",
+                       "parallelism": (f"pipeline over {world} GPUs (ILP mapping, NCCL boundary streams)" if pipeline
+                                       else f"replicas x{world}" if world > 1 else "1 GPU, 1 partition"),
                        "partitions": info["n_partitions"], "partition_mode": info["partition_mode"],
                        "launch": "CUDA graph replay of one sg_run" if graph is not None else "eager sg_run",
                        "wall_s": wall},

@@ -232,6 +232,30 @@ const char* sg_last_error(void);
 /* Library version string. */
 const char* sg_version(void);
 
+/* ---- one process per GPU (PAPER.md:552-567 with NCCL point-to-point over NVLink) ----
+ * Every rank builds the same plan (same graph, n_gpus = world size), rank 0 creates a
+ * unique id with sg_comm_unique_id and broadcasts it (e.g. torch.distributed), every
+ * rank calls sg_comm_init, then sg_run_rank.  A rank runs only the partitions mapped
+ * to it, fragment by fragment; boundary streams travel with ncclSend/ncclRecv on a
+ * library-owned stream.  `input` must be given (device pointer on `device`) on the
+ * rank whose partition consumes the graph input (sg_plan_info.input_device is that
+ * rank), `output` on the rank producing the output; other ranks may pass NULL.  The
+ * call enqueues and returns; completion is ordered on `stream`. */
+sg_status sg_comm_unique_id(uint8_t id[128]);
+sg_status sg_comm_init(sg_plan_t* p, int32_t nranks, int32_t rank, const uint8_t id[128], int32_t device);
+sg_status sg_run_rank(sg_plan_t* p, const void* input, int64_t n_iters, void* output, void* stream);
+
+/* The host-side schedule sg_run_rank issues on `rank` (for tests and tracing):
+ * op = SG_OP_LAUNCH (partition `part` over iterations [k_begin, k_end)),
+ * SG_OP_SEND / SG_OP_RECV (cut edge `edge`, `items` 4-byte items, to/from `peer`).
+ * Fills up to `cap` ops; returns the total count (< 0 on error). */
+enum { SG_OP_LAUNCH = 0, SG_OP_SEND = 1, SG_OP_RECV = 2 };
+typedef struct {
+    int32_t op, part, edge, peer;
+    int64_t fragment, k_begin, k_end, items;
+} sg_rank_op;
+int64_t sg_rank_schedule(const sg_plan_t* p, int32_t rank, int64_t n_iters, sg_rank_op* ops, int64_t cap);
+
 /* ---- planner building blocks (PAPER.md sections 3.2-3.3), for tests and tools ----
  * Topology kinds: 0 = NVSwitch star of n_gpus GPUs (uplink k and downlink k per GPU,
  * L = 2G), 1 = the 4-GPU PCIe tree of Fig. 3.3 (n_gpus must be 4). */

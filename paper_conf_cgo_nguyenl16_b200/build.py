@@ -26,9 +26,20 @@ CUDA = os.environ.get("CUDA_HOME", "/usr/local/cuda")
 NVCC = os.path.join(CUDA, "bin", "nvcc")
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 
-CPP = ["sg_graph.cpp", "sg_codegen.cpp", "sg_plan.cpp", "sg_runtime.cpp", "sg_capi.cpp"]
+CPP = ["sg_graph.cpp", "sg_codegen.cpp", "sg_plan.cpp", "sg_runtime.cpp", "sg_dist.cpp", "sg_capi.cpp"]
 CU = ["sg_aux.cu"]
 HEADERS = ["sg_internal.h", "sg_codegen.h", "sg_runtime.h", "sg_plan.h", "sg_device.cuh"]
+
+
+def _nccl_include():
+    try:
+        import nvidia.nccl
+        d = os.path.join(list(nvidia.nccl.__path__)[0], "include")
+        if os.path.exists(os.path.join(d, "nccl.h")):
+            return d
+    except Exception:
+        pass
+    return "/usr/include"
 
 
 def _embed():
@@ -64,7 +75,7 @@ def build(force: bool = False, verbose: bool = False) -> str:
         if not force and os.path.exists(obj) and os.path.getmtime(obj) >= os.path.getmtime(src):
             continue
         cmd = [NVCC, *ARCH, "-lineinfo", "-O3", "-std=c++17", "-Xcompiler", "-fPIC,-Wall,-Wno-array-bounds", "-c", src, "-o", obj,
-               "-I" + os.path.join(HERE, "..", "include")]
+               "-I" + os.path.join(HERE, "..", "include"), "-I" + _nccl_include()]
         if name.endswith(".cu"):
             cmd += ["-Xptxas", "-v"] if verbose else []
         else:

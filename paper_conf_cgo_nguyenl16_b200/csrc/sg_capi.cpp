@@ -280,6 +280,43 @@ int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst,
     return (int32_t)e.size();
 }
 
+sg_status sg_comm_unique_id(uint8_t id[128]) {
+    if (!id) return fail(SG_E_ARG, "NULL id");
+    return guard([&] { sg::nccl_unique_id(id); });
+}
+
+sg_status sg_comm_init(sg_plan_t* p, int32_t nranks, int32_t rank, const uint8_t id[128], int32_t device) {
+    if (!p || !id) return fail(SG_E_ARG, "NULL argument");
+    return guard([&] { p->plan.comm_init(nranks, rank, id, device); });
+}
+
+sg_status sg_run_rank(sg_plan_t* p, const void* input, int64_t n, void* output, void* stream) {
+    if (!p) return fail(SG_E_ARG, "NULL plan");
+    if (n < 0) return fail(SG_E_ARG, "negative n_iters");
+    if (n == 0) return SG_OK;
+    return guard([&] { p->plan.run_rank(input, n, output, (cudaStream_t)stream); });
+}
+
+int64_t sg_rank_schedule(const sg_plan_t* p, int32_t rank, int64_t n, sg_rank_op* ops, int64_t cap) {
+    if (!p || n < 0 || rank < 0 || rank >= p->plan.G) return -1;
+    try {
+        auto v = sg::rank_schedule(p->plan, rank, n, sg::fragment_size(p->plan, std::max<int64_t>(n, 1)));
+        for (int64_t i = 0; i < (int64_t)v.size() && i < cap; i++) {
+            ops[i].op = v[i].op;
+            ops[i].part = v[i].part;
+            ops[i].edge = v[i].edge;
+            ops[i].peer = v[i].peer;
+            ops[i].fragment = v[i].frag;
+            ops[i].k_begin = v[i].kb;
+            ops[i].k_end = v[i].ke;
+            ops[i].items = v[i].items;
+        }
+        return (int64_t)v.size();
+    } catch (...) {
+        return -1;
+    }
+}
+
 int64_t sg_last_launch_count(const sg_plan_t* p) { return p ? p->plan.last_launches : -1; }
 
 void sg_plan_destroy(sg_plan_t* p) { delete p; }

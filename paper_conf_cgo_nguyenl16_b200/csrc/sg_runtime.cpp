@@ -262,13 +262,6 @@ int sm_count(int dev) {
     return n;
 }
 
-struct IoBinding {
-    std::vector<const void*> in;
-    std::vector<int64_t> in_base, in_limit;
-    std::vector<void*> out;
-    std::vector<int64_t> out_base;
-};
-
 // Launch one partition kernel over iterations [kb, ke) on `stream`.
 int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int64_t ke, cudaStream_t stream,
                bool is_f32) {
@@ -331,7 +324,13 @@ int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int
 }
 }  // namespace
 
+int64_t launch_kernel(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int64_t ke, cudaStream_t stream,
+                      bool is_f32) {
+    return launch(ck, dev, io, kb, ke, stream, is_f32);
+}
+
 Plan::~Plan() {
+    dist_release();
     for (auto& r : rings) {
         for (size_t i = 0; i < r.src_slots.size(); i++) {
             if (r.src_slots[i]) { cudaSetDevice(devices[r.src_gpu]); cudaFree(r.src_slots[i]); }
@@ -386,17 +385,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
         return;
     }
     // ---- general path: fragments pipelined over partitions and GPUs
-    int64_t F = iters_per_fragment;
-    if (F <= 0) {  // auto: >= 2 full waves per kernel, ~8 fragments per GPU for pipelining
-        int64_t wave = 1;
-        for (auto& ck : kernels) wave = std::max<int64_t>(wave, (int64_t)ck.ki.tile * 148 * 2);
-        F = std::max<int64_t>(wave, (n + 8 * G - 1) / (8 * G));
-        int64_t ring_bytes_per_iter = 0;
-        for (auto& e : flat.edges)
-            if (e.src >= 0 && e.dst >= 0 && node_part[e.src] != node_part[e.dst]) ring_bytes_per_iter += 4 * e.per_iter;
-        if (ring_bytes_per_iter > 0) F = std::min<int64_t>(F, std::max<int64_t>(wave, ((int64_t)1 << 30) / ring_bytes_per_iter));
-    }
-    F = std::min(F, n);
+    int64_t F = fragment_size(*this, n);
     if (rt_ready && rt_fragment >= F) F = std::min(rt_fragment, n);
     if (!rt_ready || rt_fragment < F) {
         // (re)allocate rings for fragment size F

@@ -3,6 +3,7 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <map>
 #include <string>
 #include <vector>
 
@@ -31,6 +32,18 @@ struct CutRing {          // one boundary stream between partitions (PAPER.md:49
     int64_t slot_items = 0;
     std::vector<void*> src_slots, dst_slots;  // device buffers (dst == src when same GPU)
     std::vector<cudaEvent_t> ev_copied, ev_consumed, ev_produced;
+};
+
+struct IoBinding {
+    std::vector<const void*> in;
+    std::vector<int64_t> in_base, in_limit;
+    std::vector<void*> out;
+    std::vector<int64_t> out_base;
+};
+
+struct RankOp {
+    int32_t op, part, edge, peer;
+    int64_t frag, kb, ke, items;
 };
 
 struct GpuCtx {
@@ -72,10 +85,29 @@ struct Plan {
     size_t host_in_cap = 0, host_out_cap = 0;
     cudaStream_t host_stream = nullptr;
 
+    // one process per GPU (sg_dist.cpp)
+    void* comm = nullptr;  // ncclComm_t
+    int comm_rank = 0, comm_device = 0;
+    bool dist_ready = false;
+    int64_t dist_F = 0;
+    std::map<int, std::vector<void*>> dist_slots;
+    std::map<int, std::vector<cudaEvent_t>> dist_ev;
+    cudaStream_t dist_compute = nullptr, dist_comm = nullptr;
+    cudaEvent_t dist_join = nullptr;
+
     ~Plan();
     void run(const void* in, int64_t n, void* out, cudaStream_t stream);
     void run_host(const void* hin, int64_t n, void* hout);
+    void comm_init(int nranks, int rank, const uint8_t id[128], int device);
+    void run_rank(const void* in, int64_t n, void* out, cudaStream_t stream);
+    void dist_release();
 };
+
+int64_t launch_kernel(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int64_t ke, cudaStream_t stream,
+                      bool is_f32);
+int64_t fragment_size(const Plan& p, int64_t n);
+std::vector<RankOp> rank_schedule(const Plan& p, int rank, int64_t n, int64_t F);
+void nccl_unique_id(uint8_t out[128]);
 
 // NVRTC -> sm_100a cubin (cached by content hash in memory and on disk).
 void compile_kernel(CompiledKernel& ck, int verbose);

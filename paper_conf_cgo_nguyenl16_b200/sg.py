@@ -30,7 +30,9 @@ EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_split
            "sg_branch_end", "sg_plan_opts_default", "sg_plan", "sg_input_items", "sg_output_items",
            "sg_plan_info", "sg_plan_source", "sg_run", "sg_run_host", "sg_last_launch_count",
            "sg_plan_destroy", "sg_last_error", "sg_version", "sg_flush_l2", "sg_topology_links",
-           "sg_topology_dtlist", "sg_map_ilp", "sg_paper_model", "sg_plan_pdg"]
+           "sg_topology_dtlist", "sg_map_ilp", "sg_paper_model", "sg_plan_pdg", "sg_comm_unique_id", "sg_comm_init",
+           "sg_run_rank", "sg_rank_schedule"]
+SG_OP_LAUNCH, SG_OP_SEND, SG_OP_RECV = 0, 1, 2
 
 
 class SgError(RuntimeError):
@@ -51,6 +53,12 @@ class PlanOpts(ctypes.Structure):
                 ("virtual_gpus", ctypes.c_int32), ("devices", ctypes.POINTER(ctypes.c_int32)),
                 ("ilp_time_limit_ms", ctypes.c_int32), ("codegen_mode", ctypes.c_int32),
                 ("link_gbps", ctypes.c_double), ("link_latency_us", ctypes.c_double), ("verbose", ctypes.c_int32)]
+
+
+class RankOp(ctypes.Structure):
+    _fields_ = [("op", ctypes.c_int32), ("part", ctypes.c_int32), ("edge", ctypes.c_int32), ("peer", ctypes.c_int32),
+                ("fragment", ctypes.c_int64), ("k_begin", ctypes.c_int64), ("k_end", ctypes.c_int64),
+                ("items", ctypes.c_int64)]
 
 
 class PlanInfo(ctypes.Structure):
@@ -107,6 +115,10 @@ def lib():
                             ctypes.c_double, ctypes.c_double, ctypes.c_double, ctypes.POINTER(ctypes.c_double),
                             ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ctypes.c_double)], ctypes.c_double),
         "sg_plan_pdg": ([vp, i32, ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(ctypes.c_double)], i32),
+        "sg_comm_unique_id": ([ctypes.POINTER(ctypes.c_uint8)], ctypes.c_int),
+        "sg_comm_init": ([vp, i32, i32, ctypes.POINTER(ctypes.c_uint8), i32], ctypes.c_int),
+        "sg_run_rank": ([vp, vp, i64, vp, vp], ctypes.c_int),
+        "sg_rank_schedule": ([vp, i32, i64, ctypes.POINTER(RankOp), i64], i64),
     }
     for name, (args, res) in sig.items():
         fn = getattr(L, name)
@@ -279,6 +291,32 @@ class Plan:
         lib().sg_plan_pdg(self._h, n, a, b, c)
         return [(a[i], b[i], c[i]) for i in range(n)]
 
+    def rank_schedule(self, rank: int, n_iters: int):
+        """Host-side op list sg_run_rank issues on `rank`: dicts with op/part/edge/peer/fragment/..."""
+        cnt = lib().sg_rank_schedule(self._h, rank, n_iters, None, 0)
+        if cnt < 0:
+            raise SgError(SG_E_ARG, "bad rank / n_iters")
+        buf = (RankOp * max(1, cnt))()
+        lib().sg_rank_schedule(self._h, rank, n_iters, buf, cnt)
+        return [{"op": o.op, "part": o.part, "edge": o.edge, "peer": o.peer, "fragment": o.fragment,
+                 "k_begin": o.k_begin, "k_end": o.k_end, "items": o.items} for o in buf[:cnt]]
+
+    def comm_init(self, nranks: int, rank: int, uid: bytes, device: int):
+        arr = (ctypes.c_uint8 * 128)(*uid[:128])
+        _check(lib().sg_comm_init(self._h, nranks, rank, arr, device))
+
+    def run_rank(self, x, n_iters: int, y, stream=None):
+        """One process per GPU: run this rank's partitions; x / y only on the input / output rank."""
+        xp = 0 if x is None else (x.data_ptr() if hasattr(x, "data_ptr") else int(x))
+        yp = 0 if y is None else (y.data_ptr() if hasattr(y, "data_ptr") else int(y))
+        if stream is None:
+            import torch
+            stream = torch.cuda.current_stream().cuda_stream
+        elif hasattr(stream, "cuda_stream"):
+            stream = stream.cuda_stream
+        _check(lib().sg_run_rank(self._h, ctypes.c_void_p(xp or None), n_iters, ctypes.c_void_p(yp or None),
+                                 ctypes.c_void_p(stream)))
+
     def last_launch_count(self) -> int:
         return lib().sg_last_launch_count(self._h)
 
@@ -348,6 +386,12 @@ def paper_model(t, f, S, W, F, D, C1=38.4, C2=11.2):
     a, b, c = ctypes.c_double(), ctypes.c_double(), ctypes.c_double()
     T = lib().sg_paper_model(n, ta, fa, S, W, F, D, C1, C2, ctypes.byref(a), ctypes.byref(b), ctypes.byref(c))
     return T, a.value, b.value, c.value
+
+
+def comm_unique_id() -> bytes:
+    arr = (ctypes.c_uint8 * 128)()
+    _check(lib().sg_comm_unique_id(arr))
+    return bytes(arr)
 
 
 def version() -> str:

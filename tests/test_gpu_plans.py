@@ -168,3 +168,29 @@ def test_beamformer_full_size_sampled(oracle_lib):
     for f in list(rng.choice(n, 6, replace=False)) + [0, n - 1]:
         ref = oracle_lib.run(prog, x[24576 * f: 24576 * (f + 1)], 1)
         assert_parity(prog, y[2048 * f: 2048 * (f + 1)], ref)
+
+
+def test_run_rank_world1_nccl(oracle_lib):
+    """sg_run_rank through an NCCL communicator of one rank (the one-process-per-GPU path);
+    per-filter partitions exercise the local rings and event ordering of sg_dist.cpp."""
+    torch = _torch()
+    import os
+    import torch.distributed as dist
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan
+    if not dist.is_initialized():
+        os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+        os.environ.setdefault("MASTER_PORT", "29517")
+        dist.init_process_group("nccl", rank=0, world_size=1, device_id=torch.device("cuda", 0))
+    prog = apps.fmradio(4)
+    n = 2000
+    x = inputs.make_input("f32", oracle_lib.in_items(prog, n), 77)
+    ref = oracle_lib.run(prog, x, n)
+    for kw in (dict(), dict(partitioner="per_filter", iters_per_fragment=300)):
+        p = pipeline_plan(prog, **kw)
+        xd = torch.from_numpy(x).cuda()
+        yd = torch.empty(p.output_items(n), device="cuda")
+        p.run_rank(xd, n, yd)
+        torch.cuda.synchronize()
+        assert_parity(prog, yd.cpu().numpy(), ref)
+        p.close()
