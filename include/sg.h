@@ -140,6 +140,8 @@ typedef struct sg_plan_opts {
     double link_gbps;              /* NVLink bandwidth per direction for the ILP; 0 = 770 */
     double link_latency_us;        /* per-transfer latency Lat (Eq. III.3); 0 = 10 */
     int32_t verbose;
+    int32_t plan_only;             /* 1: stop after partitioning and mapping (no code generation,
+                                      no NVRTC); sg_run on such a plan returns SG_E_ARG */
 } sg_plan_opts;
 
 typedef struct sg_plan_info_s {

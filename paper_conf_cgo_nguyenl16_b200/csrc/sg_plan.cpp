@@ -610,6 +610,15 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     co.threads = o.threads;
     co.tile = o.tile_iters;
     for (int i = 0; i < P; i++) {
+        if (o.plan_only) {  // partitions and mapping only: keep the PEE's mode decision
+            p.kernels[i].ki.mode = register_mode_eligible(f, parts[i], nullptr) ? 1 : 2;
+            p.kernels[i].ki.tile = 1;
+            partition_boundary(f, parts[i], p.kernels[i].ki.in_edges, p.kernels[i].ki.out_edges);
+            p.part_mode[i] = p.kernels[i].ki.mode;
+            p.parts[i].mode = p.kernels[i].ki.mode;
+            p.parts[i].gpu = p.part_gpu[i];
+            continue;
+        }
         p.kernels[i].ki = generate_kernel(f, parts[i], i, co);
         compile_kernel(p.kernels[i], o.verbose);
         p.part_mode[i] = p.kernels[i].ki.mode;

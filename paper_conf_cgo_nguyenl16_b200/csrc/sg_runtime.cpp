@@ -361,6 +361,7 @@ Plan::~Plan() {
 
 void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
     if (n <= 0) return;
+    if (opts.plan_only) throw Error(SG_E_ARG, "plan was created with plan_only = 1");
     int ndev = 0;
     if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0) {
         cudaGetLastError();

@@ -52,7 +52,8 @@ class PlanOpts(ctypes.Structure):
                 ("iters_per_fragment", ctypes.c_int64), ("transport", ctypes.c_int32),
                 ("virtual_gpus", ctypes.c_int32), ("devices", ctypes.POINTER(ctypes.c_int32)),
                 ("ilp_time_limit_ms", ctypes.c_int32), ("codegen_mode", ctypes.c_int32),
-                ("link_gbps", ctypes.c_double), ("link_latency_us", ctypes.c_double), ("verbose", ctypes.c_int32)]
+                ("link_gbps", ctypes.c_double), ("link_latency_us", ctypes.c_double), ("verbose", ctypes.c_int32),
+                ("plan_only", ctypes.c_int32)]
 
 
 class RankOp(ctypes.Structure):
