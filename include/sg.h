@@ -223,6 +223,16 @@ sg_status sg_run(sg_plan_t* p, const void* input, int64_t n_iters, void* output,
 /* Same, with HOST buffers: copies in, runs, copies out, synchronises. */
 sg_status sg_run_host(sg_plan_t* p, const void* host_input, int64_t n_iters, void* host_output);
 
+/* Measured side of the PEE validation (Fig. 4.1: estimated vs
+ * measured partition time).  Runs every partition's kernel ALONE over iterations
+ * [0, n_iters), `reps` times after one warm-up launch, on zero-filled scratch
+ * boundary windows (the size sg_run's rings hold for one fragment of n_iters), and
+ * writes ns per iteration to ns_per_iter[0 .. n_partitions).  Synchronous;
+ * allocates and frees its scratch.  SG_E_ARG for n_iters <= 0, reps <= 0 or NULL;
+ * SG_E_CUDA without a device (no CPU fallback).  Compare with
+ * sg_plan_info_t.partition_time (the PEE estimate, ns per iteration). */
+sg_status sg_profile_partitions(sg_plan_t* p, int64_t n_iters, int32_t reps, double* ns_per_iter);
+
 /* Number of kernel launches the last sg_run enqueued (all devices). */
 int64_t sg_last_launch_count(const sg_plan_t* p);
 

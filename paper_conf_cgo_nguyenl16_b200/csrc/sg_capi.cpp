@@ -317,6 +317,12 @@ int64_t sg_rank_schedule(const sg_plan_t* p, int32_t rank, int64_t n, sg_rank_op
     }
 }
 
+sg_status sg_profile_partitions(sg_plan_t* p, int64_t n, int32_t reps, double* ns_per_iter) {
+    if (!p || !ns_per_iter) return fail(SG_E_ARG, "NULL argument");
+    if (n <= 0 || reps <= 0) return fail(SG_E_ARG, "n_iters and reps must be positive");
+    return guard([&] { p->plan.profile_partitions(n, reps, ns_per_iter); });
+}
+
 int64_t sg_last_launch_count(const sg_plan_t* p) { return p ? p->plan.last_launches : -1; }
 
 void sg_plan_destroy(sg_plan_t* p) { delete p; }

@@ -596,3 +596,76 @@ void Plan::run_host(const void* hin, int64_t n, void* hout) {
 }
 
 }  // namespace sg
+
+namespace sg {
+// Time every partition's kernel alone over iterations [0, n) (the measured side
+// of the PEE validation, Fig. 4.1 / PAPER.md:705-722).  Boundary streams come
+// from zero-filled scratch windows of exactly the size sg_run's rings would
+// hold for one fragment of n iterations; results in ns per iteration.
+void Plan::profile_partitions(int64_t n, int reps, double* ns_per_iter) {
+    if (n <= 0 || reps <= 0) throw Error(SG_E_ARG, "profile_partitions: n_iters and reps must be positive");
+    if (opts.plan_only) throw Error(SG_E_ARG, "plan was created with plan_only = 1");
+    int ndev = 0;
+    if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev <= 0) {
+        cudaGetLastError();
+        throw Error(SG_E_CUDA, "no CUDA device: the executor has no CPU fallback");
+    }
+    const int64_t n_in = flat.input_items(n);
+    for (size_t p = 0; p < parts.size(); p++) {
+        CompiledKernel& ck = kernels[p];
+        const int dev = devices[part_gpu[p]];
+        DevGuard dg(dev);
+        std::vector<void*> bufs;
+        auto scratch = [&](int64_t items) {
+            void* q = nullptr;
+            SG_RT(cudaMalloc(&q, (size_t)std::max<int64_t>(items, 1) * 4));
+            SG_RT(cudaMemset(q, 0, (size_t)std::max<int64_t>(items, 1) * 4));
+            bufs.push_back(q);
+            return q;
+        };
+        IoBinding io;
+        for (int e : ck.ki.in_edges) {
+            if (flat.edges[e].src < 0) {
+                io.in.push_back(scratch(n_in));
+                io.in_base.push_back(0);
+                io.in_limit.push_back(n_in);
+                continue;
+            }
+            int64_t lo, extra;
+            edge_window(flat, e, lo, extra);
+            int64_t items = flat.edges[e].per_iter * n + extra;
+            io.in.push_back(scratch(items));
+            io.in_base.push_back(lo);
+            io.in_limit.push_back(items);
+        }
+        for (int e : ck.ki.out_edges) {
+            if (flat.edges[e].dst < 0) {
+                io.out.push_back(scratch(flat.output_items(n)));
+                io.out_base.push_back(0);
+                continue;
+            }
+            int64_t lo, extra;
+            edge_window(flat, e, lo, extra);
+            io.out.push_back(scratch(flat.edges[e].per_iter * n + extra));
+            io.out_base.push_back(lo);
+        }
+        cudaStream_t s;
+        cudaEvent_t e0, e1;
+        SG_RT(cudaStreamCreateWithFlags(&s, cudaStreamNonBlocking));
+        SG_RT(cudaEventCreate(&e0));
+        SG_RT(cudaEventCreate(&e1));
+        launch(ck, dev, io, 0, n, s, flat.dtype == SG_F32);  // warm-up (module load, caches)
+        SG_RT(cudaEventRecord(e0, s));
+        for (int r = 0; r < reps; r++) launch(ck, dev, io, 0, n, s, flat.dtype == SG_F32);
+        SG_RT(cudaEventRecord(e1, s));
+        SG_RT(cudaEventSynchronize(e1));
+        float ms = 0;
+        SG_RT(cudaEventElapsedTime(&ms, e0, e1));
+        ns_per_iter[p] = (double)ms * 1e6 / ((double)reps * (double)n);
+        cudaEventDestroy(e0);
+        cudaEventDestroy(e1);
+        cudaStreamDestroy(s);
+        for (void* q : bufs) cudaFree(q);
+    }
+}
+}  // namespace sg

@@ -98,6 +98,7 @@ struct Plan {
     ~Plan();
     void run(const void* in, int64_t n, void* out, cudaStream_t stream);
     void run_host(const void* hin, int64_t n, void* hout);
+    void profile_partitions(int64_t n, int reps, double* ns_per_iter);
     void comm_init(int nranks, int rank, const uint8_t id[128], int device);
     void run_rank(const void* in, int64_t n, void* out, cudaStream_t stream);
     void dist_release();

@@ -31,7 +31,7 @@ EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_split
            "sg_plan_info", "sg_plan_source", "sg_run", "sg_run_host", "sg_last_launch_count",
            "sg_plan_destroy", "sg_last_error", "sg_version", "sg_flush_l2", "sg_topology_links",
            "sg_topology_dtlist", "sg_map_ilp", "sg_paper_model", "sg_plan_pdg", "sg_comm_unique_id", "sg_comm_init",
-           "sg_run_rank", "sg_rank_schedule"]
+           "sg_run_rank", "sg_rank_schedule", "sg_profile_partitions"]
 SG_OP_LAUNCH, SG_OP_SEND, SG_OP_RECV = 0, 1, 2
 
 
@@ -103,6 +103,7 @@ def lib():
         "sg_run": ([vp, vp, i64, vp, vp], ctypes.c_int),
         "sg_run_host": ([vp, vp, i64, vp], ctypes.c_int),
         "sg_last_launch_count": ([vp], i64),
+        "sg_profile_partitions": ([vp, i64, i32, ctypes.POINTER(ctypes.c_double)], ctypes.c_int),
         "sg_plan_destroy": ([vp], None),
         "sg_last_error": ([], ctypes.c_char_p),
         "sg_version": ([], ctypes.c_char_p),
@@ -317,6 +318,13 @@ class Plan:
             stream = stream.cuda_stream
         _check(lib().sg_run_rank(self._h, ctypes.c_void_p(xp or None), n_iters, ctypes.c_void_p(yp or None),
                                  ctypes.c_void_p(stream)))
+
+    def profile_partitions(self, n_iters: int, reps: int = 5):
+        """Measured ns/iteration of every partition's kernel run alone (PEE validation, Fig. 4.1)."""
+        k = self.info()["n_partitions"]
+        buf = (ctypes.c_double * max(1, k))()
+        _check(lib().sg_profile_partitions(self._h, n_iters, reps, buf))
+        return [buf[i] for i in range(k)]
 
     def last_launch_count(self) -> int:
         return lib().sg_last_launch_count(self._h)

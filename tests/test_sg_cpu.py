@@ -130,6 +130,12 @@ def test_run_without_gpu_fails_loudly(sg):
         with pytest.raises(sg.SgError) as e:
             p.run_host(x, 4, y)
         assert e.value.code == sg.SG_E_CUDA
+        with pytest.raises(sg.SgError) as e:
+            p.profile_partitions(4)
+        assert e.value.code == sg.SG_E_CUDA
+        with pytest.raises(sg.SgError) as e:
+            p.profile_partitions(0)
+        assert e.value.code == sg.SG_E_ARG
 
 
 # ---------------------------------------------------------------- topology
