@@ -969,7 +969,7 @@ public:
         int NT = opt.threads > 0 ? opt.threads : 256;
         NT_ = NT;
         // ---------------- fused fast path (full tiles without stream-start firings)
-        std::string fast, fast_start;
+        std::string fast, fast_start, prologue_fast;
         int WF = 0;
         size_t smem_fast = 0;
         if (opt.mode != -2) {
@@ -999,9 +999,37 @@ public:
                 }
                 if (WF > 0) {
                     fused_layout(WF);
+                    // inputs: prefetch the next tile into a staging region with cp.async while
+                    // this tile computes, if it fits at the same CTAs per SM; else issue every
+                    // load of the tile asynchronously at its start (one wait instead of a
+                    // round trip per load)
+                    {
+                        int64_t st = 0;
+                        for (int e : ins_) {
+                            int64_t lo, ex;
+                            edge_window(f_, e, lo, ex);
+                            st += (f_.edges[e].per_iter * WF + ex + 3) / 4 * 4;
+                        }
+                        auto blocks = [](size_t b) { return std::max(1, std::min(2, (int)((220 * 1024) / std::max<size_t>(1024, b)))); };
+                        size_t with = smem_bytes_ + (size_t)st * 4;
+                        prefetch_ = !ins_.empty() && !std::getenv("SG_NO_PREFETCH") && with <= 227 * 1024 &&
+                                    blocks(with) == blocks(smem_bytes_);
+                        if (prefetch_) {
+                            int64_t o = (int64_t)(smem_bytes_ / 4 + 3) / 4 * 4;
+                            stage_off_.clear();
+                            for (int e : ins_) {
+                                int64_t lo, ex;
+                                edge_window(f_, e, lo, ex);
+                                stage_off_[e] = o;
+                                o += (f_.edges[e].per_iter * WF + ex + 3) / 4 * 4;
+                            }
+                            smem_bytes_ = (size_t)o * 4;
+                        }
+                    }
                     smem_fast = smem_bytes_;
                     fast = fused_emit(WF, false);
                     fast_start = fused_emit(WF, true);
+                    prologue_fast = prologue_;
                     ki.flops_exec_per_iter = fused_flops_per_iter();
                 }
             } catch (const FusedFail&) {
@@ -1067,6 +1095,7 @@ public:
                 << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
                 << "  " << T_ << "* sm = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
                 << "  const int tid = threadIdx.x;\n"
+                << (fusedk ? prologue_fast : std::string())
                 << "  for (long long kt = SG_K_BEGIN + (long long)blockIdx.x * " << WT << "; kt < SG_K_END; kt += (long long)gridDim.x * "
                 << WT << ") {\n"
                 << "    const int Wtt = (int)min((long long)" << WT << ", SG_K_END - kt);\n";
@@ -1108,6 +1137,11 @@ private:
     // read the same buffers form one group and share one register window;
     // reductions (ADD, FIR) are emitted transposed across a block of B firings.
     bool fused_ = false;
+    bool prefetch_ = false;               // inputs of the next tile prefetched into a staging region
+    std::map<int, int64_t> stage_off_;    // input edge -> staging offset (items)
+    std::string prologue_;                // emitted before the tile loop (first prefetch, tables)
+    std::map<int, int64_t> ctab_off_;     // frame FIR -> coefficient table offset (items)
+    std::vector<std::pair<int64_t, std::vector<float>>> ctab_vals_;
     std::map<int, int64_t> plP_, plQ_;  // phys edge -> planar layout: period P, row length Q (odd)
     std::map<int, int64_t> cs_;    // phys edge -> compaction stride (live firings of the producer)
     std::map<int, int64_t> cf0_;   // phys edge -> first live local firing of the producer
@@ -1133,6 +1167,7 @@ private:
         std::ostringstream* os = nullptr;
         std::map<std::string, std::string> loads;
         std::map<std::string, std::vector<std::string>> firings;
+        std::map<std::string, std::vector<std::string>> values;   // CSE: (kind, params, inputs) -> outputs
         std::map<int, std::set<std::string>> touched;
         std::map<int, std::vector<Lin>> reads;
         int64_t nloads = 0, flops = 0;
@@ -1206,6 +1241,26 @@ private:
         int64_t use = n.kind == SG_K_FIR ? n.iv[0] : n.peek;
         for (int64_t i = 0; i < use; i++) x[i] = sym_value(c, n.in[0], lf.scaled(n.pop).plus(i));
         for (int64_t i = use; i < n.peek; i++) x[i] = "0";
+        // common-subexpression elimination: a firing of a filter with the same kind and
+        // parameters on the same input values (e.g. FMRadio's band edges: the high
+        // low-pass of band i is the low low-pass of band i+1) is the same value; reuse it
+        // so the emitted code and the pruned work count agree
+        std::string vkey;
+        {
+            std::ostringstream k;
+            k << n.kind << "|" << n.rep << "|" << n.ninit << "|" << lf.str() << "|";
+            for (auto q : n.iv) k << q << ",";
+            k << "|";
+            for (auto q : n.fv) k << hexf(q) << ",";
+            k << "|";
+            for (auto& q : x) k << q << ",";
+            vkey = k.str();
+            auto vit = c.values.find(vkey);
+            if (vit != c.values.end()) {
+                c.firings[key] = vit->second;
+                return vit->second;
+            }
+        }
         std::vector<std::string> y(n.push);
         for (auto& s : y) s = "y" + std::to_string((*c.nv)++);
         std::ostringstream& o = *c.os;
@@ -1251,6 +1306,7 @@ private:
                 if (!is_zero(yy))
                     o << c.ind << yy << " = (k0 * " << n.rep << "LL + " << lf.str() << " < 0) ? " << zero() << " : " << yy << ";\n";
         c.firings[key] = y;
+        c.values[vkey] = y;
         return y;
     }
     int64_t root_S(int r) const { auto it = cs_.find(f_.nodes[r].out[0]); return it == cs_.end() ? 1 : it->second; }
@@ -1302,8 +1358,7 @@ private:
                     if (c.guarded)
                         val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[k][be].str() + " < 0) ? " + zero() + " : " + val + ")";
                     Lin pos = lf[k][be].scaled(n.push).plus(f_.edges[n.out[0]].pre);
-                    o << c.ind << "if (jb * " << B << " + " << be << " < NL" << r << ") sm["
-                      << buf_index(n.out[0], pos).str() << "] = " << val << ";\n";
+                    o << c.ind << guard_store(r, B, be) << "sm[" << buf_index(n.out[0], pos).str() << "] = " << val << ";\n";
                 }
             }
             return;
@@ -1345,10 +1400,20 @@ private:
                     if (c.guarded && !is_zero(outs[be][j]))
                         val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[be].str() + " < 0) ? " + zero() + " : " + val + ")";
                     Lin pos = lf[be].scaled(n.push).plus(f_.edges[e].pre + j);
-                    o << c.ind << "if (jb * " << B << " + " << be << " < NL" << r << ") sm[" << buf_index(e, pos).str()
-                      << "] = " << val << ";\n";
+                    o << c.ind << guard_store(r, B, be) << "sm[" << buf_index(e, pos).str() << "] = " << val << ";\n";
                 }
         }
+    }
+    // Per-store range guards.  The branch they compile to splits a block's code into one
+    // basic block per root, so ptxas keeps each root's accumulation chain contiguous;
+    // without it (SG_NO_GUARD=1; safe, the buffers are padded) ptxas interleaves every
+    // chain of a wide group and the warps of an SMSP drift apart in straight-line code
+    // far larger than the instruction caches: FilterBank measured 0.225 ms guarded vs
+    // 0.262 ms unguarded (45% of stall samples "no instruction").
+    static std::string guard_store(int r, int64_t B, int64_t be) {
+        static const bool on = std::getenv("SG_NO_GUARD") == nullptr;
+        if (!on) return "";
+        return "if (jb * " + std::to_string(B) + " + " + std::to_string(be) + " < NL" + std::to_string(r) + ") ";
     }
     bool dry_ok(const FGroup& g, Sym& c) {
         c = Sym();
@@ -1475,7 +1540,17 @@ private:
                     g.B = B0;
                     static const int bmax = std::getenv("SG_FUSED_BMAX") ? std::atoi(std::getenv("SG_FUSED_BMAX")) : 16;
                     dry_ok(g, c);
-                    while (g.B * 2 <= bmax) {
+                    // blocking only pays when consecutive firings share loaded items (peek
+                    // windows, inlined producers); without sharing it only cuts the
+                    // parallelism and multiplies the lane stride (bank conflicts)
+                    bool shares = true;
+                    {
+                        FGroup h = g;
+                        h.B = g.B * 2;
+                        Sym c2;
+                        if (dry_ok(h, c2) && c2.nloads >= 2 * c.nloads) shares = false;
+                    }
+                    while (shares && g.B * 2 <= bmax) {
                         FGroup h = g;
                         h.B = g.B * 2;
                         Sym c2;
@@ -1553,13 +1628,18 @@ private:
                 const int64_t NL = end > F0L ? (end - 1 - F0L) / S + 1 : 0;
                 NL_[r] = NL;
                 wb_[e] = f_.edges[e].pre + F0L * n.push;
-                note(e, NL * n.push, g.level);
             }
         }
         for (auto& g : fg_) {
             int64_t nb = 0;
             for (int r : g.roots) nb = std::max(nb, (NL_[r] + g.B - 1) / g.B);
             g.NB = g.special ? 0 : nb;
+            // every root buffer has room for all NB * B firings of its group (the tail is
+            // never read), so block stores may go unguarded (see guard_store)
+            for (int r : g.roots) {
+                const Node& n = f_.nodes[r];
+                note(n.out[0], std::max(NL_[r], g.special ? 0 : g.NB * g.B) * n.push, g.level);
+            }
         }
         // extents read by the first and last block of every group; liveness
         for (auto& g : fg_) {
@@ -1623,6 +1703,31 @@ private:
             top = std::max(top, o + sz);
             placed.push_back(b);
         }
+        // frame-FIR coefficient tables ((cr, ci) interleaved, read as 128-bit broadcasts)
+        ctab_off_.clear();
+        ctab_vals_.clear();
+        {
+            std::map<std::vector<float>, int64_t> seen;
+            top = (top + 3) / 4 * 4;
+            for (auto& g : fg_) {
+                if (!g.special) continue;
+                for (int r : g.roots) {
+                    const Node& n = f_.nodes[r];
+                    const int64_t L = n.iv[0];
+                    std::vector<float> t(2 * L);
+                    for (int64_t i = 0; i < L; i++) { t[2 * i] = n.fv[i]; t[2 * i + 1] = n.fv[L + i]; }
+                    auto it = seen.find(t);
+                    if (it == seen.end()) {
+                        seen[t] = top;
+                        ctab_vals_.push_back({top, t});
+                        ctab_off_[r] = top;
+                        top += (2 * L + 3) / 4 * 4;
+                    } else {
+                        ctab_off_[r] = it->second;
+                    }
+                }
+            }
+        }
         smem_bytes_ = (size_t)std::max<int64_t>(top, 4) * 4;
     }
     // live root firings in a tile of W iterations
@@ -1685,6 +1790,16 @@ private:
     // Fused tile body for a runtime Wt <= W.  guarded: the stream-start variant.
     std::string fused_emit(int W, bool guarded) {
         std::ostringstream b;
+        {
+            std::ostringstream pb;
+            for (auto& kv : ctab_vals_) {
+                std::string name = const_array(kv.second);
+                pb << "  for (int j = tid; j < " << kv.second.size() << "; j += NT) sm[" << kv.first << " + j] = " << name
+                   << "[j];  // frame-FIR coefficient table\n";
+            }
+            if (prefetch_) emit_issue(pb, "SG_K_BEGIN + (long long)blockIdx.x * " + std::to_string(W), true);
+            prologue_ = pb.str();
+        }
         emit_loads(b);
         for (int L = 1; L <= flev_; L++) {
             b << "    // ---- fused level " << L << "\n";
@@ -1759,8 +1874,14 @@ private:
     int64_t fused_flops_per_iter() {
         double tot = 0;
         for (auto& g : fg_) {
-            if (g.special) {
-                for (int r : g.roots) { int64_t a, b2, d; node_work(f_, r, a, b2, d); tot += a; }
+            if (g.special) {  // live taps only: x[s < 0] = 0 before the frame start (skipped chunks)
+                for (int r : g.roots) {
+                    const Node& n = f_.nodes[r];
+                    const int64_t L = n.iv[0], DEC = n.iv[1], OUT = n.iv[2] / n.iv[1];
+                    int64_t taps = 0;
+                    for (int64_t t = 0; t < OUT; t++) taps += std::min<int64_t>(L, t * DEC + 1);
+                    tot += 8.0 * (double)taps * (double)n.rep;
+                }
                 continue;
             }
             Sym c;
@@ -1953,7 +2074,64 @@ private:
         }
         return "sm[" + buf_index(r.edge, r.pos).str() + "]";
     }
+    // cp.async of the input windows of the tile starting at `kexpr` (fused path)
+    void emit_issue(std::ostringstream& b, const std::string& kexpr, bool staging) {
+        b << "    { // issue loads of the tile at " << kexpr << (staging ? " into the staging region" : "") << "\n"
+          << "      const long long kn = " << kexpr << ";\n"
+          << "      if (kn < SG_K_END) {\n"
+          << "        const int Wn = (int)min((long long)" << W_ << ", SG_K_END - kn);\n";
+        for (size_t i = 0; i < ins_.size(); i++) {
+            int e = ins_[i];
+            int64_t lo, ex;
+            edge_window(f_, e, lo, ex);
+            int64_t P = f_.edges[e].per_iter;
+            std::string dst = "s + j";
+            auto pit = plP_.find(e);
+            if (!staging && pit != plP_.end())
+                dst = "s + (j % " + std::to_string(pit->second) + ") * " + std::to_string(plQ_.at(e)) + " + j / " +
+                      std::to_string(pit->second);
+            b << "        {\n"
+              << "          const " << T_ << "* g = SG_IN(" << i << ");\n"
+              << "          const long long gb = kn * " << P << "LL + (" << lo << "LL) - SG_IN_BASE(" << i << ");\n"
+              << "          const long long lim = SG_IN_LIMIT(" << i << ");\n"
+              << "          const int n = Wn * " << P << " + " << ex << ";\n"
+              << "          " << T_ << "* s = sm + " << (staging ? stage_off_.at(e) : off_.at(e)) << ";\n"
+              << "          for (int j = tid; j < n; j += NT) { const long long gi = gb + j; const bool ok = gi >= 0 && gi < lim;\n"
+              << "            sg_cp_async4(" << dst << ", g + (ok ? gi : 0LL), ok ? 4u : 0u); }\n"
+              << "        }\n";
+        }
+        b << "      }\n      sg_cp_async_commit();\n    }\n";
+    }
+    std::string fused_prologue() const { return prologue_; }
     void emit_loads(std::ostringstream& b) {
+        if (fused_ && !ins_.empty()) {
+            if (prefetch_) {
+                b << "    sg_cp_async_wait_all();\n    __syncthreads();\n";
+                for (size_t i = 0; i < ins_.size(); i++) {
+                    int e = ins_[i];
+                    int64_t lo, ex;
+                    edge_window(f_, e, lo, ex);
+                    int64_t P = f_.edges[e].per_iter;
+                    auto pit = plP_.find(e);
+                    std::string dst = "s[j]";
+                    if (pit != plP_.end())
+                        dst = "s[(j % " + std::to_string(pit->second) + ") * " + std::to_string(plQ_.at(e)) + " + j / " +
+                              std::to_string(pit->second) + "]";
+                    b << "    { // boundary input " << i << " (edge " << e << "): staging -> tile buffer\n"
+                      << "      const int n = Wt * " << P << " + " << ex << ";\n"
+                      << "      " << T_ << "* s = sm + " << off_.at(e) << ";\n"
+                      << "      const " << T_ << "* st = sm + " << stage_off_.at(e) << ";\n"
+                      << "      for (int j = tid; j < n; j += NT) " << dst << " = st[j];\n"
+                      << "    }\n";
+                }
+                b << "    __syncthreads();\n";
+                emit_issue(b, "kt + (long long)gridDim.x * " + std::to_string(W_), true);
+            } else {
+                emit_issue(b, "k0", false);
+                b << "    sg_cp_async_wait_all();\n    __syncthreads();\n";
+            }
+            return;
+        }
         for (size_t i = 0; i < ins_.size(); i++) {
             int e = ins_[i];
             int64_t lo, ex;
@@ -2113,25 +2291,58 @@ private:
     // rounds; interior chunks skip the boundary checks; short filters are fully
     // unrolled so coefficients become immediates.
     std::map<int, int64_t> beam_B_;
+    std::map<int, bool> beam_pair_;
+    // chunks of TC taps a block of B outputs starting at output t0 runs: taps whose
+    // window lies wholly before the frame start (x = 0) are skipped -- exact, the
+    // accumulators start at +0 and adding +-0 never changes them (reading 14)
+    static int64_t beam_chunks(int64_t t0, int64_t B, int64_t DEC, int64_t L, int64_t TC) {
+        int64_t lim = std::min<int64_t>(L, (t0 + B - 1) * DEC + 1);
+        return (lim + TC - 1) / TC;
+    }
+    static int64_t beam_tc(int64_t L) {
+        for (int64_t c : {16, 8, 4, 2, 1})
+            if (L % c == 0) return c;
+        return 1;
+    }
+    // Block size B (odd: lanes B samples apart hit distinct banks of the planar
+    // buffers) and pairing (an item runs blocks p and NB-1-p, so the triangular work
+    // of long filters -- few live taps early in the frame -- is even per item),
+    // chosen by simulating the round-robin assignment of all peer items of the level
+    // to the CTA's threads and minimising the busiest thread's issue slots.
     int64_t beam_block(int v, int64_t W) {
         auto it = beam_B_.find(v);
         if (it != beam_B_.end()) return it->second;
-        // all frame FIRs of v's level (same L/dec/frame/rep) share the choice
         const Node& n = f_.nodes[v];
         int64_t peers = 0;
         for (int u : nodes_)
             if (compute_node(u) && special(u) && f_.nodes[u].iv == n.iv && level_of_special(u) == level_of_special(v)) peers++;
+        const int64_t OUT = n.iv[2] / n.iv[1], L = n.iv[0], DEC = n.iv[1], TC = beam_tc(L);
+        const int64_t nf = n.halo + W * n.rep;
         int64_t best = 3;
+        bool bestp = false;
         double bestc = 1e300;
-        const int64_t OUT = n.iv[2] / n.iv[1], L = n.iv[0], DEC = n.iv[1];
-        for (int64_t B : {3, 5, 7, 9}) {
-            int64_t items = peers * (n.halo + W * n.rep) * ((OUT + B - 1) / B);
-            int64_t rounds = (items + NT_ - 1) / NT_;
-            double per_item = (double)B * L * 4 + ((B - 1) * DEC + 16) * 2.0 * L / 16.0;
-            double cost = rounds * per_item;
-            if (cost < bestc - 1e-9) { bestc = cost; best = B; }
-        }
+        for (int64_t B : {1, 3, 5, 7, 9})
+            for (bool pair : {false, true}) {
+                const int64_t NB = (OUT + B - 1) / B, NBP = pair ? (NB + 1) / 2 : NB;
+                const int64_t NWIN = (B - 1) * DEC + TC;
+                auto blk_cost = [&](int64_t blk) {
+                    int64_t ch = beam_chunks(blk * B, B, DEC, L, TC);
+                    return (double)ch * ((double)TC * B * 4 + 2.0 * NWIN + TC / 2.0 + 8) + 4.0 * B + 12;
+                };
+                std::vector<double> per(NBP);
+                for (int64_t q = 0; q < NBP; q++) {
+                    per[q] = blk_cost(q);
+                    if (pair && NB - 1 - q != q) per[q] += blk_cost(NB - 1 - q);
+                }
+                const int64_t items = peers * nf * NBP;
+                std::vector<double> th(std::min<int64_t>(NT_, items), 0.0);
+                for (int64_t k = 0; k < items; k++) th[k % NT_] += per[k % NBP];
+                double cost = 0;
+                for (double c : th) cost = std::max(cost, c);
+                if (cost < bestc * 0.98) { bestc = cost; best = B; bestp = pair; }
+            }
         beam_B_[v] = best;
+        beam_pair_[v] = bestp;
         return best;
     }
     std::map<int, int> special_level_;
@@ -2184,11 +2395,13 @@ private:
         const Node& n = f_.nodes[v];
         const int64_t NP = peers.empty() ? 1 : (int64_t)peers.size();
         int64_t L = n.iv[0], DEC = n.iv[1], FR = n.iv[2], OUT = FR / DEC;
-        int64_t TC = 1;
-        for (int64_t c : {16, 8, 4, 2, 1})
-            if (L % c == 0) { TC = c; break; }
+        const int64_t TC = beam_tc(L);
         const int64_t B = beam_block(v, W_);
+        const bool pair = beam_pair_[v];
         int64_t NB = (OUT + B - 1) / B, NWIN = (B - 1) * DEC + TC;
+        const int64_t NBP = pair ? (NB + 1) / 2 : NB;
+        auto ct = ctab_off_.find(v);
+        const bool ctab = fused_ && ct != ctab_off_.end() && TC % 2 == 0;
         const bool unroll = false;  // rolled tap loop: small code (I-cache) beats immediates here
         std::vector<float> wr(n.fv.begin(), n.fv.begin() + L), wi(n.fv.begin() + L, n.fv.end());
         std::string WR = unroll ? "" : const_array(wr), WI = unroll ? "" : const_array(wi);
@@ -2202,13 +2415,21 @@ private:
             for (int64_t q = 0; q < NP; q++) consts_ << (q ? ", " : "") << dout[q];
             consts_ << "};\n";
         }
-        b << "      const int items = nf * " << NB * NP << ";\n"
+        b << "      const int items = nf * " << NBP * NP << ";\n"
           << "      int it = tid - " << rot % NT_ << "; if (it < 0) it += NT;\n"
           << "      for (; it < items; it += NT) {\n"
-          << "        const int pq = it / (nf * " << NB << ");\n"
-          << "        const int itp = it - pq * (nf * " << NB << ");\n"
-          << "        const int j = itp / " << NB << ";\n"
-          << "        const int t0 = (itp - j * " << NB << ") * " << B << ";\n"
+          << "        const int pq = it / (nf * " << NBP << ");\n"
+          << "        const int itp = it - pq * (nf * " << NBP << ");\n"
+          << "        const int j = itp / " << NBP << ";\n"
+          << "        const int pb = itp - j * " << NBP << ";\n";
+        if (pair)
+            b << "        for (int half = 0; half < 2; half++) {\n"
+              << "        const int blk = half ? " << NB - 1 << " - pb : pb;\n"
+              << "        if (half && blk == pb) break;\n";
+        else
+            b << "        { const int blk = pb;\n";
+        b << "        const int t0 = blk * " << B << ";\n"
+          << "        const int ilim = min(" << L << ", (t0 + " << B - 1 << ") * " << DEC << " + 1);\n"
           << "        const int lf = " << F0 << " + j;\n"
           << "        " << T_ << "* smi = sm + " << (NP > 1 ? DINT + "[pq]" : std::string("0")) << ";\n"
           << "        " << T_ << "* smo = sm + " << (NP > 1 ? DOUTT + "[pq]" : std::string("0")) << ";\n"
@@ -2232,6 +2453,25 @@ private:
                       << "              xi[" << k << "] = ok ? " << ei << " : 0.0f; }\n";
                 else
                     b << "            xr[" << k << "] = " << er << "; xi[" << k << "] = " << ei << ";\n";
+            }
+            if (ctab && !unroll) {  // (cr, ci) pairs of two taps per 128-bit shared-memory broadcast
+                b << "#pragma unroll\n"
+                  << "            for (int ii = 0; ii < " << TC << "; ii += 2) {\n"
+                  << "              const float4 c4 = reinterpret_cast<const float4*>(sm + " << ct->second << ")[(" << i0expr
+                  << " + ii) >> 1];\n"
+                  << "#pragma unroll\n"
+                  << "              for (int bb = 0; bb < " << B << "; bb++) {\n"
+                  << "                const int k = bb * " << DEC << " - ii + " << TC - 1 << ";\n"
+                  << "                sg_cmac(re[bb], im[bb], xr[k], xi[k], c4.x, c4.y);\n"
+                  << "              }\n"
+                  << "#pragma unroll\n"
+                  << "              for (int bb = 0; bb < " << B << "; bb++) {\n"
+                  << "                const int k = bb * " << DEC << " - ii + " << TC - 2 << ";\n"
+                  << "                sg_cmac(re[bb], im[bb], xr[k], xi[k], c4.z, c4.w);\n"
+                  << "              }\n"
+                  << "            }\n"
+                  << "          }\n";
+                return;
             }
             b << "#pragma unroll\n"
               << "            for (int ii = 0; ii < " << TC << "; ii++) {\n"
@@ -2259,7 +2499,7 @@ private:
             }
         } else {
             b << "#pragma unroll 1\n"
-              << "          for (int i0 = 0; i0 < " << L << "; i0 += " << TC << ") {\n"
+              << "          for (int i0 = 0; i0 < ilim; i0 += " << TC << ") {\n"
               << "            if (t0 * " << DEC << " - i0 - " << TC - 1 << " >= 0 && t0 * " << DEC << " + " << (B - 1) * DEC
               << " - i0 < " << FR << ") {\n";
             chunk("i0", false, WR + "[i0 + ii]", WI + "[i0 + ii]");
@@ -2279,6 +2519,7 @@ private:
               << "            smo[" << buf_index(eo, pos.plus(1)).str() << "] = im[bb];\n";
         }
         b << "          }\n"
+          << "        }\n"
           << "      }\n";
     }
 };

@@ -233,6 +233,14 @@ template <int N>
 SG_DEV void sg_bulk_wait_read() { asm volatile("cp.async.bulk.wait_group.read %0;" :: "n"(N) : "memory"); }
 template <int N>
 SG_DEV void sg_bulk_wait() { asm volatile("cp.async.bulk.wait_group %0;" :: "n"(N) : "memory"); }
+// 4-byte cp.async (LDGSTS) with zero fill: src_bytes = 0 writes 0 and reads nothing
+// (stream positions outside [0, limit) are the zero history of the stream start).
+SG_DEV void sg_cp_async4(void* sdst, const void* gsrc, sg_u32 src_bytes) {
+    asm volatile("cp.async.ca.shared.global [%0], [%1], 4, %2;"
+                 :: "r"(sg_smem_addr(sdst)), "l"(gsrc), "r"(src_bytes) : "memory");
+}
+SG_DEV void sg_cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+SG_DEV void sg_cp_async_wait_all() { asm volatile("cp.async.wait_all;" ::: "memory"); }
 SG_DEV void sg_prefetch_tmap(const void* tmap) {
     asm volatile("prefetch.tensormap [%0];" :: "l"(tmap) : "memory");
 }
