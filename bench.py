@@ -161,6 +161,8 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-flush", action="store_true")
     ap.add_argument("--eager", action="store_true", help="launch sg_run every step instead of replaying a CUDA graph")
+    ap.add_argument("--tile", type=int, default=0, help="plan option tile_iters (0: chosen by the code generator)")
+    ap.add_argument("--threads", type=int, default=0, help="plan option threads per CTA (0: chosen)")
     ap.add_argument("--mode", default="replicas", choices=["replicas", "pipeline"],
                     help="N>1: independent replicas (default; the headline graph is HBM-bound) or the paper's "
                          "pipelined partition mapping, one process per GPU, NCCL boundary streams")
@@ -190,7 +192,12 @@ def main():
         from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan
         plan = pipeline_plan(prog)
     else:
-        plan = sg.plan(prog, 1, devices=[local])
+        kw = {}
+        if args.tile:
+            kw["tile_iters"] = args.tile
+        if args.threads:
+            kw["threads"] = args.threads
+        plan = sg.plan(prog, 1, devices=[local], **kw)
     info = plan.info()
     nin, nout = plan.input_items(n), plan.output_items(n)
     dt = torch.int32 if prog.dtype == "i32" else torch.float32

@@ -976,7 +976,8 @@ public:
             try {
                 fused_ = true;
                 fused_analyze();
-                size_t fb = opt.smem_budget > 0 ? (size_t)opt.smem_budget : (size_t)(110 * 1024);
+                size_t fb = opt.smem_budget > 0 ? (size_t)opt.smem_budget
+                                                : (size_t)((opt.tile > 0 ? 227 : 110) * 1024);  // a forced tile may use it all
                 for (int cand : fused_tile_candidates(opt.tile)) {
                     fused_layout(cand);
                     if (smem_bytes_ <= fb) { WF = cand; break; }
@@ -1168,6 +1169,8 @@ private:
         std::map<std::string, std::string> loads;
         std::map<std::string, std::vector<std::string>> firings;
         std::map<std::string, std::vector<std::string>> values;   // CSE: (kind, params, inputs) -> outputs
+        bool lockstep = false;                     // every thread runs the block (act: stores)
+        int64_t sync_every = 0, since = 0;         // fetch-locality barriers every ~sync_every FP ops
         std::map<int, std::set<std::string>> touched;
         std::map<int, std::vector<Lin>> reads;
         int64_t nloads = 0, flops = 0;
@@ -1315,51 +1318,66 @@ private:
         auto it = cf0_.find(e);
         return it == cf0_.end() ? f_.nodes[r].ninit - f_.nodes[r].halo : it->second;
     }
+    void sym_fir_chunk(Sym& c, const FGroup& g, const std::vector<int>& roots, bool emit_stores) {
+        std::ostringstream& o = *c.os;
+        const int64_t B = g.B;
+        int64_t maxL = 0;
+        std::vector<std::vector<Lin>> lf(roots.size(), std::vector<Lin>(B));
+        std::vector<std::vector<std::string>> acc(roots.size(), std::vector<std::string>(B));
+        for (size_t k = 0; k < roots.size(); k++) {
+            int r = roots[k];
+            const int64_t S = root_S(r), F0L = root_F0L(r);
+            maxL = std::max<int64_t>(maxL, f_.nodes[r].iv[0]);
+            c.node_firings[r] += B;
+            for (int64_t be = 0; be < B; be++) {
+                lf[k][be] = Lin::v("jb", S * B, F0L + S * be);
+                acc[k][be] = "a" + std::to_string((*c.nv)++);
+                if (!c.dry) o << c.ind << "float " << acc[k][be] << " = 0.0f;\n";
+            }
+        }
+        for (int64_t i = 0; i < maxL; i++)
+            for (size_t k = 0; k < roots.size(); k++) {
+                const Node& n = f_.nodes[roots[k]];
+                if (i >= n.iv[0]) continue;
+                for (int64_t be = 0; be < B; be++) {
+                    std::string x = sym_value(c, n.in[0], lf[k][be].scaled(n.pop).plus(i));
+                    if (is_zero(x)) continue;
+                    c.flops += 2;
+                    c.node_flops[roots[k]] += 2;
+                    if (!c.dry) o << c.ind << acc[k][be] << " = fmaf(" << x << ", " << hexf(n.fv[i]) << ", " << acc[k][be] << ");\n";
+                }
+            }
+        if (c.dry || !emit_stores) return;
+        for (size_t k = 0; k < roots.size(); k++) {
+            const Node& n = f_.nodes[roots[k]];
+            const int r = roots[k];
+            for (int64_t be = 0; be < B; be++) {
+                std::string val = acc[k][be];
+                if (c.guarded)
+                    val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[k][be].str() + " < 0) ? " + zero() + " : " + val + ")";
+                Lin pos = lf[k][be].scaled(n.push).plus(f_.edges[n.out[0]].pre);
+                o << c.ind << guard_store(r, B, be, c.lockstep) << "sm[" << buf_index(n.out[0], pos).str() << "] = " << val << ";\n";
+            }
+        }
+    }
     // One block of a group: roots' live firings F0L + S*(jb*B + beta), beta < B.
     void sym_block(Sym& c, const FGroup& g, bool emit_stores) {
         std::ostringstream& o = *c.os;
-        static const bool interleave = std::getenv("SG_INTERLEAVE") != nullptr;  // measured slower by default
-        bool all_fir = g.roots.size() > 1 && interleave;
+        // Sibling FIR roots (one shared window) are emitted in chunks of SG_PAIRS roots with
+        // their taps interleaved (taps outer, chunk roots and block firings inner): each warp
+        // gets that many independent accumulation chains, while the store guards between
+        // chunks keep ptxas from interleaving the whole group (which scatters the warps of an
+        // SMSP over the group's straight-line code).  SG_INTERLEAVE=1: one chunk (all roots).
+        static const int pairs_env = std::getenv("SG_PAIRS") ? std::atoi(std::getenv("SG_PAIRS")) : 2;
+        static const bool interleave = std::getenv("SG_INTERLEAVE") != nullptr;
+        bool all_fir = g.roots.size() > 1 && (interleave || pairs_env > 1);
         for (int r : g.roots) all_fir = all_fir && f_.nodes[r].kind == SG_K_FIR;
-        if (all_fir) {  // sibling FIRs: taps outer, roots and block inner -> independent chains, window loaded once
-            const int64_t B = g.B;
-            int64_t maxL = 0;
-            std::vector<std::vector<Lin>> lf(g.roots.size(), std::vector<Lin>(B));
-            std::vector<std::vector<std::string>> acc(g.roots.size(), std::vector<std::string>(B));
-            for (size_t k = 0; k < g.roots.size(); k++) {
-                int r = g.roots[k];
-                const int64_t S = root_S(r), F0L = root_F0L(r);
-                maxL = std::max<int64_t>(maxL, f_.nodes[r].iv[0]);
-                c.node_firings[r] += B;
-                for (int64_t be = 0; be < B; be++) {
-                    lf[k][be] = Lin::v("jb", S * B, F0L + S * be);
-                    acc[k][be] = "a" + std::to_string((*c.nv)++);
-                    if (!c.dry) o << c.ind << "float " << acc[k][be] << " = 0.0f;\n";
-                }
-            }
-            for (int64_t i = 0; i < maxL; i++)
-                for (size_t k = 0; k < g.roots.size(); k++) {
-                    const Node& n = f_.nodes[g.roots[k]];
-                    if (i >= n.iv[0]) continue;
-                    for (int64_t be = 0; be < B; be++) {
-                        std::string x = sym_value(c, n.in[0], lf[k][be].scaled(n.pop).plus(i));
-                        if (is_zero(x)) continue;
-                        c.flops += 2;
-                        c.node_flops[g.roots[k]] += 2;
-                        if (!c.dry) o << c.ind << acc[k][be] << " = fmaf(" << x << ", " << hexf(n.fv[i]) << ", " << acc[k][be] << ");\n";
-                    }
-                }
-            if (c.dry || !emit_stores) return;
-            for (size_t k = 0; k < g.roots.size(); k++) {
-                const Node& n = f_.nodes[g.roots[k]];
-                const int r = g.roots[k];
-                for (int64_t be = 0; be < B; be++) {
-                    std::string val = acc[k][be];
-                    if (c.guarded)
-                        val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[k][be].str() + " < 0) ? " + zero() + " : " + val + ")";
-                    Lin pos = lf[k][be].scaled(n.push).plus(f_.edges[n.out[0]].pre);
-                    o << c.ind << guard_store(r, B, be) << "sm[" << buf_index(n.out[0], pos).str() << "] = " << val << ";\n";
-                }
+        if (all_fir) {
+            const size_t P = interleave ? g.roots.size() : (size_t)pairs_env;
+            for (size_t k0 = 0; k0 < g.roots.size(); k0 += P) {
+                std::vector<int> chunk(g.roots.begin() + k0, g.roots.begin() + std::min(g.roots.size(), k0 + P));
+                sym_fir_chunk(c, g, chunk, emit_stores);
+                fetch_sync(c, 0);
             }
             return;
         }
@@ -1378,7 +1396,8 @@ private:
                     if (!c.dry) o << c.ind << "float " << acc[be] << " = 0.0f;\n";
                 }
                 c.node_firings[r] += B;
-                for (int64_t i = 0; i < terms; i++)
+                for (int64_t i = 0; i < terms; i++) {
+                    const int64_t f0 = c.flops;
                     for (int64_t be = 0; be < B; be++) {
                         std::string x = sym_value(c, n.in[0], lf[be].scaled(n.pop).plus(i));
                         if (is_zero(x)) continue;
@@ -1388,6 +1407,8 @@ private:
                         if (fir) o << c.ind << acc[be] << " = fmaf(" << x << ", " << hexf(n.fv[i]) << ", " << acc[be] << ");\n";
                         else o << c.ind << acc[be] << " = " << acc[be] << " + " << x << ";\n";
                     }
+                    fetch_sync(c, (c.flops - f0 + 1) / 2);
+                }
                 for (int64_t be = 0; be < B; be++) outs[be] = {acc[be]};
             } else {
                 for (int64_t be = 0; be < B; be++) outs[be] = sym_firing(c, r, lf[be]);
@@ -1400,8 +1421,9 @@ private:
                     if (c.guarded && !is_zero(outs[be][j]))
                         val = "((k0 * " + std::to_string(n.rep) + "LL + " + lf[be].str() + " < 0) ? " + zero() + " : " + val + ")";
                     Lin pos = lf[be].scaled(n.push).plus(f_.edges[e].pre + j);
-                    o << c.ind << guard_store(r, B, be) << "sm[" << buf_index(e, pos).str() << "] = " << val << ";\n";
+                    o << c.ind << guard_store(r, B, be, c.lockstep) << "sm[" << buf_index(e, pos).str() << "] = " << val << ";\n";
                 }
+            fetch_sync(c, 0);
         }
     }
     // Per-store range guards.  The branch they compile to splits a block's code into one
@@ -1410,8 +1432,17 @@ private:
     // chain of a wide group and the warps of an SMSP drift apart in straight-line code
     // far larger than the instruction caches: FilterBank measured 0.225 ms guarded vs
     // 0.262 ms unguarded (45% of stall samples "no instruction").
-    static std::string guard_store(int r, int64_t B, int64_t be) {
+    void fetch_sync(Sym& c, int64_t ops) {
+        if (c.dry || !c.lockstep || c.sync_every <= 0) return;
+        c.since += ops;
+        if (c.since >= c.sync_every) {
+            *c.os << c.ind << "__syncthreads();  // fetch locality\n";
+            c.since = 0;
+        }
+    }
+    static std::string guard_store(int r, int64_t B, int64_t be, bool lockstep = false) {
         static const bool on = std::getenv("SG_NO_GUARD") == nullptr;
+        if (lockstep) return "if (act && jb * " + std::to_string(B) + " + " + std::to_string(be) + " < NL" + std::to_string(r) + ") ";
         if (!on) return "";
         return "if (jb * " + std::to_string(B) + " + " + std::to_string(be) + " < NL" + std::to_string(r) + ") ";
     }
@@ -1818,13 +1849,31 @@ private:
                       << " + 1;\n"
                       << "      NBg = max(NBg, (NL" << r << " + " << g.B - 1 << ") / " << g.B << ");\n";
                 }
-                b << "      int jb = tid - " << rot % NT_ << "; if (jb < 0) jb += NT;\n"
-                  << "      for (; jb < NBg; jb += NT) {\n";
+                // lockstep: a level with one large group whose blocks fit one round runs every
+                // thread through the block once (idle threads recompute the last block and
+                // store nothing) with __syncthreads() every ~512 FP instructions, so the warps
+                // of a CTA stay within a few KB of straight-line code (instruction-fetch
+                // locality; FilterBank's levels are 35-46 KB of code each)
+                int nlev_groups = 0;
+                for (auto& h : fg_) if (h.level == L) nlev_groups++;
+                static const bool fetchbar = std::getenv("SG_FETCHBAR") != nullptr;  // measured neutral-to-worse
+                const bool lockstep = fetchbar && nlev_groups == 1 && g.NB <= NT_ && g.flops_block >= 2048;
                 Sym c;
                 c.dry = false;
                 c.os = &b;
                 c.nv = &nvar_;
                 c.guarded = guarded;
+                if (lockstep) {
+                    b << "      if (NBg > 0) {\n"
+                      << "      const bool act = tid < NBg;\n"
+                      << "      const int jb = act ? tid : NBg - 1;\n";
+                    c.lockstep = true;
+                    static const int every = std::getenv("SG_FETCHBAR_OPS") ? std::atoi(std::getenv("SG_FETCHBAR_OPS")) : 512;
+                    c.sync_every = every;
+                } else {
+                    b << "      int jb = tid - " << rot % NT_ << "; if (jb < 0) jb += NT;\n"
+                      << "      for (; jb < NBg; jb += NT) {\n";
+                }
                 sym_block(c, g, true);
                 if (c.runtime) throw FusedFail();
                 b << "      }\n    }\n";

@@ -45,13 +45,41 @@ extern "C" __global__ void f_ucst(float* out, float a0, float b0) {
     float s = 0; for (int i = 0; i < 8; i++) s += acc[i];
     out[blockIdx.x * blockDim.x + threadIdx.x] = s;
 }
+__constant__ float2 CC2[64];
+extern "C" __global__ void f_ffma2_reg(float* out, float a0, float b0) {
+    float2 x[8], c[8], acc[8];
+    for (int i = 0; i < 8; i++) { x[i] = make_float2(a0 + i + threadIdx.x, a0 - i); c[i] = make_float2(b0 * (i + 1), b0 - i); acc[i] = make_float2(0.f, 0.f); }
+    #pragma unroll 1
+    for (int it = 0; it < N_IT / 2; it++) {
+        #pragma unroll
+        for (int r = 0; r < 8; r++)
+            #pragma unroll
+            for (int i = 0; i < 8; i++) acc[i] = __ffma2_rn(x[(i + r) & 7], c[(i * 3 + r) & 7], acc[i]);
+    }
+    float s = 0; for (int i = 0; i < 8; i++) s += acc[i].x + acc[i].y;
+    out[blockIdx.x * blockDim.x + threadIdx.x] = s;
+}
+extern "C" __global__ void f_ffma2_cst(float* out, float a0, float b0) {
+    float2 x[8], acc[8];
+    for (int i = 0; i < 8; i++) { x[i] = make_float2(a0 + i + threadIdx.x, a0 - i); acc[i] = make_float2(0.f, 0.f); }
+    #pragma unroll 1
+    for (int it = 0; it < N_IT / 2; it++) {
+        #pragma unroll
+        for (int r = 0; r < 8; r++)
+            #pragma unroll
+            for (int i = 0; i < 8; i++) acc[i] = __ffma2_rn(x[(i + r) & 7], CC2[(i * 3 + r) & 63], acc[i]);
+    }
+    float s = 0; for (int i = 0; i < 8; i++) s += acc[i].x + acc[i].y;
+    out[blockIdx.x * blockDim.x + threadIdx.x] = s;
+}
 int main() {
     float* d; cudaMalloc(&d, 148 * 8 * 256 * 4);
     float h[64]; for (int i = 0; i < 64; i++) h[i] = 1.0f + i * 0.01f;
     cudaMemcpyToSymbol(CC, h, sizeof h);
+    cudaMemcpyToSymbol(CC2, h, sizeof h);
     int sm; cudaDeviceGetAttribute(&sm, cudaDevAttrMultiProcessorCount, 0);
     int clk; cudaDeviceGetAttribute(&clk, cudaDevAttrClockRate, 0);
-    struct { const char* n; void (*k)(float*, float, float); } ks[] = {{"reg3", f_reg3}, {"imm", f_imm}, {"ucst", f_ucst}};
+    struct { const char* n; void (*k)(float*, float, float); } ks[] = {{"reg3", f_reg3}, {"imm", f_imm}, {"ucst", f_ucst}, {"ffma2_reg", f_ffma2_reg}, {"ffma2_cst", f_ffma2_cst}};
     for (auto& k : ks) {
         for (int rep = 0; rep < 2; rep++) {
             cudaEvent_t a, b; cudaEventCreate(&a); cudaEventCreate(&b);
