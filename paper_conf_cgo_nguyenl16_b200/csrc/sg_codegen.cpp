@@ -988,8 +988,12 @@ public:
                 }
                 if (WF > 0 && opt.threads <= 0) {
                     fused_layout(WF);
-                    if (smem_bytes_ > 113 * 1024) {  // one CTA per SM: give it 16 warps
-                        NT_ = NT = 512;
+                    if (smem_bytes_ > 113 * 1024) {  // one CTA per SM: give it 16 warps (32 for frame
+                        // FIR partitions: their blocks fit 64 registers and the extra warps hide the
+                        // shared-memory latency of the sample windows; BeamFormer 2.69 -> 2.57 ms)
+                        bool frame = false;
+                        for (auto& g : fg_) frame = frame || g.special;
+                        NT_ = NT = frame ? 1024 : 512;
                         int W2 = 0;
                         for (int cand : fused_tile_candidates(opt.tile)) {
                             fused_layout(cand);
@@ -1141,6 +1145,7 @@ private:
     bool prefetch_ = false;               // inputs of the next tile prefetched into a staging region
     std::map<int, int64_t> stage_off_;    // input edge -> staging offset (items)
     std::string prologue_;                // emitted before the tile loop (first prefetch, tables)
+    int nctr_ = 0;                        // shared work counters used by the fused body (dynamic items)
     std::map<int, int64_t> ctab_off_;     // frame FIR -> coefficient table offset (items)
     std::vector<std::pair<int64_t, std::vector<float>>> ctab_vals_;
     std::map<int, int64_t> plP_, plQ_;  // phys edge -> planar layout: period P, row length Q (odd)
@@ -1821,6 +1826,17 @@ private:
     // Fused tile body for a runtime Wt <= W.  guarded: the stream-start variant.
     std::string fused_emit(int W, bool guarded) {
         std::ostringstream b;
+        nctr_ = 0;
+        std::ostringstream body;
+        std::string r = fused_emit_body(W, guarded, body);
+        if (nctr_ > 0)  // work counters: zeroed at tile start (the previous tile ended with a barrier,
+                        // the post-load barrier orders the reset before the first level)
+            b << "    __shared__ int sg_ctr[" << nctr_ << "];\n"
+              << "    if (tid < " << nctr_ << ") sg_ctr[tid] = 0;\n";
+        b << r;
+        return b.str();
+    }
+    std::string fused_emit_body(int W, bool guarded, std::ostringstream& b) {
         {
             std::ostringstream pb;
             for (auto& kv : ctab_vals_) {
@@ -2384,10 +2400,17 @@ private:
                     if (pair && NB - 1 - q != q) per[q] += blk_cost(NB - 1 - q);
                 }
                 const int64_t items = peers * nf * NBP;
-                std::vector<double> th(std::min<int64_t>(NT_, items), 0.0);
-                for (int64_t k = 0; k < items; k++) th[k % NT_] += per[k % NBP];
                 double cost = 0;
-                for (double c : th) cost = std::max(cost, c);
+                if (fused_ && !std::getenv("SG_STATIC_ITEMS")) {
+                    // dynamic scheduling: warps take 32-item chunks until the level is done
+                    double sum = 0, mx = 0;
+                    for (int64_t k = 0; k < items; k++) { sum += per[k % NBP]; mx = std::max(mx, per[k % NBP]); }
+                    cost = std::max(sum / NT_, mx) + mx * 0.5;
+                } else {
+                    std::vector<double> th(std::min<int64_t>(NT_, items), 0.0);
+                    for (int64_t k = 0; k < items; k++) th[k % NT_] += per[k % NBP];
+                    for (double c : th) cost = std::max(cost, c);
+                }
                 if (cost < bestc * 0.98) { bestc = cost; best = B; bestp = pair; }
             }
         beam_B_[v] = best;
@@ -2464,9 +2487,24 @@ private:
             for (int64_t q = 0; q < NP; q++) consts_ << (q ? ", " : "") << dout[q];
             consts_ << "};\n";
         }
-        b << "      const int items = nf * " << NBP * NP << ";\n"
-          << "      int it = tid - " << rot % NT_ << "; if (it < 0) it += NT;\n"
-          << "      for (; it < items; it += NT) {\n"
+        b << "      const int items = nf * " << NBP * NP << ";\n";
+        // dynamic item scheduling (fused kernels): warps grab 32 consecutive items from a
+        // shared counter, so warps the scheduler favours (highest warp id first) take more
+        // items and the level's tail is one item per thread, not a whole static share
+        const bool dyn = fused_ && !std::getenv("SG_STATIC_ITEMS");
+        if (dyn) {
+            const int slot = nctr_++;
+            b << "      for (int it0 = 0;;) {\n"
+              << "        if ((tid & 31) == 0) it0 = atomicAdd(&sg_ctr[" << slot << "], 32);\n"
+              << "        it0 = __shfl_sync(0xffffffffu, it0, 0);\n"
+              << "        if (it0 >= items) break;\n"
+              << "        const int it = it0 + (tid & 31);\n"
+              << "        if (it < items) {\n";
+        } else {
+            b << "      int it = tid - " << rot % NT_ << "; if (it < 0) it += NT;\n"
+              << "      for (; it < items; it += NT) {\n";
+        }
+        b
           << "        const int pq = it / (nf * " << NBP << ");\n"
           << "        const int itp = it - pq * (nf * " << NBP << ");\n"
           << "        const int j = itp / " << NBP << ";\n"
@@ -2475,6 +2513,8 @@ private:
             b << "        for (int half = 0; half < 2; half++) {\n"
               << "        const int blk = half ? " << NB - 1 << " - pb : pb;\n"
               << "        if (half && blk == pb) break;\n";
+        else if (dyn)  // longest blocks (most live taps) first: the dynamic tail is short
+            b << "        { const int blk = " << NB - 1 << " - pb;\n";
         else
             b << "        { const int blk = pb;\n";
         b << "        const int t0 = blk * " << B << ";\n"
@@ -2568,8 +2608,9 @@ private:
               << "            smo[" << buf_index(eo, pos.plus(1)).str() << "] = im[bb];\n";
         }
         b << "          }\n"
-          << "        }\n"
-          << "      }\n";
+          << "        }\n";
+        if (dyn) b << "        }\n";
+        b << "      }\n";
     }
 };
 
