@@ -993,7 +993,9 @@ public:
                         // shared-memory latency of the sample windows; BeamFormer 2.69 -> 2.57 ms)
                         bool frame = false;
                         for (auto& g : fg_) frame = frame || g.special;
-                        NT_ = NT = frame ? 1024 : 512;
+                        // (opt-in FFMA2 frame FIRs, SG_FFMA2=1, need the 128 registers of 512-thread
+                        // CTAs; measured slower: BeamFormer 2.88 ms vs 2.56 ms scalar at 1024 threads)
+                        NT_ = NT = (frame && !std::getenv("SG_FFMA2")) ? 1024 : 512;
                         int W2 = 0;
                         for (int cand : fused_tile_candidates(opt.tile)) {
                             fused_layout(cand);
@@ -2356,7 +2358,7 @@ private:
     // rounds; interior chunks skip the boundary checks; short filters are fully
     // unrolled so coefficients become immediates.
     std::map<int, int64_t> beam_B_;
-    std::map<int, bool> beam_pair_;
+    std::map<int, bool> beam_pair_, beam_f2_;
     // chunks of TC taps a block of B outputs starting at output t0 runs: taps whose
     // window lies wholly before the frame start (x = 0) are skipped -- exact, the
     // accumulators start at +0 and adding +-0 never changes them (reading 14)
@@ -2384,8 +2386,27 @@ private:
         const int64_t OUT = n.iv[2] / n.iv[1], L = n.iv[0], DEC = n.iv[1], TC = beam_tc(L);
         const int64_t nf = n.halo + W * n.rep;
         int64_t best = 3;
-        bool bestp = false;
+        bool bestp = false, bestf2 = false;
         double bestc = 1e300;
+        const bool dynsched = fused_ && !std::getenv("SG_STATIC_ITEMS");
+        // FFMA2 mode (fused, dynamic scheduling, coefficient table): a thread runs blocks
+        // blk and blk + 32 as the two halves of packed fp32x2 FMAs (Blackwell FFMA2)
+        if (dynsched && std::getenv("SG_FFMA2") && L % 2 == 0 && NT_ <= 512)
+            for (int64_t B : {1, 3, 5}) {
+                const int64_t NB = (OUT + B - 1) / B, NBH = (NB + 63) / 64 * 32;
+                const int64_t NWIN = (B - 1) * DEC + beam_tc(L);
+                double sum = 0, mx = 0;
+                for (int64_t q = 0; q < NBH; q++) {
+                    const int64_t a = q / 32 * 64 + q % 32, bb = std::min(a + 32, NB - 1);
+                    const int64_t ch = beam_chunks(bb * B, B, DEC, L, TC);
+                    const double c = (double)ch * ((double)TC * B * 4 + 4.0 * NWIN + TC / 2.0 + 8) + 8.0 * B + 16;
+                    sum += c;
+                    mx = std::max(mx, c);
+                }
+                sum *= (double)peers * nf;
+                const double cost = std::max(sum / NT_, mx) + mx * 0.5;
+                if (cost < bestc * 0.98) { bestc = cost; best = B; bestp = false; bestf2 = true; }
+            }
         for (int64_t B : {1, 3, 5, 7, 9})
             for (bool pair : {false, true}) {
                 const int64_t NB = (OUT + B - 1) / B, NBP = pair ? (NB + 1) / 2 : NB;
@@ -2411,10 +2432,11 @@ private:
                     for (int64_t k = 0; k < items; k++) th[k % NT_] += per[k % NBP];
                     for (double c : th) cost = std::max(cost, c);
                 }
-                if (cost < bestc * 0.98) { bestc = cost; best = B; bestp = pair; }
+                if (cost < bestc * 0.98) { bestc = cost; best = B; bestp = pair; bestf2 = false; }
             }
         beam_B_[v] = best;
         beam_pair_[v] = bestp;
+        beam_f2_[v] = bestf2;
         return best;
     }
     std::map<int, int> special_level_;
@@ -2462,6 +2484,124 @@ private:
         }
         return true;
     }
+    // FFMA2 variant of the frame FIR: item = (peer, frame, slot q); the thread computes the
+    // B-output blocks a = (q / 32) * 64 + q % 32 and a + 32 together, the two halves of
+    // packed fp32x2 registers: every tap is 4 FFMA2 (= the 8 fmaf of two sg_cmac, same
+    // order, same rounding) with the coefficient broadcast from the shared table.  Lanes
+    // stay B samples apart (odd B: distinct banks); chunks run to block a+32's triangle
+    // limit, block a's extra taps read zeros (exact, reading 14).
+    static std::string subst_s0(const std::string& e, const std::string& to) {
+        std::string r;
+        for (size_t i = 0; i < e.size();) {
+            if (e.compare(i, 2, "s0") == 0 && (i == 0 || !(isalnum((unsigned char)e[i - 1]) || e[i - 1] == '_')) &&
+                (i + 2 >= e.size() || !(isalnum((unsigned char)e[i + 2]) || e[i + 2] == '_'))) {
+                r += to;
+                i += 2;
+            } else {
+                r += e[i++];
+            }
+        }
+        return r;
+    }
+    void emit_beam_fir_f2(std::ostringstream& b, int v, int64_t F0, int64_t NP, const std::string& DINT,
+                          const std::string& DOUTT, int64_t ctoff) {
+        const Node& n = f_.nodes[v];
+        const int64_t L = n.iv[0], DEC = n.iv[1], FR = n.iv[2], OUT = FR / DEC;
+        const int64_t TC = beam_tc(L), B = beam_B_[v];
+        const int64_t NB = (OUT + B - 1) / B, NBH = (NB + 63) / 64 * 32, NWIN = (B - 1) * DEC + TC;
+        const int slot = nctr_++;
+        b << "      const int items = nf * " << NBH * NP << ";\n"
+          << "      for (int it0 = 0;;) {\n"
+          << "        if ((tid & 31) == 0) it0 = atomicAdd(&sg_ctr[" << slot << "], 32);\n"
+          << "        it0 = __shfl_sync(0xffffffffu, it0, 0);\n"
+          << "        if (it0 >= items) break;\n"
+          << "        const int it = it0 + (tid & 31);\n"
+          << "        if (it < items) {\n"
+          << "        const int pq = it / (nf * " << NBH << ");\n"
+          << "        const int itp = it - pq * (nf * " << NBH << ");\n"
+          << "        const int j = itp / " << NBH << ";\n"
+          << "        const int q = " << NBH - 1 << " - (itp - j * " << NBH << ");  // longest first\n"
+          << "        const int blka = (q >> 5) * 64 + (q & 31), blkb = blka + 32;\n"
+          << "        const int t0 = blka * " << B << ", t0b = blkb * " << B << ";\n"
+          << "        const int ilim = min(" << L << ", (t0b + " << B - 1 << ") * " << DEC << " + 1);\n"
+          << "        const int lf = " << F0 << " + j;\n"
+          << "        " << T_ << "* smi = sm + " << (NP > 1 ? DINT + "[pq]" : std::string("0")) << ";\n"
+          << "        " << T_ << "* smo = sm + " << (NP > 1 ? DOUTT + "[pq]" : std::string("0")) << ";\n"
+          << "        (void)pq; (void)smi; (void)smo;\n"
+          << "        float2 RE[" << B << "], IM[" << B << "];\n"
+          << "#pragma unroll\n"
+          << "        for (int bb = 0; bb < " << B << "; bb++) { RE[bb] = make_float2(0.0f, 0.0f); IM[bb] = RE[bb]; }\n"
+          << "        if (gf + lf >= 0) {\n"
+          << "#pragma unroll 1\n"
+          << "          for (int i0 = 0; i0 < ilim; i0 += " << TC << ") {\n"
+          << "            const int s0 = t0 * " << DEC << " - i0 - " << TC - 1 << ";\n"
+          << "            const int s0b = t0b * " << DEC << " - i0 - " << TC - 1 << ";\n"
+          << "            float2 XR[" << NWIN << "], XI[" << NWIN << "];\n"
+          << "            if (s0 >= 0 && s0b + " << NWIN - 1 << " < " << FR << ") {\n";
+        auto window = [&](bool checked) {
+            for (int64_t k = 0; k < NWIN; k++) {
+                Lin pr = Lin::v("lf", n.pop, 2 * k);
+                pr.t.push_back({"s0", 2});
+                Lin pi = pr.plus(1);
+                std::string er = "smi" + read_expr(n.in[0], pr).substr(2), ei = "smi" + read_expr(n.in[0], pi).substr(2);
+                std::string erb = subst_s0(er, "s0b"), eib = subst_s0(ei, "s0b");
+                if (checked)
+                    b << "              { const bool oa = s0 + " << k << " >= 0 && s0 + " << k << " < " << FR
+                      << ", ob = s0b + " << k << " >= 0 && s0b + " << k << " < " << FR << ";\n"
+                      << "                XR[" << k << "] = make_float2(oa ? " << er << " : 0.0f, ob ? " << erb << " : 0.0f);\n"
+                      << "                XI[" << k << "] = make_float2(oa ? " << ei << " : 0.0f, ob ? " << eib << " : 0.0f); }\n";
+                else
+                    b << "              XR[" << k << "] = make_float2(" << er << ", " << erb << "); XI[" << k << "] = make_float2(" << ei
+                      << ", " << eib << ");\n";
+            }
+        };
+        window(false);
+        b << "            } else {\n";
+        window(true);
+        b << "            }\n"
+          << "#pragma unroll\n"
+          << "            for (int ii = 0; ii < " << TC << "; ii += 2) {\n"
+          << "              const float4 c4 = reinterpret_cast<const float4*>(sm + " << ctoff << ")[(i0 + ii) >> 1];\n"
+          << "              const float2 cr0 = make_float2(c4.x, c4.x), ci0 = make_float2(c4.y, c4.y);\n"
+          << "              const float2 cr1 = make_float2(c4.z, c4.z), ci1 = make_float2(c4.w, c4.w);\n"
+          << "#pragma unroll\n"
+          << "              for (int bb = 0; bb < " << B << "; bb++) {\n"
+          << "                const int k = bb * " << DEC << " - ii + " << TC - 1 << ";\n"
+          << "                RE[bb] = __ffma2_rn(XR[k], cr0, RE[bb]);\n"
+          << "                RE[bb] = __ffma2_rn(make_float2(-XI[k].x, -XI[k].y), ci0, RE[bb]);\n"
+          << "                IM[bb] = __ffma2_rn(XR[k], ci0, IM[bb]);\n"
+          << "                IM[bb] = __ffma2_rn(XI[k], cr0, IM[bb]);\n"
+          << "              }\n"
+          << "#pragma unroll\n"
+          << "              for (int bb = 0; bb < " << B << "; bb++) {\n"
+          << "                const int k = bb * " << DEC << " - ii + " << TC - 2 << ";\n"
+          << "                RE[bb] = __ffma2_rn(XR[k], cr1, RE[bb]);\n"
+          << "                RE[bb] = __ffma2_rn(make_float2(-XI[k].x, -XI[k].y), ci1, RE[bb]);\n"
+          << "                IM[bb] = __ffma2_rn(XR[k], ci1, IM[bb]);\n"
+          << "                IM[bb] = __ffma2_rn(XI[k], cr1, IM[bb]);\n"
+          << "              }\n"
+          << "            }\n"
+          << "          }\n"
+          << "        }\n";
+        const int eo = n.out[0];
+        Lin pos = Lin::v("j", n.push, f_.edges[eo].pre + F0 * n.push);
+        pos.t.push_back({"(t0 + bb)", 2});
+        Lin posb = Lin::v("j", n.push, f_.edges[eo].pre + F0 * n.push);
+        posb.t.push_back({"(t0b + bb)", 2});
+        b << "#pragma unroll\n"
+          << "        for (int bb = 0; bb < " << B << "; bb++) {\n"
+          << "          if (t0 + bb < " << OUT << ") {\n"
+          << "            smo[" << buf_index(eo, pos).str() << "] = RE[bb].x;\n"
+          << "            smo[" << buf_index(eo, pos.plus(1)).str() << "] = IM[bb].x;\n"
+          << "          }\n"
+          << "          if (blkb < " << NB << " && t0b + bb < " << OUT << ") {\n"
+          << "            smo[" << buf_index(eo, posb).str() << "] = RE[bb].y;\n"
+          << "            smo[" << buf_index(eo, posb.plus(1)).str() << "] = IM[bb].y;\n"
+          << "          }\n"
+          << "        }\n"
+          << "        }\n"
+          << "      }\n";
+    }
     void emit_beam_fir(std::ostringstream& b, int v, int64_t F0, int64_t rot, const std::vector<int>& peers = {},
                        const std::vector<int64_t>& din = {}, const std::vector<int64_t>& dout = {}) {
         const Node& n = f_.nodes[v];
@@ -2486,6 +2626,10 @@ private:
             consts_ << "};\n__constant__ int " << DOUTT << "[" << NP << "] = {";
             for (int64_t q = 0; q < NP; q++) consts_ << (q ? ", " : "") << dout[q];
             consts_ << "};\n";
+        }
+        if (beam_f2_[v] && ctab) {
+            emit_beam_fir_f2(b, v, F0, NP, DINT, DOUTT, ct->second);
+            return;
         }
         b << "      const int items = nf * " << NBP * NP << ";\n";
         // dynamic item scheduling (fused kernels): warps grab 32 consecutive items from a
