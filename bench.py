@@ -38,6 +38,10 @@ WORKLOADS = {
     "fmradio10": dict(n=1 << 24, bound="alu", desc="FMRadio + 10-band equalizer fp32"),
     "beamformer12x4": dict(n=4096, bound="alu", desc="BeamFormer 12 channels x 4 beams fp32, 1024-sample frames"),
     "filterbank64": dict(n=1 << 20, bound="alu", desc="FilterBank 64 branches fp32 (M=8, L=32)"),
+    # second workloads of the paper's suite, not BASELINE configs
+    "bitonicrec32": dict(n=1 << 20, bound="hbm", desc="recursive BitonicSort 32-key int32, 1M iterations"),
+    "dct16": dict(n=1 << 18, bound="hbm", desc="2-D DCT-II of 16x16 fp32 blocks (row then column FIR DCTs)"),
+    "matmul16": dict(n=1 << 18, bound="hbm", desc="C = A B of streamed 16x16 fp32 matrices (MULTIPLY, ADD)"),
 }
 
 
@@ -129,7 +133,7 @@ def run_reference(args):
         return 0
     from workloads import apps
     name = args.config
-    prog = apps.CONFIGS[name]()
+    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
     vals = []
     cb = None
     for _ in range(max(1, args.warmup)):
@@ -186,7 +190,7 @@ def main():
     name = args.config
     W = WORKLOADS[name]
     n = args.iters or W["n"]
-    prog = apps.CONFIGS[name]()
+    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
     pipeline = args.mode == "pipeline" and world > 1
     if pipeline:
         from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan

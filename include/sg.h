@@ -76,6 +76,7 @@ typedef enum { SG_SPLIT_DUPLICATE = 0, SG_SPLIT_ROUNDROBIN = 1 } sg_split_kind;
  *  SG_K_BEAM_FIR         {L, dec, frame}    wr[L], wi[L]     2F/2F/2F/dec: per-frame complex FIR, zero history
  *  SG_K_BEAMFORM         {nch}              wr[nch], wi[nch] 2nch/2nch/2: complex weighted sum
  *  SG_K_MAGNITUDE        -                  -                2/2/1: sqrt(FMA(a,a,b*b))
+ *  SG_K_MULTIPLY         -                  -                2/2/1: x0 * x1 (MatMul's pairwise product)
  *
  * dtype SG_I32 admits IDENTITY, DELAY, DECIMATE, EXPAND, COMPARE_EXCHANGE, ADD.
  */
@@ -94,7 +95,8 @@ typedef enum {
     SG_K_ADD = 11,
     SG_K_BEAM_FIR = 12,
     SG_K_BEAMFORM = 13,
-    SG_K_MAGNITUDE = 14
+    SG_K_MAGNITUDE = 14,
+    SG_K_MULTIPLY = 15
 } sg_filter_kind;
 
 typedef struct {

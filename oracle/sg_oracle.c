@@ -50,10 +50,11 @@ typedef union {
 
 enum { K_IDENTITY, K_FIR, K_DELAY, K_DECIMATE, K_EXPAND, K_COMPARE_EXCHANGE, K_FFT_REORDER,
        K_COMBINE_DFT, K_FM_DEMOD, K_SUBTRACT, K_AMPLIFY, K_ADD, K_BEAM_FIR, K_BEAMFORM,
-       K_MAGNITUDE, K_COUNT };
+       K_MAGNITUDE, K_MULTIPLY, K_COUNT };
 static const char* KIND_NAMES[K_COUNT] = {
     "IDENTITY", "FIR", "DELAY", "DECIMATE", "EXPAND", "COMPARE_EXCHANGE", "FFT_REORDER",
-    "COMBINE_DFT", "FM_DEMOD", "SUBTRACT", "AMPLIFY", "ADD", "BEAM_FIR", "BEAMFORM", "MAGNITUDE"};
+    "COMBINE_DFT", "FM_DEMOD", "SUBTRACT", "AMPLIFY", "ADD", "BEAM_FIR", "BEAMFORM", "MAGNITUDE",
+    "MULTIPLY"};
 
 enum { T_FILTER, T_SPLIT_DUP, T_SPLIT_RR, T_JOIN_RR };
 
@@ -234,6 +235,7 @@ static int filter_rates(graph* g, node* n) {
         n->pop = n->peek = 2 * iv[0]; n->push = 2;
         break;
     case K_MAGNITUDE: if (g->is_i32) return ORC_E_KIND; n->pop = n->peek = 2; n->push = 1; break;
+    case K_MULTIPLY: if (g->is_i32) return ORC_E_KIND; n->pop = n->peek = 2; n->push = 1; break;
     default: return ORC_E_KIND;
     }
     if (n->kind == K_COMBINE_DFT) {
@@ -468,6 +470,7 @@ static void work(const graph* g, const node* n, const word* x, word* y) {
         y[0].f = sqrtf(fmaf(a, a, bb));
         break;
     }
+    case K_MULTIPLY: y[0].f = x[0].f * x[1].f; break;
     default: abort();
     }
 }

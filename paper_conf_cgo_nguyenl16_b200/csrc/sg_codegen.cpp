@@ -72,6 +72,7 @@ void node_work(const Flat& f, int v, int64_t& flops, int64_t& intops, int64_t& d
     case SG_K_BEAM_FIR: per = 8LL * n.iv[0] * (n.iv[2] / n.iv[1]); break;
     case SG_K_BEAMFORM: per = 8LL * n.iv[0]; break;
     case SG_K_MAGNITUDE: per = 3; break;
+    case SG_K_MULTIPLY: per = 1; break;
     case SG_K_COMPARE_EXCHANGE: intops = 2 * n.rep; break;
     default: break;
     }
@@ -344,6 +345,7 @@ protected:
                    const_array(wi) + ");";
         }
         case SG_K_MAGNITUDE: return "sg_work_magnitude(x_, y_);";
+        case SG_K_MULTIPLY: return "sg_work_multiply(x_, y_);";
         default: break;
         }
         throw Error(SG_E_UNSUPPORTED, std::string("no work function for ") + kind_name(n.kind));
@@ -1015,7 +1017,7 @@ public:
                         for (int e : ins_) {
                             int64_t lo, ex;
                             edge_window(f_, e, lo, ex);
-                            st += (f_.edges[e].per_iter * WF + ex + 3) / 4 * 4;
+                            st += (f_.edges[e].per_iter * WF + ex + 3) / 4 * 4 + 4;
                         }
                         auto blocks = [](size_t b) { return std::max(1, std::min(2, (int)((220 * 1024) / std::max<size_t>(1024, b)))); };
                         size_t with = smem_bytes_ + (size_t)st * 4;
@@ -1028,7 +1030,7 @@ public:
                                 int64_t lo, ex;
                                 edge_window(f_, e, lo, ex);
                                 stage_off_[e] = o;
-                                o += (f_.edges[e].per_iter * WF + ex + 3) / 4 * 4;
+                                o += (f_.edges[e].per_iter * WF + ex + 3) / 4 * 4 + 4;
                             }
                             smem_bytes_ = (size_t)o * 4;
                         }
@@ -1592,7 +1594,8 @@ private:
                         FGroup h = g;
                         h.B = g.B * 2;
                         Sym c2;
-                        if (!dry_ok(h, c2) || c2.flops > 2048 || c2.nloads > 96) break;
+                        static const int64_t fcap = std::getenv("SG_FUSED_FLOPCAP") ? std::atoll(std::getenv("SG_FUSED_FLOPCAP")) : 2048;
+                        if (!dry_ok(h, c2) || c2.flops > fcap || c2.nloads > 96) break;
                         g.B = h.B;
                         c = c2;
                     }
@@ -1846,7 +1849,10 @@ private:
                 pb << "  for (int j = tid; j < " << kv.second.size() << "; j += NT) sm[" << kv.first << " + j] = " << name
                    << "[j];  // frame-FIR coefficient table\n";
             }
-            if (prefetch_) emit_issue(pb, "SG_K_BEGIN + (long long)blockIdx.x * " + std::to_string(W), true);
+            if (prefetch_) {
+                pb << "  int sg_pm[" << std::max<size_t>(1, ins_.size()) << "];  // staging misalignment (items) per input\n";
+                emit_issue(pb, "SG_K_BEGIN + (long long)blockIdx.x * " + std::to_string(W), true);
+            }
             prologue_ = pb.str();
         }
         emit_loads(b);
@@ -2157,12 +2163,35 @@ private:
             if (!staging && pit != plP_.end())
                 dst = "s + (j % " + std::to_string(pit->second) + ") * " + std::to_string(plQ_.at(e)) + " + j / " +
                       std::to_string(pit->second);
+            if (staging) {
+                // 16-byte cp.async over the 16-byte-aligned superset of the window; the
+                // misalignment m (items) is kept for the staging -> tile copy; partial
+                // quads at the stream ends go item by item with zero fill
+                b << "        {\n"
+                  << "          const " << T_ << "* g = SG_IN(" << i << ");\n"
+                  << "          const long long gb = kn * " << P << "LL + (" << lo << "LL) - SG_IN_BASE(" << i << ");\n"
+                  << "          const long long lim = SG_IN_LIMIT(" << i << ");\n"
+                  << "          const int n = Wn * " << P << " + " << ex << ";\n"
+                  << "          const int m = (int)(((unsigned long long)g / 4ull + (unsigned long long)gb) & 3ull);\n"
+                  << "          sg_pm[" << i << "] = m;\n"
+                  << "          const long long ga = gb - m;\n"
+                  << "          const int nq = (n + m + 3) >> 2;\n"
+                  << "          " << T_ << "* s = sm + " << stage_off_.at(e) << ";\n"
+                  << "          for (int q = tid; q < nq; q += NT) {\n"
+                  << "            const long long gi = ga + 4LL * q;\n"
+                  << "            if (gi >= 0 && gi + 3 < lim) sg_cp_async16(s + 4 * q, g + gi);\n"
+                  << "            else for (int r = 0; r < 4; r++) { const bool ok = gi + r >= 0 && gi + r < lim;\n"
+                  << "              sg_cp_async4(s + 4 * q + r, g + (ok ? gi + r : 0LL), ok ? 4u : 0u); }\n"
+                  << "          }\n"
+                  << "        }\n";
+                continue;
+            }
             b << "        {\n"
               << "          const " << T_ << "* g = SG_IN(" << i << ");\n"
               << "          const long long gb = kn * " << P << "LL + (" << lo << "LL) - SG_IN_BASE(" << i << ");\n"
               << "          const long long lim = SG_IN_LIMIT(" << i << ");\n"
               << "          const int n = Wn * " << P << " + " << ex << ";\n"
-              << "          " << T_ << "* s = sm + " << (staging ? stage_off_.at(e) : off_.at(e)) << ";\n"
+              << "          " << T_ << "* s = sm + " << off_.at(e) << ";\n"
               << "          for (int j = tid; j < n; j += NT) { const long long gi = gb + j; const bool ok = gi >= 0 && gi < lim;\n"
               << "            sg_cp_async4(" << dst << ", g + (ok ? gi : 0LL), ok ? 4u : 0u); }\n"
               << "        }\n";
@@ -2187,7 +2216,7 @@ private:
                     b << "    { // boundary input " << i << " (edge " << e << "): staging -> tile buffer\n"
                       << "      const int n = Wt * " << P << " + " << ex << ";\n"
                       << "      " << T_ << "* s = sm + " << off_.at(e) << ";\n"
-                      << "      const " << T_ << "* st = sm + " << stage_off_.at(e) << ";\n"
+                      << "      const " << T_ << "* st = sm + " << stage_off_.at(e) << " + sg_pm[" << i << "];\n"
                       << "      for (int j = tid; j < n; j += NT) " << dst << " = st[j];\n"
                       << "    }\n";
                 }

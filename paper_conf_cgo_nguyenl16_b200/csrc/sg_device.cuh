@@ -126,6 +126,7 @@ SG_DEV void sg_work_beamform(const float (&x)[2 * NC], float (&y)[2], const floa
     y[1] = im;
 }
 
+SG_DEV void sg_work_multiply(const float (&x)[2], float (&y)[1]) { y[0] = __fmul_rn(x[0], x[1]); }
 SG_DEV void sg_work_magnitude(const float (&x)[2], float (&y)[1]) {
     const float b2 = x[1] * x[1];
     y[0] = __fsqrt_rn(fmaf(x[0], x[0], b2));
@@ -238,6 +239,9 @@ SG_DEV void sg_bulk_wait() { asm volatile("cp.async.bulk.wait_group %0;" :: "n"(
 SG_DEV void sg_cp_async4(void* sdst, const void* gsrc, sg_u32 src_bytes) {
     asm volatile("cp.async.ca.shared.global [%0], [%1], 4, %2;"
                  :: "r"(sg_smem_addr(sdst)), "l"(gsrc), "r"(src_bytes) : "memory");
+}
+SG_DEV void sg_cp_async16(void* sdst, const void* gsrc) {
+    asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" :: "r"(sg_smem_addr(sdst)), "l"(gsrc) : "memory");
 }
 SG_DEV void sg_cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
 SG_DEV void sg_cp_async_wait_all() { asm volatile("cp.async.wait_all;" ::: "memory"); }

@@ -103,3 +103,36 @@ def test_parity_bitonic_edge_sizes(oracle_lib, n):
     x = inputs.make_input("i32", 32 * n, n)
     y, _, _ = run_gpu(prog, x, n)
     assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+# ---- second workloads of the paper's suite: BitonicRec, DCT, MatMul
+EXTRA_N = {"bitonicrec32": (3 * 256 + 5, 20000), "dct16": (37, 5000), "matmul16": (41, 5000)}
+
+
+@pytest.mark.parametrize("name", list(apps.EXTRA))
+def test_parity_extra(oracle_lib, name):
+    prog = apps.EXTRA[name]()
+    for n in EXTRA_N[name]:
+        x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), inputs.SEEDS.get(name, 99) + n)
+        ref = oracle_lib.run(prog, x, n)
+        y, info, launches = run_gpu(prog, x, n)
+        assert launches >= 1
+        assert_parity(prog, y, ref)
+
+
+def test_parity_matmul_exact_small_integers(oracle_lib):
+    prog = apps.matmul(16, 16, 16)
+    n = 300
+    rng = np.random.default_rng(8)
+    x = rng.integers(-7, 8, size=512 * n).astype(np.float32)
+    y, _, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+@pytest.mark.parametrize("variant", ["ties", "sorted", "reversed"])
+def test_parity_bitonic_rec_variants(oracle_lib, variant):
+    prog = apps.bitonic_rec(32)
+    n = 1000
+    x = inputs.make_input("i32", 32 * n, 6, variant=variant)
+    y, _, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, oracle_lib.run(prog, x, n))

@@ -145,7 +145,7 @@ def _filter_pop_push(f):
         "COMBINE_DFT": (2 * iv[0], 2 * iv[0]) if iv else None, "FM_DEMOD": (1, 1), "SUBTRACT": (2, 1),
         "AMPLIFY": (1, 1), "ADD": (iv[0], 1) if iv else None,
         "BEAM_FIR": (2 * iv[2], 2 * iv[2] // iv[1]) if len(iv) >= 3 else None,
-        "BEAMFORM": (2 * iv[0], 2) if iv else None, "MAGNITUDE": (2, 1),
+        "BEAMFORM": (2 * iv[0], 2) if iv else None, "MAGNITUDE": (2, 1), "MULTIPLY": (2, 1),
     }[k]
 
 

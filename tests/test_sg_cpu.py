@@ -44,9 +44,9 @@ def test_library_is_sm100a(sg):
 
 
 # ------------------------------------------------------- SDF analysis vs oracle
-@pytest.mark.parametrize("name", list(apps.CONFIGS))
+@pytest.mark.parametrize("name", list(apps.CONFIGS) + list(apps.EXTRA))
 def test_rates_match_oracle(sg, oracle_lib, name):
-    prog = apps.CONFIGS[name]()
+    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
     r = oracle_lib.rates(prog)
     with sg.plan(prog, 1, partitioner="single", plan_only=1) as p:
         i = p.info()

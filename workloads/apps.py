@@ -14,6 +14,15 @@ StreamIt `init` block would compute.  No filter is executed here.
   fmradio(bands) FMRadio + equalizer (Fig. 4.2b, PAPER.md:736-745)
   beamformer()   12 channels x 4 beams, frame-granular FIRs (absent from PAPER.md)
   filterbank(B)  B-branch multirate filter bank (absent from PAPER.md)
+
+Second workloads from the paper's suite (Fig. 4.2 d/e/f/g,
+PAPER.md:787-833), same reading rules:
+
+  bitonic_rec(N) recursive bitonic sorter (BitonicRec, Fig. 4.2g)
+  dct2d(N)       N x N 2-D DCT-II (orthonormal), row then column 1-D DCTs (DCT, Fig. 4.2d)
+  matmul(M,K,N)  C = A B of two streamed matrices (MatMul, Fig. 4.2e/f): rows of A and
+                 columns of B are repeated / transposed by split-joins, paired, multiplied
+                 and summed (MULTIPLY, ADD)
 """
 from __future__ import annotations
 
@@ -162,6 +171,68 @@ def filterbank(branches: int = 64, M: int = 8, L: int = 32, small_int: bool = Fa
     return Program(f"filterbank{branches}{'_int' if small_int else ''}", "f32",
                    Pipeline([sj, Filter("ADD", [branches])]),
                    note="one iteration = 8 input samples -> 8 output samples")
+
+
+# ------------------------------------------------------------------- BitonicRec
+def _bsort_merge(N: int, up: bool):
+    """Bitonic merge of N keys: half-cleaner (i vs i + N/2), then merge both halves."""
+    if N == 2:
+        return _ce(up)
+    half = SplitJoin("rr", [_ce(up) for _ in range(N // 2)])       # RR(1): branch i gets i, i+N/2
+    return Pipeline([half, SplitJoin("rr", [_bsort_merge(N // 2, up), _bsort_merge(N // 2, up)],
+                                     split_w=[N // 2] * 2, join_w=[N // 2] * 2)])
+
+
+def _bsort_kernel(N: int, up: bool):
+    """Sort N keys (up: ascending): sort the halves in opposite directions, then merge."""
+    if N == 2:
+        return _ce(up)
+    halves = SplitJoin("rr", [_bsort_kernel(N // 2, up), _bsort_kernel(N // 2, not up)],
+                       split_w=[N // 2] * 2, join_w=[N // 2] * 2)
+    return Pipeline([halves, _bsort_merge(N, up)])
+
+
+def bitonic_rec(N: int = 32) -> Program:
+    return Program(f"bitonicrec{N}", "i32", Pipeline([_bsort_kernel(N, True)]),
+                   note="one iteration = one block of N int32 keys, sorted ascending (recursive form)")
+
+
+# -------------------------------------------------------------------------- DCT
+def dct_coeffs(N: int) -> List[List[float]]:
+    """Orthonormal DCT-II matrix C[k][n] = s_k cos(pi (2n+1) k / 2N), in double, rounded to f32."""
+    return [[f32((math.sqrt(1.0 / N) if k == 0 else math.sqrt(2.0 / N)) *
+                 math.cos(math.pi * (2 * n + 1) * k / (2.0 * N))) for n in range(N)] for k in range(N)]
+
+
+def _dct1d(N: int) -> SplitJoin:
+    """1-D DCT of every N consecutive items: N dot products (FIR, pop N) of the same window."""
+    C = dct_coeffs(N)
+    return SplitJoin("dup", [Filter("FIR", [N, N], C[k]) for k in range(N)])   # join RR(1): y_0..y_{N-1}
+
+
+def dct2d(N: int = 16) -> Program:
+    rows = _dct1d(N)                                              # row-major rows: R = X C^T
+    cols = SplitJoin("rr", [_dct1d(N) for _ in range(N)])        # RR(1) split: branch j = column j of R;
+    return Program(f"dct{N}", "f32", Pipeline([rows, cols]),     # RR(1) join: out[k][j] -> Y = C X C^T
+                   note="one iteration = one N x N block (row-major) -> its 2-D DCT-II (row-major)")
+
+
+# ----------------------------------------------------------------------- MatMul
+def matmul(M: int = 16, K: int = 16, N: int = 16) -> Program:
+    ident = Filter("IDENTITY")
+    a_rep = SplitJoin("dup", [ident] * N, join_w=[K] * N)               # each row of A, N times
+    b_t = SplitJoin("rr", [ident] * N, join_w=[K] * N)                  # B^T (columns of B as rows)
+    b_rep = SplitJoin("dup", [ident] * M, join_w=[K * N] * M)           # B^T, M times
+    pairs = SplitJoin("rr", [a_rep, Pipeline([b_t, b_rep])], split_w=[M * K, K * N], join_w=[1, 1])
+    return Program(f"matmul{M}x{K}x{N}", "f32", Pipeline([pairs, Filter("MULTIPLY"), Filter("ADD", [K])]),
+                   note="one iteration = A (M x K) then B (K x N), row-major -> C = A B (M x N), row-major")
+
+
+EXTRA = {
+    "bitonicrec32": lambda: bitonic_rec(32),
+    "dct16": lambda: dct2d(16),
+    "matmul16": lambda: matmul(16, 16, 16),
+}
 
 
 CONFIGS = {

@@ -25,6 +25,7 @@ SURVEY.md section 8(b)/(c)-3:
   BEAM_FIR          [L, dec, frame] / wr[L]+wi[L]   pop 2*frame push 2*frame/dec
   BEAMFORM          [nch] / wr[nch]+wi[nch]   pop 2*nch push 2
   MAGNITUDE         -                         pop 2 push 1
+  MULTIPLY          -                         pop 2 push 1
 """
 from __future__ import annotations
 
@@ -50,6 +51,7 @@ KINDS = {
     "BEAM_FIR": 12,
     "BEAMFORM": 13,
     "MAGNITUDE": 14,
+    "MULTIPLY": 15,
 }
 
 
