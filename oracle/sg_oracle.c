@@ -50,11 +50,12 @@ typedef union {
 
 enum { K_IDENTITY, K_FIR, K_DELAY, K_DECIMATE, K_EXPAND, K_COMPARE_EXCHANGE, K_FFT_REORDER,
        K_COMBINE_DFT, K_FM_DEMOD, K_SUBTRACT, K_AMPLIFY, K_ADD, K_BEAM_FIR, K_BEAMFORM,
-       K_MAGNITUDE, K_MULTIPLY, K_COUNT };
+       K_MAGNITUDE, K_MULTIPLY, K_PERMUTE, K_XOR, K_XOR_CONST, K_SBOX, K_INTO_BITS, K_BITS_TO_INT,
+       K_COUNT };
 static const char* KIND_NAMES[K_COUNT] = {
     "IDENTITY", "FIR", "DELAY", "DECIMATE", "EXPAND", "COMPARE_EXCHANGE", "FFT_REORDER",
     "COMBINE_DFT", "FM_DEMOD", "SUBTRACT", "AMPLIFY", "ADD", "BEAM_FIR", "BEAMFORM", "MAGNITUDE",
-    "MULTIPLY"};
+    "MULTIPLY", "PERMUTE", "XOR", "XOR_CONST", "SBOX", "INTO_BITS", "BITS_TO_INT"};
 
 enum { T_FILTER, T_SPLIT_DUP, T_SPLIT_RR, T_JOIN_RR };
 
@@ -236,6 +237,27 @@ static int filter_rates(graph* g, node* n) {
         break;
     case K_MAGNITUDE: if (g->is_i32) return ORC_E_KIND; n->pop = n->peek = 2; n->push = 1; break;
     case K_MULTIPLY: if (g->is_i32) return ORC_E_KIND; n->pop = n->peek = 2; n->push = 1; break;
+    /* DES (Fig. 4.2c; StreamIt bit-per-item form) */
+    case K_PERMUTE: /* {n, idx[m]}: y[k] = x[idx[k]] */
+        if (ni < 2 || iv[0] < 1) return ORC_E_KIND;
+        for (int k = 1; k < ni; k++) if (iv[k] < 0 || iv[k] >= iv[0]) return ORC_E_KIND;
+        n->pop = n->peek = iv[0]; n->push = ni - 1;
+        break;
+    case K_XOR: /* {n}: y[i] = x[i] ^ x[n+i] */
+        if (ni < 1 || iv[0] < 1 || !g->is_i32) return ORC_E_KIND;
+        n->pop = n->peek = 2 * iv[0]; n->push = iv[0];
+        break;
+    case K_XOR_CONST: /* {n, k[n]}: y[i] = x[i] ^ k[i] */
+        if (ni < 1 || iv[0] < 1 || ni != 1 + iv[0] || !g->is_i32) return ORC_E_KIND;
+        n->pop = n->peek = n->push = iv[0];
+        break;
+    case K_SBOX: /* {t[64]}: 6 bits in, 4 bits out */
+        if (ni != 64 || !g->is_i32) return ORC_E_KIND;
+        for (int k = 0; k < 64; k++) if (iv[k] < 0 || iv[k] > 15) return ORC_E_KIND;
+        n->pop = n->peek = 6; n->push = 4;
+        break;
+    case K_INTO_BITS: if (!g->is_i32) return ORC_E_KIND; n->pop = n->peek = 1; n->push = 32; break;
+    case K_BITS_TO_INT: if (!g->is_i32) return ORC_E_KIND; n->pop = n->peek = 32; n->push = 1; break;
     default: return ORC_E_KIND;
     }
     if (n->kind == K_COMBINE_DFT) {
@@ -471,6 +493,34 @@ static void work(const graph* g, const node* n, const word* x, word* y) {
         break;
     }
     case K_MULTIPLY: y[0].f = x[0].f * x[1].f; break;
+    case K_PERMUTE:
+        for (int k = 1; k < n->ni; k++) y[k - 1] = x[iv[k]];
+        break;
+    case K_XOR:
+        for (int i = 0; i < iv[0]; i++) y[i].u = x[i].u ^ x[iv[0] + i].u;
+        break;
+    case K_XOR_CONST:
+        for (int i = 0; i < iv[0]; i++) y[i].u = x[i].u ^ (uint32_t)iv[1 + i];
+        break;
+    case K_SBOX: { /* FIPS 46-3: bits b1..b6 (first popped = b1); row = b1 b6, column = b2 b3 b4 b5;
+                      the table is row-major (16 columns); output bits most significant first */
+        uint32_t b[6];
+        for (int i = 0; i < 6; i++) b[i] = x[i].u & 1u;
+        uint32_t row = 2u * b[0] + b[5];
+        uint32_t col = 8u * b[1] + 4u * b[2] + 2u * b[3] + b[4];
+        uint32_t v = (uint32_t)iv[16 * row + col];
+        for (int i = 0; i < 4; i++) y[i].u = (v >> (3 - i)) & 1u;
+        break;
+    }
+    case K_INTO_BITS: /* most significant bit first */
+        for (int k = 0; k < 32; k++) y[k].u = (x[0].u >> (31 - k)) & 1u;
+        break;
+    case K_BITS_TO_INT: {
+        uint32_t v = 0u;
+        for (int k = 0; k < 32; k++) v = 2u * v + (x[k].u & 1u);
+        y[0].u = v;
+        break;
+    }
     default: abort();
     }
 }

@@ -20,6 +20,8 @@ PAPER.md:787-833), same reading rules:
 
   bitonic_rec(N) recursive bitonic sorter (BitonicRec, Fig. 4.2g)
   dct2d(N)       N x N 2-D DCT-II (orthonormal), row then column 1-D DCTs (DCT, Fig. 4.2d)
+  des(rounds)    DES on a bit-per-item stream (Fig. 4.2a): IntoBits, IP, 16 Feistel rounds (E, key
+                 XOR, eight S-boxes in a round-robin split-join, P, XOR with L), IP^-1, BitstoInts
   matmul(M,K,N)  C = A B of two streamed matrices (MatMul, Fig. 4.2e/f): rows of A and
                  columns of B are repeated / transposed by split-joins, paired, multiplied
                  and summed (MULTIPLY, ADD)
@@ -228,10 +230,95 @@ def matmul(M: int = 16, K: int = 16, N: int = 16) -> Program:
                    note="one iteration = A (M x K) then B (K x N), row-major -> C = A B (M x N), row-major")
 
 
+# -------------------------------------------------------------------------- DES
+# FIPS 46-3 tables (1-based bit numbers, bit 1 = most significant), written as the
+# StreamIt DES init blocks hold them.  The graph works on a bit-per-item stream like
+# StreamIt's DES (IntoBits ... BitstoInts), PAPER.md:735 (Fig. 4.2a), 876.
+DES_IP = [58, 50, 42, 34, 26, 18, 10, 2, 60, 52, 44, 36, 28, 20, 12, 4,
+          62, 54, 46, 38, 30, 22, 14, 6, 64, 56, 48, 40, 32, 24, 16, 8,
+          57, 49, 41, 33, 25, 17, 9, 1, 59, 51, 43, 35, 27, 19, 11, 3,
+          61, 53, 45, 37, 29, 21, 13, 5, 63, 55, 47, 39, 31, 23, 15, 7]
+DES_E = [32, 1, 2, 3, 4, 5, 4, 5, 6, 7, 8, 9, 8, 9, 10, 11, 12, 13, 12, 13, 14, 15, 16, 17,
+         16, 17, 18, 19, 20, 21, 20, 21, 22, 23, 24, 25, 24, 25, 26, 27, 28, 29, 28, 29, 30, 31, 32, 1]
+DES_P = [16, 7, 20, 21, 29, 12, 28, 17, 1, 15, 23, 26, 5, 18, 31, 10,
+         2, 8, 24, 14, 32, 27, 3, 9, 19, 13, 30, 6, 22, 11, 4, 25]
+DES_S = [
+    [14, 4, 13, 1, 2, 15, 11, 8, 3, 10, 6, 12, 5, 9, 0, 7, 0, 15, 7, 4, 14, 2, 13, 1, 10, 6, 12, 11, 9, 5, 3, 8,
+     4, 1, 14, 8, 13, 6, 2, 11, 15, 12, 9, 7, 3, 10, 5, 0, 15, 12, 8, 2, 4, 9, 1, 7, 5, 11, 3, 14, 10, 0, 6, 13],
+    [15, 1, 8, 14, 6, 11, 3, 4, 9, 7, 2, 13, 12, 0, 5, 10, 3, 13, 4, 7, 15, 2, 8, 14, 12, 0, 1, 10, 6, 9, 11, 5,
+     0, 14, 7, 11, 10, 4, 13, 1, 5, 8, 12, 6, 9, 3, 2, 15, 13, 8, 10, 1, 3, 15, 4, 2, 11, 6, 7, 12, 0, 5, 14, 9],
+    [10, 0, 9, 14, 6, 3, 15, 5, 1, 13, 12, 7, 11, 4, 2, 8, 13, 7, 0, 9, 3, 4, 6, 10, 2, 8, 5, 14, 12, 11, 15, 1,
+     13, 6, 4, 9, 8, 15, 3, 0, 11, 1, 2, 12, 5, 10, 14, 7, 1, 10, 13, 0, 6, 9, 8, 7, 4, 15, 14, 3, 11, 5, 2, 12],
+    [7, 13, 14, 3, 0, 6, 9, 10, 1, 2, 8, 5, 11, 12, 4, 15, 13, 8, 11, 5, 6, 15, 0, 3, 4, 7, 2, 12, 1, 10, 14, 9,
+     10, 6, 9, 0, 12, 11, 7, 13, 15, 1, 3, 14, 5, 2, 8, 4, 3, 15, 0, 6, 10, 1, 13, 8, 9, 4, 5, 11, 12, 7, 2, 14],
+    [2, 12, 4, 1, 7, 10, 11, 6, 8, 5, 3, 15, 13, 0, 14, 9, 14, 11, 2, 12, 4, 7, 13, 1, 5, 0, 15, 10, 3, 9, 8, 6,
+     4, 2, 1, 11, 10, 13, 7, 8, 15, 9, 12, 5, 6, 3, 0, 14, 11, 8, 12, 7, 1, 14, 2, 13, 6, 15, 0, 9, 10, 4, 5, 3],
+    [12, 1, 10, 15, 9, 2, 6, 8, 0, 13, 3, 4, 14, 7, 5, 11, 10, 15, 4, 2, 7, 12, 9, 5, 6, 1, 13, 14, 0, 11, 3, 8,
+     9, 14, 15, 5, 2, 8, 12, 3, 7, 0, 4, 10, 1, 13, 11, 6, 4, 3, 2, 12, 9, 5, 15, 10, 11, 14, 1, 7, 6, 0, 8, 13],
+    [4, 11, 2, 14, 15, 0, 8, 13, 3, 12, 9, 7, 5, 10, 6, 1, 13, 0, 11, 7, 4, 9, 1, 10, 14, 3, 5, 12, 2, 15, 8, 6,
+     1, 4, 11, 13, 12, 3, 7, 14, 10, 15, 6, 8, 0, 5, 9, 2, 6, 11, 13, 8, 1, 4, 10, 7, 9, 5, 0, 15, 14, 2, 3, 12],
+    [13, 2, 8, 4, 6, 15, 11, 1, 10, 9, 3, 14, 5, 0, 12, 7, 1, 15, 13, 8, 10, 3, 7, 4, 12, 5, 6, 11, 0, 14, 9, 2,
+     7, 11, 4, 1, 9, 12, 14, 2, 0, 6, 10, 13, 15, 3, 5, 8, 2, 1, 14, 7, 4, 10, 8, 13, 15, 12, 9, 0, 3, 5, 6, 11],
+]
+DES_PC1 = [57, 49, 41, 33, 25, 17, 9, 1, 58, 50, 42, 34, 26, 18, 10, 2, 59, 51, 43, 35, 27, 19, 11, 3, 60, 52, 44, 36,
+           63, 55, 47, 39, 31, 23, 15, 7, 62, 54, 46, 38, 30, 22, 14, 6, 61, 53, 45, 37, 29, 21, 13, 5, 28, 20, 12, 4]
+DES_PC2 = [14, 17, 11, 24, 1, 5, 3, 28, 15, 6, 21, 10, 23, 19, 12, 4, 26, 8, 16, 7, 27, 20, 13, 2,
+           41, 52, 31, 37, 47, 55, 30, 40, 51, 45, 33, 48, 44, 49, 39, 56, 34, 53, 46, 42, 50, 36, 29, 32]
+DES_SHIFTS = [1, 1, 2, 2, 2, 2, 2, 2, 1, 2, 2, 2, 2, 2, 2, 1]
+DES_KEY = 0x133457799BBCDFF1          # default key (the classic worked example's key)
+
+
+def des_round_keys(key: int, rounds: int = 16) -> List[List[int]]:
+    """Key schedule (FIPS 46-3): PC-1, per-round left rotations of C and D, PC-2.  Round keys as
+    48 bits (most significant first).  A program constant, like a StreamIt init block."""
+    kb = [(key >> (63 - i)) & 1 for i in range(64)]
+    cd = [kb[p - 1] for p in DES_PC1]
+    c, d = cd[:28], cd[28:]
+    out = []
+    for r in range(rounds):
+        s = DES_SHIFTS[r % 16]
+        c, d = c[s:] + c[:s], d[s:] + d[:s]
+        out.append([(c + d)[p - 1] for p in DES_PC2])
+    return out
+
+
+def _des_round(k48: List[int]) -> Pipeline:
+    """One Feistel round on [L | R] (64 bits): [L | R] -> [R | L ^ P(S(E(R) ^ K))]."""
+    f = Pipeline([
+        Filter("PERMUTE", [64] + [32 + e - 1 for e in DES_E]),             # E(R): 48 bits
+        Filter("XOR_CONST", [48] + list(k48)),                              # ^ K_r
+        SplitJoin("rr", [Filter("SBOX", DES_S[j]) for j in range(8)],      # S1..S8: 6 -> 4 bits
+                  split_w=[6] * 8, join_w=[4] * 8),
+        Filter("PERMUTE", [32] + [p - 1 for p in DES_P]),                  # P
+    ])
+    fanout = SplitJoin("dup", [f, Filter("IDENTITY")], join_w=[32, 64])    # -> [f | L | R]
+    order = Filter("PERMUTE", [96] + list(range(64, 96)) + list(range(0, 64)))  # -> [R | f | L]
+    mix = SplitJoin("rr", [Filter("IDENTITY"), Filter("XOR", [32])], split_w=[32, 64], join_w=[32, 32])
+    return Pipeline([fanout, order, mix])
+
+
+def des(rounds: int = 16, key: int = DES_KEY, decrypt: bool = False) -> Program:
+    ks = des_round_keys(key, 16)[:rounds] if rounds <= 16 else [des_round_keys(key, 16)[r % 16] for r in range(rounds)]
+    if decrypt:
+        ks = ks[::-1]
+    ip_inv = [0] * 64
+    for i, p in enumerate(DES_IP):
+        ip_inv[p - 1] = i
+    kids = [Filter("INTO_BITS"), Filter("PERMUTE", [64] + [p - 1 for p in DES_IP])]
+    kids += [_des_round(k) for k in ks]
+    kids += [Filter("PERMUTE", [64] + list(range(32, 64)) + list(range(0, 32))),   # R16 L16
+             Filter("PERMUTE", [64] + ip_inv),                                      # IP^-1
+             Filter("BITS_TO_INT")]
+    return Program(f"des{rounds}", "i32", Pipeline(kids),
+                   note="one iteration = one 64-bit block as two int32 words (high word first) -> its DES "
+                        "encryption (decryption with reversed round keys)")
+
+
 EXTRA = {
     "bitonicrec32": lambda: bitonic_rec(32),
     "dct16": lambda: dct2d(16),
     "matmul16": lambda: matmul(16, 16, 16),
+    "des16": lambda: des(16),
 }
 
 

@@ -26,6 +26,12 @@ SURVEY.md section 8(b)/(c)-3:
   BEAMFORM          [nch] / wr[nch]+wi[nch]   pop 2*nch push 2
   MAGNITUDE         -                         pop 2 push 1
   MULTIPLY          -                         pop 2 push 1
+  PERMUTE           [n, idx[m]]               pop n push m: y[k] = x[idx[k]]
+  XOR               [n]                       pop 2n push n: y[i] = x[i] ^ x[n+i]        (i32)
+  XOR_CONST         [n, k[n]]                 pop n push n: y[i] = x[i] ^ k[i]           (i32)
+  SBOX              [t[64]]                   pop 6 push 4: DES S-box on bits            (i32)
+  INTO_BITS         -                         pop 1 push 32: bits, most significant first (i32)
+  BITS_TO_INT       -                         pop 32 push 1: inverse of INTO_BITS        (i32)
 """
 from __future__ import annotations
 
@@ -52,6 +58,12 @@ KINDS = {
     "BEAMFORM": 13,
     "MAGNITUDE": 14,
     "MULTIPLY": 15,
+    "PERMUTE": 16,
+    "XOR": 17,
+    "XOR_CONST": 18,
+    "SBOX": 19,
+    "INTO_BITS": 20,
+    "BITS_TO_INT": 21,
 }
 
 
