@@ -42,6 +42,7 @@ WORKLOADS = {
     "bitonicrec32": dict(n=1 << 20, bound="hbm", desc="recursive BitonicSort 32-key int32, 1M iterations"),
     "dct16": dict(n=1 << 18, bound="hbm", desc="2-D DCT-II of 16x16 fp32 blocks (row then column FIR DCTs)"),
     "matmul16": dict(n=1 << 18, bound="hbm", desc="C = A B of streamed 16x16 fp32 matrices (MULTIPLY, ADD)"),
+    "des16": dict(n=1 << 20, bound="int", desc="DES (16 rounds) on a bit-per-item int32 stream, one 64-bit block / iteration"),
 }
 
 
@@ -281,6 +282,16 @@ def main():
             roof = {"bound": "hbm", "achieved": ach, "peak": peaks["hbm_gbs"], "unit": "GB/s",
                     "frac": ach / peaks["hbm_gbs"], "traffic": None,
                     "algorithmic_bytes_per_launch": ki_bytes, "peak_source": peak_src + " copy bandwidth"}
+    elif W["bound"] == "int":
+        ops = info["intops_per_iter"]
+        if kern_ms:
+            ach = ops * n / (kern_ms / 1e3) / 1e12
+            pk = 148 * 64 * peaks.get("sm_max_mhz", 1965.0) * 1e6 / 1e12
+            roof = {"bound": "alu", "achieved": ach, "peak": pk, "unit": "Tops/s", "frac": ach / pk,
+                    "traffic": None, "algorithmic_ops_per_launch": ops * n, "ops_per_iter": ops,
+                    "ops_counting": "as written: one op per XORed bit (key XOR included), per S-box lookup, "
+                                    "per bit unpacked / packed",
+                    "peak_source": "derived: 148 SMs x 64 int32 lanes/clk (alu pipe, LOP3/SHF rate) x sm_max_mhz"}
     else:
         fl_written = _flops_per_iter(prog, info["reps"])
         fl = min(fl_written, info["flops_per_iter_pruned"]) if info["flops_per_iter_pruned"] > 0 else fl_written

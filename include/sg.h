@@ -77,6 +77,14 @@ typedef enum { SG_SPLIT_DUPLICATE = 0, SG_SPLIT_ROUNDROBIN = 1 } sg_split_kind;
  *  SG_K_BEAMFORM         {nch}              wr[nch], wi[nch] 2nch/2nch/2: complex weighted sum
  *  SG_K_MAGNITUDE        -                  -                2/2/1: sqrt(FMA(a,a,b*b))
  *  SG_K_MULTIPLY         -                  -                2/2/1: x0 * x1 (MatMul's pairwise product)
+ *  --- DES on a bit-per-item stream (Fig. 4.2a), SG_I32 only except PERMUTE:
+ *  SG_K_PERMUTE          {n, idx[m]}        -                n/n/m: y[k] = x[idx[k]], 0 <= idx < n (any dtype)
+ *  SG_K_XOR              {n}                -                2n/2n/n: y[i] = x[i] ^ x[n+i]
+ *  SG_K_XOR_CONST        {n, k[n]}          -                n/n/n: y[i] = x[i] ^ k[i]
+ *  SG_K_SBOX             {t[64]}            -                6/6/4: b_i = x[i]&1; v = t[16(2b0+b5) + 8b1+4b2+2b3+b4];
+ *                                                            y[i] = (v >> (3-i)) & 1 (FIPS 46-3 S-box, t in [0,15])
+ *  SG_K_INTO_BITS        -                  -                1/1/32: y[k] = (x >> (31-k)) & 1 (MSB first)
+ *  SG_K_BITS_TO_INT      -                  -                32/32/1: y = sum_k (x[k]&1) << (31-k)
  *
  * dtype SG_I32 admits IDENTITY, DELAY, DECIMATE, EXPAND, COMPARE_EXCHANGE, ADD.
  */
@@ -96,7 +104,13 @@ typedef enum {
     SG_K_BEAM_FIR = 12,
     SG_K_BEAMFORM = 13,
     SG_K_MAGNITUDE = 14,
-    SG_K_MULTIPLY = 15
+    SG_K_MULTIPLY = 15,
+    SG_K_PERMUTE = 16,
+    SG_K_XOR = 17,
+    SG_K_XOR_CONST = 18,
+    SG_K_SBOX = 19,
+    SG_K_INTO_BITS = 20,
+    SG_K_BITS_TO_INT = 21
 } sg_filter_kind;
 
 typedef struct {

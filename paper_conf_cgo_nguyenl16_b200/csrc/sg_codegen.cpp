@@ -54,7 +54,8 @@ static int64_t fdiv(int64_t a, int64_t b) {
 static int64_t fmodp(int64_t a, int64_t b) { return a - fdiv(a, b) * b; }
 
 bool is_view_kind(int k) {
-    return k == SG_K_IDENTITY || k == SG_K_DELAY || k == SG_K_DECIMATE || k == SG_K_EXPAND || k == SG_K_FFT_REORDER;
+    return k == SG_K_IDENTITY || k == SG_K_DELAY || k == SG_K_DECIMATE || k == SG_K_EXPAND || k == SG_K_FFT_REORDER ||
+           k == SG_K_PERMUTE;
 }
 static bool is_view_node(const Node& n) { return n.type != N_FILTER || is_view_kind(n.kind); }
 
@@ -74,6 +75,10 @@ void node_work(const Flat& f, int v, int64_t& flops, int64_t& intops, int64_t& d
     case SG_K_MAGNITUDE: per = 3; break;
     case SG_K_MULTIPLY: per = 1; break;
     case SG_K_COMPARE_EXCHANGE: intops = 2 * n.rep; break;
+    // DES bit kinds, counted as written: one op per XORed bit, one per table lookup, one per bit moved
+    case SG_K_XOR: case SG_K_XOR_CONST: intops = (int64_t)n.iv[0] * n.rep; break;
+    case SG_K_SBOX: intops = n.rep; break;
+    case SG_K_INTO_BITS: case SG_K_BITS_TO_INT: intops = 32 * n.rep; break;
     default: break;
     }
     flops = per * n.rep;
@@ -217,6 +222,14 @@ public:
                     e = u.in[0];
                     continue;
                 }
+                case SG_K_PERMUTE: {
+                    const int64_t n = u.iv[0], m = (int64_t)u.iv.size() - 1;
+                    if (!pos.divisible(m)) return {Ref::RUNTIME, e, pos};
+                    Lin q = pos.divf(m);
+                    pos = q.scaled(n).plus(u.iv[1 + pos.modc(m)]);
+                    e = u.in[0];
+                    continue;
+                }
                 case SG_K_FFT_REORDER: {
                     int64_t n = u.iv[0], F = 2 * n;
                     if (!pos.divisible(F)) return {Ref::RUNTIME, e, pos};
@@ -300,6 +313,7 @@ protected:
     std::vector<int> ins_, outs_;
     std::ostringstream consts_;
     std::map<std::vector<float>, std::string> pool_;
+    int ipool_n_ = 0;
 
     std::string const_array(const std::vector<float>& v) {
         auto it = pool_.find(v);
@@ -346,6 +360,26 @@ protected:
         }
         case SG_K_MAGNITUDE: return "sg_work_magnitude(x_, y_);";
         case SG_K_MULTIPLY: return "sg_work_multiply(x_, y_);";
+        case SG_K_XOR: return "sg_work_xor<" + std::to_string(n.iv[0]) + ">(x_, y_);";
+        case SG_K_XOR_CONST: {  // key bits folded into the code (x ^ 0 = x)
+            std::string c;
+            for (int i = 0; i < n.iv[0]; i++)
+                c += "y_[" + std::to_string(i) + "] = x_[" + std::to_string(i) + "]" +
+                     (n.iv[1 + i] ? " ^ " + std::to_string(n.iv[1 + i]) : std::string()) + "; ";
+            return c;
+        }
+        case SG_K_SBOX: {  // one 64-bit truth-table mask per output bit: bit i of t[idx] = (M_i >> idx) & 1
+            unsigned long long M[4] = {0, 0, 0, 0};
+            for (int k = 0; k < 64; k++)
+                for (int i = 0; i < 4; i++)
+                    if ((n.iv[k] >> (3 - i)) & 1) M[i] |= 1ull << k;
+            char b[160];
+            std::snprintf(b, sizeof b, "sg_work_sbox(x_, y_, 0x%016llxull, 0x%016llxull, 0x%016llxull, 0x%016llxull);",
+                          M[0], M[1], M[2], M[3]);
+            return b;
+        }
+        case SG_K_INTO_BITS: return "sg_work_into_bits(x_, y_);";
+        case SG_K_BITS_TO_INT: return "sg_work_bits_to_int(x_, y_);";
         default: break;
         }
         throw Error(SG_E_UNSUPPORTED, std::string("no work function for ") + kind_name(n.kind));
@@ -2101,6 +2135,16 @@ private:
                 s << "  const int q = sg_fdiv32(lp, " << u.iv[0] << ");\n  return (lp - q * " << u.iv[0] << ") == 0 ? "
                   << rd_name(in) << "(sm, q) : (" << T_ << ")0;\n";
                 break;
+            case SG_K_PERMUTE: {
+                const int64_t n = u.iv[0], m = (int64_t)u.iv.size() - 1;
+                std::string tab = "SG_PI" + std::to_string(ipool_n_++);
+                consts_ << "__constant__ int " << tab << "[" << m << "] = {";
+                for (int64_t k = 0; k < m; k++) consts_ << (k ? "," : "") << (k % 16 == 0 ? "\n  " : "") << u.iv[1 + k];
+                consts_ << "};\n";
+                s << "  const int q = sg_fdiv32(lp, " << m << "), o = lp - q * " << m << ";\n"
+                  << "  return " << rd_name(in) << "(sm, q * " << n << " + " << tab << "[o]);\n";
+                break;
+            }
             case SG_K_FFT_REORDER: {
                 int64_t n = u.iv[0], F = 2 * n;
                 s << "  const int q = sg_fdiv32(lp, " << F << "), o = lp - q * " << F << ";\n"

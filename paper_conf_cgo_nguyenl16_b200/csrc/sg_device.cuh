@@ -127,6 +127,33 @@ SG_DEV void sg_work_beamform(const float (&x)[2 * NC], float (&y)[2], const floa
 }
 
 SG_DEV void sg_work_multiply(const float (&x)[2], float (&y)[1]) { y[0] = __fmul_rn(x[0], x[1]); }
+// DES bit kinds (include/sg.h table); items are int32, bits are x & 1
+template <int N>
+SG_DEV void sg_work_xor(const int (&x)[2 * N], int (&y)[N]) {
+#pragma unroll
+    for (int i = 0; i < N; i++) y[i] = x[i] ^ x[N + i];
+}
+// S-box as four 64-entry truth tables: output bit i (most significant first) = (M_i >> idx) & 1,
+// idx = 16 * (2 b0 + b5) + (8 b1 + 4 b2 + 2 b3 + b4) (FIPS 46-3 row / column rule)
+SG_DEV void sg_work_sbox(const int (&x)[6], int (&y)[4], unsigned long long m0, unsigned long long m1,
+                         unsigned long long m2, unsigned long long m3) {
+    const unsigned idx = ((x[0] & 1u) << 5) | ((x[5] & 1u) << 4) | ((x[1] & 1u) << 3) | ((x[2] & 1u) << 2) |
+                         ((x[3] & 1u) << 1) | (x[4] & 1u);
+    y[0] = (int)((m0 >> idx) & 1ull);
+    y[1] = (int)((m1 >> idx) & 1ull);
+    y[2] = (int)((m2 >> idx) & 1ull);
+    y[3] = (int)((m3 >> idx) & 1ull);
+}
+SG_DEV void sg_work_into_bits(const int (&x)[1], int (&y)[32]) {
+#pragma unroll
+    for (int k = 0; k < 32; k++) y[k] = (int)(((unsigned)x[0] >> (31 - k)) & 1u);
+}
+SG_DEV void sg_work_bits_to_int(const int (&x)[32], int (&y)[1]) {
+    unsigned v = 0u;
+#pragma unroll
+    for (int k = 0; k < 32; k++) v |= ((unsigned)x[k] & 1u) << (31 - k);
+    y[0] = (int)v;
+}
 SG_DEV void sg_work_magnitude(const float (&x)[2], float (&y)[1]) {
     const float b2 = x[1] * x[1];
     y[0] = __fsqrt_rn(fmaf(x[0], x[0], b2));

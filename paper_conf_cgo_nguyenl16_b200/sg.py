@@ -25,7 +25,8 @@ SG_PART_ALGORITHM1, SG_PART_SINGLE, SG_PART_PER_FILTER, SG_PART_USER = 0, 1, 2, 
 KINDS = {"IDENTITY": 0, "FIR": 1, "DELAY": 2, "DECIMATE": 3, "EXPAND": 4, "COMPARE_EXCHANGE": 5,
          "FFT_REORDER": 6, "COMBINE_DFT": 7, "FM_DEMOD": 8, "SUBTRACT": 9, "AMPLIFY": 10, "ADD": 11,
          "BEAM_FIR": 12, "BEAMFORM": 13, "MAGNITUDE": 14,
-         "MULTIPLY": 15}
+         "MULTIPLY": 15, "PERMUTE": 16, "XOR": 17, "XOR_CONST": 18, "SBOX": 19,
+         "INTO_BITS": 20, "BITS_TO_INT": 21}
 
 EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_splitjoin", "sg_branch_begin",
            "sg_branch_end", "sg_plan_opts_default", "sg_plan", "sg_input_items", "sg_output_items",

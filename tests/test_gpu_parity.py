@@ -106,7 +106,8 @@ def test_parity_bitonic_edge_sizes(oracle_lib, n):
 
 
 # ---- second workloads of the paper's suite: BitonicRec, DCT, MatMul
-EXTRA_N = {"bitonicrec32": (3 * 256 + 5, 20000), "dct16": (37, 5000), "matmul16": (41, 5000)}
+EXTRA_N = {"bitonicrec32": (3 * 256 + 5, 20000), "dct16": (37, 5000), "matmul16": (41, 5000),
+           "des16": (3 * 256 + 5, 20000)}
 
 
 @pytest.mark.parametrize("name", list(apps.EXTRA))
@@ -135,4 +136,51 @@ def test_parity_bitonic_rec_variants(oracle_lib, variant):
     n = 1000
     x = inputs.make_input("i32", 32 * n, 6, variant=variant)
     y, _, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+# ---- DES (Fig. 4.2a): published known answers through the CUDA path
+def test_des_known_answers_gpu():
+    import json
+    import os
+    with open(os.path.join(os.path.dirname(__file__), "golden", "des_kat.json")) as f:
+        vec = json.load(f)["vectors"]
+    for v in vec:
+        k, p, c = (int(v[s], 16) for s in ("key", "plaintext", "ciphertext"))
+        for decrypt, src, dst in ((False, p, c), (True, c, p)):
+            x = np.array([src >> 32, src & 0xFFFFFFFF] * 300, dtype=np.uint32).view(np.int32)
+            y, _, _ = run_gpu(apps.des(16, k, decrypt), x, 300)
+            u = y.view(np.uint32)
+            assert all(((int(u[2 * i]) << 32) | int(u[2 * i + 1])) == dst for i in range(300)), v["cite"]
+
+
+@pytest.mark.parametrize("rounds", [1, 2, 16, 20])
+def test_des_rounds_vs_oracle(oracle_lib, rounds):
+    prog = apps.des(rounds, 0xFEDCBA9876543210)
+    n = 2 * 256 + 77
+    x = inputs.make_input("i32", oracle_lib.in_items(prog, n), 40 + rounds)
+    y, _, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+def test_permute_any_dtype(oracle_lib):
+    from workloads.spec import Filter, Pipeline, Program
+    rng = np.random.default_rng(4)
+    for dt in ("f32", "i32"):
+        idx = rng.integers(0, 12, size=9).tolist()
+        prog = Program("perm", dt, Pipeline([Filter("PERMUTE", [12] + idx), Filter("PERMUTE", [9] + idx[::-1][:9])]))
+        n = 1000
+        x = inputs.make_input(dt, 12 * n, 77)
+        y, _, _ = run_gpu(prog, x, n)
+        assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+@pytest.mark.parametrize("mode", ["staged", "general"])
+def test_des_staged_modes(oracle_lib, mode):
+    """The shared-memory (staged) code paths on a bit graph: fused roots and the general path with
+    runtime PERMUTE readers."""
+    prog = apps.des(2, 0x0E329232EA6D0D73)
+    n = 700
+    x = inputs.make_input("i32", oracle_lib.in_items(prog, n), 91)
+    y, _, _ = run_gpu(prog, x, n, codegen_mode=mode)
     assert np.array_equal(y, oracle_lib.run(prog, x, n))

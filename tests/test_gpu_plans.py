@@ -40,6 +40,7 @@ PLANS = [
     ("filterbank8", lambda: apps.filterbank(8), 500),
     ("bitonic8", lambda: apps.bitonic(8), 1000),
     ("fft16", lambda: apps.fft(16), 700),
+    ("des3", lambda: apps.des(3), 700),
     ("beamformer_small", lambda: apps.beamformer(channels=3, beams=2, frame=64, taps=8, mf_taps=16), 9),
 ])
 def test_plan_invariance(oracle_lib, name, prog_fn, n):

@@ -373,3 +373,33 @@ def test_kernel_entry_points_exist(sg, name, part):
         for q in range(p.info()["n_partitions"]):
             src = p.source(q)
             assert re.search(r'__global__ void __launch_bounds__\([^)]*\) sg_part%d(_sync)?\(' % q, src), q
+
+
+# ------------------------------------------------------------------- DES kinds
+def test_des_kind_parameters_validated(sg):
+    gi = sg.Graph("i32")
+    for kind, iv in (("PERMUTE", [4, 0, 4]), ("PERMUTE", [4]), ("XOR_CONST", [3, 1, 0]), ("SBOX", [0] * 63),
+                     ("SBOX", [16] + [0] * 63), ("XOR", [0])):
+        with pytest.raises(sg.SgError) as e:
+            gi.add_filter(kind, iv, [])
+        assert e.value.code == sg.SG_E_ARG, (kind, iv)
+    gf = sg.Graph("f32")
+    for kind, iv in (("XOR", [2]), ("SBOX", [0] * 64), ("INTO_BITS", []), ("BITS_TO_INT", []), ("XOR_CONST", [1, 1])):
+        with pytest.raises(sg.SgError) as e:
+            gf.add_filter(kind, iv, [])
+        assert e.value.code == sg.SG_E_UNSUPPORTED, kind
+    gf.add_filter("PERMUTE", [3, 2, 1, 0], [])     # PERMUTE is dtype-agnostic
+
+
+def test_des_compiles_register_and_staged(sg):
+    """DES: every PERMUTE / splitter / joiner resolves at compile time (no data-movement code), the
+    key bits are folded into the code, and the general staged path compiles the same graph."""
+    with sg.plan(apps.des(16), 1) as p:
+        info = p.info()
+        assert info["n_partitions"] == 1 and info["partition_mode"] == [1]
+        assert info["intops_per_iter"] == 16 * (48 + 32 + 8) + 64 + 64
+        src = p.source(0)
+        assert src.count("sg_work_sbox(") == 16 * 8 and "SG_PI" not in src
+    with sg.plan(apps.des(2), 1, partitioner="per_filter") as p:
+        assert p.info()["n_partitions"] > 1
+        assert any("sg_work_xor<32>" in p.source(q) for q in range(p.info()["n_partitions"]))
