@@ -39,6 +39,7 @@
 #include <map>
 #include <numeric>
 #include <set>
+#include <tuple>
 #include <sstream>
 
 namespace sg {
@@ -988,6 +989,304 @@ private:
         }
         for (size_t g = 0; g < pending.size(); g++)
             if (!stored[g]) throw Error(SG_E_UNSUPPORTED, "internal: output group never produced");
+    }
+};
+
+// ------------------------------------------------------------ bitslice mode
+// A partition whose compute filters are all bit kinds -- INTO_BITS reading the boundary input,
+// BITS_TO_INT writing the boundary output, XOR / XOR_CONST / SBOX in between -- depends only on
+// bit 0 of every inner item (XOR is bitwise, SBOX and BITS_TO_INT read x & 1).  One thread then
+// runs 32 iterations at once: an inner item is a 32-bit word whose bit j belongs to the thread's
+// j-th iteration (bitslicing across iterations), so one LOP3 does the work of 32 firings.
+// INTO_BITS / BITS_TO_INT become 32x32 bit transposes in registers; an S-box becomes a LOP3
+// circuit derived from its table at compile time (3-input cofactor functions + a mux tree);
+// XOR_CONST key bits become complement flags folded into the LUT immediates (free).
+static bool is_bit_kind(int k) {
+    return k == SG_K_INTO_BITS || k == SG_K_BITS_TO_INT || k == SG_K_XOR || k == SG_K_XOR_CONST || k == SG_K_SBOX;
+}
+
+bool bitslice_eligible(const Flat& f, const std::vector<int>& nodes, std::string* why) {
+    auto fail = [&](const std::string& s) { if (why) *why = s; return false; };
+    if (f.dtype != SG_I32) return fail("not an int32 graph");
+    if (!register_mode_eligible(f, nodes, why)) return false;
+    for (int v : nodes) {
+        const Node& n = f.nodes[v];
+        if (n.type == N_FILTER && !is_view_kind(n.kind) && !is_bit_kind(n.kind))
+            return fail(std::string("non-bit filter ") + kind_name(n.kind));
+    }
+    std::vector<int> ins, outs;
+    partition_boundary(f, nodes, ins, outs);
+    if (f.edges[ins[0]].per_iter > 8 || f.edges[outs[0]].per_iter > 8) return fail("row too wide for bitslicing");
+    return true;  // domain checks (words only at INTO_BITS / BITS_TO_INT) happen during generation
+}
+
+class BitGen : public GenBase {
+public:
+    using GenBase::GenBase;
+
+    KernelInfo run(const CodegenOpts& opt) {
+        KernelInfo ki;
+        ki.mode = 1;
+        ki.name = "sg_part" + std::to_string(part_);
+        ki.name_sync = ki.name;
+        fill_io(ki);
+        ein_ = ins_[0];
+        eout_ = outs_[0];
+        PIN_ = f_.edges[ein_].per_iter;
+        POUT_ = f_.edges[eout_].per_iter;
+        off_in_ = ki.in_lo[0];
+        off_out_ = ki.out_lo[0];
+        // output words: each must be produced by a BITS_TO_INT firing
+        std::vector<std::vector<BV>> obits(POUT_);
+        for (int64_t p = 0; p < POUT_; p++) {
+            Ref r = R_.resolve(eout_, Lin::k(off_out_ + p));
+            if (r.k != Ref::PHYS || r.edge == ein_) throw Error(SG_E_UNSUPPORTED, "bitslice: output item is not a BITS_TO_INT word");
+            const Edge& ed = f_.edges[r.edge];
+            const Node& n = f_.nodes[ed.src];
+            if (n.kind != SG_K_BITS_TO_INT) throw Error(SG_E_UNSUPPORTED, "bitslice: output not from BITS_TO_INT");
+            int64_t g = (r.pos.c - ed.pre) / n.push;
+            std::vector<BV> b(32);
+            for (int i = 0; i < 32; i++) b[i] = bit(n.in[0], g * n.pop + i);
+            obits[p] = b;
+        }
+        const int NT = opt.threads > 0 ? opt.threads : 128;
+        ki.threads = ki.threads_sync = NT;
+        ki.tile = ki.tile_sync = NT * 32;
+        ki.smem = ki.smem_sync = 0;
+        std::ostringstream s;
+        s << header("bitslice") << consts_.str() << args_struct();
+        s << "extern \"C\" __global__ void __launch_bounds__(" << NT << ", 2) " << ki.name << "(const SgArgs a) {\n"
+          << "  const int lane = threadIdx.x & 31;\n"
+          << "  const long long wstep = (long long)gridDim.x * " << NT / 32 << " * 1024;\n"
+          << "  const " << T_ << "* gin = SG_IN(0) + ((" << off_in_ << "LL) - SG_IN_BASE(0));\n"
+          << "  " << T_ << "* gout = SG_OUT(0) + ((" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
+          << "  const bool vin = " << (PIN_ == 2 || PIN_ == 4 ? "(reinterpret_cast<unsigned long long>(gin) & " + std::to_string(PIN_ * 4 - 1) + "ull) == 0" : std::string("false")) << ";\n"
+          << "  const bool vout = " << (POUT_ == 2 || POUT_ == 4 ? "(reinterpret_cast<unsigned long long>(gout) & " + std::to_string(POUT_ * 4 - 1) + "ull) == 0" : std::string("false")) << ";\n"
+          << "  for (long long wb = SG_K_BEGIN + ((long long)blockIdx.x * " << NT / 32 << " + (threadIdx.x >> 5)) * 1024; wb < SG_K_END; wb += wstep) {\n";
+        // loads: word q of iteration wb + 32 j + lane -> w<q>[j]
+        for (int64_t q = 0; q < PIN_; q++) s << "    unsigned w" << q << "[32];\n";
+        s << "#pragma unroll\n"
+          << "    for (int j = 0; j < 32; j++) {\n"
+          << "      const long long k = wb + 32 * j + lane;\n"
+          << "      if (k < SG_K_END) {\n";
+        if (PIN_ == 2 || PIN_ == 4) {
+            s << "        if (vin) {\n"
+              << "          const int" << PIN_ << " t = __ldg(reinterpret_cast<const int" << PIN_ << "*>(gin + k * " << PIN_ << "LL));\n";
+            static const char* comp[4] = {"x", "y", "z", "w"};
+            for (int64_t q = 0; q < PIN_; q++) s << "          w" << q << "[j] = (unsigned)t." << comp[q] << ";\n";
+            s << "        } else {\n";
+            for (int64_t q = 0; q < PIN_; q++) s << "          w" << q << "[j] = (unsigned)__ldg(gin + k * " << PIN_ << "LL + " << q << ");\n";
+            s << "        }\n";
+        } else {
+            for (int64_t q = 0; q < PIN_; q++) s << "        w" << q << "[j] = (unsigned)__ldg(gin + k * " << PIN_ << "LL + " << q << ");\n";
+        }
+        s << "      } else {\n";
+        for (int64_t q = 0; q < PIN_; q++) s << "        w" << q << "[j] = 0u;\n";
+        s << "      }\n    }\n";
+        for (int64_t q : used_cols_) s << "    sg_transpose32(w" << q << ");\n";
+        s << body_.str();
+        for (int64_t p = 0; p < POUT_; p++) {
+            s << "    unsigned o" << p << "[32];\n";
+            for (int i = 0; i < 32; i++) s << "    o" << p << "[" << 31 - i << "] = " << obits[p][i].expr() << ";\n";
+            s << "    sg_transpose32(o" << p << ");\n";
+        }
+        s << "#pragma unroll\n"
+          << "    for (int j = 0; j < 32; j++) {\n"
+          << "      const long long k = wb + 32 * j + lane;\n"
+          << "      if (k < SG_K_END) {\n";
+        if (POUT_ == 2 || POUT_ == 4) {
+            s << "        if (vout) {\n"
+              << "          reinterpret_cast<int" << POUT_ << "*>(gout + k * " << POUT_ << "LL)[0] = make_int" << POUT_ << "(";
+            for (int64_t p = 0; p < POUT_; p++) s << (p ? ", " : "") << "(int)o" << p << "[j]";
+            s << ");\n        } else {\n";
+            for (int64_t p = 0; p < POUT_; p++) s << "          gout[k * " << POUT_ << "LL + " << p << "] = (int)o" << p << "[j];\n";
+            s << "        }\n";
+        } else {
+            for (int64_t p = 0; p < POUT_; p++) s << "        gout[k * " << POUT_ << "LL + " << p << "] = (int)o" << p << "[j];\n";
+        }
+        s << "      }\n    }\n  }\n}\n";
+        ki.source = s.str();
+        return ki;
+    }
+
+private:
+    struct BV {  // a packed bit value: register name (or literal) and a complement flag
+        std::string s;
+        bool neg = false;
+        std::string expr() const { return neg ? "(~" + s + ")" : s; }
+        bool operator==(const BV& o) const { return s == o.s && neg == o.neg; }
+        bool operator<(const BV& o) const { return s != o.s ? s < o.s : neg < o.neg; }
+    };
+    int ein_ = -1, eout_ = -1;
+    int64_t PIN_ = 0, POUT_ = 0, off_in_ = 0, off_out_ = 0;
+    std::ostringstream body_;
+    int nv_ = 0;
+    std::set<int64_t> used_cols_;
+    std::map<std::pair<int, int64_t>, std::vector<BV>> memo_;
+    std::map<std::tuple<int, BV, BV, BV>, BV> lop_memo_;
+
+    BV fresh(const std::string& rhs) {
+        std::string v = "b" + std::to_string(nv_++);
+        body_ << "    const unsigned " << v << " = " << rhs << ";\n";
+        return {v, false};
+    }
+    static BV zero() { return {"0u", false}; }
+    static BV ones() { return {"0u", true}; }
+    // lop3 of true values A, B, C with truth table F (index A<<2 | B<<1 | C); complements folded in
+    BV lop3(int F, BV A, BV B, BV C) {
+        const int flip = (A.neg ? 4 : 0) | (B.neg ? 2 : 0) | (C.neg ? 1 : 0);
+        int L = 0;
+        for (int p = 0; p < 8; p++)
+            if ((F >> (p ^ flip)) & 1) L |= 1 << p;
+        if (L == 0x00) return zero();
+        if (L == 0xFF) return ones();
+        A.neg = B.neg = C.neg = false;
+        if (L == 0xF0) return A;
+        if (L == 0x0F) return {A.s, true};
+        if (L == 0xCC) return B;
+        if (L == 0x33) return {B.s, true};
+        if (L == 0xAA) return C;
+        if (L == 0x55) return {C.s, true};
+        auto key = std::make_tuple(L, A, B, C);
+        auto it = lop_memo_.find(key);
+        if (it != lop_memo_.end()) return it->second;
+        char b[32];
+        std::snprintf(b, sizeof b, "0x%02x", L);
+        BV r = fresh("sg_lop3<" + std::string(b) + ">(" + A.s + ", " + B.s + ", " + C.s + ")");
+        lop_memo_[key] = r;
+        return r;
+    }
+    BV mux(const BV& s, const BV& x1, const BV& x0) {  // s ? x1 : x0
+        if (x1 == x0) return x1;
+        return lop3(0xCA, s, x1, x0);
+    }
+    // S-box as a circuit: output bit i of t[idx(b)], idx = 32 b0 + 16 b5 + 8 b1 + 4 b2 + 2 b3 + b4.
+    // Three inputs feed 3-input cofactor functions (one LOP3 each), the other three drive a mux tree;
+    // the split and the mux order with the fewest gates are chosen by counting.
+    std::vector<BV> sbox(const std::vector<BV>& x, const std::vector<int32_t>& t) {
+        auto tab = [&](int out, const int b[6]) {
+            int idx = 32 * b[0] + 16 * b[5] + 8 * b[1] + 4 * b[2] + 2 * b[3] + b[4];
+            return (t[idx] >> (3 - out)) & 1;
+        };
+        int best = 1 << 30;
+        std::vector<int> bl, bs;
+        for (int m = 0; m < 64; m++) {
+            if (__builtin_popcount(m) != 3) continue;
+            std::vector<int> lv, sv;
+            for (int i = 0; i < 6; i++) (m >> i & 1 ? lv : sv).push_back(i);
+            std::sort(sv.begin(), sv.end());
+            do {
+                // count distinct non-trivial cofactors and muxes (structural, without complements)
+                std::set<int> cof;
+                std::set<std::vector<int>> muxes;
+                for (int out = 0; out < 4; out++) {
+                    std::vector<int> lvl;
+                    for (int sa = 0; sa < 8; sa++) {
+                        int u = 0;
+                        for (int p = 0; p < 8; p++) {
+                            int b[6];
+                            b[lv[0]] = p >> 2 & 1; b[lv[1]] = p >> 1 & 1; b[lv[2]] = p & 1;
+                            b[sv[0]] = sa >> 2 & 1; b[sv[1]] = sa >> 1 & 1; b[sv[2]] = sa & 1;
+                            u |= tab(out, b) << p;
+                        }
+                        int canon = std::min(u, 255 - u);
+                        if (canon != 0 && canon != 0x0F && canon != 0x33 && canon != 0x55) cof.insert(canon);
+                        lvl.push_back(u);
+                    }
+                    int id = 1000;
+                    for (int d = 2; d >= 0; d--) {
+                        std::vector<int> nx;
+                        for (size_t k = 0; k < lvl.size(); k += 2) {
+                            if (lvl[k] == lvl[k + 1]) { nx.push_back(lvl[k]); continue; }
+                            std::vector<int> key = {d, lvl[k], lvl[k + 1]};
+                            muxes.insert(key);
+                            nx.push_back(id++ + out * 100000);
+                        }
+                        lvl = nx;
+                    }
+                }
+                int cost = (int)cof.size() + (int)muxes.size();
+                if (cost < best) { best = cost; bl = lv; bs = sv; }
+            } while (std::next_permutation(sv.begin(), sv.end()));
+        }
+        std::vector<BV> y(4);
+        for (int out = 0; out < 4; out++) {
+            std::vector<BV> lvl;
+            for (int sa = 0; sa < 8; sa++) {
+                int u = 0;
+                for (int p = 0; p < 8; p++) {
+                    int b[6];
+                    b[bl[0]] = p >> 2 & 1; b[bl[1]] = p >> 1 & 1; b[bl[2]] = p & 1;
+                    b[bs[0]] = sa >> 2 & 1; b[bs[1]] = sa >> 1 & 1; b[bs[2]] = sa & 1;
+                    u |= tab(out, b) << p;
+                }
+                lvl.push_back(lop3(u, x[bl[0]], x[bl[1]], x[bl[2]]));
+            }
+            for (int d = 2; d >= 0; d--) {   // mux on bs[d]: pairs (sa with bit (2-d) = 0 / 1)
+                std::vector<BV> nx;
+                for (size_t k = 0; k < lvl.size(); k += 2) nx.push_back(mux(x[bs[d]], lvl[k + 1], lvl[k]));
+                lvl = nx;
+            }
+            y[out] = lvl[0];
+        }
+        return y;
+    }
+    // packed value of item `pos` of edge e (bit domain)
+    BV bit(int e, int64_t pos) {
+        Ref r = R_.resolve(e, Lin::k(pos));
+        if (r.k == Ref::ZERO) return zero();
+        if (r.k != Ref::PHYS) throw Error(SG_E_UNSUPPORTED, "bitslice: non-constant position");
+        if (r.edge == ein_) throw Error(SG_E_UNSUPPORTED, "bitslice: a raw input word is used as a bit");
+        const Edge& ed = f_.edges[r.edge];
+        const int u = ed.src;
+        const Node& n = f_.nodes[u];
+        const int64_t q = r.pos.c - ed.pre, g = q / n.push, j = q % n.push;
+        auto key = std::make_pair(u, g);
+        auto it = memo_.find(key);
+        if (it != memo_.end()) return it->second[j];
+        std::vector<BV> y;
+        switch (n.kind) {
+        case SG_K_INTO_BITS: {
+            Ref ri = R_.resolve(n.in[0], Lin::k(g * n.pop));
+            if (ri.k != Ref::PHYS || ri.edge != ein_) throw Error(SG_E_UNSUPPORTED, "bitslice: INTO_BITS must read the boundary input");
+            const int64_t c = ri.pos.c - off_in_;
+            if (c < 0 || c >= PIN_) throw Error(SG_E_UNSUPPORTED, "bitslice: input column out of range");
+            used_cols_.insert(c);
+            for (int b = 0; b < 32; b++) y.push_back({"w" + std::to_string(c) + "[" + std::to_string(31 - b) + "]", false});
+            break;
+        }
+        case SG_K_XOR: {
+            const int64_t nn = n.iv[0];
+            std::vector<BV> x(2 * nn);
+            for (int64_t i = 0; i < 2 * nn; i++) x[i] = bit(n.in[0], g * n.pop + i);
+            for (int64_t i = 0; i < nn; i++) {
+                BV a = x[i], b = x[nn + i];
+                if (a.s == "0u") { y.push_back({b.s, b.neg ^ a.neg}); continue; }
+                if (b.s == "0u") { y.push_back({a.s, a.neg ^ b.neg}); continue; }
+                BV r = fresh(a.s + " ^ " + b.s);
+                r.neg = a.neg ^ b.neg;
+                y.push_back(r);
+            }
+            break;
+        }
+        case SG_K_XOR_CONST:
+            for (int64_t i = 0; i < n.iv[0]; i++) {
+                BV a = bit(n.in[0], g * n.pop + i);
+                if (n.iv[1 + i] & 1) a.neg = !a.neg;
+                y.push_back(a);
+            }
+            break;
+        case SG_K_SBOX: {
+            std::vector<BV> x(6);
+            for (int i = 0; i < 6; i++) x[i] = bit(n.in[0], g * n.pop + i);
+            y = sbox(x, n.iv);
+            break;
+        }
+        default:
+            throw Error(SG_E_UNSUPPORTED, std::string("bitslice: ") + kind_name(n.kind) + " output used as a bit");
+        }
+        memo_[key] = y;
+        return y[j];
     }
 };
 
@@ -2837,6 +3136,14 @@ KernelInfo generate_kernel(const Flat& f, const std::vector<int>& nodes, int par
     int mode = opt.mode;
     if (mode == 1 && !reg_ok) throw Error(SG_E_UNSUPPORTED, "register mode not possible: " + why);
     if (mode == 0) mode = reg_ok ? 1 : 2;
+    if (mode == 1 && opt.mode == 0 && !std::getenv("SG_NO_BITSLICE") && bitslice_eligible(f, nodes, nullptr)) {
+        try {
+            BitGen g(f, nodes, part_id);
+            return g.run(opt);
+        } catch (const Error&) {
+            // bit kinds whose words cross the partition boundary (e.g. a lone XOR): plain register mode
+        }
+    }
     if (mode == 1) {
         RegGen g(f, nodes, part_id);
         return g.run(opt);

@@ -154,6 +154,26 @@ SG_DEV void sg_work_bits_to_int(const int (&x)[32], int (&y)[1]) {
     for (int k = 0; k < 32; k++) v |= ((unsigned)x[k] & 1u) << (31 - k);
     y[0] = (int)v;
 }
+// bitslice mode: any 3-input boolean function in one LOP3 (LUT index a<<2 | b<<1 | c)
+template <int LUT>
+SG_DEV unsigned sg_lop3(unsigned a, unsigned b, unsigned c) {
+    unsigned d;
+    asm("lop3.b32 %0, %1, %2, %3, %4;" : "=r"(d) : "r"(a), "r"(b), "r"(c), "n"(LUT));
+    return d;
+}
+// 32x32 bit-matrix transpose in registers: afterwards bit j of a[i] = bit i of the old a[j]
+SG_DEV void sg_transpose32(unsigned (&a)[32]) {
+#pragma unroll
+    for (unsigned s = 16, m = 0x0000FFFFu; s > 0; s >>= 1, m ^= m << s) {
+#pragma unroll
+        for (int i = 0; i < 32; i++) {
+            if (i & s) continue;
+            const unsigned t = ((a[i] >> s) ^ a[i + s]) & m;
+            a[i + s] ^= t;
+            a[i] ^= t << s;
+        }
+    }
+}
 SG_DEV void sg_work_magnitude(const float (&x)[2], float (&y)[1]) {
     const float b2 = x[1] * x[1];
     y[0] = __fsqrt_rn(fmaf(x[0], x[0], b2));

@@ -184,3 +184,34 @@ def test_des_staged_modes(oracle_lib, mode):
     x = inputs.make_input("i32", oracle_lib.in_items(prog, n), 91)
     y, _, _ = run_gpu(prog, x, n, codegen_mode=mode)
     assert np.array_equal(y, oracle_lib.run(prog, x, n))
+
+
+@pytest.mark.parametrize("n", [1, 31, 33, 1023, 1025, 3 * 4096 + 7])
+def test_des_bitslice_ragged_and_register_mode(oracle_lib, n):
+    """Bitsliced DES (32 iterations per thread, 1024 per warp) on ragged sizes, against the oracle and
+    against the thread-per-iteration register kernel."""
+    prog = apps.des(16, 0x3B3898371520F75E)
+    x = inputs.make_input("i32", oracle_lib.in_items(prog, n), 500 + n)
+    ref = oracle_lib.run(prog, x, n)
+    y, info, _ = run_gpu(prog, x, n)
+    assert np.array_equal(y, ref)
+    y2, _, _ = run_gpu(prog, x, n, codegen_mode="register")
+    assert np.array_equal(y2, ref)
+
+
+def test_des_bitslice_misaligned_buffers(oracle_lib):
+    """Input / output pointers not 8-byte aligned: the bitsliced kernel's scalar load / store path."""
+    torch = _torch()
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    prog = apps.des(16)
+    n = 5000
+    x = inputs.make_input("i32", oracle_lib.in_items(prog, n), 321)
+    ref = oracle_lib.run(prog, x, n)
+    with sg.plan(prog, 1) as p:
+        xb = torch.zeros(x.size + 1, dtype=torch.int32, device="cuda")
+        xb[1:] = torch.from_numpy(x).cuda()
+        yb = torch.full((p.output_items(n) + 1,), -7, dtype=torch.int32, device="cuda")
+        p.run(xb[1:], n, yb[1:])
+        torch.cuda.synchronize()
+        assert np.array_equal(yb[1:].cpu().numpy(), ref)
+        assert int(yb[0]) == -7

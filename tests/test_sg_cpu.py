@@ -393,11 +393,17 @@ def test_des_kind_parameters_validated(sg):
 
 def test_des_compiles_register_and_staged(sg):
     """DES: every PERMUTE / splitter / joiner resolves at compile time (no data-movement code), the
-    key bits are folded into the code, and the general staged path compiles the same graph."""
+    key bits are folded into the code, and the general staged path compiles the same graph.  The
+    default plan is the bitsliced kernel (32 iterations per thread, S-boxes as LOP3 circuits)."""
     with sg.plan(apps.des(16), 1) as p:
         info = p.info()
         assert info["n_partitions"] == 1 and info["partition_mode"] == [1]
         assert info["intops_per_iter"] == 16 * (48 + 32 + 8) + 64 + 64
+        src = p.source(0)
+        assert "(bitslice mode)" in src and "sg_transpose32(w0)" in src and "sg_transpose32(o1)" in src
+        assert 16 * 8 * 30 < src.count("sg_lop3<") < 16 * 8 * 64      # <= 64 gates per S-box
+        assert "sg_work_sbox(" not in src and "SG_PI" not in src
+    with sg.plan(apps.des(16), 1, codegen_mode="register") as p:
         src = p.source(0)
         assert src.count("sg_work_sbox(") == 16 * 8 and "SG_PI" not in src
     with sg.plan(apps.des(2), 1, partitioner="per_filter") as p:
