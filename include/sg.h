@@ -158,6 +158,13 @@ typedef struct sg_plan_opts {
     int32_t verbose;
     int32_t plan_only;             /* 1: stop after partitioning and mapping (no code generation,
                                       no NVRTC); sg_run on such a plan returns SG_E_ARG */
+    int32_t replicas;              /* hybrid replica x pipeline plans: 0 or 1 = the paper's
+                                      pipeline mapping of all partitions onto the G GPUs (Eq. III.5: each
+                                      partition on exactly one GPU); R > 1 (R | G) = R replica groups of G/R
+                                      GPUs, each holding the whole graph mapped by the ILP onto its G/R GPUs,
+                                      fragments dealt round-robin to the groups; -1 = R chosen by the cost
+                                      model max(Tmax(G/R)/R, input / output distribution over NVLink).
+                                      sg_comm_init / sg_run_rank support R = 1 only (SG_E_UNSUPPORTED). */
 } sg_plan_opts;
 
 typedef struct sg_plan_info_s {
@@ -183,6 +190,8 @@ typedef struct sg_plan_info_s {
     double flops_per_iter_written;   /* algorithmic fp32 flops per iteration as written (FMA = 2) */
     double flops_per_iter_pruned;    /* same after dead-firing / zero-tap elimination (<= written) */
     int64_t intops_per_iter;         /* algorithmic integer ops per iteration (min/max, adds) */
+    int32_t replicas;                /* replica groups R; partition_gpu[] is the mapping inside group 0,
+                                        group r runs partition p on logical GPU r * (n_gpus / R) + partition_gpu[p] */
 } sg_plan_info_t;
 
 /* ---- graph construction (the top-level stream is an implicit pipeline) ---- */

@@ -140,12 +140,15 @@ int64_t fragment_size(const Plan& p, int64_t n) {
         for (auto& e : p.flat.edges)
             if (e.src >= 0 && e.dst >= 0 && p.node_part[e.src] != p.node_part[e.dst]) ring += 4 * e.per_iter;
         if (ring > 0) F = std::min<int64_t>(F, std::max<int64_t>(wave, ((int64_t)1 << 30) / ring));
+        // replica groups: every group gets fragments (at least two rounds of R)
+        if (p.R > 1) F = std::min<int64_t>(F, std::max<int64_t>(1, (n + 2 * p.R - 1) / (2 * p.R)));
     }
     return std::max<int64_t>(1, std::min(F, n));
 }
 
 void Plan::comm_init(int nranks, int rank, const uint8_t id[128], int device) {
     if (nranks != G) throw Error(SG_E_ARG, "world size must equal the plan's n_gpus");
+    if (R != 1) throw Error(SG_E_UNSUPPORTED, "sg_run_rank supports the pipeline mapping only (replicas = 1)");
     if (rank < 0 || rank >= nranks) throw Error(SG_E_ARG, "bad rank");
     SG_RT2(cudaSetDevice(device));
     ncclUniqueId uid;

@@ -486,13 +486,10 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
 }
 
 // ============================================================ plan assembly
-void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
-    p.flat = Flat::build(g);
-    p.G = G;
-    p.opts = o;
-    const Flat& f = p.flat;
+namespace {
+// Partitions for a pipeline over Gs GPUs (Algorithm 1's cap depends on Gs).
+std::vector<std::vector<int>> make_partitions(const Flat& f, const sg_graph& g, int Gs, const sg_plan_opts& o) {
     const int N = (int)f.nodes.size();
-    // ---- partitions
     std::vector<std::vector<int>> parts;
     switch (o.partitioner) {
     case SG_PART_SINGLE: {
@@ -514,19 +511,130 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     }
     case SG_PART_ALGORITHM1: {
         double cap = 0;
-        if (G > 1) {
+        if (Gs > 1) {
             std::vector<int> all(N);
             std::iota(all.begin(), all.end(), 0);
             double sum = 0;
             for (int v = 0; v < N; v++) sum += pee_estimate(f, {v}).t;
             // G-aware cap: similar-sized partitions (goal 4)
-            cap = std::max(pee_estimate(f, all).t, sum / 4) / G * 1.25;
+            cap = std::max(pee_estimate(f, all).t, sum / 4) / Gs * 1.25;
         }
         parts = algorithm1(f, g, cap);
         break;
     }
     default: throw Error(SG_E_ARG, "unknown partitioner");
     }
+    return parts;
+}
+
+struct GroupMap {
+    std::vector<double> T;
+    std::vector<PdgEdge> pdg;
+    MapResult m;
+};
+
+// PEE times, PDG and the ILP mapping of `parts` onto Gs GPUs.
+GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, int Gs, const sg_plan_opts& o) {
+    const int N = (int)f.nodes.size(), P = (int)parts.size();
+    std::vector<int> owner(N, -1);
+    for (int i = 0; i < P; i++) for (int v : parts[i]) if (v >= 0 && v < N) owner[v] = i;
+    GroupMap gm;
+    gm.T.resize(P);
+    for (int i = 0; i < P; i++) gm.T[i] = pee_estimate(f, parts[i]).t;
+    // PDG: D_ij = sum of the weights of crossing edges (bytes / iteration)
+    std::map<std::pair<int, int>, double> D;
+    for (auto& e : f.edges) {
+        if (e.src < 0 || e.dst < 0) continue;
+        int a = owner[e.src], b = owner[e.dst];
+        if (a >= 0 && b >= 0 && a != b) D[{a, b}] += 4.0 * e.per_iter;
+    }
+    for (auto& kv : D) gm.pdg.push_back({kv.first.first, kv.first.second, kv.second});
+    gm.m.assign.assign(P, 0);
+    if (Gs > 1) {
+        Topology topo = Topology::nvswitch(Gs);
+        double bw = o.link_gbps > 0 ? o.link_gbps : 770.0;          // bytes per ns
+        double lat_us = o.link_latency_us > 0 ? o.link_latency_us : 10.0;
+        double lat = lat_us * 1e3 / 65536.0;                          // amortised per iteration (reading 12)
+        gm.m = map_partitions(gm.T, gm.pdg, topo, lat, bw, o.ilp_time_limit_ms > 0 ? o.ilp_time_limit_ms : 10000, 0);
+    } else {
+        gm.m.tmax = std::accumulate(gm.T.begin(), gm.T.end(), 0.0);
+        gm.m.optimal = true;
+    }
+    return gm;
+}
+
+// Throughput bound of R replica groups of Gs GPUs each on the NVSwitch star:
+// group r runs the group mapping `a` on GPUs r*Gs .. r*Gs+Gs-1 and 1/R of the fragments, so every
+// GPU's compute (Eq. III.4) and every link's load (Eq. III.6-III.7) is 1/R of the group's; the
+// input GPU's uplink also ships the other groups' input share and the output GPU's downlink
+// receives their output share.  Links carry Lat (Eq. III.3) only when they carry bytes, so a
+// mapping that moves nothing is not charged a transfer.
+double hybrid_cost(const Flat& f, const std::vector<double>& T, const std::vector<PdgEdge>& pdg,
+                   const std::vector<int>& a, int in_gpu, int out_gpu, int Gs, int R, const sg_plan_opts& o) {
+    const int G = Gs * R;
+    const double bw = o.link_gbps > 0 ? o.link_gbps : 770.0;
+    const double lat = (o.link_latency_us > 0 ? o.link_latency_us : 10.0) * 1e3 / 65536.0;
+    std::vector<double> comp(Gs, 0.0), up(G, 0.0), down(G, 0.0);
+    for (size_t i = 0; i < T.size(); i++) comp[a[i]] += T[i];
+    for (int r = 0; r < R; r++) {
+        for (auto& e : pdg) {
+            int k = a[e.src], h = a[e.dst];
+            if (k == h) continue;
+            up[r * Gs + k] += e.bytes / R;
+            down[r * Gs + h] += e.bytes / R;
+        }
+        if (r == 0) continue;
+        const double bi = 4.0 * (double)f.in_per_iter / R, bo = 4.0 * (double)f.out_per_iter / R;
+        up[in_gpu] += bi;
+        down[r * Gs + in_gpu] += bi;
+        up[r * Gs + out_gpu] += bo;
+        down[out_gpu] += bo;
+    }
+    double t = 0;
+    for (double c : comp) t = std::max(t, c / R);
+    for (int g = 0; g < G; g++) {
+        if (up[g] > 0) t = std::max(t, lat + up[g] / bw);
+        if (down[g] > 0) t = std::max(t, lat + down[g] / bw);
+    }
+    return t;
+}
+
+int io_gpu(const Flat& f, const std::vector<std::vector<int>>& parts, const std::vector<int>& a, int node) {
+    for (size_t i = 0; i < parts.size(); i++)
+        for (int v : parts[i]) if (v == node) return a[i];
+    return 0;
+}
+}  // namespace
+
+void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
+    p.flat = Flat::build(g);
+    p.G = G;
+    p.opts = o;
+    const Flat& f = p.flat;
+    const int N = (int)f.nodes.size();
+    // ---- replica groups (hybrid replica x pipeline; R = 1 is the paper's mapping)
+    int R = 1;
+    if (o.replicas > 1) {
+        if (G % o.replicas) throw Error(SG_E_ARG, "replicas must divide n_gpus");
+        R = o.replicas;
+    } else if (o.replicas < 0 && G > 1) {
+        double best = 0;
+        for (int r = 1; r <= G; r++) {
+            if (G % r) continue;
+            auto pr = make_partitions(f, g, G / r, o);
+            GroupMap gm = map_group(f, pr, G / r, o);
+            double c = hybrid_cost(f, gm.T, gm.pdg, gm.m.assign, io_gpu(f, pr, gm.m.assign, f.edges[f.in_edge].dst),
+                                   io_gpu(f, pr, gm.m.assign, f.edges[f.out_edge].src), G / r, r, o);
+            if (r == 1 || c < best * 0.999) { best = c; R = r; }
+        }
+    } else if (o.replicas < -1) {
+        throw Error(SG_E_ARG, "replicas must be -1 (auto), 0/1 (pipeline) or a divisor of n_gpus");
+    }
+    const int Gs = G / R;
+    p.R = R;
+    p.Gs = Gs;
+    // ---- partitions
+    std::vector<std::vector<int>> parts = make_partitions(f, g, Gs, o);
     // validate: cover, convex; order topologically
     std::vector<int> owner(N, -1);
     for (size_t i = 0; i < parts.size(); i++) {
@@ -572,30 +680,15 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         p.parts[i].t_dt = est.t_dt;
         p.part_time[i] = est.t;
     }
-    // ---- PDG: D_ij = sum of the weights of crossing edges (bytes / iteration)
-    std::map<std::pair<int, int>, double> D;
-    for (auto& e : f.edges) {
-        if (e.src < 0 || e.dst < 0) continue;
-        int a = owner[e.src], b = owner[e.dst];
-        if (a != b) D[{a, b}] += 4.0 * e.per_iter;
-    }
-    p.pdg.clear();
-    for (auto& kv : D) p.pdg.push_back({kv.first.first, kv.first.second, kv.second});
-    // ---- mapping
+    // ---- PDG and mapping inside one replica group of Gs GPUs
+    GroupMap gm = map_group(f, parts, Gs, o);
+    p.pdg = gm.pdg;
     p.part_gpu.assign(P, 0);
-    if (G > 1) {
-        Topology topo = Topology::nvswitch(G);
-        double bw = o.link_gbps > 0 ? o.link_gbps : 770.0;          // bytes per ns
-        double lat_us = o.link_latency_us > 0 ? o.link_latency_us : 10.0;
-        double lat = lat_us * 1e3 / 65536.0;                          // amortised per iteration (reading 12)
-        MapResult m = map_partitions(T, p.pdg, topo, lat, bw, o.ilp_time_limit_ms > 0 ? o.ilp_time_limit_ms : 10000, 0);
-        for (int i = 0; i < P; i++) p.part_gpu[i] = m.assign[i];
-        p.est_tmax = m.tmax;
-        p.ilp_optimal = m.optimal;
-    } else {
-        p.est_tmax = std::accumulate(T.begin(), T.end(), 0.0);
-        p.ilp_optimal = true;
-    }
+    for (int i = 0; i < P; i++) p.part_gpu[i] = gm.m.assign[i];
+    p.est_tmax = R == 1 ? gm.m.tmax
+                        : hybrid_cost(f, gm.T, gm.pdg, gm.m.assign, io_gpu(f, parts, gm.m.assign, f.edges[f.in_edge].dst),
+                                      io_gpu(f, parts, gm.m.assign, f.edges[f.out_edge].src), Gs, R, o);
+    p.ilp_optimal = gm.m.optimal;
     // ---- devices
     p.virtual_gpus = o.virtual_gpus != 0;
     p.devices.assign(G, 0);

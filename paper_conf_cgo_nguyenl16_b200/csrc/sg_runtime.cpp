@@ -373,7 +373,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
     last_launches = 0;
     const int64_t n_in = flat.input_items(n);
     // ---- fast path: one partition on one GPU, launched on the caller's stream
-    if (parts.size() == 1) {
+    if (parts.size() == 1 && R == 1) {
         CompiledKernel& ck = kernels[0];
         DevGuard dg(devices[0]);
         IoBinding io;
@@ -429,7 +429,8 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                     }
                 }
         }
-        // cut edges between partitions
+        // cut edges between partitions, one set of rings per replica group
+        for (int grp = 0; grp < R; grp++)
         for (size_t ei = 0; ei < flat.edges.size(); ei++) {
             const Edge& ed = flat.edges[ei];
             if (ed.src < 0 || ed.dst < 0) continue;
@@ -437,10 +438,11 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
             if (ps == pd) continue;
             CutRing r;
             r.edge = (int)ei;
+            r.group = grp;
             r.src_part = ps;
             r.dst_part = pd;
-            r.src_gpu = part_gpu[ps];
-            r.dst_gpu = part_gpu[pd];
+            r.src_gpu = grp * Gs + part_gpu[ps];
+            r.dst_gpu = grp * Gs + part_gpu[pd];
             edge_window(flat, (int)ei, r.lo, r.extra);
             r.per_iter = ed.per_iter;
             r.slot_items = r.per_iter * F + r.extra;
@@ -477,11 +479,12 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
         rt_fragment = F;
         rt_ready = true;
     }
-    // per partition: which rings feed it / leave it
-    std::vector<std::vector<int>> ring_in(parts.size()), ring_out(parts.size());
+    // per (group, partition): which rings feed it / leave it
+    const size_t NP = parts.size();
+    std::vector<std::vector<int>> ring_in(R * NP), ring_out(R * NP);
     for (size_t ri = 0; ri < rings.size(); ri++) {
-        ring_in[rings[ri].dst_part].push_back((int)ri);
-        ring_out[rings[ri].src_part].push_back((int)ri);
+        ring_in[rings[ri].group * NP + rings[ri].dst_part].push_back((int)ri);
+        ring_out[rings[ri].group * NP + rings[ri].src_part].push_back((int)ri);
     }
     // order every GPU after the caller's stream
     SG_RT(cudaEventRecord(user_ev, stream));
@@ -493,10 +496,14 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
     const int64_t nfrag = (n + F - 1) / F;
     for (int64_t fi = 0; fi < nfrag; fi++) {
         const int64_t ka = fi * F, kb = std::min(n, ka + F);
-        const int slot = (int)(fi % ring_depth);
+        // fragments dealt round-robin to the replica groups; rings are per group
+        const int grp = (int)(fi % R);
+        const int64_t fg = fi / R;
+        const int slot = (int)(fg % ring_depth);
         for (int p : part_order) {
             CompiledKernel& ck = kernels[p];
-            const int g = part_gpu[p];
+            const int g = grp * Gs + part_gpu[p];
+            const size_t gp = grp * NP + p;
             GpuCtx& gc = gpus[g];
             DevGuard dg(gc.dev);
             IoBinding io;
@@ -508,7 +515,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                     continue;
                 }
                 int ri = -1;
-                for (int r : ring_in[p]) if (rings[r].edge == e) ri = r;
+                for (int r : ring_in[gp]) if (rings[r].edge == e) ri = r;
                 CutRing& r = rings[ri];
                 if (r.src_gpu != r.dst_gpu) SG_RT(cudaStreamWaitEvent(gc.compute, r.ev_copied[slot], 0));
                 io.in.push_back(r.dst_slots[slot]);
@@ -522,10 +529,10 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                     continue;
                 }
                 int ri = -1;
-                for (int r : ring_out[p]) if (rings[r].edge == e) ri = r;
+                for (int r : ring_out[gp]) if (rings[r].edge == e) ri = r;
                 CutRing& r = rings[ri];
                 // slot reuse: the copy (or the same-GPU consumer) of fragment fi - depth must be done
-                if (fi >= ring_depth) {
+                if (fg >= ring_depth) {
                     if (r.src_gpu != r.dst_gpu) SG_RT(cudaStreamWaitEvent(gc.compute, r.ev_copied[slot], 0));
                     else SG_RT(cudaStreamWaitEvent(gc.compute, r.ev_consumed[slot], 0));
                 }
@@ -534,14 +541,14 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
             }
             last_launches += launch(ck, gc.dev, io, ka, kb, gc.compute, flat.dtype == SG_F32);
             // consumed slots of incoming rings are free again
-            for (int ri : ring_in[p]) SG_RT(cudaEventRecord(rings[ri].ev_consumed[slot], gc.compute));
+            for (int ri : ring_in[gp]) SG_RT(cudaEventRecord(rings[ri].ev_consumed[slot], gc.compute));
             // ship outgoing boundary streams to other GPUs (copy engine, P2P)
-            for (int ri : ring_out[p]) {
+            for (int ri : ring_out[gp]) {
                 CutRing& r = rings[ri];
                 if (r.src_gpu == r.dst_gpu) continue;
                 SG_RT(cudaEventRecord(r.ev_produced[slot], gc.compute));
                 SG_RT(cudaStreamWaitEvent(gc.copy, r.ev_produced[slot], 0));
-                if (fi >= ring_depth) SG_RT(cudaStreamWaitEvent(gc.copy, r.ev_consumed[slot], 0));
+                if (fg >= ring_depth) SG_RT(cudaStreamWaitEvent(gc.copy, r.ev_consumed[slot], 0));
                 int64_t items = r.per_iter * (kb - ka) + r.extra;
                 if (devices[r.src_gpu] == devices[r.dst_gpu])
                     SG_RT(cudaMemcpyAsync(r.dst_slots[slot], r.src_slots[slot], (size_t)items * 4,

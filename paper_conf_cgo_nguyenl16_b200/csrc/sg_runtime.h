@@ -26,6 +26,7 @@ struct CompiledKernel {
 
 struct CutRing {          // one boundary stream between partitions (a PDG edge member)
     int edge = -1;
+    int group = 0;                     // replica group owning this ring
     int src_part = -1, dst_part = -1;  // -1: graph input / output
     int src_gpu = 0, dst_gpu = 0;
     int64_t lo = 0, extra = 0, per_iter = 0;
@@ -55,6 +56,7 @@ struct GpuCtx {
 struct Plan {
     Flat flat;
     int G = 1;
+    int R = 1, Gs = 1;                     // replica groups, GPUs per group (G = R * Gs)
     sg_plan_opts opts{};
     std::vector<Partition> parts;
     std::vector<int> part_order;           // topological order of partitions

@@ -55,7 +55,7 @@ class PlanOpts(ctypes.Structure):
                 ("virtual_gpus", ctypes.c_int32), ("devices", ctypes.POINTER(ctypes.c_int32)),
                 ("ilp_time_limit_ms", ctypes.c_int32), ("codegen_mode", ctypes.c_int32),
                 ("link_gbps", ctypes.c_double), ("link_latency_us", ctypes.c_double), ("verbose", ctypes.c_int32),
-                ("plan_only", ctypes.c_int32)]
+                ("plan_only", ctypes.c_int32), ("replicas", ctypes.c_int32)]
 
 
 class RankOp(ctypes.Structure):
@@ -75,7 +75,7 @@ class PlanInfo(ctypes.Structure):
                 ("input_device", ctypes.c_int32), ("output_device", ctypes.c_int32),
                 ("iters_per_fragment", ctypes.c_int64), ("ilp_optimal", ctypes.c_int32),
                 ("flops_per_iter_written", ctypes.c_double), ("flops_per_iter_pruned", ctypes.c_double),
-                ("intops_per_iter", ctypes.c_int64)]
+                ("intops_per_iter", ctypes.c_int64), ("replicas", ctypes.c_int32)]
 
 
 def lib():
@@ -255,6 +255,7 @@ class Plan:
             "iters_per_fragment": i.iters_per_fragment, "ilp_optimal": bool(i.ilp_optimal),
             "flops_per_iter_written": i.flops_per_iter_written, "flops_per_iter_pruned": i.flops_per_iter_pruned,
             "intops_per_iter": i.intops_per_iter,
+            "replicas": i.replicas,
         }
 
     def input_items(self, n: int) -> int:

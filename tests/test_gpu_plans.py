@@ -32,6 +32,10 @@ PLANS = [
     dict(n_gpus=2, virtual_gpus=1, iters_per_fragment=128),
     dict(n_gpus=4, virtual_gpus=1, iters_per_fragment=64),
     dict(n_gpus=3, virtual_gpus=1, partitioner="per_filter", iters_per_fragment=200),
+    # hybrid replica x pipeline plans: fragments dealt round-robin to groups
+    dict(n_gpus=4, virtual_gpus=1, replicas=2, iters_per_fragment=64),
+    dict(n_gpus=4, virtual_gpus=1, replicas=4, iters_per_fragment=50),
+    dict(n_gpus=6, virtual_gpus=1, replicas=3, partitioner="per_filter", iters_per_fragment=70),
 ]
 
 
@@ -195,3 +199,18 @@ def test_run_rank_world1_nccl(oracle_lib):
         torch.cuda.synchronize()
         assert_parity(prog, yd.cpu().numpy(), ref)
         p.close()
+
+
+
+@pytest.mark.parametrize("name", ["filterbank64", "fmradio10", "beamformer12x4", "des16"])
+def test_hybrid_auto_plan_vs_oracle(oracle_lib, name):
+    """replicas = -1: the cost model picks R; whatever it picks, the output is the oracle's."""
+    _torch()
+    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
+    n = 9 if name == "beamformer12x4" else 3000
+    x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), 4321)
+    ref = oracle_lib.run(prog, x, n)
+    y, info, launches = run_gpu(prog, x, n, n_gpus=8, virtual_gpus=1, replicas=-1,
+                                iters_per_fragment=1 if name == "beamformer12x4" else 200)
+    assert_parity(prog, y, ref)
+    assert info["replicas"] >= 1 and 8 % info["replicas"] == 0

@@ -409,3 +409,33 @@ def test_des_compiles_register_and_staged(sg):
     with sg.plan(apps.des(2), 1, partitioner="per_filter") as p:
         assert p.info()["n_partitions"] > 1
         assert any("sg_work_xor<32>" in p.source(q) for q in range(p.info()["n_partitions"]))
+
+
+# ------------------------------------------------ hybrid replica x pipeline plans
+def test_hybrid_replicas_options(sg):
+    """R replica groups of G/R GPUs.  R must divide G; the paper's mapping (R = 1)
+    is the default; the auto model (-1) replicates compute-bound graphs whose input/output streams
+    are thin (FilterBank: 64 B/iteration against ~1 ns of compute) and keeps HBM-bound graphs whose
+    input would have to cross NVLink (BitonicSort: 256 B/iteration) on the input GPU."""
+    with sg.plan(apps.filterbank(64), 8, plan_only=1, virtual_gpus=1) as p:
+        assert p.info()["replicas"] == 1
+    with sg.plan(apps.filterbank(64), 8, plan_only=1, virtual_gpus=1, replicas=-1) as p:
+        i = p.info()
+        assert i["replicas"] == 8 and i["n_partitions"] == 1
+    with sg.plan(apps.bitonic(32), 8, plan_only=1, virtual_gpus=1, replicas=-1) as p:
+        assert p.info()["replicas"] == 1
+    with sg.plan(apps.filterbank(64), 8, plan_only=1, virtual_gpus=1, replicas=2) as p:
+        i = p.info()
+        assert i["replicas"] == 2 and max(i["partition_gpu"]) < 4
+    with pytest.raises(sg.SgError) as e:
+        sg.plan(apps.filterbank(8), 4, plan_only=1, virtual_gpus=1, replicas=3)
+    assert e.value.code == sg.SG_E_ARG
+
+
+def test_hybrid_estimate_scales(sg):
+    """Group-local ILP + 1/R of the fragments: with thin streams the estimate falls ~1/R."""
+    t = {}
+    for R in (1, 2, 4, 8):
+        with sg.plan(apps.filterbank(64), 8, plan_only=1, virtual_gpus=1, replicas=R, partitioner="single") as p:
+            t[R] = p.info()["est_tmax"]
+    assert t[2] < t[1] * 0.6 and t[4] < t[2] * 0.6 and t[8] < t[4] * 0.6
