@@ -352,6 +352,64 @@ static int build(graph* g, int in_edge) {
         g->nodes[jid].out[0] = oe;
         return oe;
     }
+    if (tok[0] == 'L' && tok[1] == 0) {
+        /* feedback loop ("pipeline ..., split-join ..., and feedback loop"; StreamIt
+         * form): joiner RR(jw0, jw1) merges the outer input (port 0) with the loop stream (port 1);
+         * body; splitter (duplicate, or RR(sw0, sw1)) sends port 0 out, port 1 into the loop stream,
+         * whose output returns to the joiner's port 1.  The n_enq enqueued items are the initial
+         * contents of that returning edge (the loop's delay). */
+        int jw0 = (int)next_int(g), jw1 = (int)next_int(g);
+        char sk[8];
+        next_tok(g, sk, 8);
+        int st = (sk[0] == 'D') ? T_SPLIT_DUP : T_SPLIT_RR;
+        int sw0 = 1, sw1 = 1;
+        if (st == T_SPLIT_RR) { sw0 = (int)next_int(g); sw1 = (int)next_int(g); }
+        long long nenq = next_int(g);
+        if (g->err || jw0 < 0 || jw1 < 1 || sw0 < 0 || sw1 < 1 || nenq < 0) { g->err = ORC_E_PARSE; return -1; }
+        word* enq = (word*)calloc((size_t)nenq + 1, sizeof(word));
+        for (long long k = 0; k < nenq; k++) {
+            if (g->is_i32) enq[k].i = (int32_t)next_int(g);
+            else enq[k].f = next_float(g);
+        }
+        int jid = new_node(g);
+        node* jn = &g->nodes[jid];
+        jn->type = T_JOIN_RR;
+        jn->nw = 2;
+        jn->w = (int*)calloc(2, sizeof(int));
+        jn->w[0] = jw0; jn->w[1] = jw1;
+        jn->n_in = 2; jn->n_out = 1;
+        jn->in = (int*)malloc(2 * sizeof(int));
+        jn->out = (int*)malloc(sizeof(int));
+        jn->in[0] = in_edge;
+        jn->in[1] = -1;
+        g->edges[in_edge].dst = jid;
+        int je = new_edge(g, jid);
+        g->nodes[jid].out[0] = je;
+        int be = build(g, je);                         /* body */
+        if (g->err) { free(enq); return -1; }
+        int sid = new_node(g);
+        node* sn = &g->nodes[sid];
+        sn->type = st;
+        sn->nw = 2;
+        sn->w = (int*)calloc(2, sizeof(int));
+        sn->w[0] = sw0; sn->w[1] = sw1;
+        sn->n_in = 1; sn->n_out = 2;
+        sn->in = (int*)malloc(sizeof(int));
+        sn->out = (int*)malloc(2 * sizeof(int));
+        sn->in[0] = be;
+        g->edges[be].dst = sid;
+        int oe = new_edge(g, sid);
+        int le = new_edge(g, sid);
+        g->nodes[sid].out[0] = oe;
+        g->nodes[sid].out[1] = le;
+        int re = build(g, le);                         /* loop stream */
+        if (g->err) { free(enq); return -1; }
+        g->nodes[jid].in[1] = re;
+        g->edges[re].dst = jid;
+        for (long long k = 0; k < nenq; k++) fifo_push(&g->edges[re].q, enq[k]);
+        free(enq);
+        return oe;
+    }
     g->err = ORC_E_PARSE;
     return -1;
 }
@@ -621,7 +679,12 @@ int orc_run(const char* spec, const void* input, long long n_in, void* output,
         for (long long k = 0; k < c; k++) fifo_push(qin, in[fed + k]);
         fed += c;
         if (order_seed == 0) {
-            for (int id = 0; id < g.n_nodes; id++) fire_all(&g, id, xs, ys);
+            /* sweeps in node order until nothing fires (one sweep suffices without feedback loops) */
+            long long any;
+            do {
+                any = 0;
+                for (int id = 0; id < g.n_nodes; id++) any += fire_all(&g, id, xs, ys);
+            } while (any);
         } else {
             /* reverse sweeps until nothing fires: each sweep fires downstream nodes first */
             long long any;

@@ -107,7 +107,27 @@ class SplitJoin:
             self.join_w = [1] * nb
 
 
-Stream = Union[Filter, Pipeline, SplitJoin]
+@dataclass
+class FeedbackLoop:
+    """StreamIt feedback loop: joiner RR(join_w[0], join_w[1]) merges the outer
+    input with the loop stream's output; `body`; splitter ("dup", or "rr" with split_w) sends port 0
+    out and port 1 into `loop`, whose output returns to the joiner.  `enqueue` = initial items on
+    that returning edge (the loop delay)."""
+    body: "Stream"
+    loop: "Stream"
+    join_w: List[int] = field(default_factory=lambda: [1, 1])
+    split: str = "dup"
+    split_w: Optional[List[int]] = None
+    enqueue: List[float] = field(default_factory=list)
+
+    def __post_init__(self):
+        if self.split not in ("dup", "rr"):
+            raise ValueError("split must be dup or rr")
+        if self.split == "rr" and self.split_w is None:
+            self.split_w = [1, 1]
+
+
+Stream = Union[Filter, Pipeline, SplitJoin, FeedbackLoop]
 
 
 @dataclass
@@ -130,6 +150,15 @@ class Program:
                 out.append(f"P {len(s.children)}")
                 for c in s.children:
                     emit(c)
+            elif isinstance(s, FeedbackLoop):
+                toks = ["L", str(s.join_w[0]), str(s.join_w[1]), "D" if s.split == "dup" else "R"]
+                if s.split == "rr":
+                    toks += [str(w) for w in s.split_w]
+                toks.append(str(len(s.enqueue)))
+                toks += [str(int(v)) if self.dtype == "i32" else float(f32(v)).hex() for v in s.enqueue]
+                out.append(" ".join(toks))
+                emit(s.body)
+                emit(s.loop)
             elif isinstance(s, SplitJoin):
                 nb = len(s.branches)
                 toks = ["J", "D" if s.split == "dup" else "R", str(nb)]
@@ -155,6 +184,11 @@ class Program:
             elif isinstance(s, Pipeline):
                 for c in s.children:
                     walk(c)
+            elif isinstance(s, FeedbackLoop):
+                cnt["splitters"] += 1
+                cnt["joiners"] += 1
+                walk(s.body)
+                walk(s.loop)
             else:
                 cnt["splitters"] += 1
                 cnt["joiners"] += 1
