@@ -212,6 +212,20 @@ sg_status sg_add_splitjoin(sg_graph* g, sg_split_kind kind, const int32_t* split
 sg_status sg_branch_begin(sg_graph* g, int32_t sj_id, int32_t branch);
 sg_status sg_branch_end(sg_graph* g);
 
+/* Append a feedback loop (streams compose by "pipeline ..., split-join ..., and
+ * feedback loop"; StreamIt form) to the currently open pipeline.  A joiner
+ * RR(join_w[0], join_w[1]) merges the outer input (port 0) with the loop stream's output (port 1);
+ * branch 0 is the body, branch 1 the loop stream (fill both with sg_branch_begin / sg_branch_end);
+ * a splitter (DUPLICATE, or ROUNDROBIN(split_w[0], split_w[1])) sends port 0 onwards and port 1 into
+ * the loop stream.  `enqueue` holds n_enqueue items of the graph dtype (4-byte words), the initial
+ * contents of the edge returning to the joiner (the loop delay); it is copied.  Constraints
+ * (SG_E_ARG / SG_E_UNSUPPORTED at sg_plan): join_w[1] >= 1, split_w[1] >= 1, no filter with
+ * peek > pop inside the loop, no nested feedback loops; the loop must not deadlock (SG_E_RATE).
+ * Execution: the loop runs sequentially (it carries state across iterations) as its own partition;
+ * everything around it stays data-parallel.  replicas > 1 is rejected for graphs with loops. */
+sg_status sg_add_feedbackloop(sg_graph* g, const int32_t join_w[2], sg_split_kind split, const int32_t* split_w,
+                              int32_t n_enqueue, const void* enqueue, int32_t* loop_id);
+
 /* ---- planning ---- */
 void sg_plan_opts_default(sg_plan_opts* o);
 

@@ -110,9 +110,41 @@ sg_status sg_add_splitjoin(sg_graph* g, sg_split_kind kind, const int32_t* split
     });
 }
 
+sg_status sg_add_feedbackloop(sg_graph* g, const int32_t join_w[2], sg_split_kind kind, const int32_t* split_w,
+                              int32_t n_enq, const void* enq, int32_t* loop_id) {
+    if (!g || !join_w) return fail(SG_E_ARG, "NULL argument");
+    if (kind != SG_SPLIT_DUPLICATE && kind != SG_SPLIT_ROUNDROBIN) return fail(SG_E_ARG, "bad split kind");
+    if (n_enq < 0 || (n_enq > 0 && !enq)) return fail(SG_E_ARG, "bad enqueue list");
+    return guard([&] {
+        sg::Elem e;
+        e.type = sg::E_LOOP;
+        e.split_kind = kind == SG_SPLIT_DUPLICATE ? 0 : 1;
+        e.join_w.assign(join_w, join_w + 2);
+        e.split_w.assign(2, 1);
+        if (kind == SG_SPLIT_ROUNDROBIN && split_w) e.split_w.assign(split_w, split_w + 2);
+        if (e.join_w[0] < 0 || e.join_w[1] < 1 || e.split_w[0] < 0 || e.split_w[1] < 1)
+            throw sg::Error(SG_E_ARG, "feedback loop weights: join_w = {>=0, >=1}, split_w = {>=0, >=1}");
+        if (e.join_w[0] == 0) throw sg::Error(SG_E_UNSUPPORTED, "feedback loop without outer input (join_w[0] = 0)");
+        if (kind == SG_SPLIT_ROUNDROBIN && e.split_w[0] == 0) throw sg::Error(SG_E_UNSUPPORTED, "feedback loop without output");
+        e.enq.assign((const uint32_t*)enq, (const uint32_t*)enq + n_enq);
+        int id = (int)g->elems.size();
+        g->elems.push_back(e);
+        for (int b = 0; b < 2; b++) {
+            sg::Elem p;
+            p.type = sg::E_PIPE;
+            g->elems.push_back(p);
+            g->elems[id].branches.push_back((int)g->elems.size() - 1);
+        }
+        g->elems[id].branch_done.assign(2, false);
+        current_pipe(g).kids.push_back(id);
+        if (loop_id) *loop_id = id;
+    });
+}
+
 sg_status sg_branch_begin(sg_graph* g, int32_t sj, int32_t b) {
     if (!g) return fail(SG_E_ARG, "NULL graph");
-    if (sj < 0 || sj >= (int)g->elems.size() || g->elems[sj].type != sg::E_SJ) return fail(SG_E_ARG, "not a split-join id");
+    if (sj < 0 || sj >= (int)g->elems.size() || (g->elems[sj].type != sg::E_SJ && g->elems[sj].type != sg::E_LOOP))
+        return fail(SG_E_ARG, "not a split-join or feedback-loop id");
     sg::Elem& e = g->elems[sj];
     if (b < 0 || b >= (int)e.branches.size()) return fail(SG_E_ARG, "branch out of range");
     if (e.branch_done[b]) return fail(SG_E_STRUCTURE, "branch already filled");

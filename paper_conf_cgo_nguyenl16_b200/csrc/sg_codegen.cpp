@@ -58,11 +58,24 @@ bool is_view_kind(int k) {
     return k == SG_K_IDENTITY || k == SG_K_DELAY || k == SG_K_DECIMATE || k == SG_K_EXPAND || k == SG_K_FFT_REORDER ||
            k == SG_K_PERMUTE;
 }
-static bool is_view_node(const Node& n) { return n.type != N_FILTER || is_view_kind(n.kind); }
+static bool is_view_node(const Node& n) {
+    return n.type == N_FILTER ? is_view_kind(n.kind) : n.type != N_LOOP;
+}
 
 void node_work(const Flat& f, int v, int64_t& flops, int64_t& intops, int64_t& dfma) {
     const Node& n = f.nodes[v];
     flops = intops = dfma = 0;
+    if (n.type == N_LOOP) {  // the loop graph's work per loop firing, times the loop's firings
+        const Flat& sf = *n.loop->sub;
+        for (int u = 0; u < (int)sf.nodes.size(); u++) {
+            int64_t a, b, c;
+            node_work(sf, u, a, b, c);
+            flops += a * n.rep;
+            intops += b * n.rep;
+            dfma += c * n.rep;
+        }
+        return;
+    }
     if (n.type != N_FILTER) return;
     int64_t per = 0;
     switch (n.kind) {
@@ -271,6 +284,7 @@ bool register_mode_eligible(const Flat& f, const std::vector<int>& nodes, std::s
     int64_t live = 0;
     for (int v : nodes) {
         const Node& n = f.nodes[v];
+        if (n.type == N_LOOP) return fail("feedback loop");
         if (n.halo != 0) return fail("node " + std::to_string(v) + " has a halo");
         if (n.type == N_FILTER && n.kind == SG_K_BEAM_FIR) return fail("frame FIR");
         if (n.type == N_FILTER && n.prework) return fail("prework");
@@ -1287,6 +1301,228 @@ private:
         }
         memo_[key] = y;
         return y[j];
+    }
+};
+
+// ------------------------------------------------------------ feedback loops
+// A feedback loop carries state from one iteration to the next, so its partition
+// runs sequentially: one thread executes the loop graph's static schedule firing by firing (found
+// at plan time, sg_graph.cpp go_loop), its internal FIFOs in shared memory (absolute stream
+// positions, power-of-two rings), the outer input read and the outer output written in natural
+// order.  Between launches (fragments) the FIFOs, the next firing index and a history of the last
+// `halo` firings' outputs (re-emitted when a downstream peek window reaches back) live in a plan-
+// owned state buffer, reset to the enqueued items at the start of every sg_run.
+class LoopGen : public GenBase {
+public:
+    LoopGen(const Flat& outer, int v, int part) : GenBase(*outer.nodes[v].loop->sub, all_nodes(*outer.nodes[v].loop->sub), part),
+                                                  of_(outer), v_(v), li_(*outer.nodes[v].loop) {}
+
+    static std::vector<int> all_nodes(const Flat& f) {
+        std::vector<int> a(f.nodes.size());
+        std::iota(a.begin(), a.end(), 0);
+        return a;
+    }
+    // state image layout (4-byte words): [0,2) next firing (int64), then each internal edge's ring, then history
+    static std::vector<uint32_t> initial_state(const LoopInfo& li, int64_t& hist_off, int64_t& hist_len, int64_t halo,
+                                               std::vector<int64_t>& ring_off) {
+        const Flat& sf = *li.sub;
+        int64_t o = 2;
+        ring_off.assign(sf.edges.size(), -1);
+        for (int e = 0; e < (int)sf.edges.size(); e++) {
+            if (e == sf.in_edge || e == sf.out_edge) continue;
+            ring_off[e] = o;
+            o += li.cap[e];
+        }
+        hist_off = o;
+        hist_len = 1;
+        while (hist_len < std::max<int64_t>(1, halo * li.Q)) hist_len <<= 1;
+        o += hist_len;
+        std::vector<uint32_t> img((size_t)o, 0u);
+        for (size_t k = 0; k < li.enq.size(); k++) img[ring_off[li.back] + (k & (li.cap[li.back] - 1))] = li.enq[k];
+        return img;  // DELAY prework items are zeros (already 0)
+    }
+
+    KernelInfo run() {
+        const Node& ln = of_.nodes[v_];
+        const Flat& sf = *li_.sub;
+        KernelInfo ki;
+        ki.mode = 4;
+        ki.name = "sg_part" + std::to_string(part_);
+        ki.name_sync = ki.name;
+        ki.threads = ki.threads_sync = 32;
+        ki.tile = ki.tile_sync = 1 << 30;  // one CTA
+        ki.in_edges = {ln.in[0]};
+        ki.out_edges = {ln.out[0]};
+        int64_t lo, ex;
+        edge_window(of_, ln.in[0], lo, ex);
+        ki.in_lo = {lo};
+        ki.in_extra = {ex};
+        edge_window(of_, ln.out[0], lo, ex);
+        ki.out_lo = {lo};
+        ki.out_extra = {ex};
+        const int64_t OLO = lo, OEX = ex, OPI = of_.edges[ln.out[0]].per_iter;
+        for (int u = 0; u < (int)sf.nodes.size(); u++) {
+            int64_t a, b, c;
+            node_work(sf, u, a, b, c);
+            ki.flops_per_iter += a * ln.rep;
+            ki.intops_per_iter += b * ln.rep;
+            ki.dfma_per_iter += c * ln.rep;
+        }
+        int64_t hist_off, hist_len;
+        std::vector<int64_t> roff;
+        auto img = initial_state(li_, hist_off, hist_len, ln.halo, roff);
+        ki.state_words = (int64_t)img.size();
+        ki.state_init = img;
+        // shared-memory rings
+        int64_t smem_words = 0;
+        std::vector<int64_t> soff(sf.edges.size(), -1);
+        for (int e = 0; e < (int)sf.edges.size(); e++)
+            if (roff[e] >= 0) { soff[e] = smem_words; smem_words += li_.cap[e]; }
+        ki.smem = (size_t)std::max<int64_t>(4, smem_words * 4);
+        ki.smem_sync = ki.smem;
+        // one firing of the loop = the static schedule with compile-time offsets
+        std::ostringstream body;
+        std::vector<int64_t> rd(sf.edges.size(), 0), wr(sf.edges.size(), 0);
+        for (int e = 0; e < (int)sf.edges.size(); e++) wr[e] = li_.init_level[e];
+        const std::string T = T_;
+        auto pos_ref = [&](int e, int64_t c) -> std::string {  // item at (firing-relative) position c of edge e
+            const int64_t per = sf.edges[e].per_iter;
+            if (e == sf.in_edge) return "gin[g * " + std::to_string(li_.P) + "LL + " + std::to_string(c) + "LL - in_base]";
+            return "q[" + std::to_string(soff[e]) + " + (int)((g * " + std::to_string(per) + "LL + " + std::to_string(c) +
+                   "LL) & " + std::to_string(li_.cap[e] - 1) + "LL)]";
+        };
+        for (int u : li_.sched) {
+            const Node& n = sf.nodes[u];
+            std::vector<std::string> xs;
+            for (int e : n.in) {
+                for (int64_t i = 0; i < sf.edges[e].pop; i++) xs.push_back(pos_ref(e, rd[e] + i));
+                rd[e] += sf.edges[e].pop;
+            }
+            std::vector<std::string> ys;  // per output item, in port order
+            body << "      {\n";
+            if (n.type == N_FILTER) {
+                body << "        const " << T << " x_[" << std::max<size_t>(1, xs.size()) << "] = {";
+                for (size_t i = 0; i < xs.size(); i++) body << (i ? ", " : "") << xs[i];
+                body << "};\n        " << T << " y_[" << n.push << "];\n        ";
+                body << firing_code(u) << "\n";
+                for (int64_t j = 0; j < n.push; j++) ys.push_back("y_[" + std::to_string(j) + "]");
+            } else {
+                // splitters / joiners: pure data movement
+                body << "        const " << T << " x_[" << xs.size() << "] = {";
+                for (size_t i = 0; i < xs.size(); i++) body << (i ? ", " : "") << xs[i];
+                body << "};\n";
+                if (n.type == N_SPLIT_DUP) {
+                    for (size_t k = 0; k < n.out.size(); k++) ys.push_back("x_[0]");
+                } else {
+                    for (size_t i = 0; i < xs.size(); i++) ys.push_back("x_[" + std::to_string(i) + "]");
+                }
+            }
+            // pushes: splitter RR sends consecutive items per port; DUP sends x_[0] to every port
+            size_t yi = 0;
+            for (size_t k = 0; k < n.out.size(); k++) {
+                const int e = n.out[k];
+                for (int64_t j = 0; j < sf.edges[e].push; j++, yi++) {
+                    const std::string val = n.type == N_SPLIT_DUP ? ys[k] : ys[yi];
+                    if (e == sf.out_edge) {
+                        const int64_t c = wr[e] + j;  // output item c of this firing
+                        body << "        { const long long p = g * " << li_.Q << "LL + " << c << "LL; const " << T << " val = " << val
+                             << ";\n          hist[(int)(p & " << hist_len - 1 << "LL)] = val;\n"
+                             << "          if (p >= wlo && p < whi) gout[p - out_base] = val; }\n";
+                    } else {
+                        body << "        " << pos_ref(e, wr[e] + j) << " = " << val << ";\n";
+                    }
+                }
+                wr[e] += sf.edges[e].push;
+            }
+            body << "      }\n";
+        }
+        std::ostringstream s;
+        s << header("feedback loop") << consts_.str() << args_struct_loop();
+        s << "extern \"C\" __global__ void __launch_bounds__(32, 1) " << ki.name << "(const SgArgs a) {\n"
+          << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
+          << "  " << T << "* q = reinterpret_cast<" << T << "*>(sg_smem);\n"
+          << "  " << T << "* st = reinterpret_cast<" << T << "*>(SG_STATE);\n";
+        for (int e = 0; e < (int)sf.edges.size(); e++)
+            if (roff[e] >= 0)
+                s << "  for (int i = threadIdx.x; i < " << li_.cap[e] << "; i += 32) q[" << soff[e] << " + i] = st[" << roff[e]
+                  << " + i];\n";
+        s << "  __syncwarp();\n"
+          << "  if (threadIdx.x == 0) {\n"
+          << "    " << T << "* hist = st + " << hist_off << ";\n"
+          << "    const " << T << "* gin = SG_IN(0);\n"
+          << "    const long long in_base = SG_IN_BASE(0);\n"
+          << "    " << T << "* gout = SG_OUT(0);\n"
+          << "    const long long out_base = SG_OUT_BASE(0);\n"
+          << "    const long long wlo = SG_K_BEGIN * " << OPI << "LL + (" << OLO << "LL);\n"
+          << "    const long long whi = SG_K_END * " << OPI << "LL + (" << OLO + OEX << "LL);\n"
+          << "    long long next = *reinterpret_cast<long long*>(st);\n"
+          << "    const long long g0 = SG_K_BEGIN * " << ln.rep << "LL + (" << ln.ninit - ln.halo << "LL);\n"
+          << "    const long long g1 = SG_K_END * " << ln.rep << "LL + (" << ln.ninit << "LL);\n"
+          << "    for (long long g = g0; g < g1; g++) {\n"
+          << "      if (g < next) {  // before the stream start (zeros) or already computed (history)\n"
+          << "        for (int j = 0; j < " << li_.Q << "; j++) {\n"
+          << "          const long long p = g * " << li_.Q << "LL + j;\n"
+          << "          if (p >= wlo && p < whi) gout[p - out_base] = g < 0 ? (" << T << ")0 : hist[(int)(p & " << hist_len - 1
+          << "LL)];\n"
+          << "        }\n"
+          << "        continue;\n"
+          << "      }\n"
+          << body.str()
+          << "      next = g + 1;\n"
+          << "    }\n"
+          << "    *reinterpret_cast<long long*>(st) = next;\n"
+          << "  }\n"
+          << "  __syncwarp();\n";
+        for (int e = 0; e < (int)sf.edges.size(); e++)
+            if (roff[e] >= 0)
+                s << "  for (int i = threadIdx.x; i < " << li_.cap[e] << "; i += 32) st[" << roff[e] << " + i] = q[" << soff[e]
+                  << " + i];\n";
+        s << "}\n";
+        ki.source = s.str();
+        return ki;
+    }
+
+private:
+    const Flat& of_;
+    int v_;
+    const LoopInfo& li_;
+
+    std::string args_struct_loop() {
+        // one boundary input and output (the outer edges), plus the state pointer
+        std::ostringstream s;
+        s << "struct SgArgs { long long v[8]; };\n"
+          << "#define SG_IN(i) (reinterpret_cast<const " << T_ << "*>(a.v[0]))\n"
+          << "#define SG_IN_BASE(i) (a.v[1])\n"
+          << "#define SG_IN_LIMIT(i) (a.v[2])\n"
+          << "#define SG_OUT(i) (reinterpret_cast<" << T_ << "*>(a.v[3]))\n"
+          << "#define SG_OUT_BASE(i) (a.v[4])\n"
+          << "#define SG_K_BEGIN (a.v[5])\n"
+          << "#define SG_K_END (a.v[6])\n"
+          << "#define SG_STATE (reinterpret_cast<void*>(a.v[7]))\n";
+        return s.str();
+    }
+    // one firing of filter u of the loop graph: x_ -> y_ (compute kinds via work_call; data-movement kinds inline)
+    std::string firing_code(int u) {
+        const Node& n = f_.nodes[u];
+        std::ostringstream c;
+        switch (n.kind) {
+        case SG_K_IDENTITY: case SG_K_DELAY: case SG_K_DECIMATE: c << "y_[0] = x_[0];"; break;
+        case SG_K_EXPAND:
+            c << "y_[0] = x_[0];";
+            for (int64_t j = 1; j < n.push; j++) c << " y_[" << j << "] = (" << T_ << ")0;";
+            break;
+        case SG_K_FFT_REORDER: {
+            int64_t nn = n.iv[0], o = 0;
+            for (int64_t i = 0; i < nn; i += 2) { c << "y_[" << o++ << "] = x_[" << 2 * i << "]; y_[" << o++ << "] = x_[" << 2 * i + 1 << "]; "; }
+            for (int64_t i = 1; i < nn; i += 2) { c << "y_[" << o++ << "] = x_[" << 2 * i << "]; y_[" << o++ << "] = x_[" << 2 * i + 1 << "]; "; }
+            break;
+        }
+        case SG_K_PERMUTE:
+            for (size_t k = 1; k < n.iv.size(); k++) c << "y_[" << k - 1 << "] = x_[" << n.iv[k] << "]; ";
+            break;
+        default: c << work_call(u);
+        }
+        return c.str();
     }
 };
 
@@ -3131,6 +3367,12 @@ private:
 };
 
 KernelInfo generate_kernel(const Flat& f, const std::vector<int>& nodes, int part_id, const CodegenOpts& opt) {
+    for (int v : nodes)
+        if (f.nodes[v].type == N_LOOP) {
+            if (nodes.size() != 1) throw Error(SG_E_PLAN, "a feedback loop must be a partition of its own");
+            LoopGen g(f, v, part_id);
+            return g.run();
+        }
     std::string why;
     bool reg_ok = register_mode_eligible(f, nodes, &why);
     int mode = opt.mode;

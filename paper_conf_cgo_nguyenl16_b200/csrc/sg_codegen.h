@@ -18,7 +18,7 @@ struct CodegenOpts {
 struct KernelInfo {
     std::string name;
     std::string source;       // full CUDA source (includes sg_device.cuh)
-    int mode = 0;             // 1 register (thread per iteration), 2 staged
+    int mode = 0;             // 1 register (thread per iteration), 2 staged, 4 feedback loop (sequential)
     int threads = 0;          // CTA size
     int tile = 0;             // iterations per CTA tile
     int min_blocks = 1;       // __launch_bounds__ second argument
@@ -42,6 +42,9 @@ struct KernelInfo {
     int64_t flops_exec_per_iter = -1;  // fused: algorithmic flops after dead/zero pruning (no recompute)
     std::string name_start;          // staged fused: stream-start variant (tiles with k0 < ksafe)
     int64_t ksafe = 0;
+    // feedback loop (mode 4): persistent state (4-byte words) and its image at the stream start
+    int64_t state_words = 0;
+    std::vector<uint32_t> state_init;
 };
 
 // Boundary input / output edges of a node set (sorted, deterministic).

@@ -205,6 +205,8 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
     const int64_t n_in = flat.input_items(n);
     last_launches = 0;
     std::vector<RankOp> ops = rank_schedule(*this, me, n, F);
+    for (size_t p = 0; p < parts.size(); p++)  // this rank's feedback loops restart from their enqueued items
+        if (part_gpu[p] == me && kernels[p].ki.state_words > 0) reset_state(kernels[p], dev, dist_compute);
     size_t i = 0;
     while (i < ops.size()) {
         const RankOp& o = ops[i];

@@ -24,7 +24,7 @@ struct Error : std::runtime_error {
 };
 
 // ------------------------------------------------------------------ builder
-enum ElemType { E_FILTER = 0, E_PIPE = 1, E_SJ = 2 };
+enum ElemType { E_FILTER = 0, E_PIPE = 1, E_SJ = 2, E_LOOP = 3 };
 
 struct Elem {
     ElemType type = E_FILTER;
@@ -37,8 +37,10 @@ struct Elem {
     // split-join
     int split_kind = 0;  // 0 dup, 1 rr
     std::vector<int32_t> split_w, join_w;
-    std::vector<int> branches;  // elem ids of branch pipelines
+    std::vector<int> branches;  // elem ids of branch pipelines (loop: body, loop stream)
     std::vector<bool> branch_done;
+    // feedback loop: enqueued items (raw 4-byte words)
+    std::vector<uint32_t> enq;
 };
 
 }  // namespace sg
@@ -54,7 +56,21 @@ struct sg_graph {
 namespace sg {
 
 // --------------------------------------------------------- flattened graph
-enum NodeType { N_FILTER = 0, N_SPLIT_DUP = 1, N_SPLIT_RR = 2, N_JOIN = 3 };
+enum NodeType { N_FILTER = 0, N_SPLIT_DUP = 1, N_SPLIT_RR = 2, N_JOIN = 3, N_LOOP = 4 };
+
+struct Flat;
+// A feedback loop, seen from outside as one stateful filter (N_LOOP) whose firing is one steady-state
+// iteration of the loop's own SDF graph: pop P = r_J * join_w[0], push Q = r_S * (split port-0 weight).
+struct LoopInfo {
+    std::shared_ptr<Flat> sub;          // J (node 0), body, S, loop stream; sub->in_edge / out_edge = outer ports
+    int J = 0, S = -1, back = -1;       // joiner, splitter, returning edge (loop stream -> J port 1)
+    std::vector<uint32_t> enq;          // initial contents of the returning edge
+    int64_t P = 0, Q = 0;
+    // static schedule of one firing (one steady iteration of the loop graph), found by simulation
+    std::vector<int> sched;             // sub node ids in firing order
+    std::vector<int64_t> init_level;    // per sub edge: items queued at the stream start
+    std::vector<int64_t> cap;           // per sub edge: FIFO capacity (power of two >= max live items)
+};
 
 struct Node {
     NodeType type = N_FILTER;
@@ -71,6 +87,7 @@ struct Node {
     int64_t ninit = 0;   // init-schedule firings (signed: negative = lag)
     int64_t halo = 0;    // extra firings before a range start (same for every start)
     int elem = -1;       // builder element (filters)
+    std::shared_ptr<LoopInfo> loop;  // N_LOOP only
 };
 
 struct Edge {

@@ -48,6 +48,9 @@ PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
     for (int e : outs) bytes += 4.0 * f.edges[e].per_iter;
     double flops = 0, intops = 0, dfma = 0, smem = 0;
     int levels = 0;
+    double seq = 0;  // feedback loops: one thread walks the loop schedule (~25 ns per firing)
+    for (int v : nodes)
+        if (f.nodes[v].type == N_LOOP) seq += 25e-9 * (double)f.nodes[v].rep * (double)f.nodes[v].loop->sched.size();
     for (int v : nodes) {
         int64_t a, b, c;
         node_work(f, v, a, b, c);
@@ -65,7 +68,7 @@ PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
     for (int e : ins) smem += 8.0 * f.edges[e].per_iter;
     for (int e : outs) smem += 8.0 * f.edges[e].per_iter;
     double eff = est.mode == 1 ? 0.8 : 0.5;
-    est.t_comp = flops / (kFp32 * eff) + intops / kInt + dfma * 80.0 / kFp64 + smem / kSmem;
+    est.t_comp = flops / (kFp32 * eff) + intops / kInt + dfma * 80.0 / kFp64 + smem / kSmem + seq;
     est.t_dt = bytes / kHbm;
     double bar = est.mode == 2 ? levels * 200.0 / kClk / (kTileEst * kSM * 2) : 0.0;
     est.t = (std::max(est.t_comp, est.t_dt) + bar + kLaunch / kFragIters) * 1e9;  // ns per iteration
@@ -211,6 +214,7 @@ void innermost_pipelines(const sg_graph& g, std::vector<std::vector<int>>& out) 
             for (int k : e.kids) walk(k);
             return;
         }
+        if (e.type == E_LOOP) { next++; return; }  // one N_LOOP node (its graph lives in LoopInfo::sub)
         next++;  // splitter
         for (int b : e.branches) walk(b);
         next++;  // joiner
@@ -524,6 +528,38 @@ std::vector<std::vector<int>> make_partitions(const Flat& f, const sg_graph& g, 
     }
     default: throw Error(SG_E_ARG, "unknown partitioner");
     }
+    // a feedback loop runs sequentially: it is a partition of its own.  Splitting a convex
+    // partition into {ancestors of the loop}, {loop}, {the rest} keeps every piece convex and the
+    // partition graph acyclic (no path leaves the rest and re-enters the ancestors).
+    for (bool again = true; again;) {
+        again = false;
+        for (size_t i = 0; i < parts.size() && !again; i++) {
+            if (parts[i].size() < 2) continue;
+            for (int v : parts[i]) {
+                if (f.nodes[v].type != N_LOOP) continue;
+                std::vector<char> anc(N, 0);
+                std::vector<int> st{v};
+                while (!st.empty()) {
+                    int u = st.back();
+                    st.pop_back();
+                    for (int e : f.nodes[u].in) {
+                        int w = f.edges[e].src;
+                        if (w >= 0 && !anc[w]) { anc[w] = 1; st.push_back(w); }
+                    }
+                }
+                std::vector<int> a, rest;
+                for (int u : parts[i]) {
+                    if (u == v) continue;
+                    (anc[u] ? a : rest).push_back(u);
+                }
+                parts[i] = {v};
+                if (!a.empty()) parts.push_back(a);
+                if (!rest.empty()) parts.push_back(rest);
+                again = true;
+                break;
+            }
+        }
+    }
     return parts;
 }
 
@@ -614,10 +650,14 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     const int N = (int)f.nodes.size();
     // ---- replica groups (hybrid replica x pipeline; R = 1 is the paper's mapping)
     int R = 1;
+    bool has_loop = false;
+    for (auto& n : f.nodes) has_loop |= n.type == N_LOOP;
+    if (has_loop && o.replicas > 1)
+        throw Error(SG_E_UNSUPPORTED, "replicas > 1: a feedback loop carries state from one fragment to the next");
     if (o.replicas > 1) {
         if (G % o.replicas) throw Error(SG_E_ARG, "replicas must divide n_gpus");
         R = o.replicas;
-    } else if (o.replicas < 0 && G > 1) {
+    } else if (o.replicas < 0 && G > 1 && !has_loop) {
         double best = 0;
         for (int r = 1; r <= G; r++) {
             if (G % r) continue;
@@ -705,6 +745,7 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     for (int i = 0; i < P; i++) {
         if (o.plan_only) {  // partitions and mapping only: keep the PEE's mode decision
             p.kernels[i].ki.mode = register_mode_eligible(f, parts[i], nullptr) ? 1 : 2;
+            if (parts[i].size() == 1 && f.nodes[parts[i][0]].type == N_LOOP) p.kernels[i].ki.mode = 4;
             p.kernels[i].ki.tile = 1;
             partition_boundary(f, parts[i], p.kernels[i].ki.in_edges, p.kernels[i].ki.out_edges);
             p.part_mode[i] = p.kernels[i].ki.mode;

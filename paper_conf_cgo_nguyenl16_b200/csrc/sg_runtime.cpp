@@ -276,6 +276,10 @@ int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int
     v.push_back(kb);
     v.push_back(ke);
     const KernelInfo& ki = ck.ki;
+    if (ki.state_words > 0) {
+        if ((int)ck.state.size() <= dev || !ck.state[dev]) throw Error(SG_E_CUDA, "internal: loop state not initialised");
+        v.push_back((int64_t)(uintptr_t)ck.state[dev]);
+    }
     if (ki.mode == 1 && ki.has_tma) {
         const char* in_row0 = (const char*)io.in[0] + (kb * ki.pin + ki.off_in - io.in_base[0]) * 4;
         char* out_row0 = (char*)io.out[0] + (kb * ki.pout + ki.off_out - io.out_base[0]) * 4;
@@ -329,6 +333,23 @@ int64_t launch_kernel(CompiledKernel& ck, int dev, const IoBinding& io, int64_t 
     return launch(ck, dev, io, kb, ke, stream, is_f32);
 }
 
+void reset_state(CompiledKernel& ck, int dev, cudaStream_t stream) {
+    if (ck.ki.state_words <= 0) return;
+    if ((int)ck.state.size() <= dev) {
+        ck.state.resize(dev + 1, nullptr);
+        ck.state0.resize(dev + 1, nullptr);
+    }
+    const size_t bytes = (size_t)ck.ki.state_words * 4;
+    if (!ck.state[dev]) {
+        DevGuard dg(dev);
+        SG_RT(cudaMalloc(&ck.state[dev], bytes));
+        SG_RT(cudaMalloc(&ck.state0[dev], bytes));
+        SG_RT(cudaMemcpy(ck.state0[dev], ck.ki.state_init.data(), bytes, cudaMemcpyHostToDevice));
+    }
+    DevGuard dg(dev);
+    SG_RT(cudaMemcpyAsync(ck.state[dev], ck.state0[dev], bytes, cudaMemcpyDeviceToDevice, stream));
+}
+
 Plan::~Plan() {
     dist_release();
     for (auto& r : rings) {
@@ -354,9 +375,14 @@ Plan::~Plan() {
     if (host_in_dev) { cudaSetDevice(devices[input_gpu]); cudaFree(host_in_dev); }
     if (host_out_dev) { cudaSetDevice(devices[output_gpu]); cudaFree(host_out_dev); }
     if (host_stream) { cudaSetDevice(devices[input_gpu]); cudaStreamDestroy(host_stream); }
-    for (auto& ck : kernels)
+    for (auto& ck : kernels) {
         for (size_t d = 0; d < ck.mod.size(); d++)
             if (ck.mod[d]) { cudaSetDevice((int)d); drv::api().unload(ck.mod[d]); }
+        for (size_t d = 0; d < ck.state.size(); d++) {
+            if (ck.state[d]) { cudaSetDevice((int)d); cudaFree(ck.state[d]); }
+            if (ck.state0[d]) { cudaSetDevice((int)d); cudaFree(ck.state0[d]); }
+        }
+    }
 }
 
 void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
@@ -382,6 +408,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
         io.in_limit = {n_in};
         io.out = {out};
         io.out_base = {0};
+        reset_state(ck, devices[0], stream);
         last_launches += launch(ck, devices[0], io, 0, n, stream, flat.dtype == SG_F32);
         return;
     }
@@ -493,6 +520,12 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
         SG_RT(cudaStreamWaitEvent(g.compute, user_ev, 0));
         SG_RT(cudaStreamWaitEvent(g.copy, user_ev, 0));
     }
+    // feedback loops restart from their enqueued items (R = 1 for graphs with loops)
+    for (size_t p = 0; p < parts.size(); p++)
+        if (kernels[p].ki.state_words > 0) {
+            GpuCtx& gc = gpus[part_gpu[p]];
+            reset_state(kernels[p], gc.dev, gc.compute);
+        }
     const int64_t nfrag = (n + F - 1) / F;
     for (int64_t fi = 0; fi < nfrag; fi++) {
         const int64_t ka = fi * F, kb = std::min(n, ka + F);
@@ -661,9 +694,13 @@ void Plan::profile_partitions(int64_t n, int reps, double* ns_per_iter) {
         SG_RT(cudaStreamCreateWithFlags(&s, cudaStreamNonBlocking));
         SG_RT(cudaEventCreate(&e0));
         SG_RT(cudaEventCreate(&e1));
+        reset_state(ck, dev, s);
         launch(ck, dev, io, 0, n, s, flat.dtype == SG_F32);  // warm-up (module load, caches)
         SG_RT(cudaEventRecord(e0, s));
-        for (int r = 0; r < reps; r++) launch(ck, dev, io, 0, n, s, flat.dtype == SG_F32);
+        for (int r = 0; r < reps; r++) {
+            reset_state(ck, dev, s);  // feedback loops: every repetition starts from the stream start
+            launch(ck, dev, io, 0, n, s, flat.dtype == SG_F32);
+        }
         SG_RT(cudaEventRecord(e1, s));
         SG_RT(cudaEventSynchronize(e1));
         float ms = 0;

@@ -22,6 +22,8 @@ struct CompiledKernel {
     std::vector<CUfunction> fn_sync;       // register mode: synchronous fallback; staged: stream-start variant
     std::vector<int> max_blocks_per_sm;
     std::vector<int> max_blocks_sync;
+    // feedback loop state (per device): live buffer and the stream-start image
+    std::vector<void*> state, state0;
 };
 
 struct CutRing {          // one boundary stream between partitions (a PDG edge member)
@@ -108,6 +110,8 @@ struct Plan {
 
 int64_t launch_kernel(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int64_t ke, cudaStream_t stream,
                       bool is_f32);
+// feedback-loop partitions: (allocate and) reset the persistent state to its stream-start image on `stream`
+void reset_state(CompiledKernel& ck, int dev, cudaStream_t stream);
 int64_t fragment_size(const Plan& p, int64_t n);
 std::vector<RankOp> rank_schedule(const Plan& p, int rank, int64_t n, int64_t F);
 void nccl_unique_id(uint8_t out[128]);

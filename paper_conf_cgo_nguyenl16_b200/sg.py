@@ -28,7 +28,8 @@ KINDS = {"IDENTITY": 0, "FIR": 1, "DELAY": 2, "DECIMATE": 3, "EXPAND": 4, "COMPA
          "MULTIPLY": 15, "PERMUTE": 16, "XOR": 17, "XOR_CONST": 18, "SBOX": 19,
          "INTO_BITS": 20, "BITS_TO_INT": 21}
 
-EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_splitjoin", "sg_branch_begin",
+EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_splitjoin", "sg_add_feedbackloop",
+           "sg_branch_begin",
            "sg_branch_end", "sg_plan_opts_default", "sg_plan", "sg_input_items", "sg_output_items",
            "sg_plan_info", "sg_plan_source", "sg_run", "sg_run_host", "sg_last_launch_count",
            "sg_plan_destroy", "sg_last_error", "sg_version", "sg_flush_l2", "sg_topology_links",
@@ -92,6 +93,8 @@ def lib():
         "sg_graph_create": ([ctypes.c_int, ctypes.POINTER(vp)], ctypes.c_int),
         "sg_graph_destroy": ([vp], None),
         "sg_add_filter": ([vp, ctypes.POINTER(FilterDesc), ctypes.POINTER(i32)], ctypes.c_int),
+        "sg_add_feedbackloop": ([vp, ctypes.POINTER(i32), ctypes.c_int, ctypes.POINTER(i32), i32, vp,
+                                 ctypes.POINTER(i32)], ctypes.c_int),
         "sg_add_splitjoin": ([vp, ctypes.c_int, ctypes.POINTER(i32), ctypes.POINTER(i32), i32, ctypes.POINTER(i32)],
                              ctypes.c_int),
         "sg_branch_begin": ([vp, i32, i32], ctypes.c_int),
@@ -165,6 +168,19 @@ class Graph:
         _check(lib().sg_add_splitjoin(self._h, 0 if dup else 1, sw, jw, n_branches, ctypes.byref(sj)))
         return sj.value
 
+    def add_feedbackloop(self, join_w, dup: bool, split_w=None, enqueue=()) -> int:
+        """Feedback loop; then fill branch 0 (body) and branch 1 (loop stream) with branch_begin/end."""
+        lid = ctypes.c_int32(-1)
+        jw = _i32arr(join_w)
+        sw = _i32arr(split_w) if split_w is not None else None
+        if self.dtype == "i32":
+            enq = (ctypes.c_int32 * max(1, len(enqueue)))(*[int(v) for v in enqueue])
+        else:
+            enq = (ctypes.c_float * max(1, len(enqueue)))(*[float(v) for v in enqueue])
+        _check(lib().sg_add_feedbackloop(self._h, jw, 0 if dup else 1, sw, len(enqueue), ctypes.cast(enq, ctypes.c_void_p),
+                                         ctypes.byref(lid)))
+        return lid.value
+
     def branch_begin(self, sj: int, b: int):
         _check(lib().sg_branch_begin(self._h, sj, b))
 
@@ -185,7 +201,7 @@ class Graph:
 
 def graph_from_program(prog) -> Graph:
     """Marshal a neutral workloads.spec.Program into C-ABI builder calls."""
-    from workloads.spec import Filter, Pipeline  # neutral description, no arithmetic
+    from workloads.spec import FeedbackLoop, Filter, Pipeline  # neutral description, no arithmetic
     g = Graph(prog.dtype)
 
     def emit(s):
@@ -194,6 +210,12 @@ def graph_from_program(prog) -> Graph:
         elif isinstance(s, Pipeline):
             for c in s.children:
                 emit(c)
+        elif isinstance(s, FeedbackLoop):
+            lid = g.add_feedbackloop(s.join_w, s.split == "dup", s.split_w, s.enqueue)
+            for b, br in enumerate((s.body, s.loop)):
+                g.branch_begin(lid, b)
+                emit(br)
+                g.branch_end()
         else:
             sj = g.add_splitjoin(s.split == "dup", len(s.branches), s.split_w, s.join_w)
             for b, br in enumerate(s.branches):

@@ -439,3 +439,50 @@ def test_hybrid_estimate_scales(sg):
         with sg.plan(apps.filterbank(64), 8, plan_only=1, virtual_gpus=1, replicas=R, partitioner="single") as p:
             t[R] = p.info()["est_tmax"]
     assert t[2] < t[1] * 0.6 and t[4] < t[2] * 0.6 and t[8] < t[4] * 0.6
+
+
+# ----------------------------------------------------------------- feedback loops
+@pytest.mark.parametrize("name", list(apps.FEEDBACK))
+def test_feedback_rates_and_input_items_match_oracle(sg, oracle_lib, name):
+    prog = apps.FEEDBACK[name]()
+    r = oracle_lib.rates(prog)
+    with sg.plan(prog, 1, plan_only=1) as p:
+        i = p.info()
+        assert (i["in_per_iter"], i["out_per_iter"]) == (r["in_per_iter"], r["out_per_iter"])
+        for n in (1, 2, 7, 100, 1000):
+            assert p.input_items(n) == oracle_lib.in_items(prog, n), n
+        # every loop is a partition of its own (mode 4: sequential)
+        loops = [q for q, m in enumerate(i["partition_mode"]) if m == 4]
+        assert loops and all(sum(1 for v in i["node_partition"] if v == q) == 1 for q in loops)
+
+
+def test_feedback_loop_rejections(sg):
+    from workloads.spec import FeedbackLoop, Filter, Pipeline, Program
+    def plan(fb, **kw):
+        return sg.plan(Program("x", "f32", Pipeline([fb])), kw.pop("G", 1), plan_only=1, **kw)
+    with pytest.raises(sg.SgError) as e:      # peeking filter inside the loop
+        plan(FeedbackLoop(Pipeline([Filter("ADD", [2]), Filter("FIR", [3, 1], [1.0, 1.0, 1.0])]), Filter("IDENTITY"),
+                          enqueue=[0.0]))
+    assert e.value.code == sg.SG_E_UNSUPPORTED
+    with pytest.raises(sg.SgError) as e:      # no enqueued item: the joiner waits forever
+        plan(FeedbackLoop(Filter("ADD", [2]), Filter("IDENTITY")))
+    assert e.value.code == sg.SG_E_RATE
+    with pytest.raises(sg.SgError) as e:      # rate-inconsistent loop
+        plan(FeedbackLoop(Filter("ADD", [2]), Filter("EXPAND", [2]), enqueue=[0.0]))
+    assert e.value.code == sg.SG_E_RATE
+    with pytest.raises(sg.SgError) as e:      # nested loops
+        plan(FeedbackLoop(Pipeline([Filter("ADD", [2]), FeedbackLoop(Filter("ADD", [2]), Filter("IDENTITY"),
+                                                                     enqueue=[0.0])]),
+                          Filter("IDENTITY"), enqueue=[0.0]))
+    assert e.value.code == sg.SG_E_UNSUPPORTED
+    with pytest.raises(sg.SgError) as e:      # replicas would split the loop's sequential state
+        plan(FeedbackLoop(Filter("ADD", [2]), Filter("IDENTITY"), enqueue=[0.0]), G=2, virtual_gpus=1, replicas=2)
+    assert e.value.code == sg.SG_E_UNSUPPORTED
+
+
+def test_feedback_kernel_source(sg):
+    with sg.plan(apps.echo(8), 1) as p:
+        i = p.info()
+        q = i["partition_mode"].index(4)
+        src = p.source(q)
+        assert "(feedback loop mode)" in src and "SG_STATE" in src and "sg_work_amplify" in src

@@ -33,7 +33,7 @@ import random
 from fractions import Fraction
 from typing import List, Tuple
 
-from .spec import Filter, Pipeline, Program, SplitJoin, f32
+from .spec import FeedbackLoop, Filter, Pipeline, Program, SplitJoin, f32
 
 
 # --------------------------------------------------------------------------- FFT
@@ -312,6 +312,31 @@ def des(rounds: int = 16, key: int = DES_KEY, decrypt: bool = False) -> Program:
     return Program(f"des{rounds}", "i32", Pipeline(kids),
                    note="one iteration = one 64-bit block as two int32 words (high word first) -> its DES "
                         "encryption (decryption with reversed round keys)")
+
+
+# ----------------------------------------------------------------- feedback loops
+# PAPER.md:180-182 names the feedback loop as the third composition; none of its benchmarks uses one
+# (SURVEY.md 8(f)-4).  Small programs in StreamIt's style exercise the construct:
+def echo(delay: int = 64, gain: float = 0.5, taps: int = 16) -> Program:
+    """Echo effect: y_n = x_n + gain * y_{n-delay} (an IIR comb) between two FIR smoothers."""
+    c = lowpass_coeffs(1.0, 0.25, taps)
+    return Program(f"echo{delay}", "f32", Pipeline([
+        Filter("FIR", [taps, 1], c),
+        FeedbackLoop(Filter("ADD", [2]), Filter("AMPLIFY", [], [gain]), [1, 1], "dup", enqueue=[0.0] * delay),
+        Filter("FIR", [taps, 2], c)]),
+        note="one iteration = 2 input samples -> 1 output sample (the second FIR decimates by 2)")
+
+
+def running_stats() -> Program:
+    """int32 running sum and running max side by side (split-join of two feedback loops)."""
+    rsum = FeedbackLoop(Filter("ADD", [2]), Filter("IDENTITY"), [1, 1], "dup", enqueue=[0])
+    rmax = FeedbackLoop(Filter("COMPARE_EXCHANGE", [1]), Filter("IDENTITY"), [1, 1], "rr", [1, 1],
+                        enqueue=[-2 ** 31])
+    return Program("runstats", "i32", Pipeline([SplitJoin("dup", [rsum, rmax])]),
+                   note="one iteration = 1 key -> (running sum, min(key, running max of the previous keys))")
+
+
+FEEDBACK = {"echo64": lambda: echo(64), "runstats": running_stats}
 
 
 EXTRA = {
