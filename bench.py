@@ -42,7 +42,7 @@ WORKLOADS = {
     "bitonicrec32": dict(n=1 << 20, bound="hbm", desc="recursive BitonicSort 32-key int32, 1M iterations"),
     "dct16": dict(n=1 << 18, bound="hbm", desc="2-D DCT-II of 16x16 fp32 blocks (row then column FIR DCTs)"),
     "matmul16": dict(n=1 << 18, bound="hbm", desc="C = A B of streamed 16x16 fp32 matrices (MULTIPLY, ADD)"),
-    "des16": dict(n=1 << 20, bound="int", desc="DES (16 rounds) on a bit-per-item int32 stream, one 64-bit block / iteration"),
+    "des16": dict(n=1 << 22, bound="int", desc="DES (16 rounds) on a bit-per-item int32 stream, one 64-bit block / iteration"),
 }
 
 
