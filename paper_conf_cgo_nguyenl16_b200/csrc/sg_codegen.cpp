@@ -1161,13 +1161,21 @@ private:
         if (L == 0x33) return {B.s, true};
         if (L == 0xAA) return C;
         if (L == 0x55) return {C.s, true};
+        // a function and its complement share one LOP3 (the complement becomes a flag)
+        const bool cneg = L > 255 - L;
+        if (cneg) L = 255 - L;
         auto key = std::make_tuple(L, A, B, C);
         auto it = lop_memo_.find(key);
-        if (it != lop_memo_.end()) return it->second;
-        char b[32];
-        std::snprintf(b, sizeof b, "0x%02x", L);
-        BV r = fresh("sg_lop3<" + std::string(b) + ">(" + A.s + ", " + B.s + ", " + C.s + ")");
-        lop_memo_[key] = r;
+        BV r;
+        if (it != lop_memo_.end()) {
+            r = it->second;
+        } else {
+            char b[32];
+            std::snprintf(b, sizeof b, "0x%02x", L);
+            r = fresh("sg_lop3<" + std::string(b) + ">(" + A.s + ", " + B.s + ", " + C.s + ")");
+            lop_memo_[key] = r;
+        }
+        r.neg = cneg;
         return r;
     }
     BV mux(const BV& s, const BV& x1, const BV& x0) {  // s ? x1 : x0
