@@ -1330,23 +1330,44 @@ public:
         std::iota(a.begin(), a.end(), 0);
         return a;
     }
+    // Wavefront width: firing g reads an item of edge e written by firing g' <= g - floor(init_e / T_e)
+    // (init_e = items queued at the stream start: enqueued items, DELAY prework), so the firings of any
+    // window of W = min_e floor(init_e / T_e) consecutive firings are independent and run on W lanes.
+    static int64_t wavefront(const LoopInfo& li) {
+        const Flat& sf = *li.sub;
+        int64_t W = 256;
+        for (int e = 0; e < (int)sf.edges.size(); e++)
+            if (li.init_level[e] > 0) W = std::min<int64_t>(W, li.init_level[e] / std::max<int64_t>(1, sf.edges[e].per_iter));
+        return std::max<int64_t>(1, W);
+    }
+    // ring capacity of edge e when W firings are in flight: W * T_e beyond the simulated maximum
+    static std::vector<int64_t> capacities(const LoopInfo& li, int64_t W) {
+        const Flat& sf = *li.sub;
+        std::vector<int64_t> cap(sf.edges.size(), 0);
+        for (int e = 0; e < (int)sf.edges.size(); e++) {
+            int64_t c = 1;
+            while (c < li.cap[e] + (W - 1) * sf.edges[e].per_iter) c <<= 1;
+            cap[e] = c;
+        }
+        return cap;
+    }
     // state image layout (4-byte words): [0,2) next firing (int64), then each internal edge's ring, then history
-    static std::vector<uint32_t> initial_state(const LoopInfo& li, int64_t& hist_off, int64_t& hist_len, int64_t halo,
-                                               std::vector<int64_t>& ring_off) {
+    static std::vector<uint32_t> initial_state(const LoopInfo& li, const std::vector<int64_t>& cap, int64_t& hist_off,
+                                               int64_t& hist_len, int64_t hist_items, std::vector<int64_t>& ring_off) {
         const Flat& sf = *li.sub;
         int64_t o = 2;
         ring_off.assign(sf.edges.size(), -1);
         for (int e = 0; e < (int)sf.edges.size(); e++) {
             if (e == sf.in_edge || e == sf.out_edge) continue;
             ring_off[e] = o;
-            o += li.cap[e];
+            o += cap[e];
         }
         hist_off = o;
         hist_len = 1;
-        while (hist_len < std::max<int64_t>(1, halo * li.Q)) hist_len <<= 1;
+        while (hist_len < std::max<int64_t>(1, hist_items)) hist_len <<= 1;
         o += hist_len;
         std::vector<uint32_t> img((size_t)o, 0u);
-        for (size_t k = 0; k < li.enq.size(); k++) img[ring_off[li.back] + (k & (li.cap[li.back] - 1))] = li.enq[k];
+        for (size_t k = 0; k < li.enq.size(); k++) img[ring_off[li.back] + (k & (cap[li.back] - 1))] = li.enq[k];
         return img;  // DELAY prework items are zeros (already 0)
     }
 
@@ -1357,7 +1378,6 @@ public:
         ki.mode = 4;
         ki.name = "sg_part" + std::to_string(part_);
         ki.name_sync = ki.name;
-        ki.threads = ki.threads_sync = 32;
         ki.tile = ki.tile_sync = 1 << 30;  // one CTA
         ki.in_edges = {ln.in[0]};
         ki.out_edges = {ln.out[0]};
@@ -1376,16 +1396,30 @@ public:
             ki.intops_per_iter += b * ln.rep;
             ki.dfma_per_iter += c * ln.rep;
         }
+        int64_t W = wavefront(li_);
+        if (const char* e = std::getenv("SG_LOOP_WAVEFRONT")) W = std::max<int64_t>(1, std::min<int64_t>(W, std::atoll(e)));
+        std::vector<int64_t> cap;
+        int64_t smem_words = 0;
+        for (;; W = (W + 1) / 2) {  // shrink the wavefront until the rings fit in shared memory
+            cap = capacities(li_, W);
+            smem_words = 0;
+            for (int e = 0; e < (int)sf.edges.size(); e++)
+                if (e != sf.in_edge && e != sf.out_edge) smem_words += cap[e];
+            if (smem_words * 4 <= 160 * 1024 || W == 1) break;
+        }
+        if (smem_words * 4 > 200 * 1024) throw Error(SG_E_SIZE, "feedback loop FIFOs exceed shared memory");
+        const int NT = (int)std::min<int64_t>(256, (W + 31) / 32 * 32);
+        const int64_t WB = std::min<int64_t>(W, NT);  // firings per wavefront step
+        ki.threads = ki.threads_sync = NT;
         int64_t hist_off, hist_len;
         std::vector<int64_t> roff;
-        auto img = initial_state(li_, hist_off, hist_len, ln.halo, roff);
+        auto img = initial_state(li_, cap, hist_off, hist_len, (ln.halo + WB) * li_.Q, roff);
         ki.state_words = (int64_t)img.size();
         ki.state_init = img;
-        // shared-memory rings
-        int64_t smem_words = 0;
         std::vector<int64_t> soff(sf.edges.size(), -1);
+        int64_t so = 0;
         for (int e = 0; e < (int)sf.edges.size(); e++)
-            if (roff[e] >= 0) { soff[e] = smem_words; smem_words += li_.cap[e]; }
+            if (roff[e] >= 0) { soff[e] = so; so += cap[e]; }
         ki.smem = (size_t)std::max<int64_t>(4, smem_words * 4);
         ki.smem_sync = ki.smem;
         // one firing of the loop = the static schedule with compile-time offsets
@@ -1397,7 +1431,7 @@ public:
             const int64_t per = sf.edges[e].per_iter;
             if (e == sf.in_edge) return "gin[g * " + std::to_string(li_.P) + "LL + " + std::to_string(c) + "LL - in_base]";
             return "q[" + std::to_string(soff[e]) + " + (int)((g * " + std::to_string(per) + "LL + " + std::to_string(c) +
-                   "LL) & " + std::to_string(li_.cap[e] - 1) + "LL)]";
+                   "LL) & " + std::to_string(cap[e] - 1) + "LL)]";
         };
         for (int u : li_.sched) {
             const Node& n = sf.nodes[u];
@@ -1407,16 +1441,16 @@ public:
                 rd[e] += sf.edges[e].pop;
             }
             std::vector<std::string> ys;  // per output item, in port order
-            body << "      {\n";
+            body << "        {\n";
             if (n.type == N_FILTER) {
-                body << "        const " << T << " x_[" << std::max<size_t>(1, xs.size()) << "] = {";
+                body << "          const " << T << " x_[" << std::max<size_t>(1, xs.size()) << "] = {";
                 for (size_t i = 0; i < xs.size(); i++) body << (i ? ", " : "") << xs[i];
-                body << "};\n        " << T << " y_[" << n.push << "];\n        ";
+                body << "};\n          " << T << " y_[" << n.push << "];\n          ";
                 body << firing_code(u) << "\n";
                 for (int64_t j = 0; j < n.push; j++) ys.push_back("y_[" + std::to_string(j) + "]");
             } else {
                 // splitters / joiners: pure data movement
-                body << "        const " << T << " x_[" << xs.size() << "] = {";
+                body << "          const " << T << " x_[" << xs.size() << "] = {";
                 for (size_t i = 0; i < xs.size(); i++) body << (i ? ", " : "") << xs[i];
                 body << "};\n";
                 if (n.type == N_SPLIT_DUP) {
@@ -1433,58 +1467,59 @@ public:
                     const std::string val = n.type == N_SPLIT_DUP ? ys[k] : ys[yi];
                     if (e == sf.out_edge) {
                         const int64_t c = wr[e] + j;  // output item c of this firing
-                        body << "        { const long long p = g * " << li_.Q << "LL + " << c << "LL; const " << T << " val = " << val
-                             << ";\n          hist[(int)(p & " << hist_len - 1 << "LL)] = val;\n"
-                             << "          if (p >= wlo && p < whi) gout[p - out_base] = val; }\n";
+                        body << "          { const long long p = g * " << li_.Q << "LL + " << c << "LL; const " << T
+                             << " val = " << val << ";\n            hist[(int)(p & " << hist_len - 1 << "LL)] = val;\n"
+                             << "            if (p >= wlo && p < whi) gout[p - out_base] = val; }\n";
                     } else {
-                        body << "        " << pos_ref(e, wr[e] + j) << " = " << val << ";\n";
+                        body << "          " << pos_ref(e, wr[e] + j) << " = " << val << ";\n";
                     }
                 }
                 wr[e] += sf.edges[e].push;
             }
-            body << "      }\n";
+            body << "        }\n";
         }
         std::ostringstream s;
         s << header("feedback loop") << consts_.str() << args_struct_loop();
-        s << "extern \"C\" __global__ void __launch_bounds__(32, 1) " << ki.name << "(const SgArgs a) {\n"
+        s << "// wavefront: " << WB << " independent firings per step (loop delay " << wavefront(li_) << " firings)\n"
+          << "extern \"C\" __global__ void __launch_bounds__(" << NT << ", 1) " << ki.name << "(const SgArgs a) {\n"
           << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
           << "  " << T << "* q = reinterpret_cast<" << T << "*>(sg_smem);\n"
           << "  " << T << "* st = reinterpret_cast<" << T << "*>(SG_STATE);\n";
         for (int e = 0; e < (int)sf.edges.size(); e++)
             if (roff[e] >= 0)
-                s << "  for (int i = threadIdx.x; i < " << li_.cap[e] << "; i += 32) q[" << soff[e] << " + i] = st[" << roff[e]
-                  << " + i];\n";
-        s << "  __syncwarp();\n"
-          << "  if (threadIdx.x == 0) {\n"
-          << "    " << T << "* hist = st + " << hist_off << ";\n"
-          << "    const " << T << "* gin = SG_IN(0);\n"
-          << "    const long long in_base = SG_IN_BASE(0);\n"
-          << "    " << T << "* gout = SG_OUT(0);\n"
-          << "    const long long out_base = SG_OUT_BASE(0);\n"
-          << "    const long long wlo = SG_K_BEGIN * " << OPI << "LL + (" << OLO << "LL);\n"
-          << "    const long long whi = SG_K_END * " << OPI << "LL + (" << OLO + OEX << "LL);\n"
-          << "    long long next = *reinterpret_cast<long long*>(st);\n"
-          << "    const long long g0 = SG_K_BEGIN * " << ln.rep << "LL + (" << ln.ninit - ln.halo << "LL);\n"
-          << "    const long long g1 = SG_K_END * " << ln.rep << "LL + (" << ln.ninit << "LL);\n"
-          << "    for (long long g = g0; g < g1; g++) {\n"
-          << "      if (g < next) {  // before the stream start (zeros) or already computed (history)\n"
+                s << "  for (int i = threadIdx.x; i < " << cap[e] << "; i += " << NT << ") q[" << soff[e] << " + i] = st["
+                  << roff[e] << " + i];\n";
+        s << "  const long long next0 = *reinterpret_cast<const long long*>(st);\n"
+          << "  __syncthreads();\n"
+          << "  " << T << "* hist = st + " << hist_off << ";\n"
+          << "  const " << T << "* gin = SG_IN(0);\n"
+          << "  const long long in_base = SG_IN_BASE(0);\n"
+          << "  " << T << "* gout = SG_OUT(0);\n"
+          << "  const long long out_base = SG_OUT_BASE(0);\n"
+          << "  const long long wlo = SG_K_BEGIN * " << OPI << "LL + (" << OLO << "LL);\n"
+          << "  const long long whi = SG_K_END * " << OPI << "LL + (" << OLO + OEX << "LL);\n"
+          << "  const long long g0 = SG_K_BEGIN * " << ln.rep << "LL + (" << ln.ninit - ln.halo << "LL);\n"
+          << "  const long long g1 = SG_K_END * " << ln.rep << "LL + (" << ln.ninit << "LL);\n"
+          << "  for (long long gb = g0; gb < g1; gb += " << WB << ") {\n"
+          << "    const long long g = gb + threadIdx.x;\n"
+          << "    if (threadIdx.x < " << WB << " && g < g1) {\n"
+          << "      if (g < next0) {  // before the stream start (zeros) or computed by an earlier launch (history)\n"
           << "        for (int j = 0; j < " << li_.Q << "; j++) {\n"
           << "          const long long p = g * " << li_.Q << "LL + j;\n"
           << "          if (p >= wlo && p < whi) gout[p - out_base] = g < 0 ? (" << T << ")0 : hist[(int)(p & " << hist_len - 1
           << "LL)];\n"
           << "        }\n"
-          << "        continue;\n"
-          << "      }\n"
+          << "      } else {\n"
           << body.str()
-          << "      next = g + 1;\n"
+          << "      }\n"
           << "    }\n"
-          << "    *reinterpret_cast<long long*>(st) = next;\n"
+          << "    __syncthreads();\n"
           << "  }\n"
-          << "  __syncwarp();\n";
+          << "  if (threadIdx.x == 0) *reinterpret_cast<long long*>(st) = next0 > g1 ? next0 : g1;\n";
         for (int e = 0; e < (int)sf.edges.size(); e++)
             if (roff[e] >= 0)
-                s << "  for (int i = threadIdx.x; i < " << li_.cap[e] << "; i += 32) st[" << roff[e] << " + i] = q[" << soff[e]
-                  << " + i];\n";
+                s << "  for (int i = threadIdx.x; i < " << cap[e] << "; i += " << NT << ") st[" << roff[e] << " + i] = q["
+                  << soff[e] << " + i];\n";
         s << "}\n";
         ki.source = s.str();
         return ki;
