@@ -168,6 +168,8 @@ def main():
     ap.add_argument("--eager", action="store_true", help="launch sg_run every step instead of replaying a CUDA graph")
     ap.add_argument("--tile", type=int, default=0, help="plan option tile_iters (0: chosen by the code generator)")
     ap.add_argument("--threads", type=int, default=0, help="plan option threads per CTA (0: chosen)")
+    ap.add_argument("--codegen", default="auto", choices=["auto", "register", "staged", "general"],
+                    help="plan option codegen_mode (auto: chosen by the code generator)")
     ap.add_argument("--mode", default="replicas", choices=["replicas", "pipeline"],
                     help="N>1: independent replicas (default; the headline graph is HBM-bound) or the paper's "
                          "pipelined partition mapping, one process per GPU, NCCL boundary streams")
@@ -202,6 +204,8 @@ def main():
             kw["tile_iters"] = args.tile
         if args.threads:
             kw["threads"] = args.threads
+        if args.codegen != "auto":
+            kw["codegen_mode"] = args.codegen
         plan = sg.plan(prog, 1, devices=[local], **kw)
     info = plan.info()
     nin, nout = plan.input_items(n), plan.output_items(n)

@@ -17,7 +17,8 @@ pytestmark = pytest.mark.gpu
 PROGS = {
     "runsum": lambda: Program("rsum", "i32", Pipeline([FeedbackLoop(Filter("ADD", [2]), Filter("IDENTITY"), [1, 1],
                                                                     "dup", enqueue=[0])])),
-    "echo64": apps.FEEDBACK["echo64"],
+    "echo64": apps.FEEDBACK["echo64"],           # wavefront of 64 firings (2 warps)
+    "echo300": lambda: apps.echo(300, -0.75, 8),  # wavefront capped at 256 firings
     "runstats": apps.FEEDBACK["runstats"],
     "multirate": lambda: Program("mr", "f32", Pipeline([
         Filter("FIR", [5, 1], [0.5, -1.0, 0.25, 2.0, -0.5]),
