@@ -287,15 +287,17 @@ def main():
                     "frac": ach / peaks["hbm_gbs"], "traffic": None,
                     "algorithmic_bytes_per_launch": ki_bytes, "peak_source": peak_src + " copy bandwidth"}
     elif W["bound"] == "int":
+        # DES works on one bit per item: its algorithmic ops are bit operations, and the ALU's peak in
+        # bit operations is 32 per int32 lane op (the bitsliced kernel packs 32 iterations per word)
         ops = info["intops_per_iter"]
         if kern_ms:
             ach = ops * n / (kern_ms / 1e3) / 1e12
-            pk = 148 * 64 * peaks.get("sm_max_mhz", 1965.0) * 1e6 / 1e12
-            roof = {"bound": "alu", "achieved": ach, "peak": pk, "unit": "Tops/s", "frac": ach / pk,
+            pk = 148 * 64 * 32 * peaks.get("sm_max_mhz", 1965.0) * 1e6 / 1e12
+            roof = {"bound": "alu", "achieved": ach, "peak": pk, "unit": "Tbitops/s", "frac": ach / pk,
                     "traffic": None, "algorithmic_ops_per_launch": ops * n, "ops_per_iter": ops,
-                    "ops_counting": "as written: one op per XORed bit (key XOR included), per S-box lookup, "
-                                    "per bit unpacked / packed",
-                    "peak_source": "derived: 148 SMs x 64 int32 lanes/clk (alu pipe, LOP3/SHF rate) x sm_max_mhz"}
+                    "ops_counting": "as written, in bit operations: one per XORed bit (key XOR included), one per "
+                                    "S-box lookup, one per bit unpacked / packed",
+                    "peak_source": "derived: 148 SMs x 64 int32 lanes/clk (alu pipe: LOP3/SHF) x 32 bits x sm_max_mhz"}
     else:
         fl_written = _flops_per_iter(prog, info["reps"])
         fl = min(fl_written, info["flops_per_iter_pruned"]) if info["flops_per_iter_pruned"] > 0 else fl_written

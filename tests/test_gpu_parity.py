@@ -168,7 +168,8 @@ def test_permute_any_dtype(oracle_lib):
     rng = np.random.default_rng(4)
     for dt in ("f32", "i32"):
         idx = rng.integers(0, 12, size=9).tolist()
-        prog = Program("perm", dt, Pipeline([Filter("PERMUTE", [12] + idx), Filter("PERMUTE", [9] + idx[::-1][:9])]))
+        idx2 = rng.integers(0, 9, size=13).tolist()       # 9 -> 13 items: duplicates allowed
+        prog = Program("perm", dt, Pipeline([Filter("PERMUTE", [12] + idx), Filter("PERMUTE", [9] + idx2)]))
         n = 1000
         x = inputs.make_input(dt, 12 * n, 77)
         y, _, _ = run_gpu(prog, x, n)
