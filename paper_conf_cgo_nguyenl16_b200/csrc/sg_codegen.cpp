@@ -1069,14 +1069,17 @@ public:
         ki.smem = ki.smem_sync = 0;
         std::ostringstream s;
         s << header("bitslice") << consts_.str() << args_struct();
-        s << "extern \"C\" __global__ void __launch_bounds__(" << NT << ", 2) " << ki.name << "(const SgArgs a) {\n"
+        s << "extern \"C\" __global__ void __launch_bounds__(" << NT << ", " << (NT <= 128 ? 2 : 1) << ") " << ki.name << "(const SgArgs a) {\n"
           << "  const int lane = threadIdx.x & 31;\n"
           << "  const long long wstep = (long long)gridDim.x * " << NT / 32 << " * 1024;\n"
           << "  const " << T_ << "* gin = SG_IN(0) + ((" << off_in_ << "LL) - SG_IN_BASE(0));\n"
           << "  " << T_ << "* gout = SG_OUT(0) + ((" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
           << "  const bool vin = " << (PIN_ == 2 || PIN_ == 4 ? "(reinterpret_cast<unsigned long long>(gin) & " + std::to_string(PIN_ * 4 - 1) + "ull) == 0" : std::string("false")) << ";\n"
           << "  const bool vout = " << (POUT_ == 2 || POUT_ == 4 ? "(reinterpret_cast<unsigned long long>(gout) & " + std::to_string(POUT_ * 4 - 1) + "ull) == 0" : std::string("false")) << ";\n"
-          << "  for (long long wb = SG_K_BEGIN + ((long long)blockIdx.x * " << NT / 32 << " + (threadIdx.x >> 5)) * 1024; wb < SG_K_END; wb += wstep) {\n";
+          << "  // CTA-uniform tile loop (every warp of the CTA iterates equally often: barriers are safe);\n"
+          << "  // warps past the end compute on zeros and store nothing\n"
+          << "  for (long long cb = SG_K_BEGIN + (long long)blockIdx.x * " << NT * 32 << "LL; cb < SG_K_END; cb += wstep) {\n"
+          << "    const long long wb = cb + (long long)(threadIdx.x >> 5) * 1024;\n";
         // loads: word q of iteration wb + 32 j + lane -> w<q>[j]
         for (int64_t q = 0; q < PIN_; q++) s << "    unsigned w" << q << "[32];\n";
         s << "#pragma unroll\n"
@@ -1142,6 +1145,9 @@ private:
     BV fresh(const std::string& rhs) {
         std::string v = "b" + std::to_string(nv_++);
         body_ << "    const unsigned " << v << " = " << rhs << ";\n";
+        // optional lockstep barriers: the warps of a CTA stay within one instruction-cache window
+        static const int bar = std::getenv("SG_BS_BAR") ? std::atoi(std::getenv("SG_BS_BAR")) : 0;
+        if (bar > 0 && nv_ % bar == 0) body_ << "    __syncthreads();\n";
         return {v, false};
     }
     static BV zero() { return {"0u", false}; }

@@ -13,3 +13,11 @@ ENVV= one t128 filterbank64 --threads 128
 ENVV= one default fmradio10
 ENVV="SG_PAIRS=4" one pairs4 fmradio10
 ENVV= one t512 fmradio10 --threads 512
+ENVV= one default des16
+ENVV= one t384 des16 --threads 384
+ENVV= one t256 des16 --threads 256
+ENVV="SG_BS_BAR=256" one t384bar256 des16 --threads 384
+ENVV="SG_BS_BAR=512" one t384bar512 des16 --threads 384
+ENVV="SG_BS_BAR=512" one t128bar512 des16
+timeout 900 python -m pytest tests/test_gpu_parity.py -m gpu -q -k "des or permute" > gpurun_out/$TAG/pytest_des.log 2>&1; echo "rc=$?" >> gpurun_out/$TAG/pytest_des.log
+tail -n 2 gpurun_out/$TAG/pytest_des.log

@@ -65,11 +65,12 @@ def main(rnd):
              "Main partition kernel of `bench.py --config <name> --steps 2 --warmup 3` captured with",
              "`ncu --set full --clock-control none --import-source on -k regex:sg_part0$ -s 2 -c 1`",
              "(one launch, cold caches, serialised: use for shares and counters, not as the bench value).", ""]
-    traffic = {}
-    for name in ["bitonic32", "fft64", "fmradio10", "filterbank64", "beamformer12x4"]:
+    tpath = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    traffic = json.load(open(tpath)) if os.path.exists(tpath) else {}
+    import glob
+    names = sorted(os.path.basename(r)[5:-8] for r in glob.glob(os.path.join(src, "full_*.ncu-rep")))
+    for name in names:
         rep = os.path.join(src, f"full_{name}.ncu-rep")
-        if not os.path.exists(rep):
-            continue
         d, stalls = raw(rep)
         lines.append(f"## {name}")
         lines.append("")
@@ -102,7 +103,7 @@ def main(rnd):
             lines.append(f"| {k} | {len(v)} | {sum(v) / len(v):.0f} | {sum(v) / tot:.1%} |")
         lines.append("")
     open(os.path.join(ROOT, "profiles", f"{rnd}_summary.md"), "w").write("\n".join(lines) + "\n")
-    json.dump(traffic, open(os.path.join(ROOT, "profiles", "ncu_traffic.json"), "w"), indent=1)
+    json.dump(traffic, open(tpath, "w"), indent=1)
     print("\n".join(lines))
 
 
