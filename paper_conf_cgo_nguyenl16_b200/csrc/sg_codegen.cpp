@@ -1050,10 +1050,12 @@ public:
         POUT_ = f_.edges[eout_].per_iter;
         off_in_ = ki.in_lo[0];
         off_out_ = ki.out_lo[0];
+        // a run of identical periods (cipher rounds) becomes a rolled loop over a state array
+        const bool rolled = !std::getenv("SG_BS_NOROLL") && try_roll();
         // output words: each must be produced by a BITS_TO_INT firing
         std::vector<std::vector<BV>> obits(POUT_);
         for (int64_t p = 0; p < POUT_; p++) {
-            Ref r = R_.resolve(eout_, Lin::k(off_out_ + p));
+            Ref r = cur_R_->resolve(eout_, Lin::k(off_out_ + p));
             if (r.k != Ref::PHYS || r.edge == ein_) throw Error(SG_E_UNSUPPORTED, "bitslice: output item is not a BITS_TO_INT word");
             const Edge& ed = f_.edges[r.edge];
             const Node& n = f_.nodes[ed.src];
@@ -1068,7 +1070,7 @@ public:
         ki.tile = ki.tile_sync = NT * 32;
         ki.smem = ki.smem_sync = 0;
         std::ostringstream s;
-        s << header("bitslice") << consts_.str() << args_struct();
+        s << header(rolled ? "bitslice, rolled rounds" : "bitslice") << consts_.str() << args_struct();
         s << "extern \"C\" __global__ void __launch_bounds__(" << NT << ", " << (NT <= 128 ? 2 : 1) << ") " << ki.name << "(const SgArgs a) {\n"
           << "  const int lane = threadIdx.x & 31;\n"
           << "  const long long wstep = (long long)gridDim.x * " << NT / 32 << " * 1024;\n"
@@ -1137,6 +1139,170 @@ private:
     int ein_ = -1, eout_ = -1;
     int64_t PIN_ = 0, POUT_ = 0, off_in_ = 0, off_out_ = 0;
     std::ostringstream body_;
+    // evaluation context: resolver, and (rolled loop) the edge whose items live in the state array S
+    const Resolver* cur_R_ = &R_;
+    std::unique_ptr<Resolver> rpro_, rbody_, repi_;
+    int bedge_ = -2;
+    int64_t blo_ = 0, bm_ = 0;
+    std::map<int, int64_t> keyslot_;  // XOR_CONST node of period 0 -> first slot in the per-round key table
+
+    // Edges every input -> output path crosses (pipeline boundaries), in topological order.
+    std::vector<int> cut_edges() const {
+        std::vector<char> in(f_.nodes.size(), 0);
+        for (int v : nodes_) in[v] = 1;
+        const int s0 = f_.edges[ein_].dst, t0 = f_.edges[eout_].src;
+        std::vector<int> cuts;
+        for (int e = 0; e < (int)f_.edges.size(); e++) {
+            const Edge& ed = f_.edges[e];
+            if (ed.src < 0 || ed.dst < 0 || !in[ed.src] || !in[ed.dst]) continue;
+            std::vector<char> seen(f_.nodes.size(), 0);
+            std::vector<int> st{s0};
+            seen[s0] = 1;
+            while (!st.empty()) {
+                int u = st.back();
+                st.pop_back();
+                for (int oe : f_.nodes[u].out) {
+                    if (oe == e) continue;
+                    int w = f_.edges[oe].dst;
+                    if (w >= 0 && in[w] && !seen[w]) { seen[w] = 1; st.push_back(w); }
+                }
+            }
+            if (!seen[t0]) cuts.push_back(e);
+        }
+        std::sort(cuts.begin(), cuts.end(), [&](int a, int b) { return f_.edges[a].src < f_.edges[b].src; });
+        return cuts;
+    }
+    // structural signature of the node id range [a, b] (XOR_CONST constants excluded)
+    std::vector<int64_t> signature(int a, int b) const {
+        std::vector<int64_t> sig;
+        for (int v = a; v <= b; v++) {
+            const Node& n = f_.nodes[v];
+            sig.push_back(n.type);
+            sig.push_back(n.kind);
+            sig.push_back(n.rep);
+            const size_t niv = n.type == N_FILTER && n.kind == SG_K_XOR_CONST ? 1 : n.iv.size();
+            sig.push_back((int64_t)niv);
+            for (size_t i = 0; i < niv; i++) sig.push_back(n.iv[i]);
+            for (float x : n.fv) { uint32_t w; std::memcpy(&w, &x, 4); sig.push_back(w); }
+            for (int32_t w : n.w) sig.push_back(w);
+            for (int e : n.in) {
+                const Edge& ed = f_.edges[e];
+                sig.push_back(ed.src >= a && ed.src <= b ? ed.src - a : -1);
+                sig.insert(sig.end(), {ed.sport, ed.pop, ed.peek, ed.push, ed.pre, ed.per_iter});
+            }
+            for (int e : n.out) {
+                const Edge& ed = f_.edges[e];
+                sig.push_back(ed.dst >= a && ed.dst <= b ? ed.dst - a : -1);
+                sig.push_back(ed.dport);
+            }
+        }
+        return sig;
+    }
+    static int64_t iter_lo(const Flat& f, int e) {  // first position of iteration 0 on edge e
+        const Edge& ed = f.edges[e];
+        return ed.pre + f.nodes[ed.src].ninit * ed.push;
+    }
+    // Find the longest run of >= 3 identical periods between cut edges; set up prologue / body /
+    // epilogue resolvers and emit the prologue, the state array and the rolled loop.
+    bool try_roll() {
+        std::vector<int> cuts = cut_edges();
+        const int nseg = (int)cuts.size() - 1;
+        if (nseg < 3) return false;
+        std::vector<std::vector<int64_t>> sig(nseg);
+        for (int i = 0; i < nseg; i++) {
+            const int a = f_.edges[cuts[i]].dst, b = f_.edges[cuts[i + 1]].src;
+            if (b < a) return false;
+            sig[i] = signature(a, b);
+        }
+        int bs = -1, bp = 0, bk = 0;
+        int64_t bcov = 0;
+        for (int p = 1; p <= nseg / 3; p++)
+            for (int st = 0; st + 3 * p <= nseg; st++) {
+                int k = 1;
+                while (st + (k + 1) * p <= nseg) {
+                    bool same = true;
+                    for (int t = 0; t < p && same; t++) same = sig[st + k * p + t] == sig[st + t];
+                    if (!same) break;
+                    k++;
+                }
+                const int64_t cov = (int64_t)k * (f_.edges[cuts[st + p]].src - f_.edges[cuts[st]].dst + 1);
+                if (k >= 3 && cov > bcov) { bcov = cov; bs = st; bp = p; bk = k; }
+            }
+        if (bs < 0) return false;
+        const int e0 = cuts[bs], e1 = cuts[bs + bp], eend = cuts[bs + bk * bp];
+        const int64_t m = f_.edges[e0].per_iter;
+        if (f_.edges[e1].per_iter != m || f_.edges[eend].per_iter != m || m > 256) return false;
+        const int64_t lo0 = iter_lo(f_, e0), lo1 = iter_lo(f_, e1), loend = iter_lo(f_, eend);
+        if (lo0 != lo1 || lo0 != loend) return false;
+        const int a0 = f_.edges[e0].dst, b0 = f_.edges[e1].src;   // period 0 = node ids [a0, b0]
+        const int np = b0 - a0 + 1;
+        const int aend = f_.edges[eend].dst;                       // epilogue starts here
+        std::vector<int> pro, body, epi;  // periods 1..K-1 are never evaluated (the loop replays period 0)
+        for (int v : nodes_) {
+            if (v < a0) pro.push_back(v);
+            else if (v <= b0) body.push_back(v);
+            else if (v >= aend) epi.push_back(v);
+        }
+        if (pro.empty()) return false;
+        // per-round key table (only if the XOR_CONST constants differ between rounds)
+        int64_t kw = 0;
+        std::map<int, int64_t> slots;
+        bool differ = false;
+        for (int v = a0; v <= b0; v++) {
+            const Node& n = f_.nodes[v];
+            if (n.type != N_FILTER || n.kind != SG_K_XOR_CONST) continue;
+            slots[v] = kw;
+            kw += n.iv[0];
+            for (int k = 1; k < bk; k++) differ = differ || f_.nodes[v + k * np].iv != n.iv;
+        }
+        std::vector<uint32_t> table;
+        if (differ) {
+            for (int k = 0; k < bk; k++)
+                for (auto& kv : slots) {
+                    const Node& n = f_.nodes[kv.first + k * np];
+                    for (int i = 0; i < n.iv[0]; i++) table.push_back((n.iv[1 + i] & 1) ? 0xFFFFFFFFu : 0u);
+                }
+            keyslot_ = slots;
+            consts_ << "__constant__ unsigned SG_BSKEY[" << table.size() << "] = {";
+            for (size_t i = 0; i < table.size(); i++) consts_ << (i ? "," : "") << (i % 8 == 0 ? "\n  " : "") << "0x" << std::hex << table[i] << std::dec << "u";
+            consts_ << "};\n";
+        }
+        rpro_.reset(new Resolver(f_, pro));
+        rbody_.reset(new Resolver(f_, body));
+        repi_.reset(new Resolver(f_, epi));
+        // prologue: the state at the run's start
+        cur_R_ = rpro_.get();
+        std::vector<BV> s0(m);
+        for (int64_t j = 0; j < m; j++) s0[j] = bit(e0, lo0 + j);
+        body_ << "    unsigned S[" << m << "];\n";
+        for (int64_t j = 0; j < m; j++) body_ << "    S[" << j << "] = " << s0[j].expr() << ";\n";
+        // body: one period from S to the next S
+        lop_memo_.clear();
+        const std::string pre = body_.str();
+        body_.str("");
+        cur_R_ = rbody_.get();
+        bedge_ = e0;
+        blo_ = lo0;
+        bm_ = m;
+        std::vector<BV> s1(m);
+        for (int64_t j = 0; j < m; j++) s1[j] = bit(e1, lo1 + j);
+        std::string loop = body_.str();
+        body_.str("");
+        body_ << pre << "    // " << bk << " identical rounds of " << np << " nodes, rolled\n"
+              << "#pragma unroll 1\n"
+              << "    for (int r = 0; r < " << bk << "; r++) {\n";
+        if (differ) body_ << "      const unsigned* kt = SG_BSKEY + r * " << kw << ";\n";
+        body_ << loop;
+        for (int64_t j = 0; j < m; j++) body_ << "    const unsigned n" << j << " = " << s1[j].expr() << ";\n";
+        for (int64_t j = 0; j < m; j++) body_ << "    S[" << j << "] = n" << j << ";\n";
+        body_ << "    }\n";
+        // epilogue: everything after the run reads the final S
+        lop_memo_.clear();
+        keyslot_.clear();
+        cur_R_ = repi_.get();
+        bedge_ = eend;
+        return true;
+    }
     int nv_ = 0;
     std::set<int64_t> used_cols_;
     std::map<std::pair<int, int64_t>, std::vector<BV>> memo_;
@@ -1261,9 +1427,14 @@ private:
     }
     // packed value of item `pos` of edge e (bit domain)
     BV bit(int e, int64_t pos) {
-        Ref r = R_.resolve(e, Lin::k(pos));
+        Ref r = cur_R_->resolve(e, Lin::k(pos));
         if (r.k == Ref::ZERO) return zero();
         if (r.k != Ref::PHYS) throw Error(SG_E_UNSUPPORTED, "bitslice: non-constant position");
+        if (r.edge == bedge_) {  // rolled loop: the state array
+            const int64_t j = r.pos.c - blo_;
+            if (j < 0 || j >= bm_) throw Error(SG_E_UNSUPPORTED, "bitslice: state position out of range");
+            return {"S[" + std::to_string(j) + "]", false};
+        }
         if (r.edge == ein_) throw Error(SG_E_UNSUPPORTED, "bitslice: a raw input word is used as a bit");
         const Edge& ed = f_.edges[r.edge];
         const int u = ed.src;
@@ -1297,13 +1468,21 @@ private:
             }
             break;
         }
-        case SG_K_XOR_CONST:
+        case SG_K_XOR_CONST: {
+            auto ks = keyslot_.find(u);
             for (int64_t i = 0; i < n.iv[0]; i++) {
                 BV a = bit(n.in[0], g * n.pop + i);
+                if (ks != keyslot_.end()) {  // rolled loop: this round's key bit (0 or ~0) from the key table
+                    BV r = fresh(a.s + " ^ kt[" + std::to_string(ks->second + i) + "]");
+                    r.neg = a.neg;
+                    y.push_back(r);
+                    continue;
+                }
                 if (n.iv[1 + i] & 1) a.neg = !a.neg;
                 y.push_back(a);
             }
             break;
+        }
         case SG_K_SBOX: {
             std::vector<BV> x(6);
             for (int i = 0; i < 6; i++) x[i] = bit(n.in[0], g * n.pop + i);

@@ -400,12 +400,16 @@ def test_des_compiles_register_and_staged(sg):
         assert info["n_partitions"] == 1 and info["partition_mode"] == [1]
         assert info["intops_per_iter"] == 16 * (48 + 32 + 8) + 64 + 64
         src = p.source(0)
-        assert "(bitslice mode)" in src and "sg_transpose32(w0)" in src and "sg_transpose32(o1)" in src
-        assert 16 * 8 * 30 < src.count("sg_lop3<") < 16 * 8 * 64      # <= 64 gates per S-box
+        assert "(bitslice, rolled rounds mode)" in src and "sg_transpose32(w0)" in src and "sg_transpose32(o1)" in src
+        assert "16 identical rounds" in src and "SG_BSKEY" in src      # one round's circuit, per-round key table
+        assert 8 * 30 < src.count("sg_lop3<") < 8 * 64                # <= 64 gates per S-box
         assert "sg_work_sbox(" not in src and "SG_PI" not in src
     with sg.plan(apps.des(16), 1, codegen_mode="register") as p:
         src = p.source(0)
         assert src.count("sg_work_sbox(") == 16 * 8 and "SG_PI" not in src
+    with sg.plan(apps.des(2), 1) as p:                                  # too few rounds to roll
+        src = p.source(0)
+        assert "(bitslice mode)" in src and 2 * 8 * 30 < src.count("sg_lop3<") < 2 * 8 * 64
     with sg.plan(apps.des(2), 1, partitioner="per_filter") as p:
         assert p.info()["n_partitions"] > 1
         assert any("sg_work_xor<32>" in p.source(q) for q in range(p.info()["n_partitions"]))
