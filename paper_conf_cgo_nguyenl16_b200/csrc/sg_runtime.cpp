@@ -305,6 +305,41 @@ int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int
         return 1;
     }
     int64_t launches = 0;
+    if (ki.mode == 2 && !ki.name_start.empty() && kb < ki.ksafe && !std::getenv("SG_SERIAL_START")) {
+        int64_t ks = std::min(ke, kb + ((ki.ksafe - kb + ki.tile - 1) / ki.tile) * ki.tile);
+        if (ks < ke) {
+            // stream-start tiles (guarded variant) on a side stream beside the steady-state kernel, which
+            // leaves them their CTA slots: the start tiles no longer run alone before the main launch
+            if ((int)ck.aux.size() <= dev) {
+                ck.aux.resize(dev + 1, nullptr);
+                ck.ev_fork.resize(dev + 1, nullptr);
+                ck.ev_join.resize(dev + 1, nullptr);
+            }
+            if (!ck.aux[dev]) {
+                SG_RT(cudaStreamCreateWithFlags(&ck.aux[dev], cudaStreamNonBlocking));
+                SG_RT(cudaEventCreateWithFlags(&ck.ev_fork[dev], cudaEventDisableTiming));
+                SG_RT(cudaEventCreateWithFlags(&ck.ev_join[dev], cudaEventDisableTiming));
+            }
+            const int64_t st_tiles = (ks - kb + ki.tile - 1) / ki.tile;
+            std::vector<int64_t> v2 = v;
+            v2[v2.size() - 1] = ks;
+            SG_RT(cudaEventRecord(ck.ev_fork[dev], stream));
+            SG_RT(cudaStreamWaitEvent(ck.aux[dev], ck.ev_fork[dev], 0));
+            void* p2[] = {v2.data()};
+            SG_CU(cuLaunchKernel(ck.fn_sync[dev], (unsigned)st_tiles, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
+                                 (CUstream)ck.aux[dev], p2, nullptr));
+            SG_RT(cudaEventRecord(ck.ev_join[dev], ck.aux[dev]));
+            v[v.size() - 2] = ks;
+            const int64_t tiles = (ke - ks + ki.tile - 1) / ki.tile;
+            const int64_t slots = (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev];
+            const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, slots - std::min<int64_t>(st_tiles, slots / 2)));
+            void* p1[] = {v.data()};
+            SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
+                                 (CUstream)stream, p1, nullptr));
+            SG_RT(cudaStreamWaitEvent(stream, ck.ev_join[dev], 0));
+            return 2;
+        }
+    }
     if (ki.mode == 2 && !ki.name_start.empty() && kb < ki.ksafe) {
         // stream-start tiles (firings g < 0 must emit zeros): the guarded variant
         int64_t ks = std::min(ke, kb + ((ki.ksafe - kb + ki.tile - 1) / ki.tile) * ki.tile);
@@ -381,6 +416,13 @@ Plan::~Plan() {
         for (size_t d = 0; d < ck.state.size(); d++) {
             if (ck.state[d]) { cudaSetDevice((int)d); cudaFree(ck.state[d]); }
             if (ck.state0[d]) { cudaSetDevice((int)d); cudaFree(ck.state0[d]); }
+        }
+        for (size_t d = 0; d < ck.aux.size(); d++) {
+            if (!ck.aux[d]) continue;
+            cudaSetDevice((int)d);
+            cudaStreamDestroy(ck.aux[d]);
+            cudaEventDestroy(ck.ev_fork[d]);
+            cudaEventDestroy(ck.ev_join[d]);
         }
     }
 }

@@ -24,6 +24,9 @@ struct CompiledKernel {
     std::vector<int> max_blocks_sync;
     // feedback loop state (per device): live buffer and the stream-start image
     std::vector<void*> state, state0;
+    // staged kernels: side stream + fork/join events for the stream-start variant (per device)
+    std::vector<cudaStream_t> aux;
+    std::vector<cudaEvent_t> ev_fork, ev_join;
 };
 
 struct CutRing {          // one boundary stream between partitions (a PDG edge member)

@@ -1,0 +1,8 @@
+TAG=${TAG:-ab6}
+mkdir -p gpurun_out/$TAG
+one() { tag=$1; cfg=$2; shift 2; env $ENVV timeout 600 python bench.py --config $cfg --steps 300 --no-cpu-baseline "$@" > gpurun_out/$TAG/$cfg.$tag.json 2> gpurun_out/$TAG/$cfg.$tag.err; echo "$cfg $tag $(python -c "import json,sys; d=json.loads(open('gpurun_out/$TAG/$cfg.$tag.json').read().strip().splitlines()[-1]); print('ms %.4f frac %.3f launches %d' % (d['ms_per_step'], d['roofline']['frac'], d['gpu_launches']))" 2>&1 | tail -1)"; }
+ENVV= one concurrent filterbank64
+ENVV="SG_SERIAL_START=1" one serial filterbank64
+ENVV= one concurrent fmradio10
+timeout 1500 python -m pytest tests/test_gpu_parity.py tests/test_gpu_plans.py tests/test_gpu_feedback.py -m gpu -q -x > gpurun_out/$TAG/pytest.log 2>&1; echo "rc=$?" >> gpurun_out/$TAG/pytest.log
+tail -n 2 gpurun_out/$TAG/pytest.log
