@@ -430,10 +430,12 @@ protected:
     }
     // kernel argument block: all 8-byte words
     //   in ptr[NI], in_base[NI], in_limit[NI], out ptr[NO], out_base[NO], k_begin, k_end
-    std::string args_struct() {
+    // extra = 1 (staged kernels): one more word, the runtime tile size SG_WR (<= the compiled tile)
+    std::string args_struct(int extra = 0) {
         size_t ni = ins_.size(), no = outs_.size();
         std::ostringstream s;
-        s << "struct SgArgs { long long v[" << (3 * ni + 2 * no + 2) << "]; };\n";
+        s << "struct SgArgs { long long v[" << (3 * ni + 2 * no + 2 + extra) << "]; };\n";
+        if (extra) s << "#define SG_WR ((int)a.v[" << 3 * ni + 2 * no + 2 << "])\n";
         s << "#define SG_IN(i) (reinterpret_cast<const " << T_ << "*>(a.v[(i)]))\n";
         s << "#define SG_IN_BASE(i) (a.v[" << ni << " + (i)])\n";
         s << "#define SG_IN_LIMIT(i) (a.v[" << 2 * ni << " + (i)])\n";
@@ -1892,7 +1894,7 @@ public:
         ki.fused = WF > 0;
         ki.ksafe = ksafe;
         std::ostringstream src;
-        src << header("staged") << consts_.str() << args_struct();
+        src << header("staged") << consts_.str() << args_struct(1);
         src << "#define NT " << NT << "\n";
         src << readers_.str();
         auto kernel = [&](const std::string& name, const std::string& body, bool fusedk) {
@@ -1902,9 +1904,9 @@ public:
                 << "  " << T_ << "* sm = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
                 << "  const int tid = threadIdx.x;\n"
                 << (fusedk ? prologue_fast : std::string())
-                << "  for (long long kt = SG_K_BEGIN + (long long)blockIdx.x * " << WT << "; kt < SG_K_END; kt += (long long)gridDim.x * "
-                << WT << ") {\n"
-                << "    const int Wtt = (int)min((long long)" << WT << ", SG_K_END - kt);\n";
+                << "  for (long long kt = SG_K_BEGIN + (long long)blockIdx.x * " << (fusedk ? "SG_WR" : std::to_string(WT))
+                << "; kt < SG_K_END; kt += (long long)gridDim.x * " << (fusedk ? "SG_WR" : std::to_string(WT)) << ") {\n"
+                << "    const int Wtt = (int)min((long long)" << (fusedk ? "SG_WR" : std::to_string(WT)) << ", SG_K_END - kt);\n";
             if (fusedk)
                 src << "    const long long k0 = kt;\n    const int Wt = Wtt;\n" << body << "  }\n}\n";
             else
@@ -2648,7 +2650,7 @@ private:
             }
             if (prefetch_) {
                 pb << "  int sg_pm[" << std::max<size_t>(1, ins_.size()) << "];  // staging misalignment (items) per input\n";
-                emit_issue(pb, "SG_K_BEGIN + (long long)blockIdx.x * " + std::to_string(W), true);
+                emit_issue(pb, "SG_K_BEGIN + (long long)blockIdx.x * SG_WR", true);
             }
             prologue_ = pb.str();
         }
@@ -2959,7 +2961,7 @@ private:
         b << "    { // issue loads of the tile at " << kexpr << (staging ? " into the staging region" : "") << "\n"
           << "      const long long kn = " << kexpr << ";\n"
           << "      if (kn < SG_K_END) {\n"
-          << "        const int Wn = (int)min((long long)" << W_ << ", SG_K_END - kn);\n";
+          << "        const int Wn = (int)min((long long)SG_WR, SG_K_END - kn);\n";
         for (size_t i = 0; i < ins_.size(); i++) {
             int e = ins_[i];
             int64_t lo, ex;
@@ -3028,7 +3030,7 @@ private:
                       << "    }\n";
                 }
                 b << "    __syncthreads();\n";
-                emit_issue(b, "kt + (long long)gridDim.x * " + std::to_string(W_), true);
+                emit_issue(b, "kt + (long long)gridDim.x * SG_WR", true);
             } else {
                 emit_issue(b, "k0", false);
                 b << "    sg_cp_async_wait_all();\n    __syncthreads();\n";

@@ -304,12 +304,48 @@ int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int
                              (unsigned)ki.smem_sync, (CUstream)stream, params, nullptr));
         return 1;
     }
-    int64_t launches = 0;
-    if (ki.mode == 2 && !ki.name_start.empty() && kb < ki.ksafe && !std::getenv("SG_SERIAL_START")) {
-        int64_t ks = std::min(ke, kb + ((ki.ksafe - kb + ki.tile - 1) / ki.tile) * ki.tile);
-        if (ks < ke) {
-            // stream-start tiles (guarded variant) on a side stream beside the steady-state kernel, which
-            // leaves them their CTA slots: the start tiles no longer run alone before the main launch
+    if (ki.mode != 2) {  // register / bitslice / feedback-loop kernels
+        int64_t tiles = (ke - kb + ki.tile - 1) / ki.tile;
+        int64_t grid = std::min<int64_t>(tiles, (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev]);
+        void* params[] = {v.data()};
+        SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
+                             (CUstream)stream, params, nullptr));
+        return 1;
+    }
+    // staged kernels take [.., kb, ke, WR]: WR = iterations per tile for this launch (<= the compiled tile)
+    v.push_back(ki.tile);
+    const size_t IKB = v.size() - 3, IKE = v.size() - 2, IWR = v.size() - 1;
+    const int64_t slots = (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev];
+    // steady-state launch over [a, b) on `st` with `cap` CTA slots: fused kernels get a runtime tile that
+    // makes every CTA process the same number of tiles (no straggler wave)
+    auto main_launch = [&](int64_t a, int64_t b, cudaStream_t st, int64_t cap) {
+        std::vector<int64_t> w = v;
+        w[IKB] = a;
+        w[IKE] = b;
+        int64_t wr = ki.tile;
+        const int64_t cnt = b - a;
+        if (ki.fused && !std::getenv("SG_NO_RT_TILE")) {
+            const int64_t rounds = (cnt + cap * ki.tile - 1) / (cap * ki.tile);
+            const int64_t even = (cnt + rounds * cap - 1) / (rounds * cap);
+            if (even >= (ki.tile * 3) / 4 || rounds >= 4) wr = std::max<int64_t>(1, std::min<int64_t>(ki.tile, even));
+        }
+        w[IWR] = wr;
+        const int64_t tiles = (cnt + wr - 1) / wr;
+        const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, cap));
+        void* params[] = {w.data()};
+        SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
+                             (CUstream)st, params, nullptr));
+    };
+    if (!ki.name_start.empty() && kb < ki.ksafe) {
+        // stream-start tiles (firings g < 0 must emit zeros): the guarded variant, compiled-tile sized
+        const int64_t ks = std::min(ke, kb + ((ki.ksafe - kb + ki.tile - 1) / ki.tile) * ki.tile);
+        const int64_t st_tiles = (ks - kb + ki.tile - 1) / ki.tile;
+        std::vector<int64_t> v2 = v;
+        v2[IKE] = ks;
+        void* p2[] = {v2.data()};
+        if (ks < ke && !std::getenv("SG_SERIAL_START")) {
+            // on a side stream beside the steady-state kernel, which leaves them their CTA slots:
+            // the start tiles no longer run alone before the main launch
             if ((int)ck.aux.size() <= dev) {
                 ck.aux.resize(dev + 1, nullptr);
                 ck.ev_fork.resize(dev + 1, nullptr);
@@ -320,46 +356,23 @@ int64_t launch(CompiledKernel& ck, int dev, const IoBinding& io, int64_t kb, int
                 SG_RT(cudaEventCreateWithFlags(&ck.ev_fork[dev], cudaEventDisableTiming));
                 SG_RT(cudaEventCreateWithFlags(&ck.ev_join[dev], cudaEventDisableTiming));
             }
-            const int64_t st_tiles = (ks - kb + ki.tile - 1) / ki.tile;
-            std::vector<int64_t> v2 = v;
-            v2[v2.size() - 1] = ks;
             SG_RT(cudaEventRecord(ck.ev_fork[dev], stream));
             SG_RT(cudaStreamWaitEvent(ck.aux[dev], ck.ev_fork[dev], 0));
-            void* p2[] = {v2.data()};
             SG_CU(cuLaunchKernel(ck.fn_sync[dev], (unsigned)st_tiles, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
                                  (CUstream)ck.aux[dev], p2, nullptr));
             SG_RT(cudaEventRecord(ck.ev_join[dev], ck.aux[dev]));
-            v[v.size() - 2] = ks;
-            const int64_t tiles = (ke - ks + ki.tile - 1) / ki.tile;
-            const int64_t slots = (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev];
-            const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(tiles, slots - std::min<int64_t>(st_tiles, slots / 2)));
-            void* p1[] = {v.data()};
-            SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
-                                 (CUstream)stream, p1, nullptr));
+            main_launch(ks, ke, stream, std::max<int64_t>(1, slots - std::min<int64_t>(st_tiles, slots / 2)));
             SG_RT(cudaStreamWaitEvent(stream, ck.ev_join[dev], 0));
             return 2;
         }
+        SG_CU(cuLaunchKernel(ck.fn_sync[dev], (unsigned)st_tiles, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
+                             (CUstream)stream, p2, nullptr));
+        if (ke <= ks) return 1;
+        main_launch(ks, ke, stream, slots);
+        return 2;
     }
-    if (ki.mode == 2 && !ki.name_start.empty() && kb < ki.ksafe) {
-        // stream-start tiles (firings g < 0 must emit zeros): the guarded variant
-        int64_t ks = std::min(ke, kb + ((ki.ksafe - kb + ki.tile - 1) / ki.tile) * ki.tile);
-        std::vector<int64_t> v2 = v;
-        v2[v2.size() - 1] = ks;
-        int64_t tiles = (ks - kb + ki.tile - 1) / ki.tile;
-        void* params[] = {v2.data()};
-        SG_CU(cuLaunchKernel(ck.fn_sync[dev], (unsigned)tiles, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
-                             (CUstream)stream, params, nullptr));
-        launches++;
-        kb = ks;
-        v[v.size() - 2] = kb;
-        if (ke <= kb) return launches;
-    }
-    int64_t tiles = (ke - kb + ki.tile - 1) / ki.tile;
-    int64_t grid = std::min<int64_t>(tiles, (int64_t)sm_count(dev) * ck.max_blocks_per_sm[dev]);
-    void* params[] = {v.data()};
-    SG_CU(cuLaunchKernel(ck.fn[dev], (unsigned)grid, 1, 1, (unsigned)ki.threads, 1, 1, (unsigned)ki.smem,
-                         (CUstream)stream, params, nullptr));
-    return launches + 1;
+    main_launch(kb, ke, stream, slots);
+    return 1;
 }
 }  // namespace
 
