@@ -119,7 +119,10 @@ def cpu_baseline(prog, name, target_s=10.0):
     O.run(prog, x, n0)
     rate = n0 / max(1e-6, time.perf_counter() - t)
     n = int(min(n_total, max(n0, rate * target_s)))
-    x = inputs.make_input(prog.dtype, O.in_items(prog, n), inputs.SEEDS[name])
+    # input long enough for n iterations without bisecting in_items(n) over whole-program runs:
+    # in_items(k * n0) <= k * in_items(n0) (per-iteration input plus one peek halo); extra input is unread
+    reps = -(-n // n0)
+    x = inputs.make_input(prog.dtype, reps * O.in_items(prog, n0), inputs.SEEDS[name])
     t = time.perf_counter()
     O.run(prog, x, n)
     dt = time.perf_counter() - t
