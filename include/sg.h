@@ -164,7 +164,9 @@ typedef struct sg_plan_opts {
                                       GPUs, each holding the whole graph mapped by the ILP onto its G/R GPUs,
                                       fragments dealt round-robin to the groups; -1 = R chosen by the cost
                                       model max(Tmax(G/R)/R, input / output distribution over NVLink).
-                                      sg_comm_init / sg_run_rank support R = 1 only (SG_E_UNSUPPORTED). */
+                                      With sg_comm_init / sg_run_rank, rank g * (G/R) + l is GPU l of group
+                                      g and runs fragments f with f % R == g; output fragments land on the
+                                      output rank of their group (gathering them is the caller's). */
 } sg_plan_opts;
 
 typedef struct sg_plan_info_s {

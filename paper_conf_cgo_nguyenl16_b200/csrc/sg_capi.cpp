@@ -331,7 +331,7 @@ sg_status sg_run_rank(sg_plan_t* p, const void* input, int64_t n, void* output, 
 }
 
 int64_t sg_rank_schedule(const sg_plan_t* p, int32_t rank, int64_t n, sg_rank_op* ops, int64_t cap) {
-    if (!p || n < 0 || rank < 0 || rank >= p->plan.G || p->plan.R != 1) return -1;
+    if (!p || n < 0 || rank < 0 || rank >= p->plan.G) return -1;
     try {
         auto v = sg::rank_schedule(p->plan, rank, n, sg::fragment_size(p->plan, std::max<int64_t>(n, 1)));
         for (int64_t i = 0; i < (int64_t)v.size() && i < cap; i++) {

@@ -91,6 +91,9 @@ std::vector<RankOp> rank_schedule(const Plan& p, int rank, int64_t n, int64_t F)
     std::vector<RankOp> ops;
     if (n <= 0) return ops;
     const int64_t nfrag = (n + F - 1) / F;
+    // replica groups: rank = group * Gs + local GPU; the group handles fragments f with f % R == group
+    const int grp = rank / p.Gs, base = grp * p.Gs;
+    rank %= p.Gs;
     std::vector<int> cut;
     for (int e = 0; e < (int)p.flat.edges.size(); e++) {
         const Edge& ed = p.flat.edges[e];
@@ -108,7 +111,8 @@ std::vector<RankOp> rank_schedule(const Plan& p, int rank, int64_t n, int64_t F)
         for (int e : cut) {
             const Edge& ed = p.flat.edges[e];
             if (p.part_gpu[p.node_part[ed.dst]] == rank)
-                ops.push_back({SG_OP_RECV, p.node_part[ed.dst], e, p.part_gpu[p.node_part[ed.src]], f, ka, kb, window(e, ka, kb)});
+                ops.push_back({SG_OP_RECV, p.node_part[ed.dst], e, base + p.part_gpu[p.node_part[ed.src]], f, ka, kb,
+                               window(e, ka, kb)});
         }
     };
     auto sends = [&](int64_t f) {
@@ -116,15 +120,16 @@ std::vector<RankOp> rank_schedule(const Plan& p, int rank, int64_t n, int64_t F)
         for (int e : cut) {
             const Edge& ed = p.flat.edges[e];
             if (p.part_gpu[p.node_part[ed.src]] == rank)
-                ops.push_back({SG_OP_SEND, p.node_part[ed.src], e, p.part_gpu[p.node_part[ed.dst]], f, ka, kb, window(e, ka, kb)});
+                ops.push_back({SG_OP_SEND, p.node_part[ed.src], e, base + p.part_gpu[p.node_part[ed.dst]], f, ka, kb,
+                               window(e, ka, kb)});
         }
     };
-    recvs(0);
-    for (int64_t f = 0; f < nfrag; f++) {
+    if (grp < nfrag) recvs(grp);
+    for (int64_t f = grp; f < nfrag; f += p.R) {
         int64_t ka = f * F, kb = std::min(n, ka + F);
         for (int q : p.part_order)
-            if (p.part_gpu[q] == rank) ops.push_back({SG_OP_LAUNCH, q, -1, rank, f, ka, kb, 0});
-        if (f + 1 < nfrag) recvs(f + 1);
+            if (p.part_gpu[q] == rank) ops.push_back({SG_OP_LAUNCH, q, -1, base + rank, f, ka, kb, 0});
+        if (f + p.R < nfrag) recvs(f + p.R);
         sends(f);
     }
     return ops;
@@ -148,7 +153,6 @@ int64_t fragment_size(const Plan& p, int64_t n) {
 
 void Plan::comm_init(int nranks, int rank, const uint8_t id[128], int device) {
     if (nranks != G) throw Error(SG_E_ARG, "world size must equal the plan's n_gpus");
-    if (R != 1) throw Error(SG_E_UNSUPPORTED, "sg_run_rank supports the pipeline mapping only (replicas = 1)");
     if (rank < 0 || rank >= nranks) throw Error(SG_E_ARG, "bad rank");
     SG_RT2(cudaSetDevice(device));
     ncclUniqueId uid;
@@ -163,7 +167,7 @@ void Plan::comm_init(int nranks, int rank, const uint8_t id[128], int device) {
 void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
     if (!comm) throw Error(SG_E_COMM, "sg_comm_init was not called");
     if (n <= 0) return;
-    const int me = comm_rank, dev = comm_device;
+    const int me = comm_rank % Gs, dev = comm_device;  // this rank's GPU inside its replica group
     SG_RT2(cudaSetDevice(dev));
     const int64_t F = fragment_size(*this, n);
     const int D = ring_depth;
@@ -197,14 +201,15 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
         dist_F = F;
         dist_ready = true;
     }
-    auto EV = [&](int e, int kind, int64_t f) { return dist_ev[e][kind * D + (int)(f % D)]; };
-    auto SLOT = [&](int e, int64_t f) { return dist_slots[e][(int)(f % D)]; };
+    // slots cycle over this group's fragments (f = group + R * j)
+    auto EV = [&](int e, int kind, int64_t f) { return dist_ev[e][kind * D + (int)((f / R) % D)]; };
+    auto SLOT = [&](int e, int64_t f) { return dist_slots[e][(int)((f / R) % D)]; };
     SG_RT2(cudaEventRecord(dist_join, user));
     SG_RT2(cudaStreamWaitEvent(dist_compute, dist_join, 0));
     SG_RT2(cudaStreamWaitEvent(dist_comm, dist_join, 0));
     const int64_t n_in = flat.input_items(n);
     last_launches = 0;
-    std::vector<RankOp> ops = rank_schedule(*this, me, n, F);
+    std::vector<RankOp> ops = rank_schedule(*this, comm_rank, n, F);
     for (size_t p = 0; p < parts.size(); p++)  // this rank's feedback loops restart from their enqueued items
         if (part_gpu[p] == me && kernels[p].ki.state_words > 0) reset_state(kernels[p], dev, dist_compute);
     size_t i = 0;
@@ -241,7 +246,7 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
                 int64_t lo, ex;
                 edge_window(flat, e, lo, ex);
                 bool remote = part_gpu[node_part[ed.dst]] != me;
-                if (o.frag >= D) SG_RT2(cudaStreamWaitEvent(dist_compute, EV(e, remote ? 3 : 1, o.frag), 0));
+                if (o.frag / R >= D) SG_RT2(cudaStreamWaitEvent(dist_compute, EV(e, remote ? 3 : 1, o.frag), 0));
                 io.out.push_back(SLOT(e, o.frag));
                 io.out_base.push_back(o.kb * ed.per_iter + lo);
             }
@@ -258,7 +263,7 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
         while (j < ops.size() && ops[j].op == o.op && ops[j].frag == o.frag) j++;
         for (size_t k = i; k < j; k++) {
             const RankOp& c = ops[k];
-            if (c.op == SG_OP_RECV && c.frag >= D) SG_RT2(cudaStreamWaitEvent(dist_comm, EV(c.edge, 1, c.frag), 0));
+            if (c.op == SG_OP_RECV && c.frag / R >= D) SG_RT2(cudaStreamWaitEvent(dist_comm, EV(c.edge, 1, c.frag), 0));
             if (c.op == SG_OP_SEND) SG_RT2(cudaStreamWaitEvent(dist_comm, EV(c.edge, 2, c.frag), 0));
         }
         SG_NC(nccl().gstart());

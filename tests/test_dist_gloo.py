@@ -27,7 +27,7 @@ def _free_port():
     return port
 
 
-def _worker(rank, world, port, name, n, frag, q):
+def _worker(rank, world, port, name, n, frag, q, replicas=1):
     import sys
     sys.path.insert(0, ROOT)
     try:
@@ -37,10 +37,15 @@ def _worker(rank, world, port, name, n, frag, q):
         from paper_conf_cgo_nguyenl16_b200.dist import max_over_ranks, replica_shard
         prog = {"filterbank8": lambda: apps.filterbank(8), "fmradio4": lambda: apps.fmradio(5),
                 "beamformer": lambda: apps.beamformer(channels=3, beams=2, frame=64, taps=8, mf_taps=16)}[name]()
-        with sg.plan(prog, world, iters_per_fragment=frag) as p:
+        with sg.plan(prog, world, iters_per_fragment=frag, replicas=replicas, plan_only=1) as p:
             info = p.info()
+            R = info["replicas"]
+            Gs = world // R
+            grp = rank // Gs
             ops = p.rank_schedule(rank, n)
-            mine = [q_ for q_, g in enumerate(info["partition_gpu"]) if g == rank]
+            mine = [q_ for q_, g in enumerate(info["partition_gpu"]) if g == rank % Gs]
+            for o in ops:                                            # peers stay inside the replica group
+                assert o["peer"] // Gs == grp
             launched = {}
             sent = recv = 0
             for o in ops:
@@ -61,11 +66,9 @@ def _worker(rank, world, port, name, n, frag, q):
                     assert int(t[-1]) == o["items"]                  # same size on both sides
                     recv += 1
             nfrag = (n + frag - 1) // frag
+            want = [(f * frag, min(n, (f + 1) * frag)) for f in range(grp, nfrag, R)]   # this group's fragments
             for part in mine:                                        # every fragment of every partition
-                spans = sorted(launched.get(part, []))
-                assert len(spans) == nfrag
-                assert spans[0][0] == 0 and spans[-1][1] == n
-                assert all(spans[i][1] == spans[i + 1][0] for i in range(nfrag - 1))
+                assert sorted(launched.get(part, [])) == want
             k0, k1 = replica_shard(1000, rank, world)
             tot = torch.tensor([k1 - k0])
             dist.all_reduce(tot)
@@ -79,13 +82,15 @@ def _worker(rank, world, port, name, n, frag, q):
         q.put((rank, "fail", traceback.format_exc()))
 
 
-@pytest.mark.parametrize("name,n,frag", [("filterbank8", 5000, 700), ("fmradio4", 3000, 512), ("beamformer", 40, 7)])
-def test_rank_schedules_match_over_gloo(name, n, frag):
-    world = 2
+@pytest.mark.parametrize("name,n,frag,world,replicas", [
+    ("filterbank8", 5000, 700, 2, 1), ("fmradio4", 3000, 512, 2, 1), ("beamformer", 40, 7, 2, 1),
+    # hybrid replica x pipeline plans: two groups
+    ("filterbank8", 5000, 300, 2, 2), ("fmradio4", 3000, 256, 4, 2)])
+def test_rank_schedules_match_over_gloo(name, n, frag, world, replicas):
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, name, n, frag, q)) for r in range(world)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, name, n, frag, q, replicas)) for r in range(world)]
     for p in procs:
         p.start()
     results = [q.get(timeout=240) for _ in range(world)]
