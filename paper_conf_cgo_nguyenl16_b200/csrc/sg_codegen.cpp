@@ -474,10 +474,15 @@ public:
         RIN_S_ = row_stride(PIN_);
         ROUT_S_ = row_stride(POUT_);
         body_.str("");
-        emit_body();
+        // wide rows with one dependence component (2-D DCT): node-order emission keeps every
+        // intermediate of the iteration live at once (spills); emit output groups on demand instead
+        demand_ = !std::getenv("SG_NO_DEMAND") && PIN_ + POUT_ >= 384 && n_components() == 1;
+        if (demand_) emit_body_demand();
+        else emit_body();
         const std::string VT4 = T_ == "float" ? "float4" : "int4";
         std::ostringstream src;
-        src << header("register") << consts_.str() << args_struct();
+        src << header(demand_ ? "register, demand-ordered" : "register") << consts_.str() << args_struct();
+        if (demand_) src << "#define SG_LDV(r) (*(volatile const " << T_ << "*)&SG_LD1(r))\n";
         // ---------------- variant 1: synchronous tiles (any alignment / row size)
         int bytes_per_thread = (int)((RIN_S_ + ROUT_S_) * 4);
         int NT = opt.threads;
@@ -745,6 +750,100 @@ private:
         return dval(o, e, pos);
     }
     int64_t rel_ilo_ = 0;
+    // number of output components (outputs sharing no input item are in different components)
+    int n_components() {
+        std::vector<Bits> oc(POUT_);
+        for (int64_t p = 0; p < POUT_; p++) oc[p] = cone_of(eout_, off_out_ + p);
+        std::vector<int> par(POUT_);
+        std::iota(par.begin(), par.end(), 0);
+        std::function<int(int)> find = [&](int x) { return par[x] == x ? x : par[x] = find(par[x]); };
+        for (int64_t q = 0; q < PIN_; q++) {
+            int first = -1;
+            for (int64_t p = 0; p < POUT_; p++)
+                if (oc[p][q / 64] >> (q % 64) & 1) {
+                    if (first < 0) first = (int)p;
+                    else par[find((int)p)] = find(first);
+                }
+        }
+        std::set<int> roots;
+        for (int64_t p = 0; p < POUT_; p++) roots.insert(find((int)p));
+        return (int)roots.size();
+    }
+    // ---- demand-ordered body: output groups in an order that reuses intermediates (greedy over the
+    // sets of firings they need), each group's values computed on demand (memoized firings), inputs
+    // re-read from the shared-memory row at every use (volatile: no long input live ranges)
+    bool demand_ = false;
+    std::map<std::pair<int, int64_t>, std::vector<std::string>> dm_;
+    std::string dv(int e, int64_t pos) {
+        Ref r = R_.resolve(e, Lin::k(pos));
+        if (r.k == Ref::ZERO) return "(" + T_ + ")0";
+        if (r.k != Ref::PHYS || !r.pos.is_const()) throw Error(SG_E_UNSUPPORTED, "internal: dynamic ref in register mode");
+        if (r.edge == ein_) {
+            const int64_t q = r.pos.c - off_in_;
+            if (q < 0 || q >= PIN_) throw Error(SG_E_UNSUPPORTED, "internal: register-mode input out of row");
+            return "SG_LDV(" + std::to_string(q) + ")";
+        }
+        const Edge& ed = f_.edges[r.edge];
+        const int u = ed.src;
+        const Node& n = f_.nodes[u];
+        const int64_t q = r.pos.c - ed.pre, g = q / n.push, j = q % n.push;
+        auto key = std::make_pair(u, g);
+        auto it = dm_.find(key);
+        if (it != dm_.end()) return it->second[j];
+        std::vector<std::string> xs(n.peek);
+        for (int64_t i = 0; i < n.peek; i++) xs[i] = dv(n.in[0], g * n.pop + i);
+        std::vector<std::string> ys(n.push);
+        body_ << "      " << T_ << " ";
+        for (int64_t jj = 0; jj < n.push; jj++) {
+            ys[jj] = "v" + std::to_string(nv_++);
+            body_ << (jj ? ", " : "") << ys[jj];
+        }
+        body_ << ";\n      { const " << T_ << " x_[" << n.peek << "] = {";
+        for (int64_t i = 0; i < n.peek; i++) body_ << (i ? ", " : "") << xs[i];
+        body_ << "}; " << T_ << " y_[" << n.push << "]; " << work_call(u);
+        for (int64_t jj = 0; jj < n.push; jj++) body_ << " " << ys[jj] << " = y_[" << jj << "];";
+        body_ << " }\n";
+        dm_[key] = ys;
+        return ys[j];
+    }
+    void deps_of(int e, int64_t pos, std::set<std::pair<int, int64_t>>& out) {
+        Ref r = R_.resolve(e, Lin::k(pos));
+        if (r.k == Ref::ZERO || r.edge == ein_) return;
+        const Edge& ed = f_.edges[r.edge];
+        const Node& n = f_.nodes[ed.src];
+        const int64_t g = (r.pos.c - ed.pre) / n.push;
+        if (!out.insert({ed.src, g}).second) return;
+        for (int64_t i = 0; i < n.peek; i++) deps_of(n.in[0], g * n.pop + i, out);
+    }
+    void emit_body_demand() {
+        const int gs = vout_ ? 4 : 1;
+        const int ng = (int)((POUT_ + gs - 1) / gs);
+        std::vector<std::set<std::pair<int, int64_t>>> dep(ng);
+        for (int g = 0; g < ng; g++)
+            for (int64_t p = g * gs; p < std::min<int64_t>(POUT_, (int64_t)(g + 1) * gs); p++) deps_of(eout_, off_out_ + p, dep[g]);
+        std::vector<char> done(ng, 0);
+        int cur = 0;
+        for (int step = 0; step < ng; step++) {
+            done[cur] = 1;
+            std::string v[4];
+            for (int i = 0; i < gs; i++) v[i] = dv(eout_, off_out_ + (int64_t)cur * gs + i);
+            if (vout_)
+                body_ << "      SG_ST4(" << cur << ", make_" << (T_ == "float" ? "float4" : "int4") << "(" << v[0] << ", " << v[1]
+                      << ", " << v[2] << ", " << v[3] << "));\n";
+            else
+                body_ << "      SG_ST1(" << cur << ", " << v[0] << ");\n";
+            int best = -1;
+            size_t bscore = 0;
+            for (int g = 0; g < ng; g++) {
+                if (done[g]) continue;
+                size_t sc = 0;
+                for (auto& k : dep[g]) sc += dep[cur].count(k);
+                if (best < 0 || sc > bscore) { best = g; bscore = sc; }
+            }
+            if (best < 0) break;
+            cur = best;
+        }
+    }
     bool try_inplace(KernelInfo& ki, std::ostringstream& src, const std::string& VT4) {
         if (PIN_ != POUT_ || PIN_ % 4 != 0 || PIN_ * 4 == 128 || RIN_S_ != ROUT_S_) return false;
         // components: union-find over output positions sharing an input item

@@ -1,0 +1,9 @@
+TAG=${TAG:-ab8}
+mkdir -p gpurun_out/$TAG
+one() { tag=$1; cfg=$2; shift 2; env $ENVV timeout 900 python bench.py --config $cfg --steps 300 --no-cpu-baseline "$@" > gpurun_out/$TAG/$cfg.$tag.json 2> gpurun_out/$TAG/$cfg.$tag.err; echo "$cfg $tag $(python -c "import json,sys; d=json.loads(open('gpurun_out/$TAG/$cfg.$tag.json').read().strip().splitlines()[-1]); print('ms %.4f frac %.3f launches %d' % (d['ms_per_step'], d['roofline']['frac'], d['gpu_launches']))" 2>&1 | tail -1)"; }
+timeout 900 python -m pytest tests/test_gpu_parity.py -m gpu -q -k "extra or dct" > gpurun_out/$TAG/pytest.log 2>&1; echo "rc=$?" >> gpurun_out/$TAG/pytest.log
+tail -n 2 gpurun_out/$TAG/pytest.log
+ENVV= one demand dct16
+ENVV="SG_NO_DEMAND=1" one nodemand dct16
+ENVV= one cwr fmradio10
+ENVV= one cwr filterbank64
