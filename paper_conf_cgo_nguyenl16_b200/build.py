@@ -102,7 +102,7 @@ def precompile():
     sys.path.insert(0, os.path.dirname(HERE))
     from workloads import apps
     from paper_conf_cgo_nguyenl16_b200 import sg
-    for name, mk in {**apps.CONFIGS, **apps.EXTRA}.items():
+    for name, mk in {**apps.CONFIGS, **apps.EXTRA, **apps.FEEDBACK}.items():
         prog = mk()
         with sg.plan(prog, 1) as p:
             print(f"[precompile] {name}: {p.info()['n_partitions']} partition(s), modes {p.info()['partition_mode']}")

@@ -214,3 +214,31 @@ def test_hybrid_auto_plan_vs_oracle(oracle_lib, name):
                                 iters_per_fragment=1 if name == "beamformer12x4" else 200)
     assert_parity(prog, y, ref)
     assert info["replicas"] >= 1 and 8 % info["replicas"] == 0
+
+
+def test_des_full_size_sampled(oracle_lib):
+    """DES at the bench size (2^22 blocks, bitsliced, rolled rounds): sampled blocks against the oracle
+    one by one, plus a published known-answer block planted at both ends of the stream."""
+    torch = _torch()
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    prog = apps.des(16)
+    n = 1 << 22
+    x = inputs.make_input("i32", 2 * n, inputs.SEEDS["des16"])
+    kat_p, kat_c = 0x0123456789ABCDEF, 0x85E813540F0AB405      # Grabbe's worked example (default key)
+    for k in (0, n - 1):
+        x[2 * k: 2 * k + 2] = np.array([kat_p >> 32, kat_p & 0xFFFFFFFF], dtype=np.uint32).view(np.int32)
+    with sg.plan(prog, 1) as p:
+        xd = torch.from_numpy(x).cuda()
+        yd = torch.empty_like(xd)
+        p.run(xd, n, yd)
+        torch.cuda.synchronize()
+        y = yd.cpu().numpy()
+    for k in (0, n - 1):
+        u = y[2 * k: 2 * k + 2].view(np.uint32)
+        assert (int(u[0]) << 32 | int(u[1])) == kat_c
+    rng = np.random.default_rng(11)
+    ks = np.sort(rng.choice(n, 300, replace=False))
+    blocks = np.concatenate([x[2 * k: 2 * k + 2] for k in ks])
+    ref = oracle_lib.run(prog, blocks, len(ks))
+    got = np.concatenate([y[2 * k: 2 * k + 2] for k in ks])
+    assert np.array_equal(got, ref)
