@@ -306,7 +306,8 @@ bool register_mode_eligible(const Flat& f, const std::vector<int>& nodes, std::s
         if (ex != 0 || lo != eo.pre + f.nodes[eo.src].ninit * eo.push) return fail("output window misaligned");
     }
     const Edge& ei = f.edges[ins[0]];
-    if (ei.per_iter > 256 || eo.per_iter > 256 || live > 512) return fail("iteration too large for registers");
+    if (ei.per_iter > 512 || eo.per_iter > 256 || ei.per_iter + eo.per_iter > 768 || live > 512)
+        return fail("iteration too large for registers");
     return true;
 }
 
