@@ -484,6 +484,7 @@ public:
         std::ostringstream src;
         src << header(demand_ ? "register, demand-ordered" : "register") << consts_.str() << args_struct();
         if (demand_) src << "#define SG_LDV(r) (*(volatile const " << T_ << "*)&SG_LD1(r))\n";
+        if (demand_) return run_demand(ki, src, VT4, opt);
         // ---------------- variant 1: synchronous tiles (any alignment / row size)
         int bytes_per_thread = (int)((RIN_S_ + ROUT_S_) * 4);
         int NT = opt.threads;
@@ -751,6 +752,59 @@ private:
         return dval(o, e, pos);
     }
     int64_t rel_ilo_ = 0;
+    // Demand-ordered kernels keep only the input rows in shared memory (re-read many times) and store
+    // each output group straight to global memory from registers: half the shared memory per row, so
+    // twice the warps per SM of the staged-row variants; no TMA (the rows are consumed out of order).
+    KernelInfo run_demand(KernelInfo& ki, std::ostringstream& src, const std::string& VT4, const CodegenOpts& opt) {
+        const int bytes_per_thread = (int)(RIN_S_ * 4);
+        int NT = opt.threads;
+        if (NT <= 0) {
+            NT = 256;
+            while (NT > 32 && (size_t)NT * bytes_per_thread > 100 * 1024) NT /= 2;
+        }
+        const size_t smem = (size_t)NT * bytes_per_thread;
+        const int minb = std::max(1, std::min(8, (int)((220 * 1024) / std::max<size_t>(1, smem))));
+        src << "#define SG_LD4(g) (reinterpret_cast<const " << VT4 << "*>(xr)[g])\n"
+            << "#define SG_LD1(r) (xr[r])\n"
+            << "#define SG_ST4(g, v) do { const " << VT4 << " t_ = (v); if (ga) reinterpret_cast<" << VT4
+            << "*>(yg)[g] = t_; else { yg[4 * (g)] = t_.x; yg[4 * (g) + 1] = t_.y; yg[4 * (g) + 2] = t_.z; yg[4 * (g) + 3] = t_.w; } } while (0)\n"
+            << "#define SG_ST1(g, v) (yg[g] = (v))\n";
+        src << "extern \"C\" __global__ void __launch_bounds__(" << NT << ", " << minb << ") " << ki.name_sync
+            << "(const SgArgs a) {\n"
+            << "  constexpr int NT = " << NT << ";\n"
+            << "  extern __shared__ __align__(16) unsigned char sg_smem[];\n"
+            << "  " << T_ << "* s_in = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
+            << "  const " << T_ << "* gin = SG_IN(0);\n"
+            << "  " << T_ << "* gout = SG_OUT(0);\n"
+            << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * NT; t0 < SG_K_END; t0 += (long long)gridDim.x * NT) {\n"
+            << "    const int nt = (int)min((long long)NT, SG_K_END - t0);\n"
+            << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
+            << (vin_ ? std::string("    if ((reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0)\n      sg_rows_g2s_v4<") +
+                           T_ + ", " + std::to_string(PIN_) + ", " + std::to_string(RIN_S_) + ", NT>(gsrc, s_in, nt);\n    else\n"
+                     : std::string())
+            << "      sg_rows_g2s_v1<" << T_ << ", " << PIN_ << ", " << RIN_S_ << ", NT>(gsrc, s_in, nt);\n"
+            << "    __syncthreads();\n"
+            << "    " << T_ << "* gdst = gout + (t0 * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
+            << "    const bool ga = " << (vout_ ? "(reinterpret_cast<unsigned long long>(gdst) & 15ull) == 0" : "false") << ";\n"
+            << "    (void)ga;\n"
+            << "    if (threadIdx.x < nt) {\n"
+            << "      const " << T_ << "* xr = s_in + threadIdx.x * " << RIN_S_ << ";\n"
+            << "      " << T_ << "* yg = gdst + (long long)threadIdx.x * " << POUT_ << ";\n"
+            << body_.str()
+            << "    }\n"
+            << "    __syncthreads();  // the next tile's loads reuse the rows\n"
+            << "  }\n}\n"
+            << "#undef SG_LD4\n#undef SG_LD1\n#undef SG_ST4\n#undef SG_ST1\n";
+        ki.has_tma = false;
+        ki.tma_in = ki.tma_out = 0;
+        ki.name = ki.name_sync;
+        ki.threads = ki.threads_sync = NT;
+        ki.tile = ki.tile_sync = NT;
+        ki.smem = ki.smem_sync = smem;
+        ki.min_blocks = 1;
+        ki.source = src.str();
+        return ki;
+    }
     // number of output components (outputs sharing no input item are in different components)
     int n_components() {
         std::vector<Bits> oc(POUT_);
