@@ -55,6 +55,8 @@ void partition_boundary(const Flat& f, const std::vector<int>& nodes, std::vecto
 void edge_window(const Flat& f, int e, int64_t& lo, int64_t& extra);
 
 bool register_mode_eligible(const Flat& f, const std::vector<int>& nodes, std::string* why);
+// all compute filters are bit kinds (INTO_BITS / BITS_TO_INT / XOR / XOR_CONST / SBOX): bitslice mode
+bool bitslice_eligible(const Flat& f, const std::vector<int>& nodes, std::string* why);
 
 KernelInfo generate_kernel(const Flat& f, const std::vector<int>& nodes, int part_id, const CodegenOpts& opt);
 

@@ -65,6 +65,21 @@ PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
         }
     }
     if (est.mode == 1) smem = 0;
+    if (est.mode == 1 && bitslice_eligible(f, nodes, nullptr)) {
+        // bitslice mode: one LOP3 covers 32 iterations; an S-box is a ~44-gate circuit, a word <-> bits
+        // conversion a share of a 32x32 transpose (~5 ops per bit)
+        intops = 0;
+        for (int v : nodes) {
+            const Node& n = f.nodes[v];
+            if (n.type != N_FILTER) continue;
+            switch (n.kind) {
+            case SG_K_XOR: case SG_K_XOR_CONST: intops += (double)n.rep * n.iv[0] / 32.0; break;
+            case SG_K_SBOX: intops += (double)n.rep * 44.0 / 32.0; break;
+            case SG_K_INTO_BITS: case SG_K_BITS_TO_INT: intops += (double)n.rep * 5.0; break;
+            default: break;
+            }
+        }
+    }
     for (int e : ins) smem += 8.0 * f.edges[e].per_iter;
     for (int e : outs) smem += 8.0 * f.edges[e].per_iter;
     double eff = est.mode == 1 ? 0.8 : 0.5;

@@ -18,7 +18,7 @@ sys.path.insert(0, ROOT)
 
 # iterations per measurement: enough work to fill the GPU (>= ~1 ms for the heavy graphs)
 N_ITERS = {"bitonic32": 1 << 20, "fft64": 1 << 18, "fmradio10": 1 << 22, "filterbank64": 1 << 20,
-           "beamformer12x4": 1024}
+           "beamformer12x4": 1024, "des16": 1 << 22, "bitonicrec32": 1 << 20, "dct16": 1 << 18, "matmul16": 1 << 18}
 
 
 def r2(xs, ys):
@@ -42,7 +42,7 @@ def main():
     assert torch.cuda.is_available()
     rows = []
     for name in args.configs.split(","):
-        prog = apps.CONFIGS[name]()
+        prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
         for G in [int(g) for g in args.gpus.split(",")]:
             with sg.plan(prog, G, devices=[0] * G) as p:
                 info = p.info()
