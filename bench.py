@@ -42,6 +42,8 @@ WORKLOADS = {
     "bitonicrec32": dict(n=1 << 20, bound="hbm", desc="recursive BitonicSort 32-key int32, 1M iterations"),
     "dct16": dict(n=1 << 18, bound="hbm", desc="2-D DCT-II of 16x16 fp32 blocks (row then column FIR DCTs)"),
     "matmul16": dict(n=1 << 18, bound="hbm", desc="C = A B of streamed 16x16 fp32 matrices (MULTIPLY, ADD)"),
+    # feedback loops: the comb loop is a sequential (wavefront) partition between two FIRs
+    "echo64": dict(n=1 << 22, bound="alu", desc="echo: FIR -> feedback loop y = x + 0.5 y[n-64] -> decimating FIR, fp32"),
     "des16": dict(n=1 << 22, bound="int", desc="DES (16 rounds) on a bit-per-item int32 stream, one 64-bit block / iteration"),
 }
 
@@ -137,7 +139,7 @@ def run_reference(args):
         return 0
     from workloads import apps
     name = args.config
-    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
+    prog = {**apps.CONFIGS, **apps.EXTRA, **apps.FEEDBACK}[name]()
     vals = []
     cb = None
     for _ in range(max(1, args.warmup)):
@@ -196,7 +198,7 @@ def main():
     name = args.config
     W = WORKLOADS[name]
     n = args.iters or W["n"]
-    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
+    prog = {**apps.CONFIGS, **apps.EXTRA, **apps.FEEDBACK}[name]()
     pipeline = args.mode == "pipeline" and world > 1
     if pipeline:
         from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan
@@ -369,11 +371,14 @@ def main():
 
 def _flops_per_iter(prog, reps):
     """Algorithmic fp32 flops per iteration as written (FMA = 2): program text x repetition vector."""
-    from workloads.spec import Filter, Pipeline
+    from workloads.spec import FeedbackLoop, Filter, Pipeline
     k = [0]
     tot = [0]
 
     def walk(s):
+        if isinstance(s, FeedbackLoop):   # one N_LOOP node in the product's flat graph (its work not counted)
+            k[0] += 1
+            return
         if isinstance(s, Filter):
             rep = reps[k[0]]
             k[0] += 1
