@@ -477,7 +477,8 @@ public:
         body_.str("");
         // wide rows with one dependence component (2-D DCT): node-order emission keeps every
         // intermediate of the iteration live at once (spills); emit output groups on demand instead
-        demand_ = !std::getenv("SG_NO_DEMAND") && PIN_ + POUT_ >= 384 && n_components() == 1;
+        static const int64_t dmin = std::getenv("SG_DEMAND_MIN") ? std::atoll(std::getenv("SG_DEMAND_MIN")) : 384;
+        demand_ = !std::getenv("SG_NO_DEMAND") && PIN_ + POUT_ >= dmin && n_components() == 1;
         if (demand_) emit_body_demand();
         else emit_body();
         const std::string VT4 = T_ == "float" ? "float4" : "int4";

@@ -490,3 +490,27 @@ def test_feedback_kernel_source(sg):
         q = i["partition_mode"].index(4)
         src = p.source(q)
         assert "(feedback loop mode)" in src and "SG_STATE" in src and "sg_work_amplify" in src
+
+
+def test_demand_ordered_register_kernels(sg):
+    """Wide single-component rows (2-D DCT, MatMul): demand-ordered register kernels -- inputs re-read
+    (volatile) from the shared-memory row, outputs stored straight to global memory, no TMA variant;
+    FFT (two independent 64-point components) keeps the in-place component kernel.  The row-width
+    threshold (384 items) is lowered so small shapes compile quickly (read once per process: run in a
+    subprocess)."""
+    import subprocess
+    import sys
+    code = ("import sys; sys.path.insert(0, %r)\n"
+            "from paper_conf_cgo_nguyenl16_b200 import sg\nfrom workloads import apps\n"
+            "for prog in (apps.dct2d(8), apps.matmul(8, 8, 8)):\n"
+            "    with sg.plan(prog, 1) as p:\n"
+            "        src = p.source(0)\n"
+            "        assert p.info()['partition_mode'] == [1]\n"
+            "        assert '(register, demand-ordered mode)' in src and 'SG_LDV(' in src and 'sg_tma' not in src\n"
+            "print('ok')\n") % ROOT
+    env = dict(os.environ, SG_DEMAND_MIN="100")
+    r = subprocess.run([sys.executable, "-c", code], env=env, capture_output=True, text=True, timeout=600)
+    assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-2000:]
+    with sg.plan(apps.fft(64), 1) as p:
+        src = p.source(0)
+        assert "demand-ordered" not in src and "sg_bulk_g2s" in src
