@@ -173,6 +173,8 @@ def main():
     ap.add_argument("--eager", action="store_true", help="launch sg_run every step instead of replaying a CUDA graph")
     ap.add_argument("--tile", type=int, default=0, help="plan option tile_iters (0: chosen by the code generator)")
     ap.add_argument("--threads", type=int, default=0, help="plan option threads per CTA (0: chosen)")
+    ap.add_argument("--replicas", type=int, default=1,
+                    help="--mode pipeline: replica groups (hybrid replica x pipeline plan); -1 = chosen by the cost model")
     ap.add_argument("--codegen", default="auto", choices=["auto", "register", "staged", "general"],
                     help="plan option codegen_mode (auto: chosen by the code generator)")
     ap.add_argument("--mode", default="replicas", choices=["replicas", "pipeline"],
@@ -202,7 +204,7 @@ def main():
     pipeline = args.mode == "pipeline" and world > 1
     if pipeline:
         from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan
-        plan = pipeline_plan(prog)
+        plan = pipeline_plan(prog, replicas=args.replicas)
     else:
         kw = {}
         if args.tile:
