@@ -365,7 +365,9 @@ protected:
             auto tw = twiddles(n.iv[0]);
             return "sg_work_combine_dft<" + std::to_string(n.iv[0]) + ">(x_, y_, " + tw.first + ", " + tw.second + ");";
         }
-        case SG_K_FM_DEMOD: return "sg_work_fm_demod(x_, y_, " + hexf(n.fv[0]) + ");";
+        case SG_K_FM_DEMOD:
+            return std::string(std::getenv("SG_FM_F32") ? "sg_work_fm_demod_f32" : "sg_work_fm_demod") + "(x_, y_, " +
+                   hexf(n.fv[0]) + ");";
         case SG_K_SUBTRACT: return "sg_work_subtract(x_, y_);";
         case SG_K_AMPLIFY: return "sg_work_amplify(x_, y_, " + hexf(n.fv[0]) + ");";
         case SG_K_ADD: return "sg_work_add<" + std::to_string(n.iv[0]) + ">(x_, y_);";

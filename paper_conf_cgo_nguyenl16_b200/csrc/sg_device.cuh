@@ -89,6 +89,12 @@ SG_DEV void sg_work_fm_demod(const float (&x)[2], float (&y)[1], float gain) {
     y[0] = (float)((double)gain * atan((double)p));
 }
 
+// fp32 variant (SG_FM_F32=1 at plan time): atanf (<= 2 ulp), within the fp32 tolerance, not bit-exact
+SG_DEV void sg_work_fm_demod_f32(const float (&x)[2], float (&y)[1], float gain) {
+    const float p = x[0] * x[1];
+    y[0] = gain * atanf(p);
+}
+
 SG_DEV void sg_work_subtract(const float (&x)[2], float (&y)[1]) { y[0] = x[1] - x[0]; }
 
 SG_DEV void sg_work_amplify(const float (&x)[1], float (&y)[1], float k) { y[0] = x[0] * k; }
