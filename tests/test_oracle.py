@@ -14,7 +14,8 @@ wrong sign or index, a transposed operand, a wrong rate) fails at least one:
   FIR          direct convolution: exact on small integers, Higham bound otherwise
   FilterBank   multirate identity y = sum_b F_b * up(down(H_b * delay(x))):
                exact on small integers, bounded on the benchmark coefficients
-  FMRadio      components (LPF = convolution, demod closed form, band = hi - lo)
+  FMRadio      components (LPF = convolution, demod closed form, band = hi - lo) and end to end
+               within a rigorous float32 error bound around a float64 evaluation
                and an end-to-end numpy double reference within a loose bound
   BeamFormer   numpy complex convolution / mat-vec / abs per frame
   Kahn         two schedules and three chunk sizes give bit-identical output
@@ -373,6 +374,57 @@ def test_fmradio_end_to_end_loose(oracle_lib):
     y = oracle_lib.run(prog, x, n).astype(np.float64)
     ref = _fmradio_numpy(x, n)
     assert np.linalg.norm(y - ref) / np.linalg.norm(ref) < 2e-3
+
+
+def _fmradio_bound(x, n, bands=11, taps=64, drop_band=None):
+    """FMRadio in float64 plus a rigorous elementwise bound on the float32 evaluation's error (Higham:
+    a length-L FMA dot product is within gamma_L * sum|c||x| of the exact one; the product and the
+    1-Lipschitz atan propagate first-order terms; every later rounding adds a unit roundoff)."""
+    u = 2.0 ** -24
+    gam = lambda k: k * u / (1 - k * u)
+    rate, cutoff = 250e6, 108e6
+    c1 = np.array(apps.lowpass_coeffs(rate, cutoff, taps), np.float64)
+    x = x[:379 + 5 * n].astype(np.float64)
+    X = np.array([x[5 * g:5 * g + taps] for g in range(n + 64)])
+    l1, e1 = X @ c1, gam(taps) * (np.abs(X) @ np.abs(c1))
+    a, b, ea, eb = l1[:-1], l1[1:], e1[:-1], e1[1:]
+    p = a * b
+    ep = np.abs(a) * eb + np.abs(b) * ea + ea * eb + u * (np.abs(p) + np.abs(a) * eb + np.abs(b) * ea + ea * eb)
+    gain = np.float64(np.float32(27000.0 * (rate / (10000.0 * math.pi))))
+    dm = gain * np.arctan(p)
+    edm = gain * ep + 2 * u * np.abs(dm) + 1e-14 * np.abs(dm)
+    cut = [math.exp(i * (math.log(1760.0) - math.log(55.0)) / (bands - 1) + math.log(55.0)) for i in range(bands)]
+    D = np.array([dm[k:k + taps] for k in range(n)])
+    ED = np.array([edm[k:k + taps] for k in range(n)])
+    out, err = np.zeros(n), np.zeros(n)
+    for i in range(1, bands):
+        lo = np.array(apps.lowpass_coeffs(rate, cut[i - 1], taps), np.float64)
+        hi = np.array(apps.lowpass_coeffs(rate, cut[i], taps), np.float64)
+        val = ((i - 1) - (bands - 2) / 2.0) / 5.0
+        g = np.float64(np.float32(2.0 - val if val > 0 else 2.0 + val))
+        band = D @ hi - D @ lo
+        eh = gam(taps) * (np.abs(D) @ np.abs(hi)) + ED @ np.abs(hi)
+        el = gam(taps) * (np.abs(D) @ np.abs(lo)) + ED @ np.abs(lo)
+        eband = eh + el + u * (np.abs(band) + eh + el)
+        if i != drop_band:
+            out += g * band
+        err += g * eband + u * (g * np.abs(band) + g * eband)
+    err += gam(bands - 1) * (np.abs(out) + err)
+    return out, err
+
+
+@pytest.mark.parametrize("variant", ["fmtone", "uniform"])
+def test_fmradio_end_to_end_within_error_bound(oracle_lib, variant):
+    """FMRadio end to end, pinned elementwise by the float32 error bound of _fmradio_bound; the same
+    bound rejects a dropped band (negative control), so the pin is discriminating."""
+    prog = apps.fmradio(11)
+    n = 300
+    x = inputs.make_input("f32", 379 + 5 * n, 0xF3, variant=variant)
+    y = oracle_lib.run(prog, x, n).astype(np.float64)
+    ref, err = _fmradio_bound(x, n)
+    assert np.all(np.abs(y - ref) <= err)
+    bad, _ = _fmradio_bound(x, n, drop_band=5)
+    assert np.sum(np.abs(y - bad) > err) > n // 2
 
 
 # ---------------------------------------------------------------- BeamFormer
