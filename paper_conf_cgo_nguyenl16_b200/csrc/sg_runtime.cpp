@@ -402,6 +402,9 @@ void reset_state(CompiledKernel& ck, int dev, cudaStream_t stream) {
 
 Plan::~Plan() {
     dist_release();
+    for (auto e : host_ev) cudaEventDestroy(e);
+    if (host_in_stream) cudaStreamDestroy(host_in_stream);
+    if (host_out_stream) cudaStreamDestroy(host_out_stream);
     for (auto& r : rings) {
         for (size_t i = 0; i < r.src_slots.size(); i++) {
             if (r.src_slots[i]) { cudaSetDevice(devices[r.src_gpu]); cudaFree(r.src_slots[i]); }
@@ -685,6 +688,52 @@ void Plan::run_host(const void* hin, int64_t n, void* hout) {
         host_out_dev = nullptr;
         SG_RT(cudaMalloc(&host_out_dev, bo));
         host_out_cap = bo;
+    }
+    // one partition (without a feedback loop): chunks of iterations pipelined over three streams, so
+    // the host->device copy of chunk c+1, the kernel on chunk c and the device->host copy of chunk c-1
+    // overlap (PCIe is full duplex; iterations are independent, and chunk c needs exactly the input
+    // prefix input_items(end of c)).  Otherwise: copy in, run, copy out.
+    const int NCH = std::getenv("SG_HOST_CHUNKS") ? std::atoi(std::getenv("SG_HOST_CHUNKS")) : 8;
+    if (parts.size() == 1 && R == 1 && kernels[0].ki.state_words == 0 && NCH > 1 && n >= 4 * NCH) {
+        if (!host_in_stream) {
+            SG_RT(cudaStreamCreateWithFlags(&host_in_stream, cudaStreamNonBlocking));
+            SG_RT(cudaStreamCreateWithFlags(&host_out_stream, cudaStreamNonBlocking));
+        }
+        while ((int)host_ev.size() < 2 * NCH + 1) {
+            cudaEvent_t e;
+            SG_RT(cudaEventCreateWithFlags(&e, cudaEventDisableTiming));
+            host_ev.push_back(e);
+        }
+        CompiledKernel& ck = kernels[0];
+        IoBinding io;
+        io.in = {host_in_dev};
+        io.in_base = {0};
+        io.in_limit = {flat.input_items(n)};
+        io.out = {host_out_dev};
+        io.out_base = {0};
+        reset_state(ck, din, host_stream);
+        last_launches = 0;
+        int64_t copied = 0;
+        for (int c = 0; c < NCH; c++) {
+            const int64_t ka = n * c / NCH, kb = n * (c + 1) / NCH;
+            const int64_t need = flat.input_items(kb);
+            if (need > copied) {
+                SG_RT(cudaMemcpyAsync((char*)host_in_dev + copied * 4, (const char*)hin + copied * 4,
+                                      (size_t)(need - copied) * 4, cudaMemcpyHostToDevice, host_in_stream));
+                copied = need;
+            }
+            SG_RT(cudaEventRecord(host_ev[2 * c], host_in_stream));
+            SG_RT(cudaStreamWaitEvent(host_stream, host_ev[2 * c], 0));
+            last_launches += launch_kernel(ck, din, io, ka, kb, host_stream, flat.dtype == SG_F32);
+            SG_RT(cudaEventRecord(host_ev[2 * c + 1], host_stream));
+            SG_RT(cudaStreamWaitEvent(host_out_stream, host_ev[2 * c + 1], 0));
+            const int64_t o0 = flat.output_items(ka), o1 = flat.output_items(kb);
+            SG_RT(cudaMemcpyAsync((char*)hout + o0 * 4, (const char*)host_out_dev + o0 * 4, (size_t)(o1 - o0) * 4,
+                                  cudaMemcpyDeviceToHost, host_out_stream));
+        }
+        SG_RT(cudaStreamSynchronize(host_out_stream));
+        SG_RT(cudaStreamSynchronize(host_stream));
+        return;
     }
     SG_RT(cudaMemcpyAsync(host_in_dev, hin, bi, cudaMemcpyHostToDevice, host_stream));
     run(host_in_dev, n, host_out_dev, host_stream);

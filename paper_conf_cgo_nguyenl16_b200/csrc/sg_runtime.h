@@ -91,6 +91,8 @@ struct Plan {
     void* host_out_dev = nullptr;
     size_t host_in_cap = 0, host_out_cap = 0;
     cudaStream_t host_stream = nullptr;
+    cudaStream_t host_in_stream = nullptr, host_out_stream = nullptr;  // chunked copy pipeline
+    std::vector<cudaEvent_t> host_ev;
 
     // one process per GPU (sg_dist.cpp)
     void* comm = nullptr;  // ncclComm_t

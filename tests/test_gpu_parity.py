@@ -216,3 +216,20 @@ def test_des_bitslice_misaligned_buffers(oracle_lib):
         torch.cuda.synchronize()
         assert np.array_equal(yb[1:].cpu().numpy(), ref)
         assert int(yb[0]) == -7
+
+
+@pytest.mark.parametrize("name", ["bitonic32", "fmradio10", "filterbank64", "des16", "fft64"])
+def test_run_host_chunked_pipeline(oracle_lib, name):
+    """sg_run_host with host buffers: single-partition plans pipeline chunks of iterations (copy in /
+    kernel / copy out on three streams); every chunk boundary, the stream-start tiles and the input
+    prefix each chunk needs must give the oracle's output."""
+    _torch()
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
+    n = 4099 if name != "filterbank64" else 2051
+    x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), 606)
+    ref = oracle_lib.run(prog, x, n)
+    with sg.plan(prog, 1) as p:
+        y = np.empty(p.output_items(n), dtype=np.int32 if prog.dtype == "i32" else np.float32)
+        p.run_host(x, n, y)
+    assert_parity(prog, y, ref)
