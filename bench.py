@@ -175,6 +175,8 @@ def main():
     ap.add_argument("--threads", type=int, default=0, help="plan option threads per CTA (0: chosen)")
     ap.add_argument("--replicas", type=int, default=1,
                     help="--mode pipeline: replica groups (hybrid replica x pipeline plan); -1 = chosen by the cost model")
+    ap.add_argument("--cuts", default="",
+                    help="comma-separated node ids: user partitions [0, c1), [c1, c2), ... on one GPU (A/B of splits)")
     ap.add_argument("--codegen", default="auto", choices=["auto", "register", "staged", "general"],
                     help="plan option codegen_mode (auto: chosen by the code generator)")
     ap.add_argument("--mode", default="replicas", choices=["replicas", "pipeline"],
@@ -213,6 +215,11 @@ def main():
             kw["threads"] = args.threads
         if args.codegen != "auto":
             kw["codegen_mode"] = args.codegen
+        if args.cuts:
+            cuts = [int(c) for c in args.cuts.split(",")]
+            with sg.plan(prog, 1, plan_only=1) as p0:
+                nn = p0.info()["n_nodes"]
+            kw["node_partition"] = [sum(1 for c in cuts if c <= v) for v in range(nn)]
         plan = sg.plan(prog, 1, devices=[local], **kw)
     info = plan.info()
     nin, nout = plan.input_items(n), plan.output_items(n)
