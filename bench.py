@@ -128,9 +128,24 @@ def cpu_baseline(prog, name, target_s=10.0):
     t = time.perf_counter()
     O.run(prog, x, n)
     dt = time.perf_counter() - t
-    return {"value": n / dt, "unit": "iters/s", "cores": 1, "kind": "oracle",
-            "sample": f"first {n} of {n_total} iterations of {name} (seeded input), sequential C interpreter, "
-                      f"{dt:.1f} s, gcc -O2 -ffp-contract=off"}
+    out = {"value": n / dt, "unit": "iters/s", "cores": 1, "kind": "oracle",
+           "sample": f"first {n} of {n_total} iterations of {name} (seeded input), sequential C interpreter, "
+                     f"{dt:.1f} s, gcc -O2 -ffp-contract=off"}
+    # all host cores: the same interpreter on independent chunks of iterations, one thread per core
+    # (ctypes releases the GIL during the C call); each chunk restarts at a stream start, which changes
+    # peek-halo values but not the work
+    cores = min(os.cpu_count() or 1, 64)
+    if cores > 1 and not os.environ.get("SG_ORACLE_1CORE"):
+        from concurrent.futures import ThreadPoolExecutor
+        nc = max(n0, int(rate * target_s / 2))
+        xc = inputs.make_input(prog.dtype, -(-nc // n0) * O.in_items(prog, n0), inputs.SEEDS[name])
+        t = time.perf_counter()
+        with ThreadPoolExecutor(cores) as ex:
+            list(ex.map(lambda _: O.run(prog, xc, nc), range(cores)))
+        dtc = time.perf_counter() - t
+        out.update({"value": cores * nc / dtc, "cores": cores, "value_1core": n / dt,
+                    "sample": out["sample"] + f"; all cores: {cores} threads x {nc} iterations each, {dtc:.1f} s"})
+    return out
 
 
 def run_reference(args):
