@@ -137,7 +137,8 @@ def cpu_baseline(prog, name, target_s=10.0):
     cores = min(os.cpu_count() or 1, 64)
     if cores > 1 and not os.environ.get("SG_ORACLE_1CORE"):
         from concurrent.futures import ThreadPoolExecutor
-        nc = max(n0, int(rate * target_s / 2))
+        out_per_iter = max(1, len(O.run(prog, x, 1)))
+        nc = max(n0, min(int(rate * target_s / 2), int(1e9 / (cores * 4 * out_per_iter))))  # <= 1 GB of outputs
         xc = inputs.make_input(prog.dtype, -(-nc // n0) * O.in_items(prog, n0), inputs.SEEDS[name])
         t = time.perf_counter()
         with ThreadPoolExecutor(cores) as ex:
