@@ -167,10 +167,25 @@ SG_DEV unsigned sg_lop3(unsigned a, unsigned b, unsigned c) {
     asm("lop3.b32 %0, %1, %2, %3, %4;" : "=r"(d) : "r"(a), "r"(b), "r"(c), "n"(LUT));
     return d;
 }
-// 32x32 bit-matrix transpose in registers: afterwards bit j of a[i] = bit i of the old a[j]
+// 32x32 bit-matrix transpose in registers: afterwards bit j of a[i] = bit i of the old a[j].
+// Stages 16 and 8 swap whole half-words / bytes: one byte permute per output word; stages 4, 2, 1
+// exchange masked bit groups.
 SG_DEV void sg_transpose32(unsigned (&a)[32]) {
 #pragma unroll
-    for (unsigned s = 16, m = 0x0000FFFFu; s > 0; s >>= 1, m ^= m << s) {
+    for (int i = 0; i < 16; i++) {
+        const unsigned x = a[i], y = a[i + 16];
+        a[i] = __byte_perm(x, y, 0x5410);       // [lo16(y) | lo16(x)]
+        a[i + 16] = __byte_perm(x, y, 0x7632);  // [hi16(y) | hi16(x)]
+    }
+#pragma unroll
+    for (int i = 0; i < 32; i++) {
+        if (i & 8) continue;
+        const unsigned x = a[i], y = a[i + 8];
+        a[i] = __byte_perm(x, y, 0x6240);       // bytes (y2, x2, y0, x0)
+        a[i + 8] = __byte_perm(x, y, 0x7351);   // bytes (y3, x3, y1, x1)
+    }
+#pragma unroll
+    for (unsigned s = 4, m = 0x0F0F0F0Fu; s > 0; s >>= 1, m ^= m << s) {
 #pragma unroll
         for (int i = 0; i < 32; i++) {
             if (i & s) continue;
