@@ -514,3 +514,28 @@ def test_demand_ordered_register_kernels(sg):
     with sg.plan(apps.fft(64), 1) as p:
         src = p.source(0)
         assert "demand-ordered" not in src and "sg_bulk_g2s" in src
+
+
+def test_bit_transpose_device_code_on_host(tmp_path):
+    """sg_transpose32 (the bitslice kernels' word <-> bit-plane conversion) compiled for the host from
+    sg_device.cuh, with __byte_perm emulated from its definition: bit j of a[i] must equal bit i of the
+    original a[j] for random matrices."""
+    import subprocess
+    src = open(os.path.join(ROOT, "paper_conf_cgo_nguyenl16_b200", "csrc", "sg_device.cuh")).read()
+    i = src.index("SG_DEV void sg_transpose32")
+    j = src.index("\n}\n", i) + 3
+    prog = ("#include <cstdio>\n#include <cstdlib>\n#define SG_DEV static inline\n"
+            "static unsigned __byte_perm(unsigned x, unsigned y, unsigned s) {\n"
+            "  unsigned long long v = ((unsigned long long)y << 32) | x; unsigned r = 0;\n"
+            "  for (int k = 0; k < 4; k++) r |= (unsigned)((v >> (8 * ((s >> (4 * k)) & 7))) & 0xFF) << (8 * k);\n"
+            "  return r; }\n" + src[i:j] +
+            "int main() { unsigned a[32], b[32]; int bad = 0; srand(7);\n"
+            "  for (int t = 0; t < 50; t++) { for (int i = 0; i < 32; i++) b[i] = a[i] = rand() ^ (rand() << 16);\n"
+            "    sg_transpose32(a);\n"
+            "    for (int i = 0; i < 32; i++) for (int j = 0; j < 32; j++) bad += ((a[i] >> j) & 1) != ((b[j] >> i) & 1); }\n"
+            "  printf(\"%d\\n\", bad); return 0; }\n")
+    c = tmp_path / "tr.cpp"
+    c.write_text(prog)
+    exe = tmp_path / "tr"
+    subprocess.check_call(["g++", "-O1", "-o", str(exe), str(c)])
+    assert subprocess.run([str(exe)], capture_output=True, text=True).stdout.strip() == "0"
