@@ -1776,7 +1776,7 @@ public:
         const std::string T = T_;
         auto pos_ref = [&](int e, int64_t c) -> std::string {  // item at (firing-relative) position c of edge e
             const int64_t per = sf.edges[e].per_iter;
-            if (e == sf.in_edge) return "gin[g * " + std::to_string(li_.P) + "LL + " + std::to_string(c) + "LL - in_base]";
+            if (e == sf.in_edge) return "cur[" + std::to_string(c) + "]";  // prefetched one wavefront step ahead
             return "q[" + std::to_string(soff[e]) + " + (int)((g * " + std::to_string(per) + "LL + " + std::to_string(c) +
                    "LL) & " + std::to_string(cap[e] - 1) + "LL)]";
         };
@@ -1847,8 +1847,22 @@ public:
           << "  const long long whi = SG_K_END * " << OPI << "LL + (" << OLO + OEX << "LL);\n"
           << "  const long long g0 = SG_K_BEGIN * " << ln.rep << "LL + (" << ln.ninit - ln.halo << "LL);\n"
           << "  const long long g1 = SG_K_END * " << ln.rep << "LL + (" << ln.ninit << "LL);\n"
+          << "  // the outer input of each lane's next firing is loaded one step ahead (off the serial chain)\n"
+          << "  " << T << " pf[" << li_.P << "];\n"
+          << "  {\n"
+          << "    const long long g = g0 + threadIdx.x;\n"
+          << "    if (threadIdx.x < " << WB << " && g < g1 && g >= next0)\n"
+          << "      for (int c = 0; c < " << li_.P << "; c++) pf[c] = gin[g * " << li_.P << "LL + c - in_base];\n"
+          << "  }\n"
           << "  for (long long gb = g0; gb < g1; gb += " << WB << ") {\n"
           << "    const long long g = gb + threadIdx.x;\n"
+          << "    " << T << " cur[" << li_.P << "];\n"
+          << "    for (int c = 0; c < " << li_.P << "; c++) cur[c] = pf[c];\n"
+          << "    {\n"
+          << "      const long long gn = g + " << WB << ";\n"
+          << "      if (threadIdx.x < " << WB << " && gn < g1 && gn >= next0)\n"
+          << "        for (int c = 0; c < " << li_.P << "; c++) pf[c] = gin[gn * " << li_.P << "LL + c - in_base];\n"
+          << "    }\n"
           << "    if (threadIdx.x < " << WB << " && g < g1) {\n"
           << "      if (g < next0) {  // before the stream start (zeros) or computed by an earlier launch (history)\n"
           << "        for (int j = 0; j < " << li_.Q << "; j++) {\n"
