@@ -1847,21 +1847,27 @@ public:
           << "  const long long whi = SG_K_END * " << OPI << "LL + (" << OLO + OEX << "LL);\n"
           << "  const long long g0 = SG_K_BEGIN * " << ln.rep << "LL + (" << ln.ninit - ln.halo << "LL);\n"
           << "  const long long g1 = SG_K_END * " << ln.rep << "LL + (" << ln.ninit << "LL);\n"
-          << "  // the outer input of each lane's next firing is loaded one step ahead (off the serial chain)\n"
-          << "  " << T << " pf[" << li_.P << "];\n"
-          << "  {\n"
-          << "    const long long g = g0 + threadIdx.x;\n"
+          << "  // the outer input of each lane's firings is loaded PD wavefront steps ahead (global latency\n"
+          << "  // off the serial chain: a step is a few shared-memory round trips)\n"
+          << "  constexpr int PD = 8;\n"
+          << "  " << T << " pf[PD][" << li_.P << "];\n"
+          << "#pragma unroll\n"
+          << "  for (int d = 0; d < PD; d++) {\n"
+          << "    const long long g = g0 + (long long)d * " << WB << " + threadIdx.x;\n"
           << "    if (threadIdx.x < " << WB << " && g < g1 && g >= next0)\n"
-          << "      for (int c = 0; c < " << li_.P << "; c++) pf[c] = gin[g * " << li_.P << "LL + c - in_base];\n"
+          << "      for (int c = 0; c < " << li_.P << "; c++) pf[d][c] = gin[g * " << li_.P << "LL + c - in_base];\n"
           << "  }\n"
           << "  for (long long gb = g0; gb < g1; gb += " << WB << ") {\n"
           << "    const long long g = gb + threadIdx.x;\n"
           << "    " << T << " cur[" << li_.P << "];\n"
-          << "    for (int c = 0; c < " << li_.P << "; c++) cur[c] = pf[c];\n"
+          << "    for (int c = 0; c < " << li_.P << "; c++) cur[c] = pf[0][c];\n"
+          << "#pragma unroll\n"
+          << "    for (int d = 0; d + 1 < PD; d++)\n"
+          << "      for (int c = 0; c < " << li_.P << "; c++) pf[d][c] = pf[d + 1][c];\n"
           << "    {\n"
-          << "      const long long gn = g + " << WB << ";\n"
+          << "      const long long gn = g + (long long)PD * " << WB << ";\n"
           << "      if (threadIdx.x < " << WB << " && gn < g1 && gn >= next0)\n"
-          << "        for (int c = 0; c < " << li_.P << "; c++) pf[c] = gin[gn * " << li_.P << "LL + c - in_base];\n"
+          << "        for (int c = 0; c < " << li_.P << "; c++) pf[PD - 1][c] = gin[gn * " << li_.P << "LL + c - in_base];\n"
           << "    }\n"
           << "    if (threadIdx.x < " << WB << " && g < g1) {\n"
           << "      if (g < next0) {  // before the stream start (zeros) or computed by an earlier launch (history)\n"
