@@ -261,7 +261,11 @@ const char* sg_plan_source(const sg_plan_t* p, int32_t part);
  * for every plan of the same graph (Kahn determinism). */
 sg_status sg_run(sg_plan_t* p, const void* input, int64_t n_iters, void* output, void* stream);
 
-/* Same, with HOST buffers: copies in, runs, copies out, synchronises. */
+/* Same, with HOST buffers (host_input: >= sg_input_items items; host_output: >= sg_output_items items;
+ * caller-owned; pinned memory makes the copies asynchronous): copies in, runs, copies out, synchronises
+ * before returning.  A single-partition plan without feedback loops pipelines 8 chunks of iterations
+ * over three streams (host->device copy of chunk c+1, kernel on chunk c, device->host copy of chunk
+ * c-1; SG_HOST_CHUNKS overrides the count); other plans copy in, run, copy out.  Same output as sg_run. */
 sg_status sg_run_host(sg_plan_t* p, const void* host_input, int64_t n_iters, void* host_output);
 
 /* Measured side of the PEE validation (Fig. 4.1: estimated vs
