@@ -1825,6 +1825,11 @@ public:
             }
             body << "        }\n";
         }
+        // lane-local chains: if every queued edge holds exactly one step of items (init_e == WB * T_e), a
+        // firing's cross-firing inputs come from the firing WB earlier -- the same lane, one step back
+        bool lane_local = !std::getenv("SG_LOOP_BARRIER");
+        for (int e = 0; e < (int)sf.edges.size(); e++)
+            if (li_.init_level[e] > 0 && li_.init_level[e] != WB * sf.edges[e].per_iter) lane_local = false;
         std::ostringstream s;
         s << header("feedback loop") << consts_.str() << args_struct_loop();
         s << "// wavefront: " << WB << " independent firings per step (loop delay " << wavefront(li_) << " firings)\n"
@@ -1880,8 +1885,10 @@ public:
           << body.str()
           << "      }\n"
           << "    }\n"
-          << "    __syncthreads();\n"
+          << (lane_local ? "    // every cross-firing dependency is exactly one step back on the same lane: no barrier\n"
+                         : "    __syncthreads();\n")
           << "  }\n"
+          << (lane_local ? "  __syncthreads();\n" : "")
           << "  if (threadIdx.x == 0) *reinterpret_cast<long long*>(st) = next0 > g1 ? next0 : g1;\n";
         for (int e = 0; e < (int)sf.edges.size(); e++)
             if (roff[e] >= 0)
