@@ -13,9 +13,12 @@ for fn in sorted(glob.glob(f"gpurun_out/{tag}/bench_*.json")):
     r = d.get("roofline") or {}
     c = d.get("config", {})
     rows.append((c.get("workload", fn), d["value"], d["ms_per_step"], r.get("bound"), r.get("achieved"), r.get("peak"),
-                 r.get("unit"), r.get("frac"), (d.get("cpu_baseline") or {}).get("value"), (d.get("e2e") or {}).get("value"),
+                 r.get("unit"), r.get("frac"),
+                 "%s (%s cores)" % (("%.3g" % (d.get("cpu_baseline") or {}).get("value", float("nan"))),
+                                    (d.get("cpu_baseline") or {}).get("cores")) if d.get("cpu_baseline") else None,
+                 (d.get("e2e") or {}).get("value"),
                  (d.get("clocks") or {}).get("sm_mhz")))
-print("| workload | iters/s | ms/step | bound | achieved | peak | unit | frac | oracle 1-core iters/s | e2e iters/s | SM MHz |")
+print("| workload | iters/s | ms/step | bound | achieved | peak | unit | frac | oracle iters/s (host cores) | e2e iters/s | SM MHz |")
 print("|---|---|---|---|---|---|---|---|---|---|---|")
 for w in rows:
     f = lambda x, p=3: ("%.*g" % (p, x)) if isinstance(x, (int, float)) else str(x)
