@@ -1862,17 +1862,19 @@ public:
           << "    if (threadIdx.x < " << WB << " && g < g1 && g >= next0)\n"
           << "      for (int c = 0; c < " << li_.P << "; c++) pf[d][c] = gin[g * " << li_.P << "LL + c - in_base];\n"
           << "  }\n"
-          << "  for (long long gb = g0; gb < g1; gb += " << WB << ") {\n"
+          << "  // PD steps per outer trip, unrolled: slot d is consumed and refilled at step d, so no\n"
+          << "  // register rotation ever waits on a load still in flight\n"
+          << "  for (long long gs = g0; gs < g1; gs += (long long)PD * " << WB << ") {\n"
+          << "#pragma unroll\n"
+          << "   for (int sd = 0; sd < PD; sd++) {\n"
+          << "    const long long gb = gs + (long long)sd * " << WB << ";\n"
           << "    const long long g = gb + threadIdx.x;\n"
           << "    " << T << " cur[" << li_.P << "];\n"
-          << "    for (int c = 0; c < " << li_.P << "; c++) cur[c] = pf[0][c];\n"
-          << "#pragma unroll\n"
-          << "    for (int d = 0; d + 1 < PD; d++)\n"
-          << "      for (int c = 0; c < " << li_.P << "; c++) pf[d][c] = pf[d + 1][c];\n"
+          << "    for (int c = 0; c < " << li_.P << "; c++) cur[c] = pf[sd][c];\n"
           << "    {\n"
           << "      const long long gn = g + (long long)PD * " << WB << ";\n"
           << "      if (threadIdx.x < " << WB << " && gn < g1 && gn >= next0)\n"
-          << "        for (int c = 0; c < " << li_.P << "; c++) pf[PD - 1][c] = gin[gn * " << li_.P << "LL + c - in_base];\n"
+          << "        for (int c = 0; c < " << li_.P << "; c++) pf[sd][c] = gin[gn * " << li_.P << "LL + c - in_base];\n"
           << "    }\n"
           << "    if (threadIdx.x < " << WB << " && g < g1) {\n"
           << "      if (g < next0) {  // before the stream start (zeros) or computed by an earlier launch (history)\n"
@@ -1887,6 +1889,7 @@ public:
           << "    }\n"
           << (lane_local ? "    // every cross-firing dependency is exactly one step back on the same lane: no barrier\n"
                          : "    __syncthreads();\n")
+          << "   }\n"
           << "  }\n"
           << (lane_local ? "  __syncthreads();\n" : "")
           << "  if (threadIdx.x == 0) *reinterpret_cast<long long*>(st) = next0 > g1 ? next0 : g1;\n";
