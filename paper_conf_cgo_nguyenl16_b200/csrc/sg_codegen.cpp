@@ -1774,6 +1774,19 @@ public:
         std::vector<int64_t> rd(sf.edges.size(), 0), wr(sf.edges.size(), 0);
         for (int e = 0; e < (int)sf.edges.size(); e++) wr[e] = li_.init_level[e];
         const std::string T = T_;
+        // lane-local chains: if every queued edge holds exactly one step of items (init_e == WB * T_e), a
+        // firing's cross-firing inputs come from the firing WB earlier -- the same lane, one step back
+        bool lane_local = !std::getenv("SG_LOOP_BARRIER");
+        for (int e = 0; e < (int)sf.edges.size(); e++)
+            if (li_.init_level[e] > 0 && li_.init_level[e] != WB * sf.edges[e].per_iter) lane_local = false;
+        // ... and then every item a firing reads is in a register: written earlier in the same firing
+        // (edges without initial items) or carried from the lane's previous firing (queued edges, loaded
+        // from the ring once, at the lane's first firing of the launch).  The rings of queued edges are
+        // still written, so the state saved after the launch is exact.
+        const bool fwd = lane_local && !std::getenv("SG_LOOP_NO_FWD");
+        std::ostringstream decl, carry_in, carry_out;
+        auto lv = [&](int e, int64_t c) { return "lv" + std::to_string(e) + "_" + std::to_string(c); };
+        auto cr = [&](int e, int64_t c) { return "cr" + std::to_string(e) + "_" + std::to_string(c); };
         auto pos_ref = [&](int e, int64_t c) -> std::string {  // item at (firing-relative) position c of edge e
             const int64_t per = sf.edges[e].per_iter;
             if (e == sf.in_edge) return "cur[" + std::to_string(c) + "]";  // prefetched one wavefront step ahead
@@ -1784,7 +1797,11 @@ public:
             const Node& n = sf.nodes[u];
             std::vector<std::string> xs;
             for (int e : n.in) {
-                for (int64_t i = 0; i < sf.edges[e].pop; i++) xs.push_back(pos_ref(e, rd[e] + i));
+                for (int64_t i = 0; i < sf.edges[e].pop; i++) {
+                    const int64_t c = rd[e] + i;
+                    if (!fwd || e == sf.in_edge) xs.push_back(pos_ref(e, c));
+                    else xs.push_back(li_.init_level[e] > 0 ? cr(e, c) : lv(e, c));
+                }
                 rd[e] += sf.edges[e].pop;
             }
             std::vector<std::string> ys;  // per output item, in port order
@@ -1817,19 +1834,30 @@ public:
                         body << "          { const long long p = g * " << li_.Q << "LL + " << c << "LL; const " << T
                              << " val = " << val << ";\n            hist[(int)(p & " << hist_len - 1 << "LL)] = val;\n"
                              << "            if (p >= wlo && p < whi) gout[p - out_base] = val; }\n";
-                    } else {
+                    } else if (!fwd) {
                         body << "          " << pos_ref(e, wr[e] + j) << " = " << val << ";\n";
+                    } else {
+                        decl << "        " << T << " " << lv(e, wr[e] + j) << ";\n";
+                        body << "          " << lv(e, wr[e] + j) << " = " << val << ";\n";
+                        if (li_.init_level[e] > 0)
+                            body << "          " << pos_ref(e, wr[e] + j) << " = " << lv(e, wr[e] + j) << ";\n";
                     }
                 }
                 wr[e] += sf.edges[e].push;
             }
             body << "        }\n";
         }
-        // lane-local chains: if every queued edge holds exactly one step of items (init_e == WB * T_e), a
-        // firing's cross-firing inputs come from the firing WB earlier -- the same lane, one step back
-        bool lane_local = !std::getenv("SG_LOOP_BARRIER");
-        for (int e = 0; e < (int)sf.edges.size(); e++)
-            if (li_.init_level[e] > 0 && li_.init_level[e] != WB * sf.edges[e].per_iter) lane_local = false;
+        std::ostringstream carry_decl;
+        if (fwd)
+            for (int e = 0; e < (int)sf.edges.size(); e++) {
+                if (li_.init_level[e] == 0 || e == sf.in_edge || e == sf.out_edge) continue;
+                const int64_t per = sf.edges[e].per_iter;
+                for (int64_t c = 0; c < per; c++) {
+                    carry_decl << "  " << T << " " << cr(e, c) << " = (" << T << ")0;\n";
+                    carry_in << "          " << cr(e, c) << " = " << pos_ref(e, c) << ";\n";
+                    carry_out << "        " << cr(e, c) << " = " << lv(e, WB * per + c) << ";\n";
+                }
+            }
         std::ostringstream s;
         s << header("feedback loop") << consts_.str() << args_struct_loop();
         s << "// wavefront: " << WB << " independent firings per step (loop delay " << wavefront(li_) << " firings)\n"
@@ -1855,6 +1883,7 @@ public:
           << "  // the outer input of each lane's firings is loaded PD wavefront steps ahead (global latency\n"
           << "  // off the serial chain: a step is a few shared-memory round trips)\n"
           << "  constexpr int PD = 8;\n"
+          << carry_decl.str() << (fwd ? "  bool fired = false;  // this lane's carries are in registers\n" : "")
           << "  " << T << " pf[PD][" << li_.P << "];\n"
           << "#pragma unroll\n"
           << "  for (int d = 0; d < PD; d++) {\n"
@@ -1884,7 +1913,10 @@ public:
           << "LL)];\n"
           << "        }\n"
           << "      } else {\n"
+          << (fwd ? "        if (!fired) {\n" + carry_in.str() + "          fired = true;\n        }\n" : std::string())
+          << decl.str()
           << body.str()
+          << carry_out.str()
           << "      }\n"
           << "    }\n"
           << (lane_local ? "    // every cross-firing dependency is exactly one step back on the same lane: no barrier\n"
