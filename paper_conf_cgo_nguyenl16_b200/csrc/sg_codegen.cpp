@@ -1858,6 +1858,32 @@ public:
                     carry_out << "        " << cr(e, c) << " = " << lv(e, WB * per + c) << ";\n";
                 }
             }
+        // Interior trips (every firing of the PD steps fires, prefetches in range, outputs inside the
+        // launch window, carries in registers): one straight-line block of PD steps with no per-step
+        // guards, so the address and store work of later steps overlaps the serial chain.
+        std::string fast_trip;
+        if (fwd && WB == NT) {
+            std::string fb = body.str();
+            const std::string guard = "if (p >= wlo && p < whi) ";
+            for (size_t k; (k = fb.find(guard)) != std::string::npos;) fb.erase(k, guard.size());
+            std::ostringstream ft;
+            ft << "    if (gs >= next0 && gs + 2LL * PD * " << WB << " <= g1 && gs * " << li_.Q << "LL >= wlo && (gs + (long long)PD * "
+               << WB << ") * " << li_.Q << "LL <= whi) {\n"
+               << "      if (!fired) {\n        const long long g = gs + threadIdx.x;\n" << carry_in.str()
+               << "          fired = true;\n      }\n"
+               << "#pragma unroll\n"
+               << "      for (int sd = 0; sd < PD; sd++) {\n"
+               << "        const long long g = gs + (long long)sd * " << WB << " + threadIdx.x;\n"
+               << "        " << T << " cur[" << li_.P << "];\n"
+               << "        for (int c = 0; c < " << li_.P << "; c++) cur[c] = pf[sd][c];\n"
+               << "        for (int c = 0; c < " << li_.P << "; c++) pf[sd][c] = gin[(g + (long long)PD * " << WB << ") * " << li_.P
+               << "LL + c - in_base];\n"
+               << decl.str() << fb << carry_out.str()
+               << "      }\n"
+               << "      continue;\n"
+               << "    }\n";
+            fast_trip = ft.str();
+        }
         std::ostringstream s;
         s << header("feedback loop") << consts_.str() << args_struct_loop();
         s << "// wavefront: " << WB << " independent firings per step (loop delay " << wavefront(li_) << " firings)\n"
@@ -1894,6 +1920,7 @@ public:
           << "  // PD steps per outer trip, unrolled: slot d is consumed and refilled at step d, so no\n"
           << "  // register rotation ever waits on a load still in flight\n"
           << "  for (long long gs = g0; gs < g1; gs += (long long)PD * " << WB << ") {\n"
+          << fast_trip
           << "#pragma unroll\n"
           << "   for (int sd = 0; sd < PD; sd++) {\n"
           << "    const long long gb = gs + (long long)sd * " << WB << ";\n"
