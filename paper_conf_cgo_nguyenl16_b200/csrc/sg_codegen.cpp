@@ -1863,9 +1863,9 @@ public:
         // guards, so the address and store work of later steps overlaps the serial chain.
         // PD: prefetch distance = steps per unrolled trip.  Measured on echo64 (B200, iters/s): PD 8
         // 6.2e8, 16 9.8e8, 32 1.36e9, 64 1.78e9, 128 1.89e9.  Capped so the prefetch slots stay within
-        // 64 registers and the unrolled trip within ~2048 firings.
-        int64_t PD = 64;
-        PD = std::min<int64_t>(PD, std::max<int64_t>(8, 64 / std::max<int64_t>(1, li_.P)));
+        // 128 registers and the unrolled trip within ~2048 firings.
+        int64_t PD = 128;
+        PD = std::min<int64_t>(PD, std::max<int64_t>(8, 128 / std::max<int64_t>(1, li_.P)));
         PD = std::min<int64_t>(PD, std::max<int64_t>(8, 2048 / std::max<int64_t>(1, (int64_t)li_.sched.size())));
         if (const char* e = std::getenv("SG_LOOP_PD")) PD = std::max(1, std::atoi(e));
         std::string fast_trip;
