@@ -131,14 +131,20 @@ enum {
     SG_PART_ALGORITHM1 = 0, /* the paper's Algorithm 1 with the B200 PEE */
     SG_PART_SINGLE = 1,     /* one partition (SPSG baseline) */
     SG_PART_PER_FILTER = 2, /* one partition per filter (splitters/joiners ride along) */
-    SG_PART_USER = 3        /* node_partition[] supplied by the caller */
+    SG_PART_USER = 3,       /* node_partition[] supplied by the caller */
+    SG_PART_CHAIN = 4       /* one partition per chain-fission group (needs chain_groups >= 2); nodes before
+                               the fissioned split-join join the first group, nodes after it the last */
 };
 
-/* Where boundary streams between GPUs travel (P2P). */
+/* Where boundary streams between GPUs travel (P2P) in the one-process runtime
+ * (sg_run); the one-process-per-GPU runtime (sg_run_rank) always uses NCCL send/recv and ignores it.
+ * sg_plan rejects any other value with SG_E_ARG. */
 enum {
-    SG_TRANSPORT_AUTO = 0,  /* P2P copy engine between devices; D2D copy for virtual GPUs */
-    SG_TRANSPORT_P2P = 1,   /* cudaMemcpyPeerAsync over NVLink */
-    SG_TRANSPORT_HOST = 2   /* host-staged D2H + H2D pair, as in [7] */
+    SG_TRANSPORT_AUTO = 0,  /* cudaMemcpyPeerAsync between distinct devices; D2D cudaMemcpyAsync between
+                               virtual GPUs on one device */
+    SG_TRANSPORT_P2P = 1,   /* cudaMemcpyPeerAsync for every cut edge between GPUs, virtual GPUs included */
+    SG_TRANSPORT_HOST = 2   /* host-staged pair, as in [7]: D2H into a pinned host
+                               buffer, then H2D, in order on the producer GPU's copy stream */
 };
 
 typedef struct sg_plan_opts {
@@ -167,6 +173,17 @@ typedef struct sg_plan_opts {
                                       With sg_comm_init / sg_run_rank, rank g * (G/R) + l is GPU l of group
                                       g and runs fragments f with f % R == g; output fragments land on the
                                       output rank of their group (gathering them is the caller's). */
+    int32_t chain_groups;          /* order-preserving chain fission of the largest eligible
+                                      split-join (a duplicate splitter and/or a roundrobin(1) joiner feeding
+                                      ADD(n_branches)): its branches are cut into contiguous groups; the
+                                      splitter becomes a forward chain (each group's splitter relays the
+                                      stream to the next), the joiner + ADD an accumulate chain
+                                      acc_g = ADD(acc_{g-1}, group g's outputs), bit-identical to the
+                                      sequential ADD.  0 = the planner compares the graph as written with its
+                                      fission into G/R groups (Algorithm 1 on more than one GPU only) and
+                                      keeps the smaller Tmax; -1 = never; k >= 2 = always, k groups (any
+                                      partitioner; node ids then refer to the fissioned graph, see
+                                      sg_plan_info).  SG_E_PLAN if k >= 2 and nothing is eligible. */
 } sg_plan_opts;
 
 typedef struct sg_plan_info_s {
@@ -194,6 +211,8 @@ typedef struct sg_plan_info_s {
     int64_t intops_per_iter;         /* algorithmic integer ops per iteration (min/max, adds) */
     int32_t replicas;                /* replica groups R; partition_gpu[] is the mapping inside group 0,
                                         group r runs partition p on logical GPU r * (n_gpus / R) + partition_gpu[p] */
+    int32_t chain_fission;           /* 1: the plan runs the chain-fissioned graph (sg_plan_opts.chain_groups);
+                                        n_nodes and every per-node array describe that graph */
 } sg_plan_info_t;
 
 /* ---- graph construction (the top-level stream is an implicit pipeline) ---- */
@@ -336,6 +355,16 @@ double sg_paper_model(int32_t n, const double* t, const double* f, int32_t S, in
 /* PDG of a plan: fills up to `cap` edges (partition src, dst,
  * bytes per iteration); returns the number of edges. */
 int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst, double* bytes);
+
+/* PEE inputs of partition `part` (the estimate sees the code generator's own
+ * optimisations), per steady-state iteration, written to out[0 .. min(cap, 16)):
+ *   0 kernel mode (1 register, 2 staged, 4 feedback loop; bitslice counts as 1), 1 executed fp32 flops
+ *   (after view resolution, dead-firing elimination, zero-tap pruning and CSE), 2 integer ops, 3 fp64 ops,
+ *   4 items read by live firings, 5 items written, 6 live firings, 7 boundary input bytes, 8 boundary
+ *   output bytes, 9 compute levels, 10 halo firings per tile, 11 loop firings, 12 CSE duplicate nodes,
+ *   13 frame FIRs present (0/1), 14 bitslice mode (0/1), 15 the PEE estimate (ns).
+ * Returns the number of values written, or -1 (NULL plan / bad partition). */
+int32_t sg_pee_features(const sg_plan_t* p, int32_t part, double* out, int32_t cap);
 
 /* Benchmark hygiene: evict L2 by overwriting `bytes` of device scratch memory
  * (> L2 size) and reading it back (dirty lines written back before the next

@@ -26,7 +26,7 @@ CUDA = os.environ.get("CUDA_HOME", "/usr/local/cuda")
 NVCC = os.path.join(CUDA, "bin", "nvcc")
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 
-CPP = ["sg_graph.cpp", "sg_codegen.cpp", "sg_plan.cpp", "sg_runtime.cpp", "sg_dist.cpp", "sg_capi.cpp"]
+CPP = ["sg_graph.cpp", "sg_codegen.cpp", "sg_pee.cpp", "sg_plan.cpp", "sg_runtime.cpp", "sg_dist.cpp", "sg_capi.cpp"]
 CU = ["sg_aux.cu"]
 HEADERS = ["sg_internal.h", "sg_codegen.h", "sg_runtime.h", "sg_plan.h", "sg_device.cuh"]
 

@@ -237,6 +237,7 @@ sg_status sg_plan_info(const sg_plan_t* pp, sg_plan_info_t* o) {
     o->flops_per_iter_pruned = pruned;
     o->intops_per_iter = intops;
     o->replicas = p.R;
+    o->chain_fission = p.chain_fission ? 1 : 0;
     return SG_OK;
 }
 
@@ -311,6 +312,24 @@ int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst,
         if (bytes) bytes[i] = e[i].bytes;
     }
     return (int32_t)e.size();
+}
+
+int32_t sg_pee_features(const sg_plan_t* p, int32_t part, double* out, int32_t cap) {
+    if (!p || !out || part < 0 || part >= (int32_t)p->plan.parts.size()) return -1;
+    try {
+        const sg::Plan& pl = p->plan;
+        const auto& nodes = pl.parts[part].nodes;
+        sg::PeeEstimate est = sg::pee_estimate(pl.flat, nodes);
+        const sg::PartitionWork& w = est.work;
+        const double v[16] = {(double)est.mode, w.flops, w.intops, w.dfma, w.reads, w.writes, w.firings, w.in_bytes,
+                              w.out_bytes, (double)w.levels, w.halo_firings, w.loop_firings, (double)w.cse_nodes,
+                              w.frame ? 1.0 : 0.0, est.bitslice ? 1.0 : 0.0, est.t};
+        int32_t n = std::min<int32_t>(cap, 16);
+        for (int32_t i = 0; i < n; i++) out[i] = v[i];
+        return n;
+    } catch (...) {
+        return -1;
+    }
 }
 
 sg_status sg_comm_unique_id(uint8_t id[128]) {

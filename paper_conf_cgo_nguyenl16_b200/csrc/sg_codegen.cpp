@@ -1622,8 +1622,8 @@ private:
             for (int64_t i = 0; i < 2 * nn; i++) x[i] = bit(n.in[0], g * n.pop + i);
             for (int64_t i = 0; i < nn; i++) {
                 BV a = x[i], b = x[nn + i];
-                if (a.s == "0u") { y.push_back({b.s, b.neg ^ a.neg}); continue; }
-                if (b.s == "0u") { y.push_back({a.s, a.neg ^ b.neg}); continue; }
+                if (a.s == "0u") { y.push_back({b.s, (bool)(b.neg ^ a.neg)}); continue; }
+                if (b.s == "0u") { y.push_back({a.s, (bool)(a.neg ^ b.neg)}); continue; }
                 BV r = fresh(a.s + " ^ " + b.s);
                 r.neg = a.neg ^ b.neg;
                 y.push_back(r);
@@ -1776,9 +1776,16 @@ public:
         const std::string T = T_;
         // lane-local chains: if every queued edge holds exactly one step of items (init_e == WB * T_e), a
         // firing's cross-firing inputs come from the firing WB earlier -- the same lane, one step back
+        // A slot of a ring (or of the history) is then only ever written by one lane iff its length is a
+        // multiple of the items one step writes (WB * T_e; history: WB * Q) -- otherwise lanes of different
+        // warps share slots and, with no barrier, a lagging warp could leave an older value in the saved
+        // state, so such loops keep the per-step barrier.
         bool lane_local = !std::getenv("SG_LOOP_BARRIER");
-        for (int e = 0; e < (int)sf.edges.size(); e++)
+        for (int e = 0; e < (int)sf.edges.size(); e++) {
             if (li_.init_level[e] > 0 && li_.init_level[e] != WB * sf.edges[e].per_iter) lane_local = false;
+            if (roff[e] >= 0 && cap[e] % (WB * std::max<int64_t>(1, sf.edges[e].per_iter)) != 0) lane_local = false;
+        }
+        if (hist_len % (WB * std::max<int64_t>(1, li_.Q)) != 0) lane_local = false;
         // ... and then every item a firing reads is in a register: written earlier in the same firing
         // (edges without initial items) or carried from the lane's previous firing (queued edges, loaded
         // from the ring once, at the lane's first firing of the launch).  The rings of queued edges are
@@ -1864,9 +1871,12 @@ public:
         // PD: prefetch distance = steps per unrolled trip.  Measured on echo64 (B200, iters/s): PD 8
         // 6.2e8, 16 9.8e8, 32 1.36e9, 64 1.78e9, 128 1.89e9.  Capped so the prefetch slots stay within
         // 128 registers and the unrolled trip within ~2048 firings.
+        // registers: PD * P prefetch slots <= 128 (no floor: more would spill to local memory);
+        // code size: the fast and the guarded trip are both unrolled PD steps, 2 * PD * |schedule| <= ~4096
+        // firings of straight-line code
         int64_t PD = 128;
-        PD = std::min<int64_t>(PD, std::max<int64_t>(8, 128 / std::max<int64_t>(1, li_.P)));
-        PD = std::min<int64_t>(PD, std::max<int64_t>(8, 2048 / std::max<int64_t>(1, (int64_t)li_.sched.size())));
+        PD = std::min<int64_t>(PD, std::max<int64_t>(1, 128 / std::max<int64_t>(1, li_.P)));
+        PD = std::min<int64_t>(PD, std::max<int64_t>(1, 2048 / std::max<int64_t>(1, (int64_t)li_.sched.size())));
         if (const char* e = std::getenv("SG_LOOP_PD")) PD = std::max(1, std::atoi(e));
         std::string fast_trip;
         if (fwd && WB == NT) {
@@ -1999,8 +2009,8 @@ private:
             break;
         case SG_K_FFT_REORDER: {
             int64_t nn = n.iv[0], o = 0;
-            for (int64_t i = 0; i < nn; i += 2) { c << "y_[" << o++ << "] = x_[" << 2 * i << "]; y_[" << o++ << "] = x_[" << 2 * i + 1 << "]; "; }
-            for (int64_t i = 1; i < nn; i += 2) { c << "y_[" << o++ << "] = x_[" << 2 * i << "]; y_[" << o++ << "] = x_[" << 2 * i + 1 << "]; "; }
+            for (int64_t i = 0; i < nn; i += 2, o += 2) c << "y_[" << o << "] = x_[" << 2 * i << "]; y_[" << o + 1 << "] = x_[" << 2 * i + 1 << "]; ";
+            for (int64_t i = 1; i < nn; i += 2, o += 2) c << "y_[" << o << "] = x_[" << 2 * i << "]; y_[" << o + 1 << "] = x_[" << 2 * i + 1 << "]; ";
             break;
         }
         case SG_K_PERMUTE:

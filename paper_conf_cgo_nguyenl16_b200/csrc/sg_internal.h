@@ -100,12 +100,24 @@ struct Edge {
     int64_t per_iter = 0;  // items per steady-state iteration (= rep_src * push)
 };
 
+// A split-join of the hierarchy in the flat graph: splitter, joiner, and the first node of each branch
+// (branch b = nodes [first[b], first[b + 1]), the last one ending before the joiner; branches are
+// contiguous in construction order).
+struct SjInfo {
+    int split = -1, join = -1;
+    std::vector<int> first;
+};
+
 struct Flat {
     sg_dtype dtype = SG_F32;
     std::vector<Node> nodes;  // topological (construction) order
     std::vector<Edge> edges;
     int in_edge = -1, out_edge = -1;
     int64_t in_per_iter = 0, out_per_iter = 0;
+    std::vector<std::vector<int>> pipes;  // innermost pipelines (every kid a filter), node ids in order
+    std::vector<SjInfo> sjs;              // split-joins, in construction order
+    std::vector<int> chain_first;         // chain-fissioned graph: first node id of each group (S_g); group g
+                                          // = nodes [chain_first[g], chain_first[g + 1]) (empty if not fissioned)
     // Builds from the hierarchy; throws Error.
     static Flat build(const sg_graph& g);
     void solve_rates();       // balance equations -> rep
@@ -114,6 +126,16 @@ struct Flat {
     int64_t output_items(int64_t n) const;
     bool is_physical(int e) const { return edges[e].src < 0 || nodes[edges[e].src].type == N_FILTER; }
 };
+
+// Order-preserving chain fission of split-join `sj`: its branches are cut into the
+// contiguous groups starting at branch group_first[0] = 0 < group_first[1] < ...; a duplicate
+// splitter becomes a forward chain S_1 -> S_2 -> ... (S_g feeds group g's branches and relays the
+// stream to S_{g+1}); a roundrobin(1) joiner feeding ADD(n_branches) becomes an accumulate chain
+// acc_g = ADD(acc_{g-1}, y_first(g), ..., y_last(g)) (J_g = roundrobin(1) over acc_{g-1} and group g's
+// branches), bit-identical to the sequential ADD (s = 0 + acc_{g-1} = acc_{g-1} exactly).
+// chain_fission_eligible: which of the two chains apply (0 none, bit 1 forward, bit 2 accumulate).
+int chain_fission_eligible(const Flat& f, int sj);
+Flat chain_fission(const Flat& f, int sj, const std::vector<int>& group_first);
 
 // kind metadata
 struct KindRates { int64_t peek, pop, push, prework; };

@@ -5,6 +5,8 @@
 
 #include <algorithm>
 #include <chrono>
+#include <cstdio>
+#include <cstdlib>
 #include <cmath>
 #include <functional>
 #include <numeric>
@@ -35,62 +37,66 @@ constexpr double kSmem = kSM * 128 * kClk;        // bytes/s
 constexpr double kHbm = 6.5536e12;                // bytes/s (MEASURED_PEAKS.json copy)
 constexpr double kLaunch = 4e-6;                  // s per kernel launch
 constexpr double kFragIters = 65536;              // iterations per fragment (estimate)
-constexpr int kTileEst = 64;
+constexpr double kTileEst = 64;                   // iterations per staged tile (estimate)
+// model constants, per iteration (fitted to measured partition times: see DESIGN.md, PEE)
+constexpr double kEffReg = 0.8;                   // register mode: fraction of the fp32 peak
+constexpr double kEffStaged = 0.6;                // staged fused kernels
+constexpr double kEffFrame = 0.3;                 // frame FIR kernels
+constexpr double kSmemItem = 0.0;                 // SM cycles per item read / written by live firings
+constexpr double kLevel = 1.0e-9;                 // GPU-seconds per compute level per tile (barrier + drain,
+                                                  // ~500 cycles spread over ~300 resident CTAs)
+constexpr double kLoopFiring = 25e-9;             // s per sequential loop firing
+constexpr double kFixed = 0.0;                    // ns per iteration per partition
+constexpr long long kIlpNodeBudget = 4000000;     // branch-and-bound nodes per mapping (deterministic)
 }  // namespace
 
 PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
     PeeEstimate est;
-    est.mode = register_mode_eligible(f, nodes, nullptr) ? 1 : 2;
-    std::vector<int> ins, outs;
-    partition_boundary(f, nodes, ins, outs);
-    double bytes = 0;
-    for (int e : ins) bytes += 4.0 * f.edges[e].per_iter;
-    for (int e : outs) bytes += 4.0 * f.edges[e].per_iter;
-    double flops = 0, intops = 0, dfma = 0, smem = 0;
-    int levels = 0;
-    double seq = 0;  // feedback loops: one thread walks the loop schedule (~25 ns per firing)
-    for (int v : nodes)
-        if (f.nodes[v].type == N_LOOP) seq += 25e-9 * (double)f.nodes[v].rep * (double)f.nodes[v].loop->sched.size();
-    for (int v : nodes) {
-        int64_t a, b, c;
-        node_work(f, v, a, b, c);
-        const Node& n = f.nodes[v];
-        double infl = est.mode == 2 ? (double)(n.halo + (int64_t)kTileEst * n.rep) / (double)(kTileEst * n.rep) : 1.0;
-        flops += a * infl;
-        intops += b * infl;
-        dfma += c * infl;
-        if (n.type == N_FILTER && !is_view_kind(n.kind)) {
-            levels++;
-            if (est.mode == 2) smem += 4.0 * n.rep * (n.peek + n.push) * infl;
-        }
-    }
-    if (est.mode == 1) smem = 0;
-    if (est.mode == 1 && bitslice_eligible(f, nodes, nullptr)) {
+    bool loop = false;
+    for (int v : nodes) loop = loop || f.nodes[v].type == N_LOOP;
+    est.mode = loop && nodes.size() == 1 ? 4 : (register_mode_eligible(f, nodes, nullptr) ? 1 : 2);
+    est.bitslice = est.mode == 1 && bitslice_eligible(f, nodes, nullptr);
+    est.work = partition_work(f, nodes);
+    const PartitionWork& w = est.work;
+    const double bytes = w.in_bytes + w.out_bytes;
+    double tc = 0;
+    if (est.bitslice) {
         // bitslice mode: one LOP3 covers 32 iterations; an S-box is a ~44-gate circuit, a word <-> bits
         // conversion a share of a 32x32 transpose (~5 ops per bit)
-        intops = 0;
+        double ops = 0;
         for (int v : nodes) {
             const Node& n = f.nodes[v];
             if (n.type != N_FILTER) continue;
             switch (n.kind) {
-            case SG_K_XOR: case SG_K_XOR_CONST: intops += (double)n.rep * n.iv[0] / 32.0; break;
-            case SG_K_SBOX: intops += (double)n.rep * 44.0 / 32.0; break;
-            case SG_K_INTO_BITS: case SG_K_BITS_TO_INT: intops += (double)n.rep * 5.0; break;
+            case SG_K_XOR: case SG_K_XOR_CONST: ops += (double)n.rep * n.iv[0] / 32.0; break;
+            case SG_K_SBOX: ops += (double)n.rep * 44.0 / 32.0; break;
+            case SG_K_INTO_BITS: case SG_K_BITS_TO_INT: ops += (double)n.rep * 5.0; break;
             default: break;
             }
         }
+        tc = ops / kInt;
+    } else if (est.mode == 1) {
+        // register mode: every FIFO item a register, one thread per iteration
+        tc = w.flops / (kFp32 * kEffReg) + w.intops / kInt + w.dfma * 80.0 / kFp64;
+    } else if (est.mode == 4) {
+        tc = kLoopFiring * w.loop_firings;
+    } else {
+        // staged mode: executed FP work at the fused kernels' efficiency, plus the shared-memory
+        // traffic of the live firings (reads of peek windows, writes of materialised outputs), the
+        // per-level barriers and the halo firings recomputed by every tile
+        const double eff = w.frame ? kEffFrame : kEffStaged;
+        const double recompute = 1.0 + w.halo_firings / (kTileEst * std::max(1.0, w.firings));
+        tc = (w.flops / (kFp32 * eff) + w.intops / kInt + w.dfma * 80.0 / kFp64) * recompute +
+             kSmemItem * (w.reads + w.writes) / (kSM * kClk) + kLevel * (double)w.levels / kTileEst +
+             kLoopFiring * w.loop_firings;
     }
-    for (int e : ins) smem += 8.0 * f.edges[e].per_iter;
-    for (int e : outs) smem += 8.0 * f.edges[e].per_iter;
-    double eff = est.mode == 1 ? 0.8 : 0.5;
-    est.t_comp = flops / (kFp32 * eff) + intops / kInt + dfma * 80.0 / kFp64 + smem / kSmem + seq;
-    est.t_dt = bytes / kHbm;
-    double bar = est.mode == 2 ? levels * 200.0 / kClk / (kTileEst * kSM * 2) : 0.0;
-    est.t = (std::max(est.t_comp, est.t_dt) + bar + kLaunch / kFragIters) * 1e9;  // ns per iteration
-    est.t_comp *= 1e9;
-    est.t_dt *= 1e9;
+    est.t_comp = tc * 1e9;
+    est.t_dt = bytes / kHbm * 1e9;
+    est.t = std::max(est.t_comp, est.t_dt) + kFixed;  // ns per iteration (the max() of Eq. III.8)
     return est;
 }
+
+double launch_ns_per_iter(int64_t frag) { return kLaunch / (double)(frag > 0 ? frag : (int64_t)kFragIters) * 1e9; }
 
 double paper_model(const std::vector<double>& t, const std::vector<double>& fr, int S, int W, int F, double D,
                    double C1, double C2, double* tcomp, double* tdt, double* tdb) {
@@ -136,16 +142,21 @@ namespace {
 struct PartState {
     const Flat& f;
     double cap;
+    int64_t frag = 0;
     std::vector<int> owner;                    // node -> partition id (-1 none)
     std::vector<std::vector<int>> members;     // partition id -> nodes (empty = dead)
     std::vector<double> T;
     std::vector<char> io;                      // IO-bound flag
-    explicit PartState(const Flat& fl, double c) : f(fl), cap(c), owner(fl.nodes.size(), -1) {}
+    PartState(const Flat& fl, double c, int64_t fr) : f(fl), cap(c), frag(fr), owner(fl.nodes.size(), -1) {}
 
+    mutable std::map<std::vector<int>, PeeEstimate> memo;
     double cost(const std::vector<int>& nodes, bool* io_bound = nullptr) const {
-        PeeEstimate e = pee_estimate(f, nodes);
-        if (io_bound) *io_bound = e.io_bound();
-        return e.t;
+        std::vector<int> key(nodes);
+        std::sort(key.begin(), key.end());
+        auto it = memo.find(key);
+        if (it == memo.end()) it = memo.emplace(key, pee_estimate(f, key)).first;
+        if (io_bound) *io_bound = it->second.io_bound();
+        return it->second.t + launch_ns_per_iter(frag);  // merging saves a kernel launch per fragment
     }
     int make(const std::vector<int>& nodes) {
         int id = (int)members.size();
@@ -210,40 +221,12 @@ struct PartState {
     }
 };
 
-// innermost pipelines of the hierarchy, as node-id sequences (construction order)
-void innermost_pipelines(const sg_graph& g, std::vector<std::vector<int>>& out) {
-    int next = 0;
-    std::function<void(int)> walk = [&](int id) {
-        const Elem& e = g.elems[id];
-        if (e.type == E_FILTER) { next++; return; }
-        if (e.type == E_PIPE) {
-            bool inner = !e.kids.empty();
-            for (int k : e.kids) inner &= g.elems[k].type == E_FILTER;
-            if (inner) {
-                std::vector<int> seq;
-                for (size_t i = 0; i < e.kids.size(); i++) seq.push_back(next + (int)i);
-                next += (int)e.kids.size();
-                out.push_back(seq);
-                return;
-            }
-            for (int k : e.kids) walk(k);
-            return;
-        }
-        if (e.type == E_LOOP) { next++; return; }  // one N_LOOP node (its graph lives in LoopInfo::sub)
-        next++;  // splitter
-        for (int b : e.branches) walk(b);
-        next++;  // joiner
-    };
-    walk(g.top);
-}
 }  // namespace
 
-std::vector<std::vector<int>> algorithm1(const Flat& f, const sg_graph& g, double cap) {
-    PartState S(f, cap);
-    // ---- Phase 1: inside innermost pipelines (Alg. 1 lines 2-10)
-    std::vector<std::vector<int>> pipes;
-    innermost_pipelines(g, pipes);
-    for (auto& pipe : pipes) {
+std::vector<std::vector<int>> algorithm1(const Flat& f, double cap, int64_t iters_per_fragment) {
+    PartState S(f, cap, iters_per_fragment);
+    // ---- Phase 1: inside innermost pipelines (Alg. 1 lines 2-10), recorded by Flat::build
+    for (auto& pipe : f.pipes) {
         size_t i = 0;
         while (i < pipe.size()) {
             int p = S.make({pipe[i]});
@@ -400,7 +383,7 @@ double mapping_cost(const std::vector<double>& T, const std::vector<PdgEdge>& pd
 }
 
 MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge>& pdg, const Topology& topo,
-                         double lat, double bw, int time_limit_ms, int method) {
+                         double lat, double bw, int time_limit_ms, int method, long long node_limit) {
     const int P = (int)T.size(), G = topo.G;
     MapResult best;
     best.assign.assign(P, 0);
@@ -435,6 +418,27 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
         std::vector<int> z(P, 0);
         double cz = mapping_cost(T, pdg, topo, lat, bw, z);
         if (cz < best.tmax) { best.tmax = cz; best.assign = z; }
+        // local search on the incumbent (single moves, then pairwise swaps, first improvement) so the
+        // branch and bound starts from a tight upper bound
+        for (bool improved = true; improved;) {
+            improved = false;
+            for (int i = 0; i < P && !improved; i++)
+                for (int g = 0; g < G && !improved; g++) {
+                    if (g == best.assign[i]) continue;
+                    std::vector<int> b = best.assign;
+                    b[i] = g;
+                    double c = mapping_cost(T, pdg, topo, lat, bw, b);
+                    if (c < best.tmax * (1 - 1e-12)) { best.tmax = c; best.assign = b; improved = true; }
+                }
+            for (int i = 0; i < P && !improved; i++)
+                for (int j = i + 1; j < P && !improved; j++) {
+                    if (best.assign[i] == best.assign[j]) continue;
+                    std::vector<int> b = best.assign;
+                    std::swap(b[i], b[j]);
+                    double c = mapping_cost(T, pdg, topo, lat, bw, b);
+                    if (c < best.tmax * (1 - 1e-12)) { best.tmax = c; best.assign = b; improved = true; }
+                }
+        }
     }
     bool symmetric = true;  // all GPUs interchangeable (true for the NVSwitch star)
     {
@@ -460,7 +464,8 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
     double total = suffix[0];
     std::function<void(int, int, double)> rec = [&](int k, int used, double cur) {
         if (timed_out) return;
-        if ((++nodes & 4095) == 0) {
+        if (node_limit > 0 && nodes >= node_limit) { timed_out = true; return; }  // deterministic budget
+        if ((++nodes & 4095) == 0 && time_limit_ms > 0) {
             auto ms = std::chrono::duration_cast<std::chrono::milliseconds>(std::chrono::steady_clock::now() - t0).count();
             if (ms > time_limit_ms) { timed_out = true; return; }
         }
@@ -507,7 +512,8 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
 // ============================================================ plan assembly
 namespace {
 // Partitions for a pipeline over Gs GPUs (Algorithm 1's cap depends on Gs).
-std::vector<std::vector<int>> make_partitions(const Flat& f, const sg_graph& g, int Gs, const sg_plan_opts& o) {
+// cap_mult scales Algorithm 1's G-aware cap (0: no cap).
+std::vector<std::vector<int>> make_partitions(const Flat& f, int Gs, const sg_plan_opts& o, double cap_mult = 1.0) {
     const int N = (int)f.nodes.size();
     std::vector<std::vector<int>> parts;
     switch (o.partitioner) {
@@ -528,17 +534,28 @@ std::vector<std::vector<int>> make_partitions(const Flat& f, const sg_graph& g, 
         for (auto& kv : m) parts.push_back(kv.second);
         break;
     }
+    case SG_PART_CHAIN: {  // one partition per chain-fission group; nodes before / after join the first / last
+        if (f.chain_first.empty()) throw Error(SG_E_ARG, "SG_PART_CHAIN needs a chain-fissioned graph (chain_groups >= 2)");
+        const int m = (int)f.chain_first.size();
+        parts.assign(m, {});
+        for (int v = 0; v < N; v++) {
+            int g = 0;
+            while (g + 1 < m && v >= f.chain_first[g + 1]) g++;
+            parts[g].push_back(v);
+        }
+        break;
+    }
     case SG_PART_ALGORITHM1: {
         double cap = 0;
-        if (Gs > 1) {
+        if (Gs > 1 && cap_mult > 0) {
             std::vector<int> all(N);
             std::iota(all.begin(), all.end(), 0);
             double sum = 0;
             for (int v = 0; v < N; v++) sum += pee_estimate(f, {v}).t;
             // G-aware cap: similar-sized partitions (goal 4)
-            cap = std::max(pee_estimate(f, all).t, sum / 4) / Gs * 1.25;
+            cap = std::max(pee_estimate(f, all).t, sum / 4) / Gs * 1.25 * cap_mult;
         }
-        parts = algorithm1(f, g, cap);
+        parts = algorithm1(f, cap, o.iters_per_fragment);
         break;
     }
     default: throw Error(SG_E_ARG, "unknown partitioner");
@@ -591,7 +608,7 @@ GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, in
     for (int i = 0; i < P; i++) for (int v : parts[i]) if (v >= 0 && v < N) owner[v] = i;
     GroupMap gm;
     gm.T.resize(P);
-    for (int i = 0; i < P; i++) gm.T[i] = pee_estimate(f, parts[i]).t;
+    for (int i = 0; i < P; i++) gm.T[i] = pee_estimate(f, parts[i]).t + launch_ns_per_iter(o.iters_per_fragment);
     // PDG: D_ij = sum of the weights of crossing edges (bytes / iteration)
     std::map<std::pair<int, int>, double> D;
     for (auto& e : f.edges) {
@@ -605,13 +622,121 @@ GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, in
         Topology topo = Topology::nvswitch(Gs);
         double bw = o.link_gbps > 0 ? o.link_gbps : 770.0;          // bytes per ns
         double lat_us = o.link_latency_us > 0 ? o.link_latency_us : 10.0;
-        double lat = lat_us * 1e3 / 65536.0;                          // amortised per iteration (reading 12)
-        gm.m = map_partitions(gm.T, gm.pdg, topo, lat, bw, o.ilp_time_limit_ms > 0 ? o.ilp_time_limit_ms : 10000, 0);
+        double lat = lat_us * 1e3 / (double)(o.iters_per_fragment > 0 ? o.iters_per_fragment : 65536);  // reading 12
+        // default: a deterministic node budget (plans are reproducible, so cubin caches hit); an
+        // explicit ilp_time_limit_ms is a wall-clock budget instead
+        gm.m = map_partitions(gm.T, gm.pdg, topo, lat, bw, o.ilp_time_limit_ms > 0 ? o.ilp_time_limit_ms : 0, 0,
+                              o.ilp_time_limit_ms > 0 ? 0 : kIlpNodeBudget);
     } else {
         gm.m.tmax = std::accumulate(gm.T.begin(), gm.T.end(), 0.0);
         gm.m.optimal = true;
     }
     return gm;
+}
+
+// Balanced contiguous groups of branches for chain fission: m groups minimising the largest group
+// cost (linear partition by DP over the branches' PEE times).
+std::vector<int> balanced_groups(const std::vector<double>& c, int m) {
+    const int n = (int)c.size();
+    m = std::min(m, n);
+    std::vector<double> pre(n + 1, 0.0);
+    for (int i = 0; i < n; i++) pre[i + 1] = pre[i] + c[i];
+    const double INF = 1e300;
+    // best[k][i]: first i branches in k groups; cut[k][i]: start of the k-th group
+    std::vector<std::vector<double>> best(m + 1, std::vector<double>(n + 1, INF));
+    std::vector<std::vector<int>> cut(m + 1, std::vector<int>(n + 1, 0));
+    best[0][0] = 0;
+    for (int k = 1; k <= m; k++)
+        for (int i = k; i <= n; i++)
+            for (int j = k - 1; j < i; j++) {
+                double v = std::max(best[k - 1][j], pre[i] - pre[j]);
+                if (v < best[k][i] - 1e-12) { best[k][i] = v; cut[k][i] = j; }
+            }
+    std::vector<int> first(m);
+    for (int k = m, i = n; k >= 1; k--) {
+        first[k - 1] = cut[k][i];
+        i = cut[k][i];
+    }
+    return first;
+}
+
+// The split-join chain fission applies to: eligible (forward and/or accumulate chain), most nodes.
+int fission_target(const Flat& f) {
+    int best = -1, bestn = 0;
+    for (int k = 0; k < (int)f.sjs.size(); k++) {
+        if (!chain_fission_eligible(f, k)) continue;
+        int n = f.sjs[k].join - f.sjs[k].split;
+        if (n > bestn) { bestn = n; best = k; }
+    }
+    return best;
+}
+
+Flat fissioned(const Flat& f, int sj, int m) {
+    const SjInfo& si = f.sjs[sj];
+    const int nb = (int)si.first.size();
+    std::vector<double> cost(nb);
+    for (int b = 0; b < nb; b++) {
+        std::vector<int> br;
+        for (int v = si.first[b]; v < (b + 1 < nb ? si.first[b + 1] : si.join); v++) br.push_back(v);
+        cost[b] = br.empty() ? 0.0 : pee_estimate(f, br).t;
+    }
+    return chain_fission(f, sj, balanced_groups(cost, m));
+}
+
+// Graph variants and partitionings the planner compares (pipeline of Gs GPUs): the graph as written
+// and, when a split-join is eligible, its chain fission into Gs groups; Algorithm 1
+// with the G-aware cap, twice the cap, and no cap.  The ILP objective Tmax decides (ties: the first).
+struct Candidate {
+    int variant = 0;
+    std::vector<std::vector<int>> parts;
+    double tmax = 0;
+};
+GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, int Gs, const sg_plan_opts& o);
+
+Candidate best_candidate(const std::vector<Flat>& variants, int Gs, const sg_plan_opts& o, GroupMap* gm_out) {
+    Candidate best;
+    bool have = false;
+    GroupMap bgm;
+    for (int vi = 0; vi < (int)variants.size(); vi++) {
+        std::vector<double> mults = {1.0};
+        if (o.partitioner == SG_PART_ALGORITHM1 && Gs > 1) mults = {1.0, 2.0, 0.0};
+        if (const char* env = std::getenv("SG_A1_CAPS")) {  // experiments: fixed cap multipliers ("1,2")
+            mults.clear();
+            for (const char* c = env; *c;) {
+                mults.push_back(std::atof(c));
+                while (*c && *c != ',') c++;
+                if (*c == ',') c++;
+            }
+        }
+        // a fissioned graph's groups are a candidate partitioning of their own (cap < 0 below)
+        if (o.partitioner == SG_PART_ALGORITHM1 && !variants[vi].chain_first.empty()) mults.push_back(-1.0);
+        std::set<std::vector<std::vector<int>>> seen;
+        for (double cm : mults) {
+            sg_plan_opts oc = o;
+            if (cm < 0) oc.partitioner = SG_PART_CHAIN;
+            auto parts = make_partitions(variants[vi], Gs, oc, cm);
+            auto key = parts;
+            for (auto& q : key) std::sort(q.begin(), q.end());
+            std::sort(key.begin(), key.end());
+            if (!seen.insert(key).second) continue;
+            GroupMap gm = map_group(variants[vi], parts, Gs, o);
+            if (std::getenv("SG_PLAN_DEBUG")) {
+                std::fprintf(stderr, "[sg plan] variant %d cap x%.1f: %zu partitions, Tmax %.4f ns (ilp %s) T =", vi, cm,
+                             parts.size(), gm.m.tmax, gm.m.optimal ? "optimal" : "budget");
+                for (size_t i = 0; i < parts.size() && i < 24; i++) std::fprintf(stderr, " %.3f/%zu", gm.T[i], parts[i].size());
+                std::fprintf(stderr, "\n");
+            }
+            if (!have || gm.m.tmax < best.tmax * (1 - 1e-9)) {
+                have = true;
+                best.variant = vi;
+                best.parts = parts;
+                best.tmax = gm.m.tmax;
+                bgm = gm;
+            }
+        }
+    }
+    if (gm_out) *gm_out = bgm;
+    return best;
 }
 
 // Throughput bound of R replica groups of Gs GPUs each on the NVSwitch star:
@@ -624,7 +749,8 @@ double hybrid_cost(const Flat& f, const std::vector<double>& T, const std::vecto
                    const std::vector<int>& a, int in_gpu, int out_gpu, int Gs, int R, const sg_plan_opts& o) {
     const int G = Gs * R;
     const double bw = o.link_gbps > 0 ? o.link_gbps : 770.0;
-    const double lat = (o.link_latency_us > 0 ? o.link_latency_us : 10.0) * 1e3 / 65536.0;
+    const double lat = (o.link_latency_us > 0 ? o.link_latency_us : 10.0) * 1e3 /
+                       (double)(o.iters_per_fragment > 0 ? o.iters_per_fragment : 65536);
     std::vector<double> comp(Gs, 0.0), up(G, 0.0), down(G, 0.0);
     for (size_t i = 0; i < T.size(); i++) comp[a[i]] += T[i];
     for (int r = 0; r < R; r++) {
@@ -658,11 +784,26 @@ int io_gpu(const Flat& f, const std::vector<std::vector<int>>& parts, const std:
 }  // namespace
 
 void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
-    p.flat = Flat::build(g);
+    if (o.transport < SG_TRANSPORT_AUTO || o.transport > SG_TRANSPORT_HOST)
+        throw Error(SG_E_ARG, "transport must be SG_TRANSPORT_AUTO, _P2P or _HOST");
+    if (o.chain_groups < -1 || o.chain_groups == 1) throw Error(SG_E_ARG, "chain_groups must be -1, 0 or >= 2");
+    Flat f0 = Flat::build(g);
     p.G = G;
     p.opts = o;
+    // graph variants: as written, and the order-preserving chain fission of the
+    // largest eligible split-join -- forced with chain_groups >= 2, considered by the planner for
+    // Algorithm 1 on more than one GPU (per replica group)
+    const int fsj = o.chain_groups == -1 ? -1 : fission_target(f0);
+    if (o.chain_groups >= 2 && fsj < 0) throw Error(SG_E_PLAN, "chain_groups: no eligible split-join (SURVEY.md 8(e))");
+    auto variants_for = [&](int Gs) {
+        std::vector<Flat> v;
+        if (o.chain_groups >= 2) { v.push_back(fissioned(f0, fsj, o.chain_groups)); return v; }
+        v.push_back(f0);
+        if (fsj >= 0 && Gs > 1 && o.partitioner == SG_PART_ALGORITHM1) v.push_back(fissioned(f0, fsj, Gs));
+        return v;
+    };
+    p.flat = f0;
     const Flat& f = p.flat;
-    const int N = (int)f.nodes.size();
     // ---- replica groups (hybrid replica x pipeline; R = 1 is the paper's mapping)
     int R = 1;
     bool has_loop = false;
@@ -676,10 +817,13 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         double best = 0;
         for (int r = 1; r <= G; r++) {
             if (G % r) continue;
-            auto pr = make_partitions(f, g, G / r, o);
-            GroupMap gm = map_group(f, pr, G / r, o);
-            double c = hybrid_cost(f, gm.T, gm.pdg, gm.m.assign, io_gpu(f, pr, gm.m.assign, f.edges[f.in_edge].dst),
-                                   io_gpu(f, pr, gm.m.assign, f.edges[f.out_edge].src), G / r, r, o);
+            auto vars = variants_for(G / r);
+            GroupMap gm;
+            Candidate cd = best_candidate(vars, G / r, o, &gm);
+            const Flat& fv = vars[cd.variant];
+            auto& pr = cd.parts;
+            double c = hybrid_cost(fv, gm.T, gm.pdg, gm.m.assign, io_gpu(fv, pr, gm.m.assign, fv.edges[fv.in_edge].dst),
+                                   io_gpu(fv, pr, gm.m.assign, fv.edges[fv.out_edge].src), G / r, r, o);
             if (r == 1 || c < best * 0.999) { best = c; R = r; }
         }
     } else if (o.replicas < -1) {
@@ -688,8 +832,17 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     const int Gs = G / R;
     p.R = R;
     p.Gs = Gs;
-    // ---- partitions
-    std::vector<std::vector<int>> parts = make_partitions(f, g, Gs, o);
+    // ---- graph variant + partitions (Algorithm 1 candidates compared by the ILP objective)
+    std::vector<std::vector<int>> parts;
+    GroupMap gm;
+    {
+        auto vars = variants_for(Gs);
+        Candidate cd = best_candidate(vars, Gs, o, &gm);
+        p.flat = vars[cd.variant];
+        p.chain_fission = o.chain_groups >= 2 || cd.variant == 1;
+        parts = cd.parts;
+    }
+    const int N = (int)f.nodes.size();
     // validate: cover, convex; order topologically
     std::vector<int> owner(N, -1);
     for (size_t i = 0; i < parts.size(); i++) {
@@ -736,7 +889,6 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         p.part_time[i] = est.t;
     }
     // ---- PDG and mapping inside one replica group of Gs GPUs
-    GroupMap gm = map_group(f, parts, Gs, o);
     p.pdg = gm.pdg;
     p.part_gpu.assign(P, 0);
     for (int i = 0; i < P; i++) p.part_gpu[i] = gm.m.assign[i];

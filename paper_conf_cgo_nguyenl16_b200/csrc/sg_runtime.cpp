@@ -413,6 +413,7 @@ Plan::~Plan() {
                 cudaFree(r.dst_slots[i]);
             }
         }
+        for (auto h : r.host_slots) if (h) cudaFreeHost(h);
         for (auto e : r.ev_copied) if (e) cudaEventDestroy(e);
         for (auto e : r.ev_consumed) if (e) cudaEventDestroy(e);
         for (auto e : r.ev_produced) if (e) cudaEventDestroy(e);
@@ -486,6 +487,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                     cudaFree(r.dst_slots[i]);
                 }
             }
+            for (auto h : r.host_slots) if (h) cudaFreeHost(h);
             for (auto e : r.ev_copied) cudaEventDestroy(e);
             for (auto e : r.ev_consumed) cudaEventDestroy(e);
             for (auto e : r.ev_produced) cudaEventDestroy(e);
@@ -546,6 +548,10 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                     SG_RT(cudaMalloc(&q, (size_t)r.slot_items * 4));
                 }
                 r.dst_slots.push_back(q);
+                void* h = nullptr;
+                if (opts.transport == SG_TRANSPORT_HOST && r.dst_gpu != r.src_gpu)
+                    SG_RT(cudaHostAlloc(&h, (size_t)r.slot_items * 4, cudaHostAllocPortable));
+                r.host_slots.push_back(h);
                 cudaEvent_t e1, e2, e3;
                 {
                     DevGuard dg(devices[r.dst_gpu]);
@@ -643,12 +649,19 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                 SG_RT(cudaStreamWaitEvent(gc.copy, r.ev_produced[slot], 0));
                 if (fg >= ring_depth) SG_RT(cudaStreamWaitEvent(gc.copy, r.ev_consumed[slot], 0));
                 int64_t items = r.per_iter * (kb - ka) + r.extra;
-                if (devices[r.src_gpu] == devices[r.dst_gpu])
-                    SG_RT(cudaMemcpyAsync(r.dst_slots[slot], r.src_slots[slot], (size_t)items * 4,
-                                          cudaMemcpyDeviceToDevice, gc.copy));
-                else
+                const size_t bytes = (size_t)items * 4;
+                if (opts.transport == SG_TRANSPORT_HOST) {
+                    // host-staged pair, as in [7]: D2H into pinned memory, then H2D,
+                    // in order on the producer's copy stream
+                    SG_RT(cudaMemcpyAsync(r.host_slots[slot], r.src_slots[slot], bytes, cudaMemcpyDefault, gc.copy));
+                    SG_RT(cudaMemcpyAsync(r.dst_slots[slot], r.host_slots[slot], bytes, cudaMemcpyDefault, gc.copy));
+                } else if (opts.transport == SG_TRANSPORT_P2P || devices[r.src_gpu] != devices[r.dst_gpu]) {
                     SG_RT(cudaMemcpyPeerAsync(r.dst_slots[slot], devices[r.dst_gpu], r.src_slots[slot],
-                                              devices[r.src_gpu], (size_t)items * 4, gc.copy));
+                                              devices[r.src_gpu], bytes, gc.copy));
+                } else {
+                    SG_RT(cudaMemcpyAsync(r.dst_slots[slot], r.src_slots[slot], bytes, cudaMemcpyDeviceToDevice,
+                                          gc.copy));
+                }
                 SG_RT(cudaEventRecord(r.ev_copied[slot], gc.copy));
             }
         }

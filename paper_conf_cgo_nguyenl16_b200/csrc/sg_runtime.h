@@ -37,6 +37,7 @@ struct CutRing {          // one boundary stream between partitions (PAPER.md:49
     int64_t lo = 0, extra = 0, per_iter = 0;
     int64_t slot_items = 0;
     std::vector<void*> src_slots, dst_slots;  // device buffers (dst == src when same GPU)
+    std::vector<void*> host_slots;            // SG_TRANSPORT_HOST: pinned staging buffer per slot
     std::vector<cudaEvent_t> ev_copied, ev_consumed, ev_produced;
 };
 
@@ -70,6 +71,7 @@ struct Plan {
     bool virtual_gpus = false;
     double est_tmax = 0;
     bool ilp_optimal = false;
+    bool chain_fission = false;            // p.flat is the chain-fissioned graph
     std::vector<PdgEdge> pdg;
     // info arrays
     std::vector<int64_t> reps, ninit;

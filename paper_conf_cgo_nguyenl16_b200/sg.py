@@ -20,7 +20,7 @@ _lib = None
 SG_OK, SG_E_ARG, SG_E_STRUCTURE, SG_E_RATE, SG_E_UNSUPPORTED = 0, -1, -2, -3, -4
 SG_E_NOMEM, SG_E_CUDA, SG_E_COMM, SG_E_PLAN, SG_E_SIZE = -5, -6, -7, -8, -9
 SG_F32, SG_I32 = 0, 1
-SG_PART_ALGORITHM1, SG_PART_SINGLE, SG_PART_PER_FILTER, SG_PART_USER = 0, 1, 2, 3
+SG_PART_ALGORITHM1, SG_PART_SINGLE, SG_PART_PER_FILTER, SG_PART_USER, SG_PART_CHAIN = 0, 1, 2, 3, 4
 
 KINDS = {"IDENTITY": 0, "FIR": 1, "DELAY": 2, "DECIMATE": 3, "EXPAND": 4, "COMPARE_EXCHANGE": 5,
          "FFT_REORDER": 6, "COMBINE_DFT": 7, "FM_DEMOD": 8, "SUBTRACT": 9, "AMPLIFY": 10, "ADD": 11,
@@ -34,7 +34,7 @@ EXPORTS = ["sg_graph_create", "sg_graph_destroy", "sg_add_filter", "sg_add_split
            "sg_plan_info", "sg_plan_source", "sg_run", "sg_run_host", "sg_last_launch_count",
            "sg_plan_destroy", "sg_last_error", "sg_version", "sg_flush_l2", "sg_topology_links",
            "sg_topology_dtlist", "sg_map_ilp", "sg_paper_model", "sg_plan_pdg", "sg_comm_unique_id", "sg_comm_init",
-           "sg_run_rank", "sg_rank_schedule", "sg_profile_partitions"]
+           "sg_run_rank", "sg_rank_schedule", "sg_profile_partitions", "sg_pee_features"]
 SG_OP_LAUNCH, SG_OP_SEND, SG_OP_RECV = 0, 1, 2
 
 
@@ -56,7 +56,7 @@ class PlanOpts(ctypes.Structure):
                 ("virtual_gpus", ctypes.c_int32), ("devices", ctypes.POINTER(ctypes.c_int32)),
                 ("ilp_time_limit_ms", ctypes.c_int32), ("codegen_mode", ctypes.c_int32),
                 ("link_gbps", ctypes.c_double), ("link_latency_us", ctypes.c_double), ("verbose", ctypes.c_int32),
-                ("plan_only", ctypes.c_int32), ("replicas", ctypes.c_int32)]
+                ("plan_only", ctypes.c_int32), ("replicas", ctypes.c_int32), ("chain_groups", ctypes.c_int32)]
 
 
 class RankOp(ctypes.Structure):
@@ -76,7 +76,7 @@ class PlanInfo(ctypes.Structure):
                 ("input_device", ctypes.c_int32), ("output_device", ctypes.c_int32),
                 ("iters_per_fragment", ctypes.c_int64), ("ilp_optimal", ctypes.c_int32),
                 ("flops_per_iter_written", ctypes.c_double), ("flops_per_iter_pruned", ctypes.c_double),
-                ("intops_per_iter", ctypes.c_int64), ("replicas", ctypes.c_int32)]
+                ("intops_per_iter", ctypes.c_int64), ("replicas", ctypes.c_int32), ("chain_fission", ctypes.c_int32)]
 
 
 def lib():
@@ -122,6 +122,7 @@ def lib():
                             ctypes.c_double, ctypes.c_double, ctypes.c_double, ctypes.POINTER(ctypes.c_double),
                             ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ctypes.c_double)], ctypes.c_double),
         "sg_plan_pdg": ([vp, i32, ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(ctypes.c_double)], i32),
+        "sg_pee_features": ([vp, i32, ctypes.POINTER(ctypes.c_double), i32], i32),
         "sg_comm_unique_id": ([ctypes.POINTER(ctypes.c_uint8)], ctypes.c_int),
         "sg_comm_init": ([vp, i32, i32, ctypes.POINTER(ctypes.c_uint8), i32], ctypes.c_int),
         "sg_run_rank": ([vp, vp, i64, vp, vp], ctypes.c_int),
@@ -249,7 +250,7 @@ class Plan:
             elif k == "codegen_mode" and isinstance(v, str):
                 o.codegen_mode = {"auto": 0, "register": 1, "staged": 2, "general": 3}[v]
             elif k == "partitioner" and isinstance(v, str):
-                o.partitioner = {"algorithm1": 0, "single": 1, "per_filter": 2}[v]
+                o.partitioner = {"algorithm1": 0, "single": 1, "per_filter": 2, "chain": 4}[v]
             else:
                 setattr(o, k, v)
         self._h = ctypes.c_void_p()
@@ -277,7 +278,7 @@ class Plan:
             "iters_per_fragment": i.iters_per_fragment, "ilp_optimal": bool(i.ilp_optimal),
             "flops_per_iter_written": i.flops_per_iter_written, "flops_per_iter_pruned": i.flops_per_iter_pruned,
             "intops_per_iter": i.intops_per_iter,
-            "replicas": i.replicas,
+            "replicas": i.replicas, "chain_fission": bool(i.chain_fission),
         }
 
     def input_items(self, n: int) -> int:
@@ -298,6 +299,8 @@ class Plan:
 
     def run(self, x, n_iters: int, y, stream=None):
         """x, y: CUDA tensors (or raw device pointers); enqueued on `stream` (default: torch current stream)."""
+        self._check_tensor(x, self.input_items(n_iters), "x")
+        self._check_tensor(y, self.output_items(n_iters), "y")
         xp = x.data_ptr() if hasattr(x, "data_ptr") else int(x)
         yp = y.data_ptr() if hasattr(y, "data_ptr") else int(y)
         if stream is None:
@@ -307,8 +310,27 @@ class Plan:
             stream = stream.cuda_stream
         _check(lib().sg_run(self._h, ctypes.c_void_p(xp), n_iters, ctypes.c_void_p(yp), ctypes.c_void_p(stream)))
 
+    @staticmethod
+    def _check_tensor(t, need: int, nm: str):
+        """Tensors: on a CUDA device, contiguous, 4-byte items, at least `need` of them (raw pointers: unchecked)."""
+        if not hasattr(t, "data_ptr"):
+            return
+        if not t.is_cuda:
+            raise ValueError(f"{nm}: needs a CUDA tensor")
+        if not t.is_contiguous() or t.element_size() != 4:
+            raise ValueError(f"{nm}: needs a contiguous tensor of 4-byte items")
+        if t.numel() < need:
+            raise ValueError(f"{nm}: {t.numel()} items < {need} needed")
+
     def run_host(self, x, n_iters: int, y):
         """x, y: contiguous host numpy arrays (4-byte items); copies in, runs, copies out, synchronises."""
+        for a, need, nm in ((x, self.input_items(n_iters), "x"), (y, self.output_items(n_iters), "y")):
+            if a.dtype.itemsize != 4 or not a.flags["C_CONTIGUOUS"]:
+                raise ValueError(f"{nm}: needs a C-contiguous array of 4-byte items")
+            if a.size < need:
+                raise ValueError(f"{nm}: {a.size} items < {need} needed for {n_iters} iterations")
+        if not y.flags["WRITEABLE"]:
+            raise ValueError("y: read-only array")
         _check(lib().sg_run_host(self._h, ctypes.c_void_p(x.ctypes.data), n_iters, ctypes.c_void_p(y.ctypes.data)))
 
     def pdg(self):
@@ -350,6 +372,17 @@ class Plan:
         buf = (ctypes.c_double * max(1, k))()
         _check(lib().sg_profile_partitions(self._h, n_iters, reps, buf))
         return [buf[i] for i in range(k)]
+
+    PEE_FEATURES = ["mode", "flops", "intops", "dfma", "reads", "writes", "firings", "in_bytes", "out_bytes",
+                    "levels", "halo_firings", "loop_firings", "cse_nodes", "frame", "bitslice", "est_ns"]
+
+    def pee_features(self, part: int) -> dict:
+        """PEE inputs of one partition (work after the code generator's pruning / CSE, per iteration)."""
+        buf = (ctypes.c_double * 16)()
+        n = lib().sg_pee_features(self._h, part, buf, 16)
+        if n < 0:
+            raise SgError(SG_E_ARG, "bad partition")
+        return {k: buf[i] for i, k in enumerate(self.PEE_FEATURES[:n])}
 
     def last_launch_count(self) -> int:
         return lib().sg_last_launch_count(self._h)

@@ -27,7 +27,7 @@ def _free_port():
     return port
 
 
-def _worker(rank, world, port, name, n, frag, q, replicas=1):
+def _worker(rank, world, port, name, n, frag, q, replicas=1, extra=None):
     import sys
     sys.path.insert(0, ROOT)
     try:
@@ -37,7 +37,7 @@ def _worker(rank, world, port, name, n, frag, q, replicas=1):
         from paper_conf_cgo_nguyenl16_b200.dist import max_over_ranks, replica_shard
         prog = {"filterbank8": lambda: apps.filterbank(8), "fmradio4": lambda: apps.fmradio(5),
                 "beamformer": lambda: apps.beamformer(channels=3, beams=2, frame=64, taps=8, mf_taps=16)}[name]()
-        with sg.plan(prog, world, iters_per_fragment=frag, replicas=replicas, plan_only=1) as p:
+        with sg.plan(prog, world, iters_per_fragment=frag, replicas=replicas, plan_only=1, **(extra or {})) as p:
             info = p.info()
             R = info["replicas"]
             Gs = world // R
@@ -82,15 +82,23 @@ def _worker(rank, world, port, name, n, frag, q, replicas=1):
         q.put((rank, "fail", traceback.format_exc()))
 
 
-@pytest.mark.parametrize("name,n,frag,world,replicas", [
-    ("filterbank8", 5000, 700, 2, 1), ("fmradio4", 3000, 512, 2, 1), ("beamformer", 40, 7, 2, 1),
+CHAIN = dict(chain_groups=-2, partitioner="chain")   # chain_groups = world (filled in below)
+
+
+@pytest.mark.parametrize("name,n,frag,world,replicas,extra", [
+    ("filterbank8", 5000, 700, 2, 1, None), ("fmradio4", 3000, 512, 2, 1, None), ("beamformer", 40, 7, 2, 1, None),
     # hybrid replica x pipeline plans: two groups
-    ("filterbank8", 5000, 300, 2, 2), ("fmradio4", 3000, 256, 4, 2)])
-def test_rank_schedules_match_over_gloo(name, n, frag, world, replicas):
+    ("filterbank8", 5000, 300, 2, 2, None), ("fmradio4", 3000, 256, 4, 2, None),
+    # chain fission: one group per rank, forward + accumulate streams hop rank to rank
+    ("filterbank8", 5000, 700, 2, 1, CHAIN), ("fmradio4", 3000, 256, 4, 1, CHAIN)])
+def test_rank_schedules_match_over_gloo(name, n, frag, world, replicas, extra):
+    if extra is CHAIN:
+        extra = dict(CHAIN, chain_groups=world)
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, name, n, frag, q, replicas)) for r in range(world)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, name, n, frag, q, replicas, extra))
+             for r in range(world)]
     for p in procs:
         p.start()
     results = [q.get(timeout=240) for _ in range(world)]

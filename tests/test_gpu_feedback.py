@@ -19,6 +19,10 @@ PROGS = {
                                                                     "dup", enqueue=[0])])),
     "echo64": apps.FEEDBACK["echo64"],           # wavefront of 64 firings (2 warps)
     "echo300": lambda: apps.echo(300, -0.75, 8),  # wavefront capped at 256 firings
+    # multi-warp wavefronts that are not powers of two: ring / history slots are shared between lanes
+    # of different warps, so the per-step barrier must stay (lane-local chains would race)
+    "echo96": lambda: apps.echo(96, 0.5, 8),
+    "echo100": lambda: apps.echo(100, -0.5, 8),
     "runstats": apps.FEEDBACK["runstats"],
     "multirate": lambda: Program("mr", "f32", Pipeline([
         Filter("FIR", [5, 1], [0.5, -1.0, 0.25, 2.0, -0.5]),
@@ -58,3 +62,19 @@ def test_feedback_state_resets_between_runs(oracle_lib):
             p.run(xd, n, yd)
             torch.cuda.synchronize()
             assert np.array_equal(yd.cpu().numpy(), ref)
+
+
+@pytest.mark.parametrize("name", ["echo64", "echo96", "runsum"])
+@pytest.mark.parametrize("frag", [0, 10000])
+def test_feedback_parity_long(oracle_lib, name, frag):
+    """n = 2^16 + 37 iterations: long enough that the guard-free interior trips (g1 - gs >= 2*PD*WB
+    firings) and the trip-to-trip prefetch refill run, as one fragment and as ~10k-iteration fragments
+    (state and history handed over between launches)."""
+    prog = PROGS[name]()
+    n = (1 << 16) + 37
+    x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), 91)
+    ref = oracle_lib.run(prog, x, n)
+    kw = dict(partitioner="per_filter", iters_per_fragment=frag) if frag else dict()
+    y, info, launches = run_gpu(prog, x, n, **kw)
+    assert 4 in info["partition_mode"]
+    assert_parity(prog, y, ref)

@@ -36,6 +36,10 @@ PLANS = [
     dict(n_gpus=4, virtual_gpus=1, replicas=2, iters_per_fragment=64),
     dict(n_gpus=4, virtual_gpus=1, replicas=4, iters_per_fragment=50),
     dict(n_gpus=6, virtual_gpus=1, replicas=3, partitioner="per_filter", iters_per_fragment=70),
+    # transports (include/sg.h): cudaMemcpyPeerAsync for every cut edge even between virtual GPUs of one
+    # device, and the host-staged D2H + H2D pair of [7]
+    dict(n_gpus=3, virtual_gpus=1, partitioner="per_filter", iters_per_fragment=90, transport=1),
+    dict(n_gpus=2, virtual_gpus=1, partitioner="per_filter", iters_per_fragment=150, transport=2),
 ]
 
 
@@ -183,22 +187,27 @@ def test_run_rank_world1_nccl(oracle_lib):
     import torch.distributed as dist
     from paper_conf_cgo_nguyenl16_b200 import sg
     from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan
-    if not dist.is_initialized():
+    created = not dist.is_initialized()
+    if created:
         os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
         os.environ.setdefault("MASTER_PORT", "29517")
         dist.init_process_group("nccl", rank=0, world_size=1, device_id=torch.device("cuda", 0))
-    prog = apps.fmradio(4)
-    n = 2000
-    x = inputs.make_input("f32", oracle_lib.in_items(prog, n), 77)
-    ref = oracle_lib.run(prog, x, n)
-    for kw in (dict(), dict(partitioner="per_filter", iters_per_fragment=300)):
-        p = pipeline_plan(prog, **kw)
-        xd = torch.from_numpy(x).cuda()
-        yd = torch.empty(p.output_items(n), device="cuda")
-        p.run_rank(xd, n, yd)
-        torch.cuda.synchronize()
-        assert_parity(prog, yd.cpu().numpy(), ref)
-        p.close()
+    try:
+        prog = apps.fmradio(4)
+        n = 2000
+        x = inputs.make_input("f32", oracle_lib.in_items(prog, n), 77)
+        ref = oracle_lib.run(prog, x, n)
+        for kw in (dict(), dict(partitioner="per_filter", iters_per_fragment=300)):
+            p = pipeline_plan(prog, **kw)
+            xd = torch.from_numpy(x).cuda()
+            yd = torch.empty(p.output_items(n), device="cuda")
+            p.run_rank(xd, n, yd)
+            torch.cuda.synchronize()
+            assert_parity(prog, yd.cpu().numpy(), ref)
+            p.close()
+    finally:
+        if created:
+            dist.destroy_process_group()
 
 
 
