@@ -5,12 +5,17 @@
 
 One step = one sg_run() over the whole workload (replayed as a CUDA graph) (all of SURVEY.md 8(a)'s timed
 rows: tile loads, filter execution, stores; plus boundary streams when the plan
-has several partitions/GPUs).  Default workload: BASELINE.json configs[1],
-BitonicSort 32-key int32, 2^20 iterations, one GPU.  Inputs resident in HBM;
-L2 flushed (256 MiB write + read-back with our sg_flush_l2 kernels) before every
-timed step, outside the per-step CUDA-event window.  Under torchrun (N > 1) every rank
-runs an independent replica on its own GPU ("replicas only" for this HBM-bound
-graph); value = all ranks' iterations / max-over-ranks time.
+has several partitions/GPUs).  Default workload: the largest graph of BASELINE.json
+(configs[4], FilterBank 64 branches fp32, the north star's "largest graph"), 2^20
+iterations on one GPU.  Inputs resident in HBM; L2 flushed (256 MiB write + read-back
+with our sg_flush_l2 kernels) before every timed step, outside the per-step CUDA-event
+window.  Under torchrun (N > 1) the default is the paper's pipelined mapping
+(--mode pipeline): every rank builds the same plan for N GPUs (Algorithm 1 + ILP; for
+FilterBank the chain-fission groups) and runs its partitions with NCCL
+boundary streams (sg_run_rank), 2^24 iterations per step so the fragment pipeline
+fills; value = iterations / max-over-ranks time ("strong").  --mode replicas runs N
+independent replicas instead ("weak").  --config fft64 also reports BASELINE's 4096
+iterations (CUDA-graph replay) next to the 2^20 roofline run.
 
 --impl reference times the oracle (the plain sequential CPU interpreter in
 oracle/, as it stands) on the host cores, on a bounded sample of the workload.
@@ -181,7 +186,7 @@ def main():
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=3000)
     ap.add_argument("--warmup", type=int, default=20)
-    ap.add_argument("--config", default="bitonic32", choices=list(WORKLOADS))
+    ap.add_argument("--config", default="filterbank64", choices=list(WORKLOADS))
     ap.add_argument("--impl", default="sg", choices=["sg", "reference"])
     ap.add_argument("--iters", type=int, default=0, help="override iterations per step")
     ap.add_argument("--no-cpu-baseline", action="store_true")
@@ -195,9 +200,9 @@ def main():
                     help="comma-separated node ids: user partitions [0, c1), [c1, c2), ... on one GPU (A/B of splits)")
     ap.add_argument("--codegen", default="auto", choices=["auto", "register", "staged", "general"],
                     help="plan option codegen_mode (auto: chosen by the code generator)")
-    ap.add_argument("--mode", default="replicas", choices=["replicas", "pipeline"],
-                    help="N>1: independent replicas (default; the headline graph is HBM-bound) or the paper's "
-                         "pipelined partition mapping, one process per GPU, NCCL boundary streams")
+    ap.add_argument("--mode", default="pipeline", choices=["replicas", "pipeline"],
+                    help="N>1: the paper's pipelined partition mapping (default), one process per GPU, NCCL "
+                         "boundary streams; or independent replicas")
     args = ap.parse_args()
     if args.warmup < 3:
         args.warmup = 3
@@ -217,9 +222,11 @@ def main():
     torch.cuda.set_device(local)
     name = args.config
     W = WORKLOADS[name]
-    n = args.iters or W["n"]
-    prog = {**apps.CONFIGS, **apps.EXTRA, **apps.FEEDBACK}[name]()
     pipeline = args.mode == "pipeline" and world > 1
+    # pipelined runs need many fragments per GPU (fill / drain F / (F + G - 1))
+    n = args.iters or (max(W["n"], 1 << 24) if pipeline and W["bound"] == "alu" and name != "beamformer12x4"
+                       else W["n"])
+    prog = {**apps.CONFIGS, **apps.EXTRA, **apps.FEEDBACK}[name]()
     if pipeline:
         from paper_conf_cgo_nguyenl16_b200.dist import pipeline_plan
         plan = pipeline_plan(prog, replicas=args.replicas)
@@ -351,7 +358,31 @@ def main():
 
     # end to end through the public C ABI with HOST buffers (pinned), copies inside the timed region
     e2e = None
-    if not pipeline:
+    if pipeline:
+        # one process per GPU: the input rank copies the step's input in from pinned host memory, the
+        # output rank copies the output back; wall clock between barriers, max over ranks
+        xh = x_host.pin_memory()
+        yh = torch.empty(nout, dtype=dt).pin_memory()
+        is_in, is_out = local == info["input_device"], local == info["output_device"]
+        k2 = max(3, min(10, args.steps))
+        torch.cuda.synchronize()
+        dist.barrier()
+        t0 = time.perf_counter()
+        for _ in range(k2):
+            if is_in:
+                x.copy_(xh, non_blocking=True)
+            plan.run_rank(x, n, y, stream)
+            if is_out:
+                yh.copy_(y, non_blocking=True)
+            torch.cuda.synchronize()
+        dist.barrier()
+        e2e_s = (time.perf_counter() - t0) / k2
+        from paper_conf_cgo_nguyenl16_b200.dist import max_over_ranks
+        e2e_s = max_over_ranks(e2e_s, device=f"cuda:{local}")
+        e2e = {"value": n / e2e_s, "unit": "iters/s", "h2d_bytes_per_step": nin * 4, "d2h_bytes_per_step": nout * 4,
+               "steps": k2, "timing": "host wall clock between barriers around H2D (input rank) + sg_run_rank + "
+                                      "D2H (output rank), max over ranks"}
+    else:
         xh = x_host.pin_memory()
         yh = torch.empty(nout, dtype=dt).pin_memory()
         xnp, ynp = xh.numpy(), yh.numpy()
@@ -363,6 +394,30 @@ def main():
         e2e_s = (time.perf_counter() - t0) / k2
         e2e = {"value": world * n / e2e_s, "unit": "iters/s", "h2d_bytes_per_step": nin * 4,
                "d2h_bytes_per_step": nout * 4, "steps": k2, "timing": "host wall clock around sg_run_host"}
+
+    # FFT: BASELINE.json configs[0] is 4096 iterations (8 MiB of traffic, ~1 us at the roof, L2-resident):
+    # reported as given, 1000 back-to-back replays of a CUDA graph of one sg_run, no flush in between
+    at_config = None
+    if name == "fft64" and not pipeline and world == 1:
+        n4 = 4096
+        y4 = torch.empty(plan.output_items(n4), dtype=dt, device=f"cuda:{local}")
+        g4 = torch.cuda.CUDAGraph()
+        gs4 = torch.cuda.Stream()
+        with torch.cuda.graph(g4, stream=gs4):
+            plan.run(x, n4, y4, torch.cuda.current_stream())
+        for _ in range(20):
+            g4.replay()
+        torch.cuda.synchronize()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        for _ in range(1000):
+            g4.replay()
+        e1.record(stream)
+        torch.cuda.synchronize()
+        ms4 = e0.elapsed_time(e1) / 1000
+        at_config = {"iters_per_step": n4, "value": n4 / (ms4 / 1e3), "unit": "iters/s", "ms_per_step": ms4,
+                     "steps": 1000, "note": "BASELINE.json configs[0] size: CUDA-graph replays back to back, "
+                                            "L2-resident (8 MiB), not flushed"}
 
     cb = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
@@ -378,12 +433,14 @@ def main():
                        "items_per_s_out": value * info["out_per_iter"],
                        "l2": "flushed before every step (256 MiB sg_flush_l2: write + read back), outside the event window"
                        if not args.no_flush else "not flushed",
+                       "chain_fission": info["chain_fission"], "partition_gpu": info["partition_gpu"],
                        "parallelism": (f"pipeline over {world} GPUs (ILP mapping, NCCL boundary streams)" if pipeline
                                        else f"replicas x{world}" if world > 1 else "1 GPU, 1 partition"),
                        "partitions": info["n_partitions"], "partition_mode": info["partition_mode"],
                        "launch": "CUDA graph replay of one sg_run" if graph is not None else "eager sg_run",
                        "wall_s": wall},
             "roofline": roof, "cpu_baseline": cb, "e2e": e2e,
+            **({"at_config_size": at_config} if at_config else {}),
             "gpu_launches": args.steps * (launches_per_step + (0 if args.no_flush else 2)),
             "clocks": clocks,
         }

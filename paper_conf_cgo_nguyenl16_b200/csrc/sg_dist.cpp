@@ -99,11 +99,12 @@ std::vector<RankOp> rank_schedule(const Plan& p, int rank, int64_t n, int64_t F)
         const Edge& ed = p.flat.edges[e];
         if (ed.src < 0 || ed.dst < 0) continue;
         int ps = p.node_part[ed.src], pd = p.node_part[ed.dst];
-        if (ps != pd && p.part_gpu[ps] != p.part_gpu[pd]) cut.push_back(e);
+        // one message per shared ring (a duplicated stream crosses to a GPU once): its representative
+        if (ps != pd && p.part_gpu[ps] != p.part_gpu[pd] && p.ring_rep[e] == e) cut.push_back(e);
     }
     auto window = [&](int e, int64_t ka, int64_t kb) {
         int64_t lo, ex;
-        edge_window(p.flat, e, lo, ex);
+        p.cut_window(e, lo, ex);
         return p.flat.edges[e].per_iter * (kb - ka) + ex;
     };
     auto recvs = [&](int64_t f) {
@@ -184,8 +185,9 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
             if (ed.src < 0 || ed.dst < 0) continue;
             int ps = node_part[ed.src], pd = node_part[ed.dst];
             if (ps == pd || (part_gpu[ps] != me && part_gpu[pd] != me)) continue;
+            if (ring_rep[e] != e) continue;  // shares its representative's slots
             int64_t lo, ex;
-            edge_window(flat, e, lo, ex);
+            cut_window(e, lo, ex);
             for (int s = 0; s < D; s++) {
                 void* q = nullptr;
                 SG_RT2(cudaMalloc(&q, (size_t)(ed.per_iter * F + ex) * 4));
@@ -202,8 +204,8 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
         dist_ready = true;
     }
     // slots cycle over this group's fragments (f = group + R * j)
-    auto EV = [&](int e, int kind, int64_t f) { return dist_ev[e][kind * D + (int)((f / R) % D)]; };
-    auto SLOT = [&](int e, int64_t f) { return dist_slots[e][(int)((f / R) % D)]; };
+    auto EV = [&](int e, int kind, int64_t f) { return dist_ev[ring_rep[e]][kind * D + (int)((f / R) % D)]; };
+    auto SLOT = [&](int e, int64_t f) { return dist_slots[ring_rep[e]][(int)((f / R) % D)]; };
     SG_RT2(cudaEventRecord(dist_join, user));
     SG_RT2(cudaStreamWaitEvent(dist_compute, dist_join, 0));
     SG_RT2(cudaStreamWaitEvent(dist_comm, dist_join, 0));
@@ -228,7 +230,7 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
                     continue;
                 }
                 int64_t lo, ex;
-                edge_window(flat, e, lo, ex);
+                cut_window(e, lo, ex);
                 bool remote = part_gpu[node_part[ed.src]] != me;
                 SG_RT2(cudaStreamWaitEvent(dist_compute, EV(e, remote ? 0 : 2, o.frag), 0));
                 io.in.push_back(SLOT(e, o.frag));
@@ -244,7 +246,7 @@ void Plan::run_rank(const void* in, int64_t n, void* out, cudaStream_t user) {
                     continue;
                 }
                 int64_t lo, ex;
-                edge_window(flat, e, lo, ex);
+                cut_window(e, lo, ex);
                 bool remote = part_gpu[node_part[ed.dst]] != me;
                 if (o.frag / R >= D) SG_RT2(cudaStreamWaitEvent(dist_compute, EV(e, remote ? 3 : 1, o.frag), 0));
                 io.out.push_back(SLOT(e, o.frag));

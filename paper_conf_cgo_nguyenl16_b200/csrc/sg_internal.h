@@ -152,7 +152,10 @@ struct Topology {
     static Topology pcie_tree4();  // Fig. 3.3
 };
 
-struct PdgEdge { int src, dst; double bytes; };
+// PDG edge: bytes per iteration from partition src to partition dst.  `data` >= 0
+// names the stream a duplicate splitter copies (its node id): edges with the same `data` carry the
+// same items, so a link carries them once per destination GPU (SURVEY.md 8(c)-4 reading 15).
+struct PdgEdge { int src, dst; double bytes; int data = -1; };
 
 struct Partition {
     std::vector<int> nodes;  // node ids (sorted, topological)

@@ -11,6 +11,7 @@
 #include <functional>
 #include <numeric>
 #include <set>
+#include <tuple>
 
 #include "sg_codegen.h"
 
@@ -371,9 +372,11 @@ double mapping_cost(const std::vector<double>& T, const std::vector<PdgEdge>& pd
                     double bw, const std::vector<int>& a) {
     std::vector<double> gl(topo.G, 0.0), ll(topo.L, 0.0);
     for (size_t i = 0; i < T.size(); i++) gl[a[i]] += T[i];                       // III.4
-    for (auto& e : pdg) {                                                          // III.6-III.7
+    std::set<std::tuple<int, int, int>> shipped;                                   // duplicated data: once per
+    for (auto& e : pdg) {                                                          // III.6-III.7 (src, dst) GPU
         int k = a[e.src], h = a[e.dst];
         if (k == h) continue;
+        if (e.data >= 0 && !shipped.insert(std::make_tuple(e.data, k, h)).second) continue;
         for (int l = 0; l < topo.L; l++) if (topo.carries(l, k, h)) ll[l] += e.bytes;
     }
     double tmax = 0;
@@ -445,15 +448,17 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
         Topology s = Topology::nvswitch(G);
         symmetric = s.L == topo.L && s.dt == topo.dt;
     }
-    std::vector<std::vector<std::pair<int, double>>> adj(P);  // edges to earlier-ordered partitions
+    struct Adj { int other; double bytes; bool out; int data; };
+    std::vector<std::vector<Adj>> adj(P);  // edges to earlier-ordered partitions
     std::vector<int> rank(P);
     for (int k = 0; k < P; k++) rank[ord[k]] = k;
     for (auto& e : pdg) {
         if (e.src == e.dst) continue;
         int later = rank[e.src] > rank[e.dst] ? e.src : e.dst;
         int other = later == e.src ? e.dst : e.src;
-        adj[later].push_back({other, later == e.src ? e.bytes : -e.bytes});  // sign: direction
+        adj[later].push_back({other, e.bytes, later == e.src, e.data});
     }
+    std::map<std::tuple<int, int, int>, int> shipped;  // (data, src GPU, dst GPU) -> edges carrying it
     std::vector<double> suffix(P + 1, 0.0);
     for (int k = P - 1; k >= 0; k--) suffix[k] = suffix[k + 1] + T[ord[k]];
     std::vector<int> a(P, -1);
@@ -484,11 +489,17 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
             gl[g] += T[i];
             double c = std::max(cur, gl[g]);
             std::vector<std::pair<int, double>> touched;
+            std::vector<std::tuple<int, int, int>> counted;
             for (auto& pr : adj[i]) {
-                int j = pr.first;
-                double D = std::fabs(pr.second);
-                int src = pr.second >= 0 ? g : a[j], dst = pr.second >= 0 ? a[j] : g;
+                int j = pr.other;
+                double D = pr.bytes;
+                int src = pr.out ? g : a[j], dst = pr.out ? a[j] : g;
                 if (src == dst) continue;
+                if (pr.data >= 0) {
+                    auto key = std::make_tuple(pr.data, src, dst);
+                    counted.push_back(key);
+                    if (shipped[key]++ > 0) continue;  // the same duplicated stream already crosses this pair
+                }
                 for (int l = 0; l < topo.L; l++)
                     if (topo.carries(l, src, dst)) {
                         ll[l] += D;
@@ -497,6 +508,7 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
                     }
             }
             rec(k + 1, std::max(used, g + 1), c);
+            for (auto& key : counted) shipped[key]--;
             for (auto& t : touched) ll[t.first] -= t.second;
             gl[g] -= T[i];
             a[i] = -1;
@@ -610,13 +622,24 @@ GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, in
     gm.T.resize(P);
     for (int i = 0; i < P; i++) gm.T[i] = pee_estimate(f, parts[i]).t + launch_ns_per_iter(o.iters_per_fragment);
     // PDG: D_ij = sum of the weights of crossing edges (bytes / iteration)
-    std::map<std::pair<int, int>, double> D;
+    // edges out of a duplicate splitter carry the splitter's input stream: one data id per splitter
+    std::map<std::tuple<int, int, int>, double> D;
     for (auto& e : f.edges) {
         if (e.src < 0 || e.dst < 0) continue;
         int a = owner[e.src], b = owner[e.dst];
-        if (a >= 0 && b >= 0 && a != b) D[{a, b}] += 4.0 * e.per_iter;
+        if (a < 0 || b < 0 || a == b) continue;
+        const int data = f.nodes[e.src].type == N_SPLIT_DUP ? e.src : -1;
+        if (data >= 0) D[std::make_tuple(a, b, data)] = 4.0 * e.per_iter;  // once per destination partition
+        else D[std::make_tuple(a, b, -1)] += 4.0 * e.per_iter;
     }
-    for (auto& kv : D) gm.pdg.push_back({kv.first.first, kv.first.second, kv.second});
+    for (auto& kv : D) {
+        PdgEdge pe;
+        pe.src = std::get<0>(kv.first);
+        pe.dst = std::get<1>(kv.first);
+        pe.data = std::get<2>(kv.first);
+        pe.bytes = kv.second;
+        gm.pdg.push_back(pe);
+    }
     gm.m.assign.assign(P, 0);
     if (Gs > 1) {
         Topology topo = Topology::nvswitch(Gs);
@@ -754,9 +777,11 @@ double hybrid_cost(const Flat& f, const std::vector<double>& T, const std::vecto
     std::vector<double> comp(Gs, 0.0), up(G, 0.0), down(G, 0.0);
     for (size_t i = 0; i < T.size(); i++) comp[a[i]] += T[i];
     for (int r = 0; r < R; r++) {
+        std::set<std::tuple<int, int, int>> shipped;
         for (auto& e : pdg) {
             int k = a[e.src], h = a[e.dst];
             if (k == h) continue;
+            if (e.data >= 0 && !shipped.insert(std::make_tuple(e.data, k, h)).second) continue;
             up[r * Gs + k] += e.bytes / R;
             down[r * Gs + h] += e.bytes / R;
         }
@@ -896,6 +921,37 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
                         : hybrid_cost(f, gm.T, gm.pdg, gm.m.assign, io_gpu(f, parts, gm.m.assign, f.edges[f.in_edge].dst),
                                       io_gpu(f, parts, gm.m.assign, f.edges[f.out_edge].src), Gs, R, o);
     p.ilp_optimal = gm.m.optimal;
+    // ---- rings: a duplicated stream crosses to a GPU once (PDG data ids, reading 15)
+    p.ring_rep.assign(f.edges.size(), -1);
+    p.ring_lo.assign(f.edges.size(), 0);
+    p.ring_extra.assign(f.edges.size(), 0);
+    {
+        std::map<std::pair<int, int>, int> first;  // (dup splitter, destination GPU) -> representative edge
+        for (int e = 0; e < (int)f.edges.size(); e++) {
+            const Edge& ed = f.edges[e];
+            if (ed.src < 0 || ed.dst < 0) continue;
+            const int ps = owner[ed.src], pd = owner[ed.dst];
+            if (ps == pd) continue;
+            int rep = e;
+            const int hg = p.part_gpu[pd];
+            if (f.nodes[ed.src].type == N_SPLIT_DUP && p.part_gpu[ps] != hg) {
+                auto it = first.find({ed.src, hg});
+                if (it == first.end()) first[{ed.src, hg}] = e;
+                else rep = it->second;
+            }
+            p.ring_rep[e] = rep;
+            int64_t lo, ex;
+            edge_window(f, e, lo, ex);
+            if (rep == e) {
+                p.ring_lo[e] = lo;
+                p.ring_extra[e] = ex;
+            } else {  // union [min lo, max(lo + extra)) -- members have the same items per iteration
+                const int64_t hi = std::max(p.ring_lo[rep] + p.ring_extra[rep], lo + ex);
+                p.ring_lo[rep] = std::min(p.ring_lo[rep], lo);
+                p.ring_extra[rep] = hi - p.ring_lo[rep];
+            }
+        }
+    }
     // ---- devices
     p.virtual_gpus = o.virtual_gpus != 0;
     p.devices.assign(G, 0);

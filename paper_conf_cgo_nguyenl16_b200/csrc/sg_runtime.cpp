@@ -524,15 +524,19 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
             const Edge& ed = flat.edges[ei];
             if (ed.src < 0 || ed.dst < 0) continue;
             int ps = node_part[ed.src], pd = node_part[ed.dst];
-            if (ps == pd) continue;
+            if (ps == pd || ring_rep[ei] != (int)ei) continue;  // members of a shared ring: below
             CutRing r;
             r.edge = (int)ei;
             r.group = grp;
             r.src_part = ps;
             r.dst_part = pd;
+            for (size_t ej = 0; ej < flat.edges.size(); ej++)
+                if (ring_rep[ej] == (int)ei && std::find(r.dst_parts.begin(), r.dst_parts.end(),
+                                                         node_part[flat.edges[ej].dst]) == r.dst_parts.end())
+                    r.dst_parts.push_back(node_part[flat.edges[ej].dst]);
             r.src_gpu = grp * Gs + part_gpu[ps];
             r.dst_gpu = grp * Gs + part_gpu[pd];
-            edge_window(flat, (int)ei, r.lo, r.extra);
+            cut_window((int)ei, r.lo, r.extra);
             r.per_iter = ed.per_iter;
             r.slot_items = r.per_iter * F + r.extra;
             for (int s = 0; s < ring_depth; s++) {
@@ -576,7 +580,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
     const size_t NP = parts.size();
     std::vector<std::vector<int>> ring_in(R * NP), ring_out(R * NP);
     for (size_t ri = 0; ri < rings.size(); ri++) {
-        ring_in[rings[ri].group * NP + rings[ri].dst_part].push_back((int)ri);
+        for (int dp : rings[ri].dst_parts) ring_in[rings[ri].group * NP + dp].push_back((int)ri);
         ring_out[rings[ri].group * NP + rings[ri].src_part].push_back((int)ri);
     }
     // order every GPU after the caller's stream
@@ -614,7 +618,8 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                     continue;
                 }
                 int ri = -1;
-                for (int r : ring_in[gp]) if (rings[r].edge == e) ri = r;
+                for (int r : ring_in[gp]) if (rings[r].edge == ring_rep[e]) ri = r;
+                if (ri < 0) throw Error(SG_E_PLAN, "internal: no ring for cut edge " + std::to_string(e));
                 CutRing& r = rings[ri];
                 if (r.src_gpu != r.dst_gpu) SG_RT(cudaStreamWaitEvent(gc.compute, r.ev_copied[slot], 0));
                 io.in.push_back(r.dst_slots[slot]);
@@ -628,7 +633,8 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                     continue;
                 }
                 int ri = -1;
-                for (int r : ring_out[gp]) if (rings[r].edge == e) ri = r;
+                for (int r : ring_out[gp]) if (rings[r].edge == ring_rep[e]) ri = r;
+                if (ri < 0) throw Error(SG_E_PLAN, "internal: no ring for cut edge " + std::to_string(e));
                 CutRing& r = rings[ri];
                 // slot reuse: the copy (or the same-GPU consumer) of fragment fi - depth must be done
                 if (fg >= ring_depth) {

@@ -30,9 +30,10 @@ struct CompiledKernel {
 };
 
 struct CutRing {          // one boundary stream between partitions (a PDG edge member)
-    int edge = -1;
+    int edge = -1;                     // representative cut edge (Plan::ring_rep)
     int group = 0;                     // replica group owning this ring
     int src_part = -1, dst_part = -1;  // -1: graph input / output
+    std::vector<int> dst_parts;        // every consumer partition (a duplicated stream shipped once)
     int src_gpu = 0, dst_gpu = 0;
     int64_t lo = 0, extra = 0, per_iter = 0;
     int64_t slot_items = 0;
@@ -73,6 +74,16 @@ struct Plan {
     bool ilp_optimal = false;
     bool chain_fission = false;            // p.flat is the chain-fissioned graph
     std::vector<PdgEdge> pdg;
+    // cut edges: the edge whose ring carries this edge's items (itself, or -- for outputs of one duplicate
+    // splitter whose consumers sit on the same other GPU -- the lowest such edge: the stream is shipped
+    // once per destination GPU, SURVEY.md 8(c)-4 reading 15); -1 for edges inside a partition
+    std::vector<int> ring_rep;
+    std::vector<int64_t> ring_lo, ring_extra;  // per representative: union of its members' windows
+    void cut_window(int e, int64_t& lo, int64_t& extra) const {
+        const int r = ring_rep.empty() || ring_rep[e] < 0 ? e : ring_rep[e];
+        if (!ring_lo.empty() && ring_rep[e] >= 0) { lo = ring_lo[r]; extra = ring_extra[r]; return; }
+        edge_window(flat, e, lo, extra);
+    }
     // info arrays
     std::vector<int64_t> reps, ninit;
     std::vector<int32_t> node_type, node_kind, node_part, part_gpu, part_mode;

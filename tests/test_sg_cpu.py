@@ -574,9 +574,11 @@ def test_chain_fission_structure(sg, name, m):
         kinds = i["node_kind"]
         assert kinds.count(sg.KINDS["ADD"]) == i0["node_kind"].count(sg.KINDS["ADD"]) + m - 1
         hop = 64.0 if name == "filterbank64" else 8.0
-        pdg = p.pdg()
-        assert len(pdg) == m - 1 and all(b == hop for _, _, b in pdg)
-        assert sorted((a, b) for a, b, _ in pdg) == [(g, g + 1) for g in range(m - 1)]
+        per_pair = {}
+        for a, b, nbytes in p.pdg():      # the forward stream (a duplicate splitter's data) and the accumulator
+            per_pair[(a, b)] = per_pair.get((a, b), 0.0) + nbytes
+        assert sorted(per_pair) == [(g, g + 1) for g in range(m - 1)]
+        assert all(v == hop for v in per_pair.values())
 
 
 def test_chain_fission_rejections(sg):
@@ -602,7 +604,10 @@ def test_planner_picks_chain_for_filterbank(sg, G):
         assert sorted(i["partition_gpu"]) == list(range(G))
         t = i["partition_time"]
         assert max(t) < 1.1 * min(t)
-        assert all(b == 64.0 for _, _, b in p.pdg())
+        per_pair = {}
+        for a, b, nbytes in p.pdg():
+            per_pair[(a, b)] = per_pair.get((a, b), 0.0) + nbytes
+        assert len(per_pair) == G - 1 and all(v == 64.0 for v in per_pair.values())
 
 
 # ------------------------------------------------------------ PEE work
@@ -636,3 +641,26 @@ def test_pee_counts_dead_firings_and_zero_taps_by_hand(sg):
     with sg.plan(cse, 1, plan_only=1, partitioner="single") as p:
         f = p.pee_features(0)
         assert f["cse_nodes"] == 1 and f["flops"] == 6 + 2
+
+
+def test_pdg_counts_duplicated_stream_once_per_gpu(sg):
+    """PDG reading 15: the branches of a duplicate splitter placed on another GPU
+    receive its stream once.  FilterBank 8 with the splitter on GPU 0 and all branches on GPU 1: the
+    4-byte x 8 items/iteration input crosses once (32 B), not once per branch (8 x 32 B); the rank
+    schedule sends one message per fragment for the whole split."""
+    prog = apps.filterbank(8)
+    with sg.plan(prog, 1, plan_only=1, partitioner="single") as p0:
+        n_nodes = p0.info()["n_nodes"]
+    part = [1] * n_nodes
+    part[0] = 0                                   # the duplicate splitter alone in partition 0
+    with sg.plan(prog, 2, plan_only=1, virtual_gpus=1, node_partition=part, link_gbps=1e6,
+                 link_latency_us=0.001, iters_per_fragment=1000) as p:
+        i = p.info()
+        assert i["partition_gpu"][0] != i["partition_gpu"][1]
+        dup = [e for e in p.pdg() if e[0] == 0]
+        assert len(dup) == 1 and dup[0][2] == 32.0
+        src_rank, dst_rank = i["partition_gpu"][0], i["partition_gpu"][1]
+        recvs = [o for o in p.rank_schedule(dst_rank, 3000) if o["op"] == sg.SG_OP_RECV]
+        assert len(recvs) == 3 and all(o["items"] >= 8 * 1000 for o in recvs)
+        sends = [o for o in p.rank_schedule(src_rank, 3000) if o["op"] == sg.SG_OP_SEND]
+        assert len(sends) == 3                    # one message per fragment (3 fragments of 1000)
