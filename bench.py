@@ -47,6 +47,7 @@ WORKLOADS = {
     "bitonicrec32": dict(n=1 << 20, bound="hbm", desc="recursive BitonicSort 32-key int32, 1M iterations"),
     "dct16": dict(n=1 << 18, bound="hbm", desc="2-D DCT-II of 16x16 fp32 blocks (row then column FIR DCTs)"),
     "matmul16": dict(n=1 << 18, bound="hbm", desc="C = A B of streamed 16x16 fp32 matrices (MULTIPLY, ADD)"),
+    "matmul3_16": dict(n=1 << 18, bound="hbm", desc="MatMul3: blocked C = sum_d A_d B_d, 16x16 fp32, 4 K-blocks"),
     # feedback loops: the comb loop is a sequential (wavefront) partition between two FIRs
     "echo64": dict(n=1 << 22, bound="alu", desc="echo: FIR -> feedback loop y = x + 0.5 y[n-64] -> decimating FIR, fp32"),
     "des16": dict(n=1 << 22, bound="int", desc="DES (16 rounds) on a bit-per-item int32 stream, one 64-bit block / iteration"),
@@ -198,6 +199,9 @@ def main():
                     help="--mode pipeline: replica groups (hybrid replica x pipeline plan); -1 = chosen by the cost model")
     ap.add_argument("--cuts", default="",
                     help="comma-separated node ids: user partitions [0, c1), [c1, c2), ... on one GPU (A/B of splits)")
+    ap.add_argument("--chain", type=int, default=0,
+                    help="1 GPU: plan option chain_groups (chain fission of the largest eligible split-join, one "
+                         "partition); 0 = as planned")
     ap.add_argument("--codegen", default="auto", choices=["auto", "register", "staged", "general"],
                     help="plan option codegen_mode (auto: chosen by the code generator)")
     ap.add_argument("--mode", default="pipeline", choices=["replicas", "pipeline"],
@@ -238,6 +242,9 @@ def main():
             kw["threads"] = args.threads
         if args.codegen != "auto":
             kw["codegen_mode"] = args.codegen
+        if args.chain:
+            kw["chain_groups"] = args.chain
+            kw["partitioner"] = "single"
         if args.cuts:
             cuts = [int(c) for c in args.cuts.split(",")]
             with sg.plan(prog, 1, plan_only=1) as p0:

@@ -2947,6 +2947,34 @@ private:
                 for (auto& h : fg_) if (h.level == L) nlev_groups++;
                 static const bool fetchbar = std::getenv("SG_FETCHBAR") != nullptr;  // measured neutral-to-worse
                 const bool lockstep = fetchbar && nlev_groups == 1 && g.NB <= NT_ && g.flops_block >= 2048;
+                // warp sub-groups: a group of many sibling roots (FilterBank: 64 FIR_H on one window) is
+                // split into K contiguous root ranges, warp w running range w mod K over every block, so
+                // each warp scheduler streams ~1/K of the level's straight-line code (instruction-fetch
+                // locality: L0 ~6 KB, L1.5 ~32 KB per SM) at the cost of K reloads of the shared window
+                static const int ksub_env = std::getenv("SG_SUBGROUPS") ? std::atoi(std::getenv("SG_SUBGROUPS")) : 0;
+                const int ksub = ksub_env;
+                if (!lockstep && ksub > 1 && (int)g.roots.size() >= 2 * ksub && NT_ % (32 * ksub) == 0) {
+                    b << "      const int sgw = (tid >> 5) % " << ksub << ";\n"
+                      << "      const int tsg = ((tid >> 5) / " << ksub << ") * 32 + (tid & 31);\n";
+                    const size_t nr = g.roots.size();
+                    for (int q = 0; q < ksub; q++) {
+                        FGroup h = g;
+                        h.roots.assign(g.roots.begin() + nr * q / ksub, g.roots.begin() + nr * (q + 1) / ksub);
+                        Sym cq;
+                        cq.dry = false;
+                        cq.os = &b;
+                        cq.nv = &nvar_;
+                        cq.guarded = guarded;
+                        b << "      " << (q ? "else " : "") << "if (sgw == " << q << ") {\n"
+                          << "      for (int jb = tsg; jb < NBg; jb += " << NT_ / ksub << ") {\n";
+                        sym_block(cq, h, true);
+                        if (cq.runtime) throw FusedFail();
+                        b << "      }\n      }\n";
+                    }
+                    b << "    }\n";
+                    rot += g.NB;
+                    continue;
+                }
                 Sym c;
                 c.dry = false;
                 c.os = &b;

@@ -106,7 +106,7 @@ def test_parity_bitonic_edge_sizes(oracle_lib, n):
 
 
 # ---- second workloads of the paper's suite: BitonicRec, DCT, MatMul
-EXTRA_N = {"bitonicrec32": (3 * 256 + 5, 20000), "dct16": (37, 5000), "matmul16": (41, 5000),
+EXTRA_N = {"bitonicrec32": (3 * 256 + 5, 20000), "dct16": (37, 5000), "matmul16": (41, 5000), "matmul3_16": (29, 3000),
            "des16": (3 * 256 + 5, 20000)}
 
 

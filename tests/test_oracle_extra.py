@@ -134,6 +134,33 @@ def test_matmul_identity_and_permutation(oracle_lib):
     assert np.array_equal(y[1], A[:, ::-1])
 
 
+@pytest.mark.parametrize("M,K,N,D", [(16, 16, 16, 4), (3, 6, 5, 2), (4, 8, 2, 8)])
+def test_matmul3_vs_numpy(oracle_lib, M, K, N, D):
+    """MatMul3 (blocked): each of the D block dot products within gamma(K/D), their sum within one more
+    gamma(D) -- bounded by gamma(K/D + D) |A| |B|."""
+    prog = apps.matmul_block(M, K, N, D)
+    n = 5
+    x = inputs.make_input("f32", (M * K + K * N) * n, M * 1000 + K * 100 + N * 10 + D)
+    y = oracle_lib.run(prog, x, n).reshape(n, M, N).astype(np.float64)
+    for i, (A, B) in enumerate(_mm_blocks(x, M, K, N, n)):
+        bound = gamma(K // D + D) * (np.abs(A) @ np.abs(B)) + 1e-30
+        assert np.all(np.abs(y[i] - A @ B) <= bound)
+
+
+def test_matmul3_exact_small_integers_and_block_order(oracle_lib):
+    """Exact on small integers; and with D = 1 the blocked graph is MatMul2 bit for bit (same order)."""
+    M, K, N = 16, 16, 16
+    n = 4
+    rng = np.random.default_rng(31)
+    x = rng.integers(-7, 8, size=(M * K + K * N) * n).astype(np.float32)
+    y = oracle_lib.run(apps.matmul_block(M, K, N, 4), x, n).reshape(n, M, N)
+    for i, (A, B) in enumerate(_mm_blocks(x, M, K, N, n)):
+        assert np.array_equal(y[i], (A @ B).astype(np.float32))
+    xf = inputs.make_input("f32", (M * K + K * N) * n, 5)
+    assert oracle_lib.run(apps.matmul_block(M, K, N, 1), xf, n).tobytes() == oracle_lib.run(
+        apps.matmul(M, K, N), xf, n).tobytes()
+
+
 def test_multiply_is_float32_product(oracle_lib):
     prog = Program("mul", "f32", Pipeline([Filter("MULTIPLY")]))
     x = inputs.make_input("f32", 2 * 1000, 4)

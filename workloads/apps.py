@@ -230,6 +230,26 @@ def matmul(M: int = 16, K: int = 16, N: int = 16) -> Program:
                    note="one iteration = A (M x K) then B (K x N), row-major -> C = A B (M x N), row-major")
 
 
+def matmul_block(M: int = 16, K: int = 16, N: int = 16, D: int = 4) -> Program:
+    """MatMul3 (Fig. 4.2f, 1210; the paper gives no structure): StreamIt's blocked form of the
+    product [DECISION].  K is cut into D blocks of K/D; branch d selects A[:, block d] and B[block d, :]
+    (a PERMUTE of the iteration's A | B items), forms the block product with the MatMul2 core (pairs,
+    MULTIPLY, ADD(K/D)), and the D partial products are summed element-wise: duplicate split -> D branches
+    -> roundrobin(1) join -> ADD(D).  Rounding order: each block's dot product, then the block sums."""
+    assert K % D == 0
+    Kc = K // D
+    branches = []
+    for d in range(D):
+        idx = [i * K + d * Kc + k for i in range(M) for k in range(Kc)]                  # A[:, block d]
+        idx += [M * K + (d * Kc + k) * N + j for k in range(Kc) for j in range(N)]      # B[block d, :]
+        core = matmul(M, Kc, N).top
+        branches.append(Pipeline([Filter("PERMUTE", [M * K + K * N] + idx)] + list(core.children)))
+    return Program(f"matmul3_{M}x{K}x{N}_d{D}", "f32",
+                   Pipeline([SplitJoin("dup", branches, join_w=[1] * D), Filter("ADD", [D])]),
+                   note="one iteration = A (M x K) then B (K x N), row-major -> C = sum over D K-blocks of "
+                        "A_d B_d (M x N), row-major")
+
+
 # -------------------------------------------------------------------------- DES
 # FIPS 46-3 tables (1-based bit numbers, bit 1 = most significant), written as the
 # StreamIt DES init blocks hold them.  The graph works on a bit-per-item stream like
@@ -343,6 +363,7 @@ EXTRA = {
     "bitonicrec32": lambda: bitonic_rec(32),
     "dct16": lambda: dct2d(16),
     "matmul16": lambda: matmul(16, 16, 16),
+    "matmul3_16": lambda: matmul_block(16, 16, 16, 4),
     "des16": lambda: des(16),
 }
 

@@ -39,7 +39,7 @@ def keys_i32(seed: int, count: int, start: int = 0) -> np.ndarray:
 # Per-config default seeds.
 SEEDS = {"fft64": 0xF0F1, "bitonic32": 0xB170, "fmradio10": 0xF3,
          "beamformer12x4": 0xBEA3, "filterbank64": 0xFB64,
-         "bitonicrec32": 0xB1C, "dct16": 0xDC7, "matmul16": 0x3A7, "des16": 0xDE5, "echo64": 0xEC0}
+         "bitonicrec32": 0xB1C, "dct16": 0xDC7, "matmul16": 0x3A7, "matmul3_16": 0x3A3, "des16": 0xDE5, "echo64": 0xEC0}
 
 
 def make_input(dtype: str, count: int, seed: int, variant: str = "uniform", block: int = 32) -> np.ndarray:
