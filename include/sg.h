@@ -362,7 +362,11 @@ int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst,
  *   (after view resolution, dead-firing elimination, zero-tap pruning and CSE), 2 integer ops, 3 fp64 ops,
  *   4 items read by live firings, 5 items written, 6 live firings, 7 boundary input bytes, 8 boundary
  *   output bytes, 9 compute levels, 10 halo firings per tile, 11 loop firings, 12 CSE duplicate nodes,
- *   13 frame FIRs present (0/1), 14 bitslice mode (0/1), 15 the PEE estimate (ns).
+ *   13 frame FIRs present (0/1), 14 bitslice mode (0/1), 15 the plan's estimate T(p) (ns; sg_plan_info's
+ *   partition_time), 16 boundary input edges, 17 boundary output edges, 18 items of one iteration at the
+ *   boundary (register mode: one thread's row); from the generated kernel (-1 for plan_only plans):
+ *   19 staged fused path taken (0/1), 20 iterations per tile, 21 threads per CTA, 22 dynamic shared memory
+ *   bytes, 23 CUDA source bytes.
  * Returns the number of values written, or -1 (NULL plan / bad partition). */
 int32_t sg_pee_features(const sg_plan_t* p, int32_t part, double* out, int32_t cap);
 

@@ -2888,7 +2888,11 @@ private:
             }
             scored.push_back({tile / (double)W, (int)W});
         }
-        std::sort(scored.begin(), scored.end());
+        // equal cost per iteration (e.g. a partition of views only, no compute level): the larger tile
+        // amortises the per-tile halo, barriers and loop overhead
+        std::sort(scored.begin(), scored.end(), [](const std::pair<double, int>& a, const std::pair<double, int>& b) {
+            return a.first != b.first ? a.first < b.first : a.second > b.second;
+        });
         std::vector<int> out;
         for (auto& p : scored) out.push_back(p.second);
         return out;

@@ -170,6 +170,9 @@ PartitionWork partition_work(const Flat& f, const std::vector<int>& nodes) {
     partition_boundary(f, nodes, ins, outs);
     for (int e : ins) w.in_bytes += 4.0 * f.edges[e].per_iter;
     for (int e : outs) w.out_bytes += 4.0 * f.edges[e].per_iter;
+    w.in_edges = (int)ins.size();
+    w.out_edges = (int)outs.size();
+    w.row_items = (w.in_bytes + w.out_bytes) / 4.0;
     // a reference iteration far from the stream start (every firing index positive)
     int64_t K = 1;
     for (int v : nodes) {

@@ -17,6 +17,8 @@ struct PartitionWork {
     double reads = 0, writes = 0;             // items read (non-zero peek items) / written by live firings
     double firings = 0;                       // live firings
     double in_bytes = 0, out_bytes = 0;       // boundary streams
+    int in_edges = 0, out_edges = 0;          // boundary edges (each a load / store stream of its own)
+    double row_items = 0;                     // register mode: items of one iteration held by one thread
     double halo_firings = 0;                  // firings recomputed per tile (peek halos)
     double loop_firings = 0;                  // feedback loops: sequential firings per iteration
     int levels = 0;                           // longest chain of compute nodes

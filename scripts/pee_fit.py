@@ -21,7 +21,7 @@ sys.path.insert(0, ROOT)
 sys.path.insert(0, os.path.join(ROOT, "scripts"))
 
 
-def features(rows):
+def features(rows, plan_only=1):
     from paper_conf_cgo_nguyenl16_b200 import sg
     from pee_calibrate import program
     out = []
@@ -38,7 +38,7 @@ def features(rows):
         kw.pop("partitioner", None)
         if r.get("chain_fission") and kw.get("chain_groups", 0) < 2:
             kw["chain_groups"] = r["G"]        # the planner fissions into G / replicas = G groups
-        with sg.plan(program(r["config"]), r["G"], plan_only=1, **kw) as p:
+        with sg.plan(program(r["config"]), r["G"], plan_only=plan_only, **kw) as p:
             info = p.info()
             for k in range(info["n_partitions"]):
                 f = p.pee_features(k)

@@ -13,6 +13,8 @@ runtime):
 Each output must be BIT-IDENTICAL to the one-partition output (Kahn determinism; every rewrite is
 order-preserving), and sampled windows plus the stream start must match the oracle.
 """
+import zlib
+
 import numpy as np
 import pytest
 
@@ -22,6 +24,8 @@ from test_gpu_parity import assert_parity
 pytestmark = pytest.mark.gpu
 
 N_FULL = {"filterbank64": 1 << 20, "fmradio10": 1 << 24, "beamformer12x4": 4096}
+# input items for n iterations (closed forms; the oracle's in_items bisects whole runs)
+IN_ITEMS = {"filterbank64": lambda n: 8 * n, "fmradio10": lambda n: 379 + 5 * n, "beamformer12x4": lambda n: 24576 * n}
 CASES = [("filterbank64", 2), ("filterbank64", 4), ("filterbank64", 8),
          ("beamformer12x4", 2), ("beamformer12x4", 4), ("fmradio10", 2)]
 
@@ -44,7 +48,7 @@ def _run(prog, xd, n, n_gpus, **kw):
 
 
 def _sampled_vs_oracle(oracle_lib, name, prog, x, y, n):
-    rng = np.random.default_rng(hash(name) % 1000)
+    rng = np.random.default_rng(zlib.crc32(name.encode()))
     if name == "filterbank64":       # 8 in / 8 out per iteration; FIR memory < 8 iterations
         warm, m = 8, 16
         for s in list(rng.choice(n - m - warm, 12, replace=False)) + [n - m - warm]:
@@ -67,7 +71,7 @@ def test_pipelined_plans_full_size(oracle_lib, name, G):
     torch = _torch()
     prog = apps.CONFIGS[name]()
     n = N_FULL[name]
-    x = inputs.make_input("f32", oracle_lib.in_items(prog, n), inputs.SEEDS[name])
+    x = inputs.make_input("f32", IN_ITEMS[name](n), inputs.SEEDS[name])
     xd = torch.from_numpy(x).cuda()
     base, _ = _run(prog, xd, n, 1)
     _sampled_vs_oracle(oracle_lib, name, prog, x, base, n)
