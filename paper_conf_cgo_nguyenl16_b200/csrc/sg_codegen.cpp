@@ -487,7 +487,10 @@ public:
         std::ostringstream src;
         src << header(demand_ ? "register, demand-ordered" : "register") << consts_.str() << args_struct();
         if (demand_) src << "#define SG_LDV(r) (*(volatile const " << T_ << "*)&SG_LD1(r))\n";
-        if (demand_) return run_demand(ki, src, VT4, opt);
+        if (demand_) {
+            ki.reg_variant = 2;
+            return run_demand(ki, src, VT4, opt);
+        }
         // ---------------- variant 1: synchronous tiles (any alignment / row size)
         int bytes_per_thread = (int)((RIN_S_ + ROUT_S_) * 4);
         int NT = opt.threads;
@@ -544,6 +547,7 @@ public:
         ki.off_in = off_in_;
         ki.off_out = off_out_;
         if (opt.mode != -1 && try_inplace(ki, src, VT4)) {
+            ki.reg_variant = 1;
             // in-place component kernel generated
         } else if (ki.tma_in && ki.tma_out && opt.mode != -1) {
             auto stage_bytes = [&](int lay, int64_t P, int64_t RS, int rows) -> int64_t {

@@ -39,6 +39,8 @@ struct KernelInfo {
     int threads_sync = 0, tile_sync = 0;
     size_t smem_sync = 0;
     bool fused = false;              // staged mode: fused fast path present
+    int reg_variant = 0;             // register mode: 0 TMA / synchronous rows, 1 in-place components (bulk
+                                     // copies), 2 demand-ordered wide single-component rows
     int64_t flops_exec_per_iter = -1;  // fused: algorithmic flops after dead/zero pruning (no recompute)
     std::string name_start;          // staged fused: stream-start variant (tiles with k0 < ksafe)
     int64_t ksafe = 0;

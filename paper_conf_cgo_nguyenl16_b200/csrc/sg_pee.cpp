@@ -21,6 +21,9 @@
 // those firings (the shared-memory traffic of the staged kernels).
 #include <algorithm>
 #include <cstring>
+#include <functional>
+#include <map>
+#include <set>
 #include <unordered_map>
 #include <unordered_set>
 
@@ -156,7 +159,7 @@ void firing_work(const Flat& f, int v, int64_t nz, double& fl, double& io, doubl
 }
 }  // namespace
 
-PartitionWork partition_work(const Flat& f, const std::vector<int>& nodes) {
+PartitionWork partition_work(const Flat& f, const std::vector<int>& nodes, bool components) {
     PartitionWork w;
     const int N = (int)f.nodes.size();
     std::vector<char> in(N, 0);
@@ -232,6 +235,51 @@ PartitionWork partition_work(const Flat& f, const std::vector<int>& nodes) {
                 }
             }
         }
+    }
+    // ---- 1b. dependence components of one iteration (register mode picks its kernel variant by them:
+    // one wide component -> the demand-ordered kernel): outputs whose cones share an input item
+    if (components) {
+        std::map<std::pair<int, int64_t>, int> id;
+        std::vector<int> uf;
+        auto get = [&](int e, int64_t pos) {
+            auto it = id.find({e, pos});
+            if (it != id.end()) return it->second;
+            int k = (int)uf.size();
+            uf.push_back(k);
+            id[{e, pos}] = k;
+            return k;
+        };
+        std::function<int(int)> find = [&](int x) { return uf[x] == x ? x : uf[x] = find(uf[x]); };
+        auto unite = [&](int a, int b) { a = find(a); b = find(b); if (a != b) uf[a] = b; };
+        std::vector<int> out_ids;
+        for (int e : outs) {
+            const Edge& ed = f.edges[e];
+            const Node& s0 = f.nodes[ed.src];
+            const int64_t p0 = ed.pre + (s0.ninit + K * s0.rep) * ed.push;
+            for (int64_t i = 0; i < ed.per_iter; i++) {
+                const int me = get(-2 - e, p0 + i);
+                out_ids.push_back(me);
+                std::set<std::pair<int, int64_t>> seen;
+                std::vector<Item> st{R.resolve(e, p0 + i)};
+                while (!st.empty()) {
+                    Item x = st.back();
+                    st.pop_back();
+                    if (x.k != Item::PHYS) continue;
+                    int u;
+                    int64_t g;
+                    producer(x, u, g);
+                    if (u < 0) { unite(me, get(x.edge, x.pos)); continue; }
+                    if (!seen.insert({u, g}).second) continue;
+                    for (int ie : f.nodes[u].in) {
+                        const Edge& ied = f.edges[ie];
+                        for (int64_t q = 0; q < ied.peek; q++) st.push_back(R.resolve(ie, g * ied.pop + q));
+                    }
+                }
+            }
+        }
+        std::set<int> roots;
+        for (int o : out_ids) roots.insert(find(o));
+        w.components = (int)roots.size();
     }
     // ---- 2. work per live firing, zero taps pruned, CSE duplicates skipped (producers first)
     std::unordered_map<int, int> cls;           // node -> class representative

@@ -36,19 +36,51 @@ constexpr double kInt = kSM * 64 * kClk;          // int min/max per s
 constexpr double kFp64 = 37e12;                   // flop/s
 constexpr double kSmem = kSM * 128 * kClk;        // bytes/s
 constexpr double kHbm = 6.5536e12;                // bytes/s (MEASURED_PEAKS.json copy)
-constexpr double kLaunch = 4e-6;                  // s per kernel launch
+constexpr double kLaunch = 10e-6;                 // s per kernel launch incl. ramp / tail (fitted: c_l)
 constexpr double kFragIters = 65536;              // iterations per fragment (estimate)
-constexpr double kTileEst = 64;                   // iterations per staged tile (estimate)
-// model constants, per iteration (fitted to measured partition times: see DESIGN.md, PEE)
-constexpr double kEffReg = 0.8;                   // register mode: fraction of the fp32 peak
-constexpr double kEffStaged = 0.6;                // staged fused kernels
-constexpr double kEffFrame = 0.3;                 // frame FIR kernels
-constexpr double kSmemItem = 0.0;                 // SM cycles per item read / written by live firings
-constexpr double kLevel = 1.0e-9;                 // GPU-seconds per compute level per tile (barrier + drain,
-                                                  // ~500 cycles spread over ~300 resident CTAs)
 constexpr double kLoopFiring = 25e-9;             // s per sequential loop firing
-constexpr double kFixed = 0.0;                    // ns per iteration per partition
 constexpr long long kIlpNodeBudget = 4000000;     // branch-and-bound nodes per mapping (deterministic)
+
+// Model constants, fitted by least squares on log time to 399 measured partitions (scripts/pee_fit.py
+// over profiles/pee_corpus_r02.json; the paper fits its C1, C2 the same way).  Two
+// sets: the plan-time estimate (Algorithm 1, ILP; kernel variant and tile inferred from the work), and
+// the estimate refined with the generated kernel's own decisions (fused path, tile, variant).
+struct PeeModel {
+    double e_reg;      // register mode: fraction of the fp32 peak
+    double c_row;      // register rows: ns per (items of one iteration)^2 (one thread holds the row)
+    double c_demand;   // demand-ordered wide single-component rows: ns per items^2
+    double e_staged;   // staged fused kernels: fraction of the fp32 peak
+    double e_frame;    // frame FIRs
+    double e_general;  // staged general path (fused path declined)
+    double c_edge;     // ns per boundary edge per tile
+    double c_level;    // ns per compute level per tile
+};
+constexpr PeeModel kPlanModel{0.8, 2.839e-6, 1.392e-5, 0.6069, 0.3068, 0.6069, 5.878, 0.09224};
+constexpr PeeModel kKernelModel{0.8, 2.741e-6, 1.128e-5, 0.9937, 0.3469, 0.07126, 0.9232, 7.397};
+
+struct KernelShape {  // the code generator's decisions the model needs
+    bool demand = false, inplace = false, fused = true;
+    double tile = 1;
+};
+
+double model_ns(const PartitionWork& w, int mode, bool bitslice, double bitslice_ops, const KernelShape& k,
+                const PeeModel& m) {
+    const double hbm = (w.in_bytes + w.out_bytes) / kHbm * 1e9;
+    if (bitslice) return std::max(bitslice_ops / kInt * 1e9, hbm);
+    if (mode == 4) return std::max(kLoopFiring * w.loop_firings * 1e9, hbm);
+    if (mode == 1) {
+        const double row2 = w.row_items * w.row_items;
+        if (k.demand) return std::max(hbm, m.c_demand * row2);
+        const double tc = (w.flops / (kFp32 * m.e_reg) + w.intops / kInt + w.dfma * 80.0 / kFp64) * 1e9;
+        return std::max({tc, hbm, k.inplace ? 0.0 : m.c_row * row2});
+    }
+    const double e = k.fused ? (w.frame ? m.e_frame : m.e_staged) : m.e_general;
+    const double W = std::max(1.0, k.tile);
+    const double recompute = 1.0 + w.halo_firings / (W * std::max(1.0, w.firings));
+    const double tc = (w.flops / (kFp32 * e) + w.intops / kInt + w.dfma * 80.0 / kFp64) * recompute * 1e9 +
+                      kLoopFiring * w.loop_firings * 1e9;
+    return std::max(tc, hbm) + m.c_edge * (w.in_edges + w.out_edges) / W + m.c_level * (w.levels + 1) / W;
+}
 }  // namespace
 
 PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
@@ -57,44 +89,42 @@ PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
     for (int v : nodes) loop = loop || f.nodes[v].type == N_LOOP;
     est.mode = loop && nodes.size() == 1 ? 4 : (register_mode_eligible(f, nodes, nullptr) ? 1 : 2);
     est.bitslice = est.mode == 1 && bitslice_eligible(f, nodes, nullptr);
-    est.work = partition_work(f, nodes);
+    est.work = partition_work(f, nodes, est.mode == 1 && !est.bitslice);
     const PartitionWork& w = est.work;
-    const double bytes = w.in_bytes + w.out_bytes;
-    double tc = 0;
     if (est.bitslice) {
         // bitslice mode: one LOP3 covers 32 iterations; an S-box is a ~44-gate circuit, a word <-> bits
         // conversion a share of a 32x32 transpose (~5 ops per bit)
-        double ops = 0;
         for (int v : nodes) {
             const Node& n = f.nodes[v];
             if (n.type != N_FILTER) continue;
             switch (n.kind) {
-            case SG_K_XOR: case SG_K_XOR_CONST: ops += (double)n.rep * n.iv[0] / 32.0; break;
-            case SG_K_SBOX: ops += (double)n.rep * 44.0 / 32.0; break;
-            case SG_K_INTO_BITS: case SG_K_BITS_TO_INT: ops += (double)n.rep * 5.0; break;
+            case SG_K_XOR: case SG_K_XOR_CONST: est.bitslice_ops += (double)n.rep * n.iv[0] / 32.0; break;
+            case SG_K_SBOX: est.bitslice_ops += (double)n.rep * 44.0 / 32.0; break;
+            case SG_K_INTO_BITS: case SG_K_BITS_TO_INT: est.bitslice_ops += (double)n.rep * 5.0; break;
             default: break;
             }
         }
-        tc = ops / kInt;
-    } else if (est.mode == 1) {
-        // register mode: every FIFO item a register, one thread per iteration
-        tc = w.flops / (kFp32 * kEffReg) + w.intops / kInt + w.dfma * 80.0 / kFp64;
-    } else if (est.mode == 4) {
-        tc = kLoopFiring * w.loop_firings;
-    } else {
-        // staged mode: executed FP work at the fused kernels' efficiency, plus the shared-memory
-        // traffic of the live firings (reads of peek windows, writes of materialised outputs), the
-        // per-level barriers and the halo firings recomputed by every tile
-        const double eff = w.frame ? kEffFrame : kEffStaged;
-        const double recompute = 1.0 + w.halo_firings / (kTileEst * std::max(1.0, w.firings));
-        tc = (w.flops / (kFp32 * eff) + w.intops / kInt + w.dfma * 80.0 / kFp64) * recompute +
-             kSmemItem * (w.reads + w.writes) / (kSM * kClk) + kLevel * (double)w.levels / kTileEst +
-             kLoopFiring * w.loop_firings;
     }
-    est.t_comp = tc * 1e9;
-    est.t_dt = bytes / kHbm * 1e9;
-    est.t = std::max(est.t_comp, est.t_dt) + kFixed;  // ns per iteration (the max() of Eq. III.8)
+    // the kernel shape the code generator will pick, inferred: register rows of one wide dependence
+    // component are demand-ordered (>= 384 items, sg_codegen.cpp), several components run in place;
+    // staged tiles hold ~150k live firings' worth of iterations (frame FIRs: one frame)
+    KernelShape k;
+    k.demand = est.mode == 1 && w.row_items >= 384 && w.components == 1;
+    k.inplace = est.mode == 1 && w.components > 1;
+    k.tile = w.frame ? 1.0 : std::min(4096.0, std::max(1.0, 150000.0 / std::max(1.0, w.firings)));
+    est.t = model_ns(w, est.mode, est.bitslice, est.bitslice_ops, k, kPlanModel);
+    est.t_dt = (w.in_bytes + w.out_bytes) / kHbm * 1e9;
+    est.t_comp = est.t;
     return est;
+}
+
+double pee_refine(const PeeEstimate& est, const KernelInfo& ki) {
+    KernelShape k;
+    k.demand = ki.mode == 1 && ki.reg_variant == 2;
+    k.inplace = ki.mode == 1 && ki.reg_variant == 1;
+    k.fused = ki.mode != 2 || ki.fused;
+    k.tile = std::max(1, ki.tile);
+    return model_ns(est.work, est.mode, est.bitslice, est.bitslice_ops, k, kKernelModel);
 }
 
 double launch_ns_per_iter(int64_t frag) { return kLaunch / (double)(frag > 0 ? frag : (int64_t)kFragIters) * 1e9; }
@@ -405,9 +435,35 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
         return best;
     }
     // branch and bound: partitions by decreasing T; LPT incumbent
+    // interchangeable partitions (same T, the same PDG edges to the same other partitions, none between
+    // them): classes; members are branched consecutively and in non-decreasing GPU order (symmetry
+    // breaking: sorting a consecutive run of identical jobs keeps first-use GPU labels valid)
+    std::vector<int> cls(P);
+    {
+        std::vector<std::vector<std::tuple<int, double, int, int>>> sig(P);
+        for (auto& e : pdg) {
+            if (e.src == e.dst) continue;
+            sig[e.src].push_back(std::make_tuple(e.dst, e.bytes, 1, e.data));
+            sig[e.dst].push_back(std::make_tuple(e.src, e.bytes, 0, e.data));
+        }
+        for (auto& v : sig) std::sort(v.begin(), v.end());
+        std::map<std::pair<double, std::vector<std::tuple<int, double, int, int>>>, int> ids;
+        for (int i = 0; i < P; i++) {
+            auto key = std::make_pair(T[i], sig[i]);
+            auto it = ids.find(key);
+            cls[i] = it == ids.end() ? (ids[key] = i) : it->second;
+        }
+        for (auto& e : pdg)  // members adjacent to each other are not interchangeable
+            if (e.src != e.dst && cls[e.src] == cls[e.dst]) {
+                const int c = cls[e.src];
+                for (int i = 0; i < P; i++) if (cls[i] == c) cls[i] = i;
+            }
+    }
     std::vector<int> ord(P);
     std::iota(ord.begin(), ord.end(), 0);
-    std::stable_sort(ord.begin(), ord.end(), [&](int x, int y) { return T[x] > T[y]; });
+    std::stable_sort(ord.begin(), ord.end(), [&](int x, int y) {
+        return T[x] != T[y] ? T[x] > T[y] : cls[x] < cls[y];
+    });
     {
         std::vector<int> a(P, 0);
         std::vector<double> gl(G, 0);
@@ -484,7 +540,8 @@ MapResult map_partitions(const std::vector<double>& T, const std::vector<PdgEdge
         }
         int i = ord[k];
         int gmax = symmetric ? std::min(G - 1, used) : G - 1;
-        for (int g = 0; g <= gmax; g++) {
+        const int gmin = k > 0 && cls[ord[k - 1]] == cls[i] ? a[ord[k - 1]] : 0;
+        for (int g = gmin; g <= gmax; g++) {
             a[i] = g;
             gl[g] += T[i];
             double c = std::max(cur, gl[g]);
@@ -712,7 +769,7 @@ Flat fissioned(const Flat& f, int sj, int m) {
 struct Candidate {
     int variant = 0;
     std::vector<std::vector<int>> parts;
-    double tmax = 0;
+    double tmax = 0, maxload = 0;
 };
 GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, int Gs, const sg_plan_opts& o);
 
@@ -749,7 +806,13 @@ Candidate best_candidate(const std::vector<Flat>& variants, int Gs, const sg_pla
                 for (size_t i = 0; i < parts.size() && i < 24; i++) std::fprintf(stderr, " %.3f/%zu", gm.T[i], parts[i].size());
                 std::fprintf(stderr, "\n");
             }
-            if (!have || gm.m.tmax < best.tmax * (1 - 1e-9)) {
+            // ties on Tmax (e.g. every candidate bound by the same link): the smaller largest GPU load
+            std::vector<double> load(Gs, 0.0);
+            for (size_t i = 0; i < parts.size(); i++) load[gm.m.assign[i]] += gm.T[i];
+            const double maxload = *std::max_element(load.begin(), load.end());
+            const bool tie = have && std::fabs(gm.m.tmax - best.tmax) <= 1e-9 * std::max(1.0, best.tmax);
+            if (!have || gm.m.tmax < best.tmax * (1 - 1e-9) || (tie && maxload < best.maxload * (1 - 1e-9))) {
+                best.maxload = maxload;
                 have = true;
                 best.variant = vi;
                 best.parts = parts;
@@ -905,9 +968,10 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     p.part_time.assign(P, 0.0);
     p.part_mode.assign(P, 0);
     std::vector<double> T(P);
+    std::vector<PeeEstimate> ests(P);
     for (int i = 0; i < P; i++) {
         p.parts[i].nodes = parts[i];
-        PeeEstimate est = pee_estimate(f, parts[i]);
+        PeeEstimate est = ests[i] = pee_estimate(f, parts[i]);
         p.parts[i].t_est = T[i] = est.t;
         p.parts[i].t_comp = est.t_comp;
         p.parts[i].t_dt = est.t_dt;
@@ -983,6 +1047,8 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         p.parts[i].gpu = p.part_gpu[i];
         p.parts[i].tile = p.kernels[i].ki.tile;
         p.parts[i].threads = p.kernels[i].ki.threads;
+        // the PEE with the generated kernel's own decisions (static discrepancy)
+        p.parts[i].t_est = p.part_time[i] = pee_refine(ests[i], p.kernels[i].ki);
     }
     // ---- info arrays
     p.reps.resize(N);

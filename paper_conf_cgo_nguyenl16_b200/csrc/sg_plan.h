@@ -19,22 +19,28 @@ struct PartitionWork {
     double in_bytes = 0, out_bytes = 0;       // boundary streams
     int in_edges = 0, out_edges = 0;          // boundary edges (each a load / store stream of its own)
     double row_items = 0;                     // register mode: items of one iteration held by one thread
+    int components = 0;                       // register-eligible: independent dependence components of an
+                                              // iteration (outputs sharing no input item); 0 otherwise
     double halo_firings = 0;                  // firings recomputed per tile (peek halos)
     double loop_firings = 0;                  // feedback loops: sequential firings per iteration
     int levels = 0;                           // longest chain of compute nodes
     int cse_nodes = 0;                        // compute nodes found identical to an earlier one
     bool frame = false;                       // contains frame FIRs (BEAM_FIR)
 };
-PartitionWork partition_work(const Flat& f, const std::vector<int>& nodes);
+PartitionWork partition_work(const Flat& f, const std::vector<int>& nodes, bool components = false);
 
 struct PeeEstimate {
     double t = 0, t_comp = 0, t_dt = 0;
     int mode = 0;
     bool bitslice = false;
+    double bitslice_ops = 0;  // bitslice mode: 32-lane ALU ops per iteration
     PartitionWork work;
     bool io_bound() const { return t_dt >= t_comp; }
 };
 PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes);
+// The estimate refined with the generated kernel's own decisions (fused path, tile, register variant):
+// ns per iteration, steady state (no launch term).
+double pee_refine(const PeeEstimate& est, const KernelInfo& ki);
 double launch_ns_per_iter(int64_t iters_per_fragment);  // per-fragment kernel launch, amortised per iteration
 
 // The paper's analytic model Eq. III.8-III.12, kept as a

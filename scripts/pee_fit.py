@@ -21,7 +21,7 @@ sys.path.insert(0, ROOT)
 sys.path.insert(0, os.path.join(ROOT, "scripts"))
 
 
-def features(rows, plan_only=1):
+def features(rows, plan_only=0):
     from paper_conf_cgo_nguyenl16_b200 import sg
     from pee_calibrate import program
     out = []
@@ -42,8 +42,11 @@ def features(rows, plan_only=1):
             info = p.info()
             for k in range(info["n_partitions"]):
                 f = p.pee_features(k)
+                # the estimate of a kernel run alone over n iterations: steady state + one launch (ramp, tail)
                 f.update(config=r["config"], G=r["G"], kw=r["kw"], part=k, meas=r["meas_ns_per_iter"][k],
-                         est=info["partition_time"][k], nodes=sum(1 for q in info["node_partition"] if q == k))
+                         est_steady=info["partition_time"][k], n=r["n_iters"],
+                         est=info["partition_time"][k] + LAUNCH_NS / r["n_iters"],
+                         nodes=sum(1 for q in info["node_partition"] if q == k))
                 out.append(f)
     os.environ.pop("SG_A1_CAPS", None)
     return out
@@ -56,6 +59,8 @@ def r2(xs, ys):
     sxy = sum((x - mx) * (y - my) for x, y in zip(xs, ys))
     return (sxy * sxy / (sxx * syy)) if sxx > 0 and syy > 0 else float("nan")
 
+
+LAUNCH_NS = 10e3   # sg_plan.cpp kLaunch: one kernel launch including ramp-up and tail
 
 # staged-mode model (sg_plan.cpp pee_estimate), all times in ns per iteration
 FP32 = 148 * 128 * 2 * 1.9e9

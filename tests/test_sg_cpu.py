@@ -664,3 +664,20 @@ def test_pdg_counts_duplicated_stream_once_per_gpu(sg):
         assert len(recvs) == 3 and all(o["items"] >= 8 * 1000 for o in recvs)
         sends = [o for o in p.rank_schedule(src_rank, 3000) if o["op"] == sg.SG_OP_SEND]
         assert len(sends) == 3                    # one message per fragment (3 fragments of 1000)
+
+
+@pytest.mark.parametrize("name", list(apps.CONFIGS))
+@pytest.mark.parametrize("G", [2, 4, 8])
+def test_ilp_exact_for_every_config(sg, name, G):
+    """The branch and bound (Eq. III.1-III.7) proves optimality for every BASELINE
+    config at G = 2/4/8 within its deterministic node budget (the paper: Gurobi within 10 s,
+    PAPER.md:651-652); HBM-bound graphs stay one partition (any NVLink cut is slower than one GPU,
+    SURVEY.md 8(e)); FMRadio takes the 8 B/iteration chain cut at G = 2."""
+    with sg.plan(apps.CONFIGS[name](), G, plan_only=1, virtual_gpus=1, replicas=1) as p:
+        i = p.info()
+        assert i["ilp_optimal"]
+        if name in ("fft64", "bitonic32"):
+            assert i["n_partitions"] == 1
+        if name == "fmradio10" and G == 2:
+            assert i["chain_fission"] and i["n_partitions"] == 2
+            assert sum(b for _, _, b in p.pdg()) == 8.0
