@@ -2552,6 +2552,9 @@ private:
             if (boundary || comp.size() != 1) continue;
             int v = *comp.begin();
             if (special(v)) continue;
+            // opt-in (A/B): keep an accumulate chain's partial sums materialised, one level per group
+            static const bool keep_acc = std::getenv("SG_KEEP_ACC") != nullptr;
+            if (keep_acc && f_.nodes[u].kind == SG_K_ADD && f_.nodes[v].kind == SG_K_ADD) continue;
             inl_.insert(u);
             FGroup g;
             g.roots = {v};

@@ -34,6 +34,7 @@ struct PeeEstimate {
     int mode = 0;
     bool bitslice = false;
     double bitslice_ops = 0;  // bitslice mode: 32-lane ALU ops per iteration
+    bool fused = true;        // staged mode: the fused path is expected (every view map affine)
     PartitionWork work;
     bool io_bound() const { return t_dt >= t_comp; }
 };
