@@ -321,7 +321,9 @@ def main():
     peaks, peak_src = measured_peaks()
     # kernel duration: CUDA events around the launch on its stream (one kernel per step here)
     # one partition => every launch of the step is this partition's kernel (main + stream-start variant)
-    kern_ms = statistics.median(step_ms) if info["n_partitions"] == 1 else None
+    # one GPU, several partitions: the step's kernels run back to back on one device; the roofline is
+    # then that of the whole step (every launch is one of the plan's partition kernels)
+    kern_ms = statistics.median(step_ms) if (info["n_partitions"] == 1 or (world == 1 and not pipeline)) else None
     ki_bytes = (info["in_per_iter"] + info["out_per_iter"]) * 4 * n
     roof = None
     if W["bound"] == "hbm":
@@ -354,6 +356,10 @@ def main():
                     "flops_counting": "as written" if fl == fl_written else
                     "pruned (dead firings and zero taps eliminated by the code generator)",
                     "peak_source": "derived: 148 SMs x 128 FP32 lanes x 2 x sm_max_mhz (FFMA)"}
+    if roof is not None:
+        roof["scope"] = ("the partition kernel (one launch per step, plus the stream-start variant beside it)"
+                         if info["n_partitions"] == 1 else
+                         f"the whole step: {info['n_partitions']} partition kernels back to back on one GPU")
     prof = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     if roof is not None and os.path.exists(prof):
         try:

@@ -2026,6 +2026,137 @@ private:
     }
 };
 
+// --------------------------------------------------------------- gather mode
+// A partition of views only (splitters, joiners, IDENTITY / DELAY / DECIMATE / EXPAND / PERMUTE /
+// FFT_REORDER; e.g. the transposing join of a 2-D DCT, a joiner + duplicate splitter between the channel
+// and beam halves of BeamFormer) computes nothing: every output position is one input position (or a
+// zero).  Such a kernel is a straight global-to-global gather -- a grid-stride loop over the output
+// window, each position resolved through the views by generated index arithmetic (64-bit positions,
+// floor division), no tiles, no shared memory.  Positions outside an input's window (the stream start,
+// prework) read as zero, exactly what the producer's firings g < 0 emit.
+class GatherGen : public GenBase {
+public:
+    using GenBase::GenBase;
+
+    KernelInfo run() {
+        KernelInfo ki;
+        ki.mode = 5;
+        ki.name = "sg_part" + std::to_string(part_);
+        ki.name_sync = ki.name;
+        fill_io(ki);
+        ki.threads = ki.threads_sync = 256;
+        ki.tile = ki.tile_sync = 64;  // iterations per grid-stride unit (grid sizing only)
+        ki.smem = ki.smem_sync = 0;
+        ki.min_blocks = 1;
+        for (int e : outs_) reader(e);
+        std::ostringstream src;
+        src << header("gather") << consts_.str() << args_struct();
+        src << "__device__ __forceinline__ long long sg_fdiv64(long long a, long long b) {\n"
+            << "  const long long q = a / b; return (a % b != 0 && ((a < 0) != (b < 0))) ? q - 1 : q;\n}\n";
+        for (auto& r : order_) src << body_.at(r);
+        src << "extern \"C\" __global__ void __launch_bounds__(256) " << ki.name << "(const SgArgs a) {\n"
+            << "  const long long step = (long long)gridDim.x * 256;\n";
+        for (size_t oi = 0; oi < outs_.size(); oi++) {
+            const int e = outs_[oi];
+            const Edge& ed = f_.edges[e];
+            src << "  { // boundary output " << oi << " (edge " << e << ")\n"
+                << "    " << T_ << "* g = SG_OUT(" << oi << ");\n"
+                << "    const long long ob = SG_OUT_BASE(" << oi << ");\n"
+                << "    const long long p0 = SG_K_BEGIN * " << ed.per_iter << "LL + (" << ki.out_lo[oi] << "LL);\n"
+                << "    const long long p1 = SG_K_END * " << ed.per_iter << "LL + (" << ki.out_lo[oi] + ki.out_extra[oi]
+                << "LL);\n"
+                << "    for (long long p = p0 + (long long)blockIdx.x * 256 + threadIdx.x; p < p1; p += step)\n"
+                << "      g[p - ob] = " << name(e) << "(a, p);\n"
+                << "  }\n";
+        }
+        src << "}\n";
+        ki.source = src.str();
+        return ki;
+    }
+
+private:
+    std::map<int, std::string> body_;
+    std::vector<int> order_;  // callees first
+    std::string name(int e) { return "sg_rdg" + std::to_string(e); }
+
+    void reader(int e) {
+        if (body_.count(e)) return;
+        body_[e] = "";
+        std::ostringstream s;
+        s << "__device__ __forceinline__ " << T_ << " " << name(e) << "(const SgArgs& a, long long p) {\n";
+        const Edge& ed = f_.edges[e];
+        const int i = (int)(std::find(ins_.begin(), ins_.end(), e) - ins_.begin());
+        std::vector<int> deps;
+        if (i < (int)ins_.size()) {  // a boundary input: its window, zero outside
+            s << "  const long long q = p - SG_IN_BASE(" << i << ");\n"
+              << "  return (q >= 0 && q < SG_IN_LIMIT(" << i << ")) ? SG_IN(" << i << ")[q] : (" << T_ << ")0;\n";
+        } else {
+            const Node& u = f_.nodes[ed.src];
+            switch (u.type) {
+            case N_SPLIT_DUP: s << "  return " << name(u.in[0]) << "(a, p);\n"; deps.push_back(u.in[0]); break;
+            case N_SPLIT_RR: {
+                int64_t w = u.w[ed.sport], P = 0;
+                for (int k = 0; k < ed.sport; k++) P += u.w[k];
+                s << "  const long long q = sg_fdiv64(p, " << w << "LL), r = p - q * " << w << "LL;\n"
+                  << "  return " << name(u.in[0]) << "(a, q * " << u.wsum << "LL + " << P << "LL + r);\n";
+                deps.push_back(u.in[0]);
+                break;
+            }
+            case N_JOIN: {
+                s << "  const long long q = sg_fdiv64(p, " << u.wsum << "LL), o = p - q * " << u.wsum << "LL;\n";
+                int64_t P = 0;
+                for (size_t b = 0; b < u.w.size(); b++) {
+                    s << "  if (o < " << P + u.w[b] << "LL) return " << name(u.in[b]) << "(a, q * " << u.w[b] << "LL + o - "
+                      << P << "LL);\n";
+                    deps.push_back(u.in[b]);
+                    P += u.w[b];
+                }
+                s << "  return (" << T_ << ")0;\n";
+                break;
+            }
+            case N_FILTER: {
+                const int in = u.in[0];
+                deps.push_back(in);
+                switch (u.kind) {
+                case SG_K_IDENTITY: s << "  return " << name(in) << "(a, p);\n"; break;
+                case SG_K_DELAY: s << "  return " << name(in) << "(a, p - " << u.iv[0] << "LL);\n"; break;
+                case SG_K_DECIMATE: s << "  return " << name(in) << "(a, p * " << u.iv[0] << "LL);\n"; break;
+                case SG_K_EXPAND:
+                    s << "  const long long q = sg_fdiv64(p, " << u.iv[0] << "LL);\n  return (p - q * " << u.iv[0]
+                      << "LL) == 0 ? " << name(in) << "(a, q) : (" << T_ << ")0;\n";
+                    break;
+                case SG_K_PERMUTE: {
+                    const int64_t n = u.iv[0], m = (int64_t)u.iv.size() - 1;
+                    const std::string tab = "SG_GP" + std::to_string(e);
+                    consts_ << "__constant__ int " << tab << "[" << m << "] = {";
+                    for (int64_t k = 0; k < m; k++) consts_ << (k ? "," : "") << (k % 16 == 0 ? "\n  " : "") << u.iv[1 + k];
+                    consts_ << "};\n";
+                    s << "  const long long q = sg_fdiv64(p, " << m << "LL), o = p - q * " << m << "LL;\n"
+                      << "  return " << name(in) << "(a, q * " << n << "LL + " << tab << "[o]);\n";
+                    break;
+                }
+                case SG_K_FFT_REORDER: {
+                    const int64_t n = u.iv[0], F = 2 * n;
+                    s << "  const long long q = sg_fdiv64(p, " << F << "LL), o = p - q * " << F << "LL;\n"
+                      << "  const long long m = o >> 1, r = o & 1;\n"
+                      << "  const long long sc = m < " << n / 2 << " ? 2 * m : 2 * (m - " << n / 2 << ") + 1;\n"
+                      << "  return " << name(in) << "(a, q * " << F << "LL + 2 * sc + r);\n";
+                    break;
+                }
+                default: throw Error(SG_E_UNSUPPORTED, "internal: gather through a compute filter");
+                }
+                break;
+            }
+            default: throw Error(SG_E_UNSUPPORTED, "internal: gather through a feedback loop");
+            }
+        }
+        s << "}\n";
+        for (int d : deps) reader(d);  // callees first
+        body_[e] = s.str();
+        order_.push_back(e);
+    }
+};
+
 // -------------------------------------------------------------- staged mode
 class StageGen : public GenBase {
 public:
@@ -3924,6 +4055,14 @@ KernelInfo generate_kernel(const Flat& f, const std::vector<int>& nodes, int par
     if (mode == 1) {
         RegGen g(f, nodes, part_id);
         return g.run(opt);
+    }
+    if (mode == 2 && opt.mode == 0 && !std::getenv("SG_NO_GATHER")) {
+        bool views_only = true;
+        for (int v : nodes) views_only = views_only && is_view_node(f.nodes[v]);
+        if (views_only) {
+            GatherGen g(f, nodes, part_id);
+            return g.run();
+        }
     }
     StageGen g(f, nodes, part_id);
     CodegenOpts o2 = opt;

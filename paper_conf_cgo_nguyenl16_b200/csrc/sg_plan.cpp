@@ -119,9 +119,11 @@ PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
     k.demand = est.mode == 1 && w.row_items >= 384 && w.components == 1;
     k.inplace = est.mode == 1 && w.components > 1;
     k.tile = w.frame ? 1.0 : std::min(4096.0, std::max(1.0, 150000.0 / std::max(1.0, w.firings)));
-    // the fused staged path declines for partitions of views only and for gathers of many boundary
-    // streams (runtime index readers: the general path) -- observed over the corpus
-    est.fused = k.fused = est.mode != 2 || ((w.flops + w.intops + w.dfma) > 0 && w.in_edges <= kFusedMaxInEdges);
+    // staged partitions: views only -> the gather kernel (HBM-bound like the fused path); with compute,
+    // the fused path declines for merges of many boundary streams (runtime index readers: the general
+    // path) -- observed over the corpus
+    const bool compute = (w.flops + w.intops + w.dfma + w.loop_firings) > 0;
+    est.fused = k.fused = est.mode != 2 || !compute || w.in_edges <= kFusedMaxInEdges;
     if (!k.fused) {  // the general path's tile: every buffer of the tile in ~100 KB of shared memory
         double W = 1;
         while (W < 1024 && 2 * W * 8.0 * std::max(1.0, w.row_items) <= 100.0 * 1024) W *= 2;
@@ -137,7 +139,7 @@ double pee_refine(const PeeEstimate& est, const KernelInfo& ki) {
     KernelShape k;
     k.demand = ki.mode == 1 && ki.reg_variant == 2;
     k.inplace = ki.mode == 1 && ki.reg_variant == 1;
-    k.fused = ki.mode != 2 || ki.fused;
+    k.fused = ki.mode != 2 || ki.fused;  // mode 5 (gather) is priced like the fused path
     k.tile = std::max(1, ki.tile);
     return model_ns(est.work, est.mode, est.bitslice, est.bitslice_ops, k, kModel);
 }

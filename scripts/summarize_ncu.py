@@ -5,8 +5,8 @@
 
 Reads gpurun_out/<round>/full_<config>.ncu-rep (ncu --set full of the main
 partition kernel of `bench.py --config <config>`) and
-gpurun_out/<round>/launches_bitonic32.csv (the launch list), writes
-profiles/<round>_summary.md, profiles/<round>_bitonic32_launches.csv and
+gpurun_out/<round>/launches_<config>.csv (launch lists), writes
+profiles/<round>_summary.md, profiles/<round>_<config>_launches.csv and
 profiles/ncu_traffic.json (DRAM bytes per launch, read by bench.py).
 """
 import csv
@@ -86,15 +86,15 @@ def main(rnd):
                              to_bytes(*d["dram__bytes_write.sum"]), "source": f"profiles/{rnd}_summary.md"}
         except Exception:
             pass
-    launches = os.path.join(src, "launches_bitonic32.csv")
-    if os.path.exists(launches):
+    for launches in sorted(glob.glob(os.path.join(src, "launches_*.csv"))):
+        cfg = os.path.basename(launches)[len("launches_"):-4]
         txt = open(launches).read()
-        open(os.path.join(ROOT, "profiles", f"{rnd}_bitonic32_launches.csv"), "w").write(txt)
+        open(os.path.join(ROOT, "profiles", f"{rnd}_{cfg}_launches.csv"), "w").write(txt)
         rows = [r for r in csv.reader(io.StringIO(txt)) if len(r) > 10 and r[0].isdigit()]
         per = {}
         for r in rows:
             per.setdefault(r[4], []).append(float(r[-1].replace(",", "")))
-        lines.append("## launch list (bitonic32, `bench.py --steps 5 --warmup 3`)")
+        lines.append(f"## launch list ({cfg}, `bench.py --config {cfg} --steps 5 --warmup 3`)")
         lines.append("")
         tot = sum(sum(v) for v in per.values()) or 1
         lines.append("| kernel | launches | mean ns | share of GPU time |")
