@@ -790,13 +790,15 @@ struct Candidate {
 };
 GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, int Gs, const sg_plan_opts& o);
 
-Candidate best_candidate(const std::vector<Flat>& variants, int Gs, const sg_plan_opts& o, GroupMap* gm_out) {
+Candidate best_candidate(const std::vector<Flat>& variants, int Gs, const sg_plan_opts& o, GroupMap* gm_out,
+                         std::vector<std::pair<Candidate, GroupMap>>* all = nullptr) {
     Candidate best;
     bool have = false;
     GroupMap bgm;
     for (int vi = 0; vi < (int)variants.size(); vi++) {
         std::vector<double> mults = {1.0};
         if (o.partitioner == SG_PART_ALGORITHM1 && Gs > 1) mults = {1.0, 2.0, 0.0};
+        if (o.partitioner == SG_PART_ALGORITHM1 && vi == 0) mults.push_back(-2.0);  // one partition
         if (const char* env = std::getenv("SG_A1_CAPS")) {  // experiments: fixed cap multipliers ("1,2")
             mults.clear();
             for (const char* c = env; *c;) {
@@ -810,7 +812,8 @@ Candidate best_candidate(const std::vector<Flat>& variants, int Gs, const sg_pla
         std::set<std::vector<std::vector<int>>> seen;
         for (double cm : mults) {
             sg_plan_opts oc = o;
-            if (cm < 0) oc.partitioner = SG_PART_CHAIN;
+            if (cm == -1.0) oc.partitioner = SG_PART_CHAIN;
+            if (cm == -2.0) oc.partitioner = SG_PART_SINGLE;
             auto parts = make_partitions(variants[vi], Gs, oc, cm);
             auto key = parts;
             for (auto& q : key) std::sort(q.begin(), q.end());
@@ -829,6 +832,14 @@ Candidate best_candidate(const std::vector<Flat>& variants, int Gs, const sg_pla
             const double maxload = *std::max_element(load.begin(), load.end());
             // a plan of several partitions is charged the PEE's noise margin against one partition
             const double score = gm.m.tmax * (parts.size() > 1 ? 1.0 + kSplitMargin : 1.0);
+            if (all) {
+                Candidate c;
+                c.variant = vi;
+                c.parts = parts;
+                c.tmax = score;
+                c.maxload = maxload;
+                all->push_back({c, gm});
+            }
             const bool tie = have && std::fabs(score - best.tmax) <= 1e-9 * std::max(1.0, best.tmax);
             if (!have || score < best.tmax * (1 - 1e-9) || (tie && maxload < best.maxload * (1 - 1e-9))) {
                 best.maxload = maxload;
@@ -841,7 +852,22 @@ Candidate best_candidate(const std::vector<Flat>& variants, int Gs, const sg_pla
         }
     }
     if (gm_out) *gm_out = bgm;
+    if (all)  // best first (the order the planner falls back in when a partition cannot be generated)
+        std::stable_sort(all->begin(), all->end(), [](const std::pair<Candidate, GroupMap>& a,
+                                                      const std::pair<Candidate, GroupMap>& b) {
+            return a.first.tmax != b.first.tmax ? a.first.tmax < b.first.tmax : a.first.maxload < b.first.maxload;
+        });
     return best;
+}
+
+// Eq. III.1-III.7 objective of a given mapping inside one group of Gs GPUs (same link model as map_group)
+double group_tmax(const std::vector<double>& T, const std::vector<PdgEdge>& pdg, const std::vector<int>& a, int Gs,
+                  const sg_plan_opts& o) {
+    if (Gs <= 1) return std::accumulate(T.begin(), T.end(), 0.0);
+    const double bw = o.link_gbps > 0 ? o.link_gbps : 770.0;
+    const double lat = (o.link_latency_us > 0 ? o.link_latency_us : 10.0) * 1e3 /
+                       (o.iters_per_fragment > 0 ? (double)o.iters_per_fragment : kFragIters);
+    return mapping_cost(T, pdg, Topology::nvswitch(Gs), lat, bw, a);
 }
 
 // Throughput bound of R replica groups of Gs GPUs each on the NVSwitch star:
@@ -889,6 +915,11 @@ int io_gpu(const Flat& f, const std::vector<std::vector<int>>& parts, const std:
     return 0;
 }
 }  // namespace
+
+namespace {
+void assemble_plan(Plan& p, std::vector<std::vector<int>> parts, const GroupMap& gm, int G, int R, int Gs,
+                   const sg_plan_opts& o);
+}
 
 void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     if (o.transport < SG_TRANSPORT_AUTO || o.transport > SG_TRANSPORT_HOST)
@@ -939,16 +970,54 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     const int Gs = G / R;
     p.R = R;
     p.Gs = Gs;
-    // ---- graph variant + partitions (Algorithm 1 candidates compared by the ILP objective)
-    std::vector<std::vector<int>> parts;
-    GroupMap gm;
-    {
-        auto vars = variants_for(Gs);
-        Candidate cd = best_candidate(vars, Gs, o, &gm);
-        p.flat = vars[cd.variant];
-        p.chain_fission = o.chain_groups >= 2 || cd.variant == 1;
-        parts = cd.parts;
+    // ---- graph variant + partitions (Algorithm 1 candidates compared by the ILP objective); a candidate
+    // with a partition the code generator cannot fit (SG_E_SIZE: shared memory) yields to the next one
+    auto vars = variants_for(Gs);
+    std::vector<std::pair<Candidate, GroupMap>> cands;
+    best_candidate(vars, Gs, o, nullptr, &cands);
+    // After code generation the estimate is refined with the kernels' own decisions; a plan whose refined
+    // Tmax exceeds its planning score by more than half also has the one-partition candidate (and the next
+    // few) generated, and the smallest refined Tmax wins -- the planner never keeps a cut the generated code
+    // shows to be slower than what it had to compare with.
+    auto attempt = [&](size_t ci) -> bool {
+        try {
+            p.flat = vars[cands[ci].first.variant];
+            p.chain_fission = o.chain_groups >= 2 || cands[ci].first.variant == 1;
+            assemble_plan(p, cands[ci].first.parts, cands[ci].second, G, R, Gs, o);
+            return true;
+        } catch (const Error& e) {
+            if (e.code != SG_E_SIZE) throw;
+            return false;
+        }
+    };
+    int best_ci = -1;
+    double best_ref = 0;
+    size_t tried = 0;
+    double single_score = 0;  // the one-partition candidate's planning score
+    for (auto& c : cands) if (c.first.parts.size() == 1) single_score = c.first.tmax;
+    for (size_t ci = 0; ci < cands.size() && tried < 4; ci++) {
+        if (!attempt(ci)) continue;
+        tried++;
+        const bool cut = cands[ci].first.parts.size() > 1;
+        if (o.plan_only || (p.est_tmax <= cands[ci].first.tmax * 1.5 &&
+                            (!cut || single_score <= 0 || p.est_tmax <= 0.9 * single_score)))
+            return;
+        if (best_ci < 0 || p.est_tmax < best_ref) { best_ci = (int)ci; best_ref = p.est_tmax; }
     }
+    for (size_t ci = 0; ci < cands.size(); ci++)  // the one-partition candidate, if not yet tried
+        if (cands[ci].first.parts.size() == 1 && (int)ci != best_ci && attempt(ci)) {
+            if (best_ci < 0 || p.est_tmax < best_ref) { best_ci = (int)ci; best_ref = p.est_tmax; }
+            break;
+        }
+    if (best_ci < 0) throw Error(SG_E_SIZE, "no candidate partitioning fits the code generator's shared memory");
+    if (!attempt((size_t)best_ci)) throw Error(SG_E_SIZE, "internal: candidate no longer fits");
+}
+
+namespace {
+// Partitions -> ordered, mapped, generated plan (the graph variant is p.flat).
+void assemble_plan(Plan& p, std::vector<std::vector<int>> parts, const GroupMap& gm, int G, int R, int Gs,
+                   const sg_plan_opts& o) {
+    const Flat& f = p.flat;
     const int N = (int)f.nodes.size();
     // validate: cover, convex; order topologically
     std::vector<int> owner(N, -1);
@@ -1043,6 +1112,7 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     p.output_gpu = p.part_gpu[owner[f.edges[f.out_edge].src]];
     p.iters_per_fragment = o.iters_per_fragment;
     // ---- code generation + NVRTC (one kernel per partition)
+    p.kernels.clear();
     p.kernels.resize(P);
     CodegenOpts co;
     co.mode = o.codegen_mode;
@@ -1069,6 +1139,13 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         // the PEE with the generated kernel's own decisions (static discrepancy)
         p.parts[i].t_est = p.part_time[i] = pee_refine(ests[i], p.kernels[i].ki);
     }
+    if (!o.plan_only) {  // Tmax of this mapping with the refined partition times
+        std::vector<double> Tr(P);
+        for (int i = 0; i < P; i++) Tr[i] = p.part_time[i] + launch_ns_per_iter(o.iters_per_fragment);
+        p.est_tmax = R == 1 ? group_tmax(Tr, gm.pdg, gm.m.assign, Gs, o)
+                            : hybrid_cost(f, Tr, gm.pdg, gm.m.assign, io_gpu(f, parts, gm.m.assign, f.edges[f.in_edge].dst),
+                                          io_gpu(f, parts, gm.m.assign, f.edges[f.out_edge].src), Gs, R, o);
+    }
     // ---- info arrays
     p.reps.resize(N);
     p.ninit.resize(N);
@@ -1083,5 +1160,6 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         p.node_part[v] = owner[v];
     }
 }
+}  // namespace
 
 }  // namespace sg

@@ -8,7 +8,8 @@ tests/test_gpu_sanitize.py).
 Families: TMA register rows (BitonicSort), bulk-copy in-place components (FFT), staged fused with
 prefetch (FMRadio, FilterBank), staged general path, bitslice with rolled rounds (DES), feedback loops
 (lane-local wavefront and the per-step-barrier wavefront), multi-fragment rings on virtual GPUs
-(per-filter partitions and chain fission), frame FIRs (BeamFormer), demand-ordered register rows (DCT).
+(per-filter partitions and chain fission), frame FIRs (BeamFormer), demand-ordered register rows (DCT),
+gather kernels of partitions of views only.
 """
 import argparse
 import os
@@ -34,7 +35,8 @@ def cases():
         "rings_chain": (lambda: apps.filterbank(8), 900, dict(n_gpus=2, virtual_gpus=1, chain_groups=2,
                                                               partitioner="chain", iters_per_fragment=200)),
         "frame_fir": (lambda: apps.beamformer(channels=3, beams=2, frame=64, taps=8, mf_taps=16), 5, {}),
-        "demand_register": (lambda: apps.dct2d(16), 300, {}),
+        "demand_register": (lambda: apps.dct2d(16), 300, dict(partitioner="single")),
+        "gather_views": (lambda: apps.fmradio(4), 600, dict(partitioner="per_filter", iters_per_fragment=150)),
     }
 
 

@@ -14,7 +14,8 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 
 @pytest.mark.parametrize("tool,case", [("memcheck", "tma_register"), ("memcheck", "staged_fused_fb"),
                                        ("memcheck", "rings_chain"), ("racecheck", "staged_fused_fm"),
-                                       ("racecheck", "loop_barrier"), ("synccheck", "bitslice_rolled")])
+                                       ("racecheck", "loop_barrier"), ("synccheck", "bitslice_rolled"),
+                                       ("memcheck", "gather_views")])
 def test_compute_sanitizer_clean(tool, case):
     import torch
     if not torch.cuda.is_available():
