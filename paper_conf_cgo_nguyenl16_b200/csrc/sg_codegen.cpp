@@ -2045,7 +2045,11 @@ public:
         ki.name_sync = ki.name;
         fill_io(ki);
         ki.threads = ki.threads_sync = 256;
-        ki.tile = ki.tile_sync = 64;  // iterations per grid-stride unit (grid sizing only)
+        // iterations per grid-stride unit (grid sizing only): ~16k output items each, so a launch gets
+        // enough CTAs to fill the GPU whatever the iteration size (BeamFormer: 49 152 items per frame)
+        int64_t items = 0;
+        for (int e : outs_) items += f_.edges[e].per_iter;
+        ki.tile = ki.tile_sync = (int)std::max<int64_t>(1, std::min<int64_t>(64, 16384 / std::max<int64_t>(1, items)));
         ki.smem = ki.smem_sync = 0;
         ki.min_blocks = 1;
         for (int e : outs_) reader(e);
@@ -2065,8 +2069,15 @@ public:
                 << "    const long long p0 = SG_K_BEGIN * " << ed.per_iter << "LL + (" << ki.out_lo[oi] << "LL);\n"
                 << "    const long long p1 = SG_K_END * " << ed.per_iter << "LL + (" << ki.out_lo[oi] + ki.out_extra[oi]
                 << "LL);\n"
-                << "    for (long long p = p0 + (long long)blockIdx.x * 256 + threadIdx.x; p < p1; p += step)\n"
-                << "      g[p - ob] = " << name(e) << "(a, p);\n"
+                << "    // four positions per trip, loads first: four gathers in flight per thread\n"
+                << "    for (long long p = p0 + (long long)blockIdx.x * 256 + threadIdx.x; p < p1; p += 4 * step) {\n"
+                << "      " << T_ << " v[4];\n"
+                << "#pragma unroll\n"
+                << "      for (int u = 0; u < 4; u++) { const long long q = p + u * step; v[u] = q < p1 ? " << name(e)
+                << "(a, q) : (" << T_ << ")0; }\n"
+                << "#pragma unroll\n"
+                << "      for (int u = 0; u < 4; u++) { const long long q = p + u * step; if (q < p1) g[q - ob] = v[u]; }\n"
+                << "    }\n"
                 << "  }\n";
         }
         src << "}\n";
