@@ -323,7 +323,9 @@ def main():
     # one partition => every launch of the step is this partition's kernel (main + stream-start variant)
     # one GPU, several partitions: the step's kernels run back to back on one device; the roofline is
     # then that of the whole step (every launch is one of the plan's partition kernels)
-    kern_ms = statistics.median(step_ms) if (info["n_partitions"] == 1 or (world == 1 and not pipeline)) else None
+    # (feedback loops excepted: their partition is a serial chain, bounded by latency, not by a roof)
+    serial = 4 in info["partition_mode"]
+    kern_ms = statistics.median(step_ms) if (info["n_partitions"] == 1 or (world == 1 and not pipeline and not serial)) else None
     ki_bytes = (info["in_per_iter"] + info["out_per_iter"]) * 4 * n
     roof = None
     if W["bound"] == "hbm":

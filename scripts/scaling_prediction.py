@@ -2,7 +2,8 @@
 """Multi-GPU scaling predicted from measured partition times (one B200; the pool has no multi-GPU box).
 
 For each BASELINE multi-GPU config and G = 1, 2, 4, 8 the planner's pipelined plan (replicas = 1,
-Algorithm 1 + ILP, chain fission considered -- SURVEY.md 8(e)) is built; every partition's kernel is
+Algorithm 1 + ILP, chain fission considered -- SURVEY.md 8(e)) and its hybrid replica x pipeline plan
+(replicas = -1; the input on one GPU) are built; every partition's kernel is
 timed alone at the bench's per-step iteration count (sg_profile_partitions), and the throughput of the
 G-GPU pipeline is bounded by ("Tmax ... determines the application throughput"):
 
@@ -43,19 +44,33 @@ def main():
         n = N[name]
         x = torch.from_numpy(inputs.make_input("f32", IN_ITEMS[name](n), 7)).cuda()
         base = None
-        for G in (1, 2, 4, 8):
-            with sg.plan(prog, G, virtual_gpus=1, replicas=1) as p:
+        for G, R in ((1, 1), (2, 1), (4, 1), (8, 1), (2, -1), (4, -1), (8, -1)):
+            with sg.plan(prog, G, virtual_gpus=1, replicas=R) as p:
                 info = p.info()
+                if R == -1 and info["replicas"] == 1:
+                    continue                           # the auto model kept the pipeline: row above
                 meas = p.profile_partitions(n, 5)
-                load = [0.0] * G
+                Rr = info["replicas"]
+                Gs = G // Rr
+                load = [0.0] * Gs
                 for k, g in enumerate(info["partition_gpu"]):
-                    load[g] += meas[k]
+                    load[g] += meas[k] / Rr             # each group runs 1/R of the fragments
                 up, down = [0.0] * G, [0.0] * G
-                for a, b, nbytes in p.pdg():          # sg_plan_pdg: per (partition pair, stream)
-                    ga, gb = info["partition_gpu"][a], info["partition_gpu"][b]
-                    if ga != gb:
-                        up[ga] += nbytes
-                        down[gb] += nbytes
+                for r in range(Rr):
+                    for a, b, nbytes in p.pdg():      # sg_plan_pdg: per (partition pair, stream)
+                        ga, gb = info["partition_gpu"][a], info["partition_gpu"][b]
+                        if ga != gb:
+                            up[r * Gs + ga] += nbytes / Rr
+                            down[r * Gs + gb] += nbytes / Rr
+                    if r:  # other groups' input / output cross the links of group 0's input / output GPU
+                        # (node 0 consumes the graph input, the last node produces the output)
+                        gin = info["partition_gpu"][info["node_partition"][0]]
+                        gout = info["partition_gpu"][info["node_partition"][-1]]
+                        bi, bo = 4.0 * info["in_per_iter"] / Rr, 4.0 * info["out_per_iter"] / Rr
+                        up[gin] += bi
+                        down[r * Gs + gin] += bi
+                        up[r * Gs + gout] += bo
+                        down[gout] += bo
                 comp = max(load)
                 link = max(up + down) / LINK_GBS    # ns per iteration (bytes / (GB/s) = ns)
                 if G == 1:
@@ -71,7 +86,7 @@ def main():
                 e1.record()
                 torch.cuda.synchronize()
                 virt = e0.elapsed_time(e1) / 3 * 1e6 / n
-                row = {"config": name, "G": G, "n_iters": n, "partitions": info["n_partitions"],
+                row = {"config": name, "G": G, "replicas": Rr, "n_iters": n, "partitions": info["n_partitions"],
                        "chain_fission": info["chain_fission"], "partition_gpu": info["partition_gpu"],
                        "partition_ns": meas, "max_gpu_ns": comp, "link_ns": link,
                        "pred_speedup_compute": base / comp, "pred_speedup": base / max(comp, link),
@@ -85,11 +100,11 @@ def main():
              "times; link bound = the busiest NVSwitch link's PDG bytes / 900 GB/s; predicted speedup = "
              "T(1 GPU) / max(compute, link).  `virtual run` = the whole plan run on G virtual GPUs of this one "
              "device (fragment pipeline overhead vs the summed partition times).", "",
-             "| config | G | partitions | chain | busiest GPU ns/iter | link ns/iter | speedup (compute) | "
-             "speedup (compute + links) | x linear | virtual run / sum of partitions |", "|---|---|---|---|---|---|---|---|---|---|"]
+             "| config | G | replica groups | partitions | chain | busiest GPU ns/iter | link ns/iter | speedup (compute) | "
+             "speedup (compute + links) | x linear | virtual run / sum of partitions |", "|---|---|---|---|---|---|---|---|---|---|---|"]
     for r in rows:
-        lines.append("| %s | %d | %d | %s | %.4g | %.4g | %.2f | %.2f | %.2f | %.2f |" % (
-            r["config"], r["G"], r["partitions"], "yes" if r["chain_fission"] else "no", r["max_gpu_ns"],
+        lines.append("| %s | %d | %d | %d | %s | %.4g | %.4g | %.2f | %.2f | %.2f | %.2f |" % (
+            r["config"], r["G"], r["replicas"], r["partitions"], "yes" if r["chain_fission"] else "no", r["max_gpu_ns"],
             r["link_ns"], r["pred_speedup_compute"], r["pred_speedup"], r["pred_speedup"] / r["G"],
             r["virtual_run_ns"] / r["sum_partition_ns"]))
     open(args.out + ".md", "w").write("\n".join(lines) + "\n")
