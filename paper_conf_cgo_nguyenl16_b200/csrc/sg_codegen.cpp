@@ -2063,6 +2063,7 @@ public:
         for (size_t oi = 0; oi < outs_.size(); oi++) {
             const int e = outs_[oi];
             const Edge& ed = f_.edges[e];
+            if (emit_periodic(src, oi, e, ki)) continue;
             src << "  { // boundary output " << oi << " (edge " << e << ")\n"
                 << "    " << T_ << "* g = SG_OUT(" << oi << ");\n"
                 << "    const long long ob = SG_OUT_BASE(" << oi << ");\n"
@@ -2089,6 +2090,53 @@ private:
     std::map<int, std::string> body_;
     std::vector<int> order_;  // callees first
     std::string name(int e) { return "sg_rdg" + std::to_string(e); }
+
+    // Periodic form: the smallest period P (dividing the output's items per iteration, <= 256) for which
+    // output position k*P + c resolves, for every residue c, to an affine position a_c*k + b_c of one
+    // boundary input (or to a zero): each thread then copies one whole period with compile-time maps --
+    // no per-item division or branch chain.  Returns false when no such period exists.
+    bool emit_periodic(std::ostringstream& src, size_t oi, int e, const KernelInfo& ki) {
+        const int64_t per = f_.edges[e].per_iter;
+        for (int64_t P = 1; P <= std::min<int64_t>(per, 256); P++) {
+            if (per % P) continue;
+            struct M { int in = -1; int64_t a = 0, b = 0; };
+            std::vector<M> maps(P);
+            bool ok = true;
+            for (int64_t c = 0; c < P && ok; c++) {
+                Ref r = R_.resolve(e, Lin::v("k", P, c));
+                if (r.k == Ref::ZERO) continue;
+                if (r.k == Ref::RUNTIME) { ok = false; break; }
+                const int i = (int)(std::find(ins_.begin(), ins_.end(), r.edge) - ins_.begin());
+                if (i >= (int)ins_.size()) { ok = false; break; }
+                for (auto& t : r.pos.t) if (t.first != "k") ok = false;
+                maps[c].in = i;
+                maps[c].a = r.pos.coef("k");
+                maps[c].b = r.pos.c;
+            }
+            if (!ok) continue;
+            src << "  { // boundary output " << oi << " (edge " << e << "): period " << P << ", affine per residue\n"
+                << "    " << T_ << "* g = SG_OUT(" << oi << ");\n"
+                << "    const long long ob = SG_OUT_BASE(" << oi << ");\n"
+                << "    const long long p0 = SG_K_BEGIN * " << per << "LL + (" << ki.out_lo[oi] << "LL);\n"
+                << "    const long long p1 = SG_K_END * " << per << "LL + (" << ki.out_lo[oi] + ki.out_extra[oi] << "LL);\n"
+                << "    const long long kb = sg_fdiv64(p0, " << P << "LL), ke = sg_fdiv64(p1 + " << P - 1 << "LL, " << P << "LL);\n"
+                << "    for (long long k = kb + (long long)blockIdx.x * 256 + threadIdx.x; k < ke; k += step) {\n"
+                << "      const long long pb = k * " << P << "LL;\n";
+            for (int64_t c = 0; c < P; c++) {
+                const M& m = maps[c];
+                if (m.in < 0) { src << "      const " << T_ << " v" << c << " = (" << T_ << ")0;\n"; continue; }
+                src << "      " << T_ << " v" << c << ";\n"
+                    << "      { const long long q = " << m.a << "LL * k + (" << m.b << "LL) - SG_IN_BASE(" << m.in << ");\n"
+                    << "        v" << c << " = (q >= 0 && q < SG_IN_LIMIT(" << m.in << ")) ? SG_IN(" << m.in << ")[q] : (" << T_
+                    << ")0; }\n";
+            }
+            for (int64_t c = 0; c < P; c++)
+                src << "      if (pb + " << c << " >= p0 && pb + " << c << " < p1) g[pb + " << c << " - ob] = v" << c << ";\n";
+            src << "    }\n  }\n";
+            return true;
+        }
+        return false;
+    }
 
     void reader(int e) {
         if (body_.count(e)) return;
@@ -2252,7 +2300,8 @@ public:
                     prologue_fast = prologue_;
                     ki.flops_exec_per_iter = fused_flops_per_iter();
                 }
-            } catch (const FusedFail&) {
+            } catch (const FusedFail& ff) {
+                if (std::getenv("SG_FUSED_DEBUG")) std::fprintf(stderr, "[sg codegen] partition %d: fused path declined (%s)\n", part_, ff.why);
                 WF = 0;
                 fast.clear();
             }
@@ -2790,7 +2839,7 @@ private:
                         g.B = B;
                         if (dry_ok(g, c)) { B0 = B; break; }
                     }
-                    if (!B0) throw FusedFail();
+                    if (!B0) throw FusedFail{"site 1"};
                     g.B = B0;
                     static const int bmax = std::getenv("SG_FUSED_BMAX") ? std::atoi(std::getenv("SG_FUSED_BMAX")) : 16;
                     dry_ok(g, c);
@@ -2912,12 +2961,12 @@ private:
                         auto it = cs_.find(e);
                         if (it != cs_.end() && it->second > 1) {
                             int64_t q = pos - f_.edges[e].pre - cf0_.at(e);
-                            if (fmodp(q, it->second) != 0) throw FusedFail();
+                            if (fmodp(q, it->second) != 0) throw FusedFail{"site 2"};
                             idx = fdiv(q, it->second);
                         } else {
                             idx = pos - wb_.at(e);
                         }
-                        if (idx < 0) throw FusedFail();
+                        if (idx < 0) throw FusedFail{"site 3"};
                         bufs[e].size = std::max(bufs[e].size, idx + 1);
                     }
             }
@@ -3121,7 +3170,7 @@ private:
                         b << "      " << (q ? "else " : "") << "if (sgw == " << q << ") {\n"
                           << "      for (int jb = tsg; jb < NBg; jb += " << NT_ / ksub << ") {\n";
                         sym_block(cq, h, true);
-                        if (cq.runtime) throw FusedFail();
+                        if (cq.runtime) throw FusedFail{"site 4"};
                         b << "      }\n      }\n";
                     }
                     b << "    }\n";
@@ -3145,7 +3194,7 @@ private:
                       << "      for (; jb < NBg; jb += NT) {\n";
                 }
                 sym_block(c, g, true);
-                if (c.runtime) throw FusedFail();
+                if (c.runtime) throw FusedFail{"site 5"};
                 b << "      }\n    }\n";
                 rot += g.NB;
             }
@@ -3374,21 +3423,23 @@ private:
         for (int d : deps) gen_reader(d);  // callees first
         readers_ << s.str();
     }
-    struct FusedFail {};
+    struct FusedFail {
+        const char* why = "";
+    };
     // shared-memory index of position `pos` of physical edge e in the current layout
     Lin buf_index(int e, const Lin& pos) {
         auto pit = plP_.find(e);
         if (fused_ && pit != plP_.end() && pit->second > 1) {  // planar: [P][Q], Q odd
             const int64_t P = pit->second, Q = plQ_.at(e);
             Lin j = pos.plus(-wb_.at(e));
-            if (!j.divisible(P)) throw FusedFail();
+            if (!j.divisible(P)) throw FusedFail{"site 6"};
             return j.divf(P).plus(j.modc(P) * Q + off_.at(e));
         }
         auto it = cs_.find(e);
         if (fused_ && it != cs_.end() && it->second > 1) {
             const Edge& ed = f_.edges[e];
             Lin q = pos.plus(-(ed.pre + cf0_.at(e)));
-            if (!q.divisible(it->second) || q.modc(it->second) != 0) throw FusedFail();
+            if (!q.divisible(it->second) || q.modc(it->second) != 0) throw FusedFail{"site 7"};
             return q.divf(it->second).plus(off_.at(e));
         }
         return pos.plus(off_.at(e) - wb_.at(e));
@@ -3397,7 +3448,17 @@ private:
         Ref r = R_.resolve(e, pos);
         if (r.k == Ref::ZERO) return "(" + T_ + ")0";
         if (r.k == Ref::RUNTIME) {
-            if (fused_) throw FusedFail();
+            if (fused_) {
+                // a view map that is not affine in the loop index (e.g. the transposing joins of a 2-D DCT
+                // in a store): generated index readers over dense, uncompacted buffers
+                std::set<int> src;
+                R_.sources(r.edge, src);
+                for (int pe : src) {
+                    const bool dense = materialised(pe) && off_.count(pe) && wb_.count(pe) &&
+                                       !(cs_.count(pe) && cs_.at(pe) > 1) && !(plP_.count(pe) && plP_.at(pe) > 1);
+                    if (!dense) throw FusedFail{"site 8"};
+                }
+            }
             gen_reader(r.edge);
             return rd_name(r.edge) + "(sm, " + r.pos.str() + ")";
         }

@@ -233,3 +233,29 @@ def test_run_host_chunked_pipeline(oracle_lib, name):
         y = np.empty(p.output_items(n), dtype=np.int32 if prog.dtype == "i32" else np.float32)
         p.run_host(x, n, y)
     assert_parity(prog, y, ref)
+
+
+def test_parity_dct_staged_fused(oracle_lib):
+    """2-D DCT in staged mode: the fused path stores through the transposing joins with generated index
+    readers over dense buffers (a view map not affine in the store loop)."""
+    prog = apps.dct2d(16)
+    for n in (37, 3001):
+        x = inputs.make_input("f32", 256 * n, 4242 + n)
+        ref = oracle_lib.run(prog, x, n)
+        y, info, _ = run_gpu(prog, x, n, codegen_mode="staged", partitioner="single")
+        assert info["partition_mode"] == [2]
+        assert_parity(prog, y, ref)
+
+
+@pytest.mark.parametrize("G", [2, 4])
+def test_parity_gather_partitions(oracle_lib, G):
+    """Partitions of views only run as gather kernels (periodic affine copies or generic index chains):
+    BeamFormer's channel-to-beam join + duplicate, per-filter splits of FMRadio and FFT."""
+    for prog, n in ((apps.beamformer(channels=4, beams=2, frame=64, taps=8, mf_taps=16), 7),
+                    (apps.fmradio(5), 900), (apps.fft(16), 500)):
+        x = inputs.make_input("f32", oracle_lib.in_items(prog, n), 77 + G)
+        ref = oracle_lib.run(prog, x, n)
+        y, info, _ = run_gpu(prog, x, n, n_gpus=G, virtual_gpus=1, partitioner="per_filter",
+                             iters_per_fragment=max(1, n // 3))
+        assert 5 in info["partition_mode"]
+        assert_parity(prog, y, ref)
