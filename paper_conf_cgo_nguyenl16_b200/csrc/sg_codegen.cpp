@@ -2481,7 +2481,14 @@ private:
     std::string sym_value(Sym& c, int e, const Lin& pos) {
         Ref r = R_.resolve(e, pos);
         if (r.k == Ref::ZERO) return "0";
-        if (r.k == Ref::RUNTIME) { c.runtime = true; return "0"; }
+        if (r.k == Ref::RUNTIME) {
+            static const bool dbg = std::getenv("SG_FUSED_DEBUG") != nullptr;
+            if (dbg && !c.runtime)
+                std::fprintf(stderr, "[sg codegen] runtime view: edge %d position %s (resolved to edge %d at %s)\n", e,
+                             pos.str().c_str(), r.edge, r.pos.str().c_str());
+            c.runtime = true;
+            return "0";
+        }
         int pe = r.edge;
         const Edge& ed = f_.edges[pe];
         if (materialised(pe)) {
