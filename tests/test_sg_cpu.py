@@ -681,3 +681,17 @@ def test_ilp_exact_for_every_config(sg, name, G):
         if name == "fmradio10" and G == 2:
             assert i["chain_fission"] and i["n_partitions"] == 2
             assert sum(b for _, _, b in p.pdg()) == 8.0
+
+
+@pytest.mark.parametrize("name,G", [("beamformer12x4", 2), ("beamformer12x4", 4), ("dct16", 2)])
+def test_planner_never_keeps_a_cut_worse_than_one_partition(sg, name, G):
+    """After code generation the PEE is refined with the kernels' own decisions; a
+    candidate the code generator cannot fit (shared memory) or whose refined Tmax is not better than one
+    partition yields to the next candidate: the plan's refined estimate never exceeds one partition's."""
+    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
+    with sg.plan(prog, 1, partitioner="single") as p1:
+        t1 = p1.info()["est_tmax"]
+    with sg.plan(prog, G, virtual_gpus=1, replicas=1) as p:
+        i = p.info()
+        assert i["est_tmax"] <= t1 * 1.0001
+        assert all(t > 0 for t in i["partition_time"])
