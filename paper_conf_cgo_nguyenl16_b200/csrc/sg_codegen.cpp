@@ -2091,13 +2091,15 @@ private:
     std::vector<int> order_;  // callees first
     std::string name(int e) { return "sg_rdg" + std::to_string(e); }
 
-    // Periodic form: the smallest period P (dividing the output's items per iteration, <= 256) for which
+    // Periodic form: the smallest period P (dividing the output's items per iteration, <= 32) for which
     // output position k*P + c resolves, for every residue c, to an affine position a_c*k + b_c of one
     // boundary input (or to a zero): each thread then copies one whole period with compile-time maps --
-    // no per-item division or branch chain.  Returns false when no such period exists.
+    // no per-item division or branch chain.  Longer periods keep the generic form: a thread copying a whole
+    // period of P items makes a warp's accesses P items apart (uncoalesced), while the generic loop maps
+    // consecutive threads to consecutive output positions.  Returns false when no such period exists.
     bool emit_periodic(std::ostringstream& src, size_t oi, int e, const KernelInfo& ki) {
         const int64_t per = f_.edges[e].per_iter;
-        for (int64_t P = 1; P <= std::min<int64_t>(per, 256); P++) {
+        for (int64_t P = 1; P <= std::min<int64_t>(per, 32); P++) {
             if (per % P) continue;
             struct M { int in = -1; int64_t a = 0, b = 0; };
             std::vector<M> maps(P);
