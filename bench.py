@@ -204,6 +204,9 @@ def main():
                          "partition); 0 = as planned")
     ap.add_argument("--codegen", default="auto", choices=["auto", "register", "staged", "general"],
                     help="plan option codegen_mode (auto: chosen by the code generator)")
+    ap.add_argument("--force-pipeline", action="store_true",
+                    help="run the one-process-per-GPU pipelined path (sg_run_rank, NCCL) even on one GPU (a check "
+                         "of the multi-GPU bench path on a one-GPU box)")
     ap.add_argument("--mode", default="pipeline", choices=["replicas", "pipeline"],
                     help="N>1: the paper's pipelined partition mapping (default), one process per GPU, NCCL "
                          "boundary streams; or independent replicas")
@@ -221,12 +224,17 @@ def main():
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
-    if world > 1:
+    if args.force_pipeline and world == 1:
+        os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+        os.environ.setdefault("MASTER_PORT", "29531")
+        os.environ.setdefault("RANK", "0")
+        os.environ.setdefault("WORLD_SIZE", "1")
+    if world > 1 or args.force_pipeline:
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     torch.cuda.set_device(local)
     name = args.config
     W = WORKLOADS[name]
-    pipeline = args.mode == "pipeline" and world > 1
+    pipeline = args.mode == "pipeline" and (world > 1 or args.force_pipeline)
     # pipelined runs need many fragments per GPU (fill / drain F / (F + G - 1))
     n = args.iters or (max(W["n"], 1 << 24) if pipeline and W["bound"] == "alu" and name != "beamformer12x4"
                        else W["n"])
@@ -291,7 +299,7 @@ def main():
 
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
     sampler = ClockSampler(local)
-    if world > 1:
+    if dist.is_initialized():
         dist.barrier()
     torch.cuda.synchronize()
     sampler.start()
@@ -305,7 +313,7 @@ def main():
         ev[k][1].record(stream)
     torch.cuda.synchronize()
     wall = time.perf_counter() - wall0
-    if world > 1:
+    if dist.is_initialized():
         dist.barrier()
     clocks = sampler.stop()
     step_ms = [a.elapsed_time(b) for a, b in ev]
@@ -461,7 +469,7 @@ def main():
         }
         print(json.dumps(line))
     plan.close()
-    if world > 1:
+    if dist.is_initialized():
         dist.destroy_process_group()
     return 0
 
