@@ -733,7 +733,9 @@ GroupMap map_group(const Flat& f, const std::vector<std::vector<int>>& parts, in
 
 // Balanced contiguous groups of branches for chain fission: m groups minimising the largest group
 // cost (linear partition by DP over the branches' PEE times).
-std::vector<int> balanced_groups(const std::vector<double>& c, int m) {
+// head / tail: work outside the split-join that lands on the first / last group (SG_PART_CHAIN puts the
+// nodes before the split-join into group 0 and those after it into the last group).
+std::vector<int> balanced_groups(const std::vector<double>& c, int m, double head = 0.0, double tail = 0.0) {
     const int n = (int)c.size();
     m = std::min(m, n);
     std::vector<double> pre(n + 1, 0.0);
@@ -746,7 +748,8 @@ std::vector<int> balanced_groups(const std::vector<double>& c, int m) {
     for (int k = 1; k <= m; k++)
         for (int i = k; i <= n; i++)
             for (int j = k - 1; j < i; j++) {
-                double v = std::max(best[k - 1][j], pre[i] - pre[j]);
+                const double extra = (k == 1 ? head : 0.0) + (k == m && i == n ? tail : 0.0);
+                double v = std::max(best[k - 1][j], pre[i] - pre[j] + extra);
                 if (v < best[k][i] - 1e-12) { best[k][i] = v; cut[k][i] = j; }
             }
     std::vector<int> first(m);
@@ -777,7 +780,19 @@ Flat fissioned(const Flat& f, int sj, int m) {
         for (int v = si.first[b]; v < (b + 1 < nb ? si.first[b + 1] : si.join); v++) br.push_back(v);
         cost[b] = br.empty() ? 0.0 : pee_estimate(f, br).t;
     }
-    return chain_fission(f, sj, balanced_groups(cost, m));
+    std::vector<int> head, tail;
+    for (int v = 0; v < si.split; v++) head.push_back(v);
+    for (int v = si.join + 1; v < (int)f.nodes.size(); v++) tail.push_back(v);
+    // head / tail priced by their own work only (alone they would be partitions with the split-join's
+    // boundary streams, which they are not inside a group)
+    auto work_ns = [&](const std::vector<int>& nodes) {
+        if (nodes.empty()) return 0.0;
+        const PartitionWork w = partition_work(f, nodes);
+        return (w.flops / (kFp32 * kModel.e_staged) + w.intops / kInt + w.dfma * 80.0 / kFp64 +
+                kLoopFiring * w.loop_firings) * 1e9;
+    };
+    const double th = work_ns(head), tt = work_ns(tail);
+    return chain_fission(f, sj, balanced_groups(cost, m, th, tt));
 }
 
 // Graph variants and partitionings the planner compares (pipeline of Gs GPUs): the graph as written
