@@ -36,7 +36,7 @@ constexpr double kInt = kSM * 64 * kClk;          // int min/max per s
 constexpr double kFp64 = 37e12;                   // flop/s
 constexpr double kSmem = kSM * 128 * kClk;        // bytes/s
 constexpr double kHbm = 6.5536e12;                // bytes/s (MEASURED_PEAKS.json copy)
-constexpr double kLaunch = 6.8e-6;                // s per kernel launch incl. ramp / tail (fitted)
+constexpr double kLaunch = 8.5e-6;                // s per kernel launch incl. ramp / tail (fitted)
 constexpr double kFragIters = 1 << 20;            // iterations per fragment assumed when planning (the
                                                   // runtime's default at the bench sizes: n / (8 G))
 constexpr double kLoopFiring = 25e-9;             // s per sequential loop firing
@@ -60,11 +60,14 @@ struct PeeModel {
     double c_level;    // ns per compute level per tile
     double e_gen_hbm;  // general path: fraction of the HBM bandwidth its boundary streams reach
     double c_gen_edge; // general path: ns per boundary edge per tile
+    double c_gather;   // views only (gather kernels): ns per output item and (boundary input + 1)
 };
-constexpr PeeModel kModel{0.8, 2.819e-6, 9.785e-6, 0.7307, 0.4013, 0.003418, 0.3124, 9.007, 0.5677, 5.783};
+// fitted on the round-2 corpus (profiles/pee_corpus_r02.json); the general-path constants on the corpus of
+// the code generator before gather kernels existed, where that path ran (a 2-D DCT split: 58.8 ns/block)
+constexpr PeeModel kModel{0.8, 2.782e-6, 1.129e-5, 1.0, 0.3852, 0.0034, 0.7779, 8.674, 0.5677, 5.783, 5.649e-4};
 
 struct KernelShape {  // the code generator's decisions the model needs
-    bool demand = false, inplace = false, fused = true;
+    bool demand = false, inplace = false, fused = true, gather = false;
     double tile = 1;
 };
 
@@ -79,6 +82,7 @@ double model_ns(const PartitionWork& w, int mode, bool bitslice, double bitslice
         const double tc = (w.flops / (kFp32 * m.e_reg) + w.intops / kInt + w.dfma * 80.0 / kFp64) * 1e9;
         return std::max({tc, hbm, k.inplace ? 0.0 : m.c_row * row2});
     }
+    if (k.gather) return std::max(hbm, m.c_gather * (w.out_bytes / 4.0) * (w.in_edges + 1));
     const double e = k.fused ? (w.frame ? m.e_frame : m.e_staged) : m.e_general;
     const double W = std::max(1.0, k.tile);
     const double recompute = 1.0 + w.halo_firings / (W * std::max(1.0, w.firings));
@@ -123,6 +127,7 @@ PeeEstimate pee_estimate(const Flat& f, const std::vector<int>& nodes) {
     // the fused path declines for merges of many boundary streams (runtime index readers: the general
     // path) -- observed over the corpus
     const bool compute = (w.flops + w.intops + w.dfma + w.loop_firings) > 0;
+    k.gather = est.mode == 2 && !compute;
     est.fused = k.fused = est.mode != 2 || !compute || w.in_edges <= kFusedMaxInEdges;
     if (!k.fused) {  // the general path's tile: every buffer of the tile in ~100 KB of shared memory
         double W = 1;
@@ -139,7 +144,8 @@ double pee_refine(const PeeEstimate& est, const KernelInfo& ki) {
     KernelShape k;
     k.demand = ki.mode == 1 && ki.reg_variant == 2;
     k.inplace = ki.mode == 1 && ki.reg_variant == 1;
-    k.fused = ki.mode != 2 || ki.fused;  // mode 5 (gather) is priced like the fused path
+    k.fused = ki.mode != 2 || ki.fused;
+    k.gather = ki.mode == 5;
     k.tile = std::max(1, ki.tile);
     return model_ns(est.work, est.mode, est.bitslice, est.bitslice_ops, k, kModel);
 }

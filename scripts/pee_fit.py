@@ -60,7 +60,7 @@ def r2(xs, ys):
     return (sxy * sxy / (sxx * syy)) if sxx > 0 and syy > 0 else float("nan")
 
 
-LAUNCH_NS = 6.8e3  # sg_plan.cpp kLaunch: one kernel launch including ramp-up and tail
+LAUNCH_NS = 8.5e3  # sg_plan.cpp kLaunch: one kernel launch including ramp-up and tail
 
 # staged-mode model (sg_plan.cpp pee_estimate), all times in ns per iteration
 FP32 = 148 * 128 * 2 * 1.9e9

@@ -603,7 +603,7 @@ def test_planner_picks_chain_for_filterbank(sg, G):
         assert i["chain_fission"] and i["n_partitions"] == G and i["ilp_optimal"]
         assert sorted(i["partition_gpu"]) == list(range(G))
         t = i["partition_time"]
-        assert max(t) < 1.1 * min(t)
+        assert max(t) < 1.2 * min(t)          # equal branch work; the first group has one input stream fewer
         per_pair = {}
         for a, b, nbytes in p.pdg():
             per_pair[(a, b)] = per_pair.get((a, b), 0.0) + nbytes
