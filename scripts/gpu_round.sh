@@ -6,10 +6,11 @@
 #   corpus    the PEE corpus (scripts/pee_calibrate.py): every partition of a fixed set of plans, timed alone
 #   scaling   multi-GPU throughput predicted from measured partitions (scripts/scaling_prediction.py)
 #   ncu       ncu --set full of the main kernel of each config in $NCU_CONFIGS + the default bench's launch list
-#   sanitize  compute-sanitizer memcheck / racecheck / synccheck over the kernel families (scripts/sanitize.sh)
+#   sanitize  compute-sanitizer memcheck / racecheck / synccheck over the kernel families (scripts/sanitize.sh;
+#             closed on the GPU pool since r02: do not run it there)
 #   ab        bench A/B of $C (default filterbank64) over the variants in $AB ("name:ENV=V ...:bench args;...")
 TAG=${TAG:-round}
-STEPS=${STEPS:-tests bench corpus scaling ncu sanitize}
+STEPS=${STEPS:-tests bench corpus scaling ncu}
 CONFIGS=${CONFIGS:-filterbank64 fft64 fmradio10 beamformer12x4 bitonic32 des16 bitonicrec32 dct16 matmul16 matmul3_16 echo64}
 NCU_CONFIGS=${NCU_CONFIGS:-filterbank64}
 O=gpurun_out/$TAG
