@@ -199,6 +199,9 @@ def main():
                     help="--mode pipeline: replica groups (hybrid replica x pipeline plan); -1 = chosen by the cost model")
     ap.add_argument("--cuts", default="",
                     help="comma-separated node ids: user partitions [0, c1), [c1, c2), ... on one GPU (A/B of splits)")
+    ap.add_argument("--node-partition", default="",
+                    help="comma-separated partition id per node: user partitions on one GPU (A/B of non-contiguous "
+                         "splits)")
     ap.add_argument("--chain", type=int, default=0,
                     help="1 GPU: plan option chain_groups (chain fission of the largest eligible split-join, one "
                          "partition); 0 = as planned")
@@ -258,6 +261,8 @@ def main():
             with sg.plan(prog, 1, plan_only=1) as p0:
                 nn = p0.info()["n_nodes"]
             kw["node_partition"] = [sum(1 for c in cuts if c <= v) for v in range(nn)]
+        if args.node_partition:
+            kw["node_partition"] = [int(c) for c in args.node_partition.split(",")]
         plan = sg.plan(prog, 1, devices=[local], **kw)
     info = plan.info()
     nin, nout = plan.input_items(n), plan.output_items(n)
@@ -458,7 +463,8 @@ def main():
                        if not args.no_flush else "not flushed",
                        "chain_fission": info["chain_fission"], "partition_gpu": info["partition_gpu"],
                        "parallelism": (f"pipeline over {world} GPUs (ILP mapping, NCCL boundary streams)" if pipeline
-                                       else f"replicas x{world}" if world > 1 else "1 GPU, 1 partition"),
+                                       else f"replicas x{world}" if world > 1
+                                       else f"1 GPU, {info['n_partitions']} partition(s)"),
                        "partitions": info["n_partitions"], "partition_mode": info["partition_mode"],
                        "launch": "CUDA graph replay of one sg_run" if graph is not None else "eager sg_run",
                        "wall_s": wall},

@@ -369,7 +369,9 @@ int32_t sg_plan_pdg(const sg_plan_t* p, int32_t cap, int32_t* src, int32_t* dst,
  *   bytes, 23 CUDA source bytes, 24 register-mode variant (0 TMA / synchronous rows, 1 in-place components,
  *   2 demand-ordered wide rows); 25 dependence components of one iteration (register-eligible partitions);
  *   26 the plan-time expectation of 19 (staged: views only (gather) or at most 8 boundary input streams),
- *   27 the generated kernel's mode (1 register/bitslice, 2 staged, 4 feedback loop, 5 gather).
+ *   27 the generated kernel's mode (1 register/bitslice, 2 staged, 4 feedback loop, 5 gather), 28 the
+ *   fused kernel's frame-FIR parallel efficiency (ideal FFMA issue / the code generator's simulated issue
+ *   of its sliding-window levels; 1 without frame FIRs).
  * Returns the number of values written, or -1 (NULL plan / bad partition). */
 int32_t sg_pee_features(const sg_plan_t* p, int32_t part, double* out, int32_t cap);
 

@@ -323,15 +323,16 @@ int32_t sg_pee_features(const sg_plan_t* p, int32_t part, double* out, int32_t c
         const sg::PartitionWork& w = est.work;
         const sg::KernelInfo& ki = pl.kernels[part].ki;
         const bool gen = !pl.opts.plan_only;
-        const double v[28] = {(double)est.mode, w.flops, w.intops, w.dfma, w.reads, w.writes, w.firings, w.in_bytes,
+        const double v[29] = {(double)est.mode, w.flops, w.intops, w.dfma, w.reads, w.writes, w.firings, w.in_bytes,
                               w.out_bytes, (double)w.levels, w.halo_firings, w.loop_firings, (double)w.cse_nodes,
                               w.frame ? 1.0 : 0.0, est.bitslice ? 1.0 : 0.0, pl.part_time[part], (double)w.in_edges,
                               (double)w.out_edges, w.row_items,
                               gen ? (ki.fused ? 1.0 : 0.0) : -1.0, gen ? (double)ki.tile : -1.0,
                               gen ? (double)ki.threads : -1.0, gen ? (double)ki.smem : -1.0,
                               gen ? (double)ki.source.size() : -1.0, gen ? (double)ki.reg_variant : -1.0,
-                              (double)w.components, est.fused ? 1.0 : 0.0, gen ? (double)ki.mode : -1.0};
-        int32_t n = std::min<int32_t>(cap, 28);
+                              (double)w.components, est.fused ? 1.0 : 0.0, gen ? (double)ki.mode : -1.0,
+                              gen ? ki.par_eff : -1.0};
+        int32_t n = std::min<int32_t>(cap, 29);
         for (int32_t i = 0; i < n; i++) out[i] = v[i];
         return n;
     } catch (...) {

@@ -2258,7 +2258,8 @@ public:
                         for (auto& g : fg_) frame = frame || g.special;
                         // (opt-in FFMA2 frame FIRs, SG_FFMA2=1, need the 128 registers of 512-thread
                         // CTAs; measured slower: BeamFormer 2.88 ms vs 2.56 ms scalar at 1024 threads)
-                        NT_ = NT = (frame && !std::getenv("SG_FFMA2")) ? 1024 : 512;
+                        // (the sliding-window frame FIRs hold R-sample windows per plane: 512 threads)
+                        NT_ = NT = (frame && !std::getenv("SG_FFMA2") && !beam_slide_on()) ? 1024 : 512;
                         int W2 = 0;
                         for (int cand : fused_tile_candidates(opt.tile)) {
                             fused_layout(cand);
@@ -2301,6 +2302,23 @@ public:
                     fast_start = fused_emit(WF, true);
                     prologue_fast = prologue_;
                     ki.flops_exec_per_iter = fused_flops_per_iter();
+                    // frame-FIR levels: parallel efficiency of the chosen blocking (sliding-window form)
+                    // and the level to split before when one level cannot fill the CTA
+                    {
+                        double id = 0, co = 0, worst = 2.0;
+                        int wl = 0;
+                        for (auto& kv : beam_slide_) {
+                            if (kv.second.B <= 0 || kv.second.cost <= 0) continue;
+                            id += kv.second.ideal;
+                            co += kv.second.cost;
+                            const double e = kv.second.ideal / kv.second.cost;
+                            const int lv = level_.count(kv.first) ? level_.at(kv.first) : 0;
+                            if (e < worst) { worst = e; wl = lv; }
+                        }
+                        if (co > 0) ki.par_eff = std::min(1.0, id / co);
+                        ki.split_level = (worst < 0.6 && wl > 1) ? wl : 0;
+                        for (int u : nodes_) ki.node_level.push_back({u, node_level_of(u)});
+                    }
                 }
             } catch (const FusedFail& ff) {
                 if (std::getenv("SG_FUSED_DEBUG")) std::fprintf(stderr, "[sg codegen] partition %d: fused path declined (%s)\n", part_, ff.why);
@@ -2916,6 +2934,7 @@ private:
     void fused_layout(int W) {
         W_ = W;
         beam_B_.clear();
+        beam_slide_.clear();
         off_.clear();
         wb_.clear();
         size_.clear();
@@ -3794,6 +3813,23 @@ private:
         beam_f2_[v] = bestf2;
         return best;
     }
+    // fused level of a node of the partition: compute nodes their level, views the largest level of the
+    // compute nodes feeding them (a cut at a level boundary is then convex)
+    int node_level_of(int u) {
+        const Node& n = f_.nodes[u];
+        if (compute_node(u)) return level_.count(u) ? level_.at(u) : 0;
+        int L = 0;
+        for (int e : n.in) {
+            std::set<int> src;
+            R_.sources(e, src);
+            for (int pe : src) {
+                const int s = f_.edges[pe].src;
+                if (s >= 0 && std::find(nodes_.begin(), nodes_.end(), s) != nodes_.end() && compute_node(s))
+                    L = std::max(L, level_.count(s) ? level_.at(s) : 0);
+            }
+        }
+        return L;
+    }
     std::map<int, int> special_level_;
     int level_of_special(int v) {
         auto it = special_level_.find(v);
@@ -3957,6 +3993,245 @@ private:
           << "        }\n"
           << "      }\n";
     }
+    // ---- sliding-window frame FIR (fused kernels; the default, SG_BEAM_NOSLIDE=1 restores the chunked form)
+    // An item is (peer, firing, block of B consecutive outputs t0..t0+B-1).  At tap i output t0+b reads
+    // sample (t0+b)*DEC - i, so from one tap to the next the lane needs ONE new sample (per plane): the
+    // window lives in R registers per plane, sample S0 + rel (S0 = t0*DEC - i0, i0 = first tap of an
+    // R-tap group) in slot rel mod R -- compile-time slots, no register moves.  Per tap and lane: 4B FFMA,
+    // 2 scalar shared loads (re, im; lanes B*DEC samples apart), one constant-cache coefficient pair.
+    // Taps run i = 0..L-1 per output in the FIR's order (bit-identical to the chunked form); groups past
+    // the block's triangle limit (x[s < 0] = 0, reading 14) are skipped, so L % R == 0.
+    struct BeamSlide { int64_t B = 0, R = 0, PF = 2; bool pair = false; double cost = 0, ideal = 0; };
+    std::map<int, BeamSlide> beam_slide_;
+    static bool beam_slide_on() { return std::getenv("SG_BEAM_NOSLIDE") == nullptr; }
+    BeamSlide beam_slide_cfg(int v) {
+        auto it = beam_slide_.find(v);
+        if (it != beam_slide_.end()) return it->second;
+        const Node& n = f_.nodes[v];
+        int64_t peers = 0;
+        for (int u : nodes_)
+            if (compute_node(u) && special(u) && f_.nodes[u].iv == n.iv && level_of_special(u) == level_of_special(v)) peers++;
+        const int64_t L = n.iv[0], DEC = n.iv[1], OUT = n.iv[2] / n.iv[1];
+        const int64_t nf = n.halo + (int64_t)W_ * n.rep;
+        const int64_t nwarps = std::max(1, NT_ / 32);
+        BeamSlide best;
+        double bestc = 1e300;
+        // A/B override: SG_BEAM_B="level/B,level/B" (odd B) for the frame FIRs of the given fused levels
+        int64_t bforce = 0;
+        if (const char* e = std::getenv("SG_BEAM_B")) {
+            const std::string sp(e);
+            const int lv = level_of_special(v);
+            for (size_t p = 0; p < sp.size();) {
+                size_t q = sp.find(',', p);
+                if (q == std::string::npos) q = sp.size();
+                const std::string tok = sp.substr(p, q - p);
+                const size_t c = tok.find('/');
+                if (c != std::string::npos && std::atoi(tok.substr(0, c).c_str()) == lv) bforce = std::atoll(tok.c_str() + c + 1);
+                p = q + 1;
+            }
+        }
+        for (int64_t B = 1; B <= 15; B += 2) {
+            if (bforce && B != bforce) continue;
+            BeamSlide c;
+            c.B = B;
+            static const int64_t pf_env = std::getenv("SG_BEAM_PF") ? std::atoll(std::getenv("SG_BEAM_PF")) : 0;
+            if (pf_env > 0) c.PF = pf_env;
+            for (int64_t R : {4, 8, 16, 32})
+                if (R >= (B - 1) * DEC + c.PF + 1 && L % R == 0) { c.R = R; break; }
+            if (c.R == 0 || 2 * c.R + 2 * B > (NT_ <= 512 ? 104 : 44)) continue;  // register budget
+            for (bool pair : {false, true}) {
+                const int64_t NB = (OUT + B - 1) / B, NBP = pair ? (NB + 1) / 2 : NB;
+                auto blk_cost = [&](int64_t blk) {
+                    int64_t lim = std::min<int64_t>(L, (blk * B + B - 1) * DEC + 1);
+                    lim = std::min<int64_t>(L, (lim + c.R - 1) / c.R * c.R);
+                    return (double)lim * (4.0 * B + 3.5) + 4.0 * B + 40.0;
+                };
+                std::vector<double> per(NBP);
+                for (int64_t q = 0; q < NBP; q++) {
+                    const int64_t blk = pair ? q : NB - 1 - q;  // longest first
+                    per[q] = blk_cost(blk);
+                    if (pair && NB - 1 - q != q) per[q] += blk_cost(NB - 1 - q);
+                }
+                // dynamic scheduling: warps take 32 consecutive items; list-schedule the chunks
+                const int64_t items = peers * nf * NBP;
+                std::vector<double> wl(nwarps, 0.0);
+                for (int64_t k0 = 0; k0 < items; k0 += 32) {
+                    double cmax = 0;
+                    for (int64_t k = k0; k < std::min(items, k0 + 32); k++)
+                        cmax = std::max(cmax, per[pair ? k / (peers * nf) : k % NBP]);  // item order as emitted
+                    *std::min_element(wl.begin(), wl.end()) += cmax;
+                }
+                // a warp issues at most one instruction per cycle; warp w shares scheduler w % 4,
+                // which needs about four busy warps to hide the FFMA / shared-load latencies (measured on
+                // BeamFormer's matched filter: B = 1 over 16 warps beats B = 3 over 11, 2.37 vs 2.59 ms)
+                // (co-resident CTAs of the same kernel -- shared memory permitting -- add their warps)
+                const double ctas = (double)std::max(1, std::min(2, (int)((220 * 1024) / std::max<size_t>(1024, smem_bytes_))));
+                double cost = *std::max_element(wl.begin(), wl.end());
+                for (int s = 0; s < 4; s++) {
+                    double t = 0;
+                    int busy = 0;
+                    for (int64_t w = s; w < nwarps; w += 4) { t += wl[w]; busy += wl[w] > 0; }
+                    cost = std::max(cost, t / std::min(1.0, busy * ctas / 4.0));
+                }
+                if (cost < bestc * 0.98) { bestc = cost; best = c; best.pair = pair; best.cost = cost; }
+            }
+        }
+        // the level's pure FFMA issue (live taps, 4 FFMA per complex tap, 32 lanes, 4 schedulers): the
+        // parallel efficiency ideal / cost feeds the PEE (pee_refine) and the planner's level split
+        double taps = 0;
+        for (int64_t t = 0; t < OUT; t++) taps += (double)std::min<int64_t>(L, t * DEC + 1);
+        best.ideal = taps * 4.0 * (double)(peers * nf) / 128.0;
+        beam_slide_[v] = best;
+        return best;
+    }
+    std::map<std::vector<float>, std::string> beam_ct_;
+    std::string beam_const_table(const Node& n) {
+        auto it = beam_ct_.find(n.fv);
+        if (it != beam_ct_.end()) return it->second;
+        const int64_t L = n.iv[0];
+        std::string nm = "SG_CTS" + std::to_string(nvar_++);
+        consts_ << "__constant__ float2 " << nm << "[" << L << "] = {";
+        for (int64_t i = 0; i < L; i++)
+            consts_ << (i ? ", " : "") << "{" << hexf(n.fv[i]) << ", " << hexf(n.fv[L + i]) << "}";
+        consts_ << "};\n";
+        beam_ct_[n.fv] = nm;
+        return nm;
+    }
+    void emit_beam_fir_slide(std::ostringstream& b, int v, int64_t F0, int64_t rot, int64_t NP, const std::string& DINT,
+                             const std::string& DOUTT) {
+        const Node& n = f_.nodes[v];
+        const int64_t L = n.iv[0], DEC = n.iv[1], FR = n.iv[2], OUT = FR / DEC;
+        const BeamSlide cfg = beam_slide_cfg(v);
+        const int64_t B = cfg.B, R = cfg.R, PF = cfg.PF;
+        const int64_t NB = (OUT + B - 1) / B, NBP = cfg.pair ? (NB + 1) / 2 : NB;
+        static const bool ct_smem = std::getenv("SG_BEAM_CT_SMEM") != nullptr;
+        auto ct = ctab_off_.find(v);
+        std::string coef;  // expression of the (cr, ci) pair of tap `i0 + u`
+        if (ct_smem && ct != ctab_off_.end())
+            coef = "reinterpret_cast<const float2*>(sm + " + std::to_string(ct->second) + ")";
+        else
+            coef = beam_const_table(n);
+        auto slot = [&](int64_t rel) { return ((rel % R) + R) % R; };
+        auto sample = [&](int64_t rel, bool im, const std::string& var) {  // shared-memory read of sample var + rel
+            Lin p = Lin::v("lf", n.pop, 2 * rel + (im ? 1 : 0));
+            p.t.push_back({var, 2});
+            return "smi" + read_expr(n.in[0], p).substr(2);
+        };
+        b << "      const int items = nf * " << NBP * NP << ";  // sliding window: B = " << B << ", R = " << R
+          << (cfg.pair ? ", paired blocks" : "") << "\n";
+        // Every lane of a warp runs the same tap groups (trip count = the warp's largest triangle limit;
+        // a lane's extra taps read x[s < 0] = 0, exact by DESIGN.md reading 14), so the tap index is
+        // warp-uniform: the coefficient pair is a uniform-register operand of the FFMAs (LDCU), not a
+        // third vector register.  Items past the end are clamped to a valid one and not stored.
+        const int slot_c = nctr_++;
+        (void)rot;
+        b << "      for (int it0 = 0;;) {\n"
+          << "        if ((tid & 31) == 0) it0 = atomicAdd(&sg_ctr[" << slot_c << "], 32);\n"
+          << "        it0 = __shfl_sync(0xffffffffu, it0, 0);\n"
+          << "        if (it0 >= items) break;\n"
+          << "        const int itr = it0 + (tid & 31);\n"
+          << "        const bool valid = itr < items;\n"
+          << "        const int it = valid ? itr : items - 1;\n";
+        // paired blocks (long triangular filters): block-pair-major order, so the lanes of a warp run pairs
+        // of nearly equal triangle limits (the warp's trip count is its largest limit)
+        static const bool pmajor = std::getenv("SG_BEAM_PMAJOR") ? std::atoi(std::getenv("SG_BEAM_PMAJOR")) != 0 : true;
+        if (cfg.pair && pmajor)
+            b << "        const int pb = it / (nf * " << NP << ");\n"
+              << "        const int itq = it - pb * (nf * " << NP << ");\n"
+              << "        const int pq = itq / nf;\n"
+              << "        const int j = itq - pq * nf;\n";
+        else
+            b << "        const int pq = it / (nf * " << NBP << ");\n"
+              << "        const int itp = it - pq * (nf * " << NBP << ");\n"
+              << "        const int j = itp / " << NBP << ";\n"
+              << "        const int pb = itp - j * " << NBP << ";\n";
+        b
+          << "        const int lf = " << F0 << " + j;\n"
+          << "        const bool live = valid && gf + lf >= 0;  // firings before the stream start emit zeros\n"
+          << "        " << T_ << "* smi = sm + " << (NP > 1 ? DINT + "[pq]" : std::string("0")) << ";\n"
+          << "        " << T_ << "* smo = sm + " << (NP > 1 ? DOUTT + "[pq]" : std::string("0")) << ";\n"
+          << "        (void)pq; (void)smi; (void)smo;\n";
+        if (cfg.pair)
+            b << "#pragma unroll 1\n"
+              << "        for (int half = 0; half < 2; half++) {\n"
+              << "        const int blk = half ? " << NB - 1 << " - pb : pb;\n"
+              << "        const bool hs = valid && !(half && blk == pb), hv = hs && live;\n";
+        else
+            b << "        { const int blk = " << NB - 1 << " - pb;  // longest first\n"
+              << "        const bool hs = valid, hv = live;\n";
+        b << "        const int t0 = blk * " << B << ";\n"
+          << "        const int S0 = t0 * " << DEC << ";\n"
+          << "        const int ilim = min(" << L << ", (min(" << L << ", S0 + " << (B - 1) * DEC << " + 1) + " << R - 1
+          << ") / " << R << " * " << R << ");\n"
+          << "        const int ilimw = __reduce_max_sync(0xffffffffu, hv ? ilim : 0);\n"
+          << "        float re[" << B << "], im[" << B << "];\n";
+        for (int64_t bb = 0; bb < B; bb++) b << "        re[" << bb << "] = 0.0f; im[" << bb << "] = 0.0f;\n";
+        b << "        {\n"
+          << "          float xr[" << R << "], xi[" << R << "];\n";
+        // prologue: rel in [-(PF-1), (B-1)*DEC] relative to S0
+        auto prologue = [&](bool checked) {
+            for (int64_t rel = -(PF - 1); rel <= (B - 1) * DEC; rel++) {
+                const int64_t s = slot(rel);
+                if (checked)
+                    b << "            { const int s = S0 + " << rel << "; const bool ok = s >= 0 && s < " << FR << ";\n"
+                      << "              xr[" << s << "] = ok ? " << sample(rel, false, "S0") << " : 0.0f;\n"
+                      << "              xi[" << s << "] = ok ? " << sample(rel, true, "S0") << " : 0.0f; }\n";
+                else
+                    b << "            xr[" << s << "] = " << sample(rel, false, "S0") << "; xi[" << s << "] = "
+                      << sample(rel, true, "S0") << ";\n";
+            }
+        };
+        // guard decisions are warp-uniform too (one lane near the frame start would otherwise split the warp
+        // into a serialised few-lane pass over the guarded copy; the guarded copy is exact for every lane)
+        b << "          if (__all_sync(0xffffffffu, S0 - " << PF - 1 << " >= 0 && S0 + " << (B - 1) * DEC << " < " << FR
+          << ")) {\n";
+        prologue(false);
+        b << "          } else {\n";
+        prologue(true);
+        b << "          }\n"
+          << "#pragma unroll 1\n"
+          << "          for (int i0 = 0; i0 < ilimw; i0 += " << R << ") {\n"
+          << "            const int sb = S0 - i0;\n";
+        auto body = [&](bool checked) {
+            for (int64_t u = 0; u < R; u++) {
+                const int64_t rl = -(u + PF), sl = slot(rl);
+                b << "            { const float2 c = " << coef << "[i0 + " << u << "];\n";
+                if (checked)
+                    b << "              { const bool ok = sb - " << u + PF << " >= 0;\n"
+                      << "                xr[" << sl << "] = ok ? " << sample(rl, false, "sb") << " : 0.0f;\n"
+                      << "                xi[" << sl << "] = ok ? " << sample(rl, true, "sb") << " : 0.0f; }\n";
+                else
+                    b << "              xr[" << sl << "] = " << sample(rl, false, "sb") << "; xi[" << sl << "] = "
+                      << sample(rl, true, "sb") << ";\n";
+                for (int64_t bb = 0; bb < B; bb++) {
+                    const int64_t s = slot(bb * DEC - u);
+                    b << "              sg_cmac(re[" << bb << "], im[" << bb << "], xr[" << s << "], xi[" << s
+                      << "], c.x, c.y);\n";
+                }
+                b << "            }\n";
+            }
+        };
+        b << "            if (__all_sync(0xffffffffu, sb - " << R - 1 + PF << " >= 0)) {\n";
+        body(false);
+        b << "            } else {\n";
+        body(true);
+        b << "            }\n"
+          << "          }\n"
+          << "        }\n";
+        const int eo = n.out[0];
+        Lin pos = Lin::v("j", n.push, f_.edges[eo].pre + F0 * n.push);
+        pos.t.push_back({"(t0 + bb)", 2});
+        b << "        if (hs) {\n"
+          << "#pragma unroll\n"
+          << "        for (int bb = 0; bb < " << B << "; bb++)\n"
+          << "          if (t0 + bb < " << OUT << ") {\n"
+          << "            smo[" << buf_index(eo, pos).str() << "] = hv ? re[bb] : 0.0f;\n"
+          << "            smo[" << buf_index(eo, pos.plus(1)).str() << "] = hv ? im[bb] : 0.0f;\n"
+          << "          }\n"
+          << "        }\n"
+          << "        }\n"
+          << "      }\n";
+    }
     void emit_beam_fir(std::ostringstream& b, int v, int64_t F0, int64_t rot, const std::vector<int>& peers = {},
                        const std::vector<int64_t>& din = {}, const std::vector<int64_t>& dout = {}) {
         const Node& n = f_.nodes[v];
@@ -3981,6 +4256,10 @@ private:
             consts_ << "};\n__constant__ int " << DOUTT << "[" << NP << "] = {";
             for (int64_t q = 0; q < NP; q++) consts_ << (q ? ", " : "") << dout[q];
             consts_ << "};\n";
+        }
+        if (fused_ && beam_slide_on() && !std::getenv("SG_FFMA2") && beam_slide_cfg(v).B > 0) {
+            emit_beam_fir_slide(b, v, F0, rot, NP, DINT, DOUTT);
+            return;
         }
         if (beam_f2_[v] && ctab) {
             emit_beam_fir_f2(b, v, F0, NP, DINT, DOUTT, ct->second);

@@ -42,6 +42,7 @@ constexpr double kFragIters = 1 << 20;            // iterations per fragment ass
 constexpr double kLoopFiring = 25e-9;             // s per sequential loop firing
 constexpr long long kIlpNodeBudget = 4000000;     // branch-and-bound nodes per mapping (deterministic)
 constexpr int kFusedMaxInEdges = 8;               // staged: more boundary inputs -> general path expected
+constexpr double kFrameParRef = 1.0;               // par_eff the fitted e_frame corresponds to
 constexpr double kSplitMargin = 0.05;             // a cut must beat one partition by more than the PEE's noise
 
 // Model constants, fitted by least squares on log time to the partition corpus measured on the B200
@@ -69,6 +70,7 @@ constexpr PeeModel kModel{0.8, 2.782e-6, 1.129e-5, 1.0, 0.3852, 0.0034, 0.7779, 
 struct KernelShape {  // the code generator's decisions the model needs
     bool demand = false, inplace = false, fused = true, gather = false;
     double tile = 1;
+    double par_eff = 1;  // frame-FIR levels: the code generator's simulated parallel efficiency
 };
 
 double model_ns(const PartitionWork& w, int mode, bool bitslice, double bitslice_ops, const KernelShape& k,
@@ -83,7 +85,7 @@ double model_ns(const PartitionWork& w, int mode, bool bitslice, double bitslice
         return std::max({tc, hbm, k.inplace ? 0.0 : m.c_row * row2});
     }
     if (k.gather) return std::max(hbm, m.c_gather * (w.out_bytes / 4.0) * (w.in_edges + 1));
-    const double e = k.fused ? (w.frame ? m.e_frame : m.e_staged) : m.e_general;
+    const double e = k.fused ? (w.frame ? m.e_frame * k.par_eff : m.e_staged) : m.e_general;
     const double W = std::max(1.0, k.tile);
     const double recompute = 1.0 + w.halo_firings / (W * std::max(1.0, w.firings));
     const double tc = (w.flops / (kFp32 * e) + w.intops / kInt + w.dfma * 80.0 / kFp64) * recompute * 1e9 +
@@ -147,6 +149,7 @@ double pee_refine(const PeeEstimate& est, const KernelInfo& ki) {
     k.fused = ki.mode != 2 || ki.fused;
     k.gather = ki.mode == 5;
     k.tile = std::max(1, ki.tile);
+    k.par_eff = ki.fused ? std::max(0.05, ki.par_eff / kFrameParRef) : 1.0;
     return model_ns(est.work, est.mode, est.bitslice, est.bitslice_ops, k, kModel);
 }
 
@@ -1011,6 +1014,39 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
             return false;
         }
     };
+    // One GPU: a fused kernel whose frame-FIR level cannot fill the CTA (the code generator's simulated
+    // parallel efficiency, KernelInfo::split_level) is also tried as two partitions cut at that level
+    // boundary (convex: levels rise along every edge); the refined estimates decide (static discrepancy,
+    // the estimate sees the code generator's own decisions).
+    auto level_split = [&]() {
+        if (o.plan_only || Gs != 1 || R != 1 || p.parts.size() != 1 || o.partitioner != SG_PART_ALGORITHM1 ||
+            std::getenv("SG_NO_LEVEL_SPLIT"))
+            return;
+        const int sl = p.kernels[0].ki.split_level;
+        const std::vector<std::pair<int, int>> nlev = p.kernels[0].ki.node_level;
+        if (sl <= 1 || nlev.empty()) return;
+        std::vector<std::vector<int>> parts(2);
+        for (auto& nl : nlev) parts[nl.second >= sl ? 1 : 0].push_back(nl.first);
+        if (parts[0].empty() || parts[1].empty()) return;
+        const double one = p.est_tmax;
+        const std::vector<std::vector<int>> single{p.parts[0].nodes};
+        const Flat fsave = p.flat;
+        const bool chain = p.chain_fission;
+        try {
+            GroupMap gm = map_group(p.flat, parts, 1, o);
+            assemble_plan(p, parts, gm, G, R, Gs, o);
+            if (std::getenv("SG_PLAN_DEBUG"))
+                std::fprintf(stderr, "[sg plan] level split before level %d: %.3f ns vs one partition %.3f ns\n",
+                             sl, p.est_tmax, one);
+            if (p.est_tmax < one * (1.0 - kSplitMargin)) return;
+        } catch (const Error& e) {
+            if (e.code != SG_E_SIZE) throw;
+        }
+        p.flat = fsave;
+        p.chain_fission = chain;
+        GroupMap gm1 = map_group(p.flat, single, 1, o);
+        assemble_plan(p, single, gm1, G, R, Gs, o);
+    };
     int best_ci = -1;
     double best_ref = 0;
     size_t tried = 0;
@@ -1021,8 +1057,10 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         tried++;
         const bool cut = cands[ci].first.parts.size() > 1;
         if (o.plan_only || (p.est_tmax <= cands[ci].first.tmax * 1.5 &&
-                            (!cut || single_score <= 0 || p.est_tmax <= 0.9 * single_score)))
+                            (!cut || single_score <= 0 || p.est_tmax <= 0.9 * single_score))) {
+            level_split();
             return;
+        }
         if (best_ci < 0 || p.est_tmax < best_ref) { best_ci = (int)ci; best_ref = p.est_tmax; }
     }
     for (size_t ci = 0; ci < cands.size(); ci++)  // the one-partition candidate, if not yet tried
@@ -1032,6 +1070,7 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
         }
     if (best_ci < 0) throw Error(SG_E_SIZE, "no candidate partitioning fits the code generator's shared memory");
     if (!attempt((size_t)best_ci)) throw Error(SG_E_SIZE, "internal: candidate no longer fits");
+    level_split();
 }
 
 namespace {

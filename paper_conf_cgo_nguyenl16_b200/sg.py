@@ -376,12 +376,12 @@ class Plan:
     PEE_FEATURES = ["mode", "flops", "intops", "dfma", "reads", "writes", "firings", "in_bytes", "out_bytes",
                     "levels", "halo_firings", "loop_firings", "cse_nodes", "frame", "bitslice", "est_ns",
                     "in_edges", "out_edges", "row_items", "fused", "tile", "threads", "smem", "source_bytes",
-                    "reg_variant", "components", "fused_expected", "kernel_mode"]
+                    "reg_variant", "components", "fused_expected", "kernel_mode", "par_eff"]
 
     def pee_features(self, part: int) -> dict:
         """PEE inputs of one partition (work after the code generator's pruning / CSE, per iteration)."""
-        buf = (ctypes.c_double * 28)()
-        n = lib().sg_pee_features(self._h, part, buf, 28)
+        buf = (ctypes.c_double * 29)()
+        n = lib().sg_pee_features(self._h, part, buf, 29)
         if n < 0:
             raise SgError(SG_E_ARG, "bad partition")
         return {k: buf[i] for i, k in enumerate(self.PEE_FEATURES[:n])}
