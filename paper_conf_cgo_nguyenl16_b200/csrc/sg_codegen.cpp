@@ -486,7 +486,13 @@ public:
         const std::string VT4 = T_ == "float" ? "float4" : "int4";
         std::ostringstream src;
         src << header(demand_ ? "register, demand-ordered" : "register") << consts_.str() << args_struct();
-        if (demand_) src << "#define SG_LDV(r) (*(volatile const " << T_ << "*)&SG_LD1(r))\n";
+        // input re-reads: plain loads (the compiler may keep a run's inputs in registers) for rows of at most
+        // 256 items, volatile (no long live ranges) above -- measured DCT 16x16 0.40 -> 0.33 ms plain, MatMul 16
+        // (512-item rows) 0.70 -> 0.72 ms plain; SG_DEMAND_VOL=0/1 forces either
+        const bool dvol = std::getenv("SG_DEMAND_VOL") ? std::atoi(std::getenv("SG_DEMAND_VOL")) != 0 : PIN_ > 256;
+        if (demand_)
+            src << (!dvol ? "#define SG_LDV(r) (SG_LD1(r))\n"
+                          : "#define SG_LDV(r) (*(volatile const " + T_ + "*)&SG_LD1(r))\n");
         if (demand_) {
             ki.reg_variant = 2;
             return run_demand(ki, src, VT4, opt);
@@ -763,16 +769,24 @@ private:
     // each output group straight to global memory from registers: half the shared memory per row, so
     // twice the warps per SM of the staged-row variants; no TMA (the rows are consumed out of order).
     KernelInfo run_demand(KernelInfo& ki, std::ostringstream& src, const std::string& VT4, const CodegenOpts& opt) {
-        const int bytes_per_thread = (int)(RIN_S_ * 4);
+        const int bytes_per_row = (int)(RIN_S_ * 4);
+        const int K = demand_K_;
         int NT = opt.threads;
         if (NT <= 0) {
             NT = 256;
-            while (NT > 32 && (size_t)NT * bytes_per_thread > 100 * 1024) NT /= 2;
+            while (NT > 32 * K && (size_t)(NT / K) * bytes_per_row > 100 * 1024) NT /= 2;
         }
-        const size_t smem = (size_t)NT * bytes_per_thread;
-        const int minb = std::max(1, std::min(8, (int)((220 * 1024) / std::max<size_t>(1, smem))));
-        src << "#define SG_LD4(g) (reinterpret_cast<const " << VT4 << "*>(xr)[g])\n"
-            << "#define SG_LD1(r) (xr[r])\n"
+        if (NT % (32 * K) != 0) throw Error(SG_E_ARG, "threads must be a multiple of 32 x the demand runs");
+        const int TR = NT / K;  // iterations (rows) per tile
+        // rows stored transposed (item q of row r at q * (TR + 1) + r): the lanes of a warp -- consecutive
+        // rows -- read item q from consecutive banks (row-major rows 4 items apart were a 4-way conflict
+        // on every one of DCT 16x16's 4 096 input re-reads per block)
+        const int ST = TR + 1;
+        const size_t smem = (size_t)PIN_ * ST * 4;
+        // CTAs per SM the shared memory allows, but never below 128 registers per thread (the demand
+        // bodies' live sets: DCT 16x16 at 42 registers spilled 9 KB per thread)
+        const int minb = std::max(1, std::min({8, (int)((220 * 1024) / std::max<size_t>(1, smem)), 65536 / (NT * 128)}));
+        src << "#define SG_LD1(r) (xr[(r) * " << ST << "])\n"
             << "#define SG_ST4(g, v) do { const " << VT4 << " t_ = (v); if (ga) reinterpret_cast<" << VT4
             << "*>(yg)[g] = t_; else { yg[4 * (g)] = t_.x; yg[4 * (g) + 1] = t_.y; yg[4 * (g) + 2] = t_.z; yg[4 * (g) + 3] = t_.w; } } while (0)\n"
             << "#define SG_ST1(g, v) (yg[g] = (v))\n";
@@ -783,32 +797,49 @@ private:
             << "  " << T_ << "* s_in = reinterpret_cast<" << T_ << "*>(sg_smem);\n"
             << "  const " << T_ << "* gin = SG_IN(0);\n"
             << "  " << T_ << "* gout = SG_OUT(0);\n"
-            << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * NT; t0 < SG_K_END; t0 += (long long)gridDim.x * NT) {\n"
-            << "    const int nt = (int)min((long long)NT, SG_K_END - t0);\n"
+            << "  constexpr int TR = " << TR << ";  // rows per tile: " << K << " warp(s) per 32 rows, one demand run each\n"
+            << "  const int q_ = (threadIdx.x >> 5) % " << K << ";\n"
+            << "  const int r_ = (threadIdx.x >> 5) / " << K << " * 32 + (threadIdx.x & 31);\n"
+            << "  (void)q_;\n"
+            << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * TR; t0 < SG_K_END; t0 += (long long)gridDim.x * TR) {\n"
+            << "    const int nt = (int)min((long long)TR, SG_K_END - t0);\n"
             << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
-            << (vin_ ? std::string("    if ((reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0)\n      sg_rows_g2s_v4<") +
-                           T_ + ", " + std::to_string(PIN_) + ", " + std::to_string(RIN_S_) + ", NT>(gsrc, s_in, nt);\n    else\n"
-                     : std::string())
-            << "      sg_rows_g2s_v1<" << T_ << ", " << PIN_ << ", " << RIN_S_ << ", NT>(gsrc, s_in, nt);\n"
+            << (PIN_ % 4 == 0 ? std::string("    if ((reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0) {\n") +
+                   "      for (int i = threadIdx.x; i < nt * " + std::to_string(PIN_ / 4) + "; i += NT) {\n" +
+                   "        const int row = i / " + std::to_string(PIN_ / 4) + ", c = i - row * " + std::to_string(PIN_ / 4) + ";\n" +
+                   "        const " + VT4 + " v = __ldg(reinterpret_cast<const " + VT4 + "*>(gsrc) + i);\n" +
+                   "        " + T_ + "* d = s_in + 4 * c * " + std::to_string(ST) + " + row;\n" +
+                   "        d[0] = v.x; d[" + std::to_string(ST) + "] = v.y; d[" + std::to_string(2 * ST) + "] = v.z; d[" +
+                   std::to_string(3 * ST) + "] = v.w;\n" +
+                   "      }\n    } else\n"
+                                : std::string())
+            << "    for (int i = threadIdx.x; i < nt * " << PIN_ << "; i += NT) {\n"
+            << "      const int row = i / " << PIN_ << ", q = i - row * " << PIN_ << ";\n"
+            << "      s_in[q * " << ST << " + row] = gsrc[i];\n"
+            << "    }\n"
             << "    __syncthreads();\n"
             << "    " << T_ << "* gdst = gout + (t0 * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
             << "    const bool ga = " << (vout_ ? "(reinterpret_cast<unsigned long long>(gdst) & 15ull) == 0" : "false") << ";\n"
             << "    (void)ga;\n"
-            << "    if (threadIdx.x < nt) {\n"
-            << "      const " << T_ << "* xr = s_in + threadIdx.x * " << RIN_S_ << ";\n"
-            << "      " << T_ << "* yg = gdst + (long long)threadIdx.x * " << POUT_ << ";\n"
-            << body_.str()
-            << "    }\n"
+            << "    if (r_ < nt) {\n"
+            << "      const " << T_ << "* xr = s_in + r_;\n"
+            << "      " << T_ << "* yg = gdst + (long long)r_ * " << POUT_ << ";\n";
+        for (int k = 0; k < K; k++)
+            src << (K > 1 ? std::string(k ? "      } else if (q_ == " : "      if (q_ == ") + std::to_string(k) + ") {\n" : std::string())
+                << dbodies_[k];
+        if (K > 1) src << "      }\n";
+        src << "    }\n"
             << "    __syncthreads();  // the next tile's loads reuse the rows\n"
             << "  }\n}\n"
-            << "#undef SG_LD4\n#undef SG_LD1\n#undef SG_ST4\n#undef SG_ST1\n";
+            << "#undef SG_LD1\n#undef SG_ST4\n#undef SG_ST1\n";
         ki.has_tma = false;
         ki.tma_in = ki.tma_out = 0;
         ki.name = ki.name_sync;
         ki.threads = ki.threads_sync = NT;
-        ki.tile = ki.tile_sync = NT;
+        ki.tile = ki.tile_sync = TR;
         ki.smem = ki.smem_sync = smem;
         ki.min_blocks = 1;
+        ki.demand_runs = K;
         ki.source = src.str();
         return ki;
     }
@@ -877,6 +908,12 @@ private:
         if (!out.insert({ed.src, g}).second) return;
         for (int64_t i = 0; i < n.peek; i++) deps_of(n.in[0], g * n.pop + i, out);
     }
+    // The output groups are split into K contiguous runs of the demand order (about equal new-firing work
+    // each; a run recomputes what an earlier run had memoized) -- one body per run, run by its own warps:
+    // K warps share one iteration's input row, so a CTA holds NT / K rows instead of NT and the SM K times
+    // more warps (DCT 16x16: one row of 1 KB per thread held it to 6 warps per SM).
+    std::vector<std::string> dbodies_;
+    int demand_K_ = 1;
     void emit_body_demand() {
         const int gs = vout_ ? 4 : 1;
         const int ng = (int)((POUT_ + gs - 1) / gs);
@@ -884,16 +921,11 @@ private:
         for (int g = 0; g < ng; g++)
             for (int64_t p = g * gs; p < std::min<int64_t>(POUT_, (int64_t)(g + 1) * gs); p++) deps_of(eout_, off_out_ + p, dep[g]);
         std::vector<char> done(ng, 0);
+        std::vector<int> order;
         int cur = 0;
         for (int step = 0; step < ng; step++) {
             done[cur] = 1;
-            std::string v[4];
-            for (int i = 0; i < gs; i++) v[i] = dv(eout_, off_out_ + (int64_t)cur * gs + i);
-            if (vout_)
-                body_ << "      SG_ST4(" << cur << ", make_" << (T_ == "float" ? "float4" : "int4") << "(" << v[0] << ", " << v[1]
-                      << ", " << v[2] << ", " << v[3] << "));\n";
-            else
-                body_ << "      SG_ST1(" << cur << ", " << v[0] << ");\n";
+            order.push_back(cur);
             int best = -1;
             size_t bscore = 0;
             for (int g = 0; g < ng; g++) {
@@ -905,6 +937,50 @@ private:
             if (best < 0) break;
             cur = best;
         }
+        // K: four runs (64 rows per 256-thread CTA), more when the transposed rows would not fit ~200 KB of
+        // shared memory (SG_DEMAND_K overrides); measured: DCT 16x16 K = 1/2/4/8 -> 0.82/0.66/0.40/1.03 ms,
+        // MatMul 16 1.40/0.89/0.70/0.91 ms per 2^18 iterations
+        int K = 4;
+        while (K < 32 && (int64_t)PIN_ * (256 / K + 1) * 4 > 200 * 1024) K *= 2;
+        if (const char* e = std::getenv("SG_DEMAND_K")) K = std::max(1, std::atoi(e));
+        K = std::max(1, std::min(K, (int)order.size()));
+        while (K > 1 && 256 % (32 * K) != 0) K--;
+        // new firings per group along the order (one run's memo), then K runs of about equal work
+        std::set<std::pair<int, int64_t>> seen;
+        std::vector<double> w(order.size());
+        double tot = 0;
+        for (size_t i = 0; i < order.size(); i++) {
+            size_t nw = 0;
+            for (auto& k : dep[order[i]]) nw += seen.insert(k).second;
+            w[i] = (double)nw + 1.0;
+            tot += w[i];
+        }
+        std::vector<size_t> start{0};
+        double acc = 0;
+        for (size_t i = 0; i < order.size() && (int)start.size() < K; i++) {
+            acc += w[i];
+            if (acc >= tot * (double)start.size() / K && i + 1 < order.size()) start.push_back(i + 1);
+        }
+        K = (int)start.size();
+        start.push_back(order.size());
+        demand_K_ = K;
+        dbodies_.clear();
+        for (int k = 0; k < K; k++) {
+            dm_.clear();
+            body_.str("");
+            for (size_t i = start[k]; i < start[k + 1]; i++) {
+                const int g = order[i];
+                std::string v[4];
+                for (int j = 0; j < gs; j++) v[j] = dv(eout_, off_out_ + (int64_t)g * gs + j);
+                if (vout_)
+                    body_ << "      SG_ST4(" << g << ", make_" << (T_ == "float" ? "float4" : "int4") << "(" << v[0] << ", " << v[1]
+                          << ", " << v[2] << ", " << v[3] << "));\n";
+                else
+                    body_ << "      SG_ST1(" << g << ", " << v[0] << ");\n";
+            }
+            dbodies_.push_back(body_.str());
+        }
+        body_.str("");
     }
     bool try_inplace(KernelInfo& ki, std::ostringstream& src, const std::string& VT4) {
         if (PIN_ != POUT_ || PIN_ % 4 != 0 || PIN_ * 4 == 128 || RIN_S_ != ROUT_S_) return false;

@@ -43,6 +43,7 @@ struct KernelInfo {
                                      // copies), 2 demand-ordered wide single-component rows
     int64_t flops_exec_per_iter = -1;  // fused: algorithmic flops after dead/zero pruning (no recompute)
     std::string name_start;          // staged fused: stream-start variant (tiles with k0 < ksafe)
+    int demand_runs = 1;             // register demand-ordered: warps (output-group runs) per iteration row
     double par_eff = 1.0;            // fused frame-FIR levels: ideal FFMA issue / simulated issue (<= 1)
     int split_level = 0;             // > 0: a frame-FIR level that cannot fill the CTA starts at this level
     std::vector<std::pair<int, int>> node_level;  // fused: (flat node, level) of every node of the partition

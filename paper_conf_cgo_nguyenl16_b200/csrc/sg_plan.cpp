@@ -65,7 +65,9 @@ struct PeeModel {
 };
 // fitted on the round-2 corpus (profiles/pee_corpus_r02.json); the general-path constants on the corpus of
 // the code generator before gather kernels existed, where that path ran (a 2-D DCT split: 58.8 ns/block)
-constexpr PeeModel kModel{0.8, 2.782e-6, 1.129e-5, 1.0, 0.3852, 0.0034, 0.7779, 8.674, 0.5677, 5.783, 5.649e-4};
+// e_frame and c_demand re-centred on the corpus of the sliding-window frame FIRs (which report their parallel
+// efficiency, e_frame x par_eff) and of the four-run transposed-row demand kernels (profiles/pee_corpus_r02b.json)
+constexpr PeeModel kModel{0.8, 2.782e-6, 4.6e-6, 1.0, 0.534, 0.0034, 0.7779, 8.674, 0.5677, 5.783, 5.649e-4};
 
 struct KernelShape {  // the code generator's decisions the model needs
     bool demand = false, inplace = false, fused = true, gather = false;

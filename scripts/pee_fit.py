@@ -83,6 +83,9 @@ def main():
     ap.add_argument("corpus")
     ap.add_argument("--fit", action="store_true")
     ap.add_argument("--out", default="")
+    ap.add_argument("--fit-frame", action="store_true",
+                    help="report the e_frame (sg_plan.cpp kModel) that centres the frame-FIR partitions' "
+                         "measured / estimated ratio at 1 (geometric mean), given their par_eff")
     args = ap.parse_args()
     rows = json.load(open(args.corpus))
     F = features(rows)
@@ -99,6 +102,14 @@ def main():
         print("fitted staged constants (eff, eff_frame, level s, smem cycles/item, fixed ns):", list(sol.x))
         for f in S:
             f["fit"] = staged_model(sol.x, f)
+    if args.fit_frame:
+        fr = [f for f in F if f["frame"] and f["mode"] == 2]
+        if fr:
+            g = math.exp(sum(math.log(f["meas"] / f["est"]) for f in fr) / len(fr))
+            print("frame partitions: %d, geometric-mean measured / estimated %.3f -> e_frame x %.3f" % (len(fr), g, 1 / g))
+            for f in fr:
+                print("  %s G=%d part %d par_eff %.3f est %.1f meas %.1f" % (f["config"], f["G"], f["part"],
+                                                                           f.get("par_eff", 1), f["est"], f["meas"]))
     est = [f["est"] for f in F]
     mea = [f["meas"] for f in F]
     ratios = sorted(m / e for e, m in zip(est, mea))
