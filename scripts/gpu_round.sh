@@ -35,9 +35,11 @@ for step in $STEPS; do
     cat $O/scaling_prediction.md ;;
   ncu)
     for c in $NCU_CONFIGS; do
-      timeout 900 ncu --set full --clock-control none --import-source on -k regex:"sg_part0$" -s 3 -c 1 \
+      python bench.py --config $c --steps 2 --warmup 3 --no-cpu-baseline > $O/plain_$c.log 2>&1 &&
+      timeout 900 ncu --set full --clock-control none --import-source on -k regex:"sg_part[0-9]+$" -s 3 -c ${NCU_C:-2} \
         -o $O/full_$c python bench.py --config $c --steps 2 --warmup 3 --no-cpu-baseline > $O/ncu_$c.log 2>&1
     done
+    python bench.py --steps 5 --warmup 3 --no-cpu-baseline > $O/plain_default.log 2>&1 &&
     timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none -c 60 --csv \
       --log-file $O/launches_filterbank64.csv python bench.py --steps 5 --warmup 3 --no-cpu-baseline > /dev/null 2>&1 ;;
   sanitize)
