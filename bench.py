@@ -376,7 +376,9 @@ def main():
                          if info["n_partitions"] == 1 else
                          f"the whole step: {info['n_partitions']} partition kernels back to back on one GPU")
     prof = os.path.join(ROOT, "profiles", "ncu_traffic.json")
-    if roof is not None and os.path.exists(prof):
+    # (per-launch DRAM bytes of one kernel; a multi-partition step launches each kernel once per fragment,
+    # so only one-partition steps carry it -- the profiles/ summary lists every kernel's own)
+    if roof is not None and os.path.exists(prof) and info["n_partitions"] == 1:
         try:
             tr = json.load(open(prof)).get(name)
             if tr:

@@ -4102,7 +4102,12 @@ private:
                 if (q == std::string::npos) q = sp.size();
                 const std::string tok = sp.substr(p, q - p);
                 const size_t c = tok.find('/');
-                if (c != std::string::npos && std::atoi(tok.substr(0, c).c_str()) == lv) bforce = std::atoll(tok.c_str() + c + 1);
+                // "level/B", or "t<taps>x<dec>/B" for every frame FIR of that shape
+                const bool shape = !tok.empty() && tok[0] == 't';
+                const std::string key = tok.substr(shape ? 1 : 0, c == std::string::npos ? 0 : c - (shape ? 1 : 0));
+                const bool hit = shape ? key == std::to_string(n.iv[0]) + "x" + std::to_string(n.iv[1])
+                                       : std::atoi(key.c_str()) == lv;
+                if (c != std::string::npos && hit) bforce = std::atoll(tok.c_str() + c + 1);
                 p = q + 1;
             }
         }

@@ -67,7 +67,7 @@ struct PeeModel {
 // the code generator before gather kernels existed, where that path ran (a 2-D DCT split: 58.8 ns/block)
 // e_frame and c_demand re-centred on the corpus of the sliding-window frame FIRs (which report their parallel
 // efficiency, e_frame x par_eff) and of the four-run transposed-row demand kernels (profiles/pee_corpus_r02b.json)
-constexpr PeeModel kModel{0.8, 2.782e-6, 4.6e-6, 1.0, 0.534, 0.0034, 0.7779, 8.674, 0.5677, 5.783, 5.649e-4};
+constexpr PeeModel kModel{0.8, 2.782e-6, 4.6e-6, 1.0, 0.595, 0.0034, 0.7779, 8.674, 0.5677, 5.783, 5.649e-4};
 
 struct KernelShape {  // the code generator's decisions the model needs
     bool demand = false, inplace = false, fused = true, gather = false;
@@ -1021,7 +1021,7 @@ void build_plan(Plan& p, const sg_graph& g, int G, const sg_plan_opts& o) {
     // boundary (convex: levels rise along every edge); the refined estimates decide (static discrepancy,
     // the estimate sees the code generator's own decisions).
     auto level_split = [&]() {
-        if (o.plan_only || Gs != 1 || R != 1 || p.parts.size() != 1 || o.partitioner != SG_PART_ALGORITHM1 ||
+        if (o.plan_only || Gs != 1 || p.parts.size() != 1 || o.partitioner != SG_PART_ALGORITHM1 ||
             std::getenv("SG_NO_LEVEL_SPLIT"))
             return;
         const int sl = p.kernels[0].ki.split_level;

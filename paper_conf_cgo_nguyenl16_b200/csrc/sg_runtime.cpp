@@ -403,6 +403,7 @@ void reset_state(CompiledKernel& ck, int dev, cudaStream_t stream) {
 Plan::~Plan() {
     dist_release();
     for (auto e : host_ev) cudaEventDestroy(e);
+    for (auto e : pipe_ev) cudaEventDestroy(e);
     if (host_in_stream) cudaStreamDestroy(host_in_stream);
     if (host_out_stream) cudaStreamDestroy(host_out_stream);
     for (auto& r : rings) {
@@ -597,12 +598,32 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
             reset_state(kernels[p], gc.dev, gc.compute);
         }
     const int64_t nfrag = (n + F - 1) / F;
+    // host pipeline (run_host): fragment fi's input prefix arrives on host_in_stream before the partition
+    // reading the graph input runs it; its outputs leave on host_out_stream once the writing partition is done
+    const bool pipe = pipe_hin != nullptr && R == 1;
+    int64_t piped_in = 0;
+    if (pipe)
+        while ((int64_t)pipe_ev.size() < 2 * nfrag) {
+            cudaEvent_t e;
+            SG_RT(cudaEventCreateWithFlags(&e, cudaEventDisableTiming));
+            pipe_ev.push_back(e);
+        }
     for (int64_t fi = 0; fi < nfrag; fi++) {
         const int64_t ka = fi * F, kb = std::min(n, ka + F);
         // fragments dealt round-robin to the replica groups; rings are per group
         const int grp = (int)(fi % R);
         const int64_t fg = fi / R;
         const int slot = (int)(fg % ring_depth);
+        if (pipe) {
+            const int64_t need = flat.input_items(kb);
+            if (need > piped_in) {
+                DevGuard dg(devices[input_gpu]);
+                SG_RT(cudaMemcpyAsync((char*)in + piped_in * 4, (const char*)pipe_hin + piped_in * 4,
+                                      (size_t)(need - piped_in) * 4, cudaMemcpyHostToDevice, host_in_stream));
+                piped_in = need;
+            }
+            SG_RT(cudaEventRecord(pipe_ev[2 * fi], host_in_stream));
+        }
         for (int p : part_order) {
             CompiledKernel& ck = kernels[p];
             const int g = grp * Gs + part_gpu[p];
@@ -610,8 +631,10 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
             GpuCtx& gc = gpus[g];
             DevGuard dg(gc.dev);
             IoBinding io;
+            bool writes_out = false;
             for (int e : ck.ki.in_edges) {
                 if (flat.edges[e].src < 0) {  // graph input (resident on this GPU: input_gpu)
+                    if (pipe) SG_RT(cudaStreamWaitEvent(gc.compute, pipe_ev[2 * fi], 0));
                     io.in.push_back(in);
                     io.in_base.push_back(0);
                     io.in_limit.push_back(n_in);
@@ -630,6 +653,7 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                 if (flat.edges[e].dst < 0) {
                     io.out.push_back(out);
                     io.out_base.push_back(0);
+                    writes_out = true;
                     continue;
                 }
                 int ri = -1;
@@ -645,6 +669,13 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
                 io.out_base.push_back(ka * r.per_iter + r.lo);
             }
             last_launches += launch(ck, gc.dev, io, ka, kb, gc.compute, flat.dtype == SG_F32);
+            if (pipe && writes_out) {
+                SG_RT(cudaEventRecord(pipe_ev[2 * fi + 1], gc.compute));
+                SG_RT(cudaStreamWaitEvent(host_out_stream, pipe_ev[2 * fi + 1], 0));
+                const int64_t o0 = flat.output_items(ka), o1 = flat.output_items(kb);
+                SG_RT(cudaMemcpyAsync((char*)pipe_hout + o0 * 4, (const char*)out + o0 * 4, (size_t)(o1 - o0) * 4,
+                                      cudaMemcpyDeviceToHost, host_out_stream));
+            }
             // consumed slots of incoming rings are free again
             for (int ri : ring_in[gp]) SG_RT(cudaEventRecord(rings[ri].ev_consumed[slot], gc.compute));
             // ship outgoing boundary streams to other GPUs (copy engine, P2P)
@@ -751,6 +782,30 @@ void Plan::run_host(const void* hin, int64_t n, void* hout) {
                                   cudaMemcpyDeviceToHost, host_out_stream));
         }
         SG_RT(cudaStreamSynchronize(host_out_stream));
+        SG_RT(cudaStreamSynchronize(host_stream));
+        return;
+    }
+    bool loops = false;
+    for (auto& k : kernels) loops = loops || k.ki.state_words > 0;
+    if (parts.size() > 1 && R == 1 && G == 1 && !loops && NCH > 1) {
+        // several partitions: the fragment pipeline itself carries the copies (see run())
+        if (!host_in_stream) {
+            SG_RT(cudaStreamCreateWithFlags(&host_in_stream, cudaStreamNonBlocking));
+            SG_RT(cudaStreamCreateWithFlags(&host_out_stream, cudaStreamNonBlocking));
+        }
+        pipe_hin = hin;
+        pipe_hout = hout;
+        try {
+            run(host_in_dev, n, host_out_dev, host_stream);
+        } catch (...) {
+            pipe_hin = nullptr;
+            pipe_hout = nullptr;
+            throw;
+        }
+        pipe_hin = nullptr;
+        pipe_hout = nullptr;
+        SG_RT(cudaStreamSynchronize(host_out_stream));
+        SG_RT(cudaStreamSynchronize(host_in_stream));
         SG_RT(cudaStreamSynchronize(host_stream));
         return;
     }

@@ -106,6 +106,11 @@ struct Plan {
     cudaStream_t host_stream = nullptr;
     cudaStream_t host_in_stream = nullptr, host_out_stream = nullptr;  // chunked copy pipeline
     std::vector<cudaEvent_t> host_ev;
+    // set by run_host for a multi-partition plan: run() copies each fragment's input prefix in and its
+    // output range out on the host streams, interleaved with the fragment pipeline
+    const void* pipe_hin = nullptr;
+    void* pipe_hout = nullptr;
+    std::vector<cudaEvent_t> pipe_ev;
 
     // one process per GPU (sg_dist.cpp)
     void* comm = nullptr;  // ncclComm_t

@@ -36,7 +36,7 @@ for step in $STEPS; do
   ncu)
     for c in $NCU_CONFIGS; do
       python bench.py --config $c --steps 2 --warmup 3 --no-cpu-baseline > $O/plain_$c.log 2>&1 &&
-      timeout 900 ncu --set full --clock-control none --import-source on -k regex:"sg_part[0-9]+$" -s 3 -c ${NCU_C:-2} \
+      timeout 900 ncu --set full --clock-control none --import-source on -k regex:"sg_part[0-9]+(_sync)?$" -s 3 -c ${NCU_C:-2} \
         -o $O/full_$c python bench.py --config $c --steps 2 --warmup 3 --no-cpu-baseline > $O/ncu_$c.log 2>&1
     done
     python bench.py --steps 5 --warmup 3 --no-cpu-baseline > $O/plain_default.log 2>&1 &&

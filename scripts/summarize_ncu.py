@@ -38,9 +38,23 @@ UNITS = {"Gbyte": 1e9, "Mbyte": 1e6, "Kbyte": 1e3, "byte": 1.0}
 
 
 def raw(rep):
+    """One (metrics, stalls) pair per distinct kernel of the capture (the first launch of each)."""
     out = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
     rows = list(csv.reader(io.StringIO(out)))
-    h, units, v = rows[0], rows[1], rows[2]
+    h, units = rows[0], rows[1]
+    res, seen = [], set()
+    for v in rows[2:]:
+        if len(v) != len(h):
+            continue
+        k = v[h.index("Kernel Name")] if "Kernel Name" in h else str(len(res))
+        if k in seen:
+            continue
+        seen.add(k)
+        res.append((k,) + one(h, units, v))
+    return res
+
+
+def one(h, units, v):
     d = {h[i]: (v[i], units[i]) for i in range(len(h))}
     stalls = []
     for k, (x, _) in d.items():
@@ -63,7 +77,8 @@ def main(rnd):
     os.makedirs(os.path.join(ROOT, "profiles"), exist_ok=True)
     lines = [f"# ncu summary, round {rnd}", "",
              "Main partition kernel of `bench.py --config <name> --steps 2 --warmup 3` captured with",
-             "`ncu --set full --clock-control none --import-source on -k regex:sg_part0$ -s 2 -c 1`",
+             "`ncu --set full --clock-control none --import-source on -k regex:sg_part[0-9]+$ -s 3 -c 2` (every",
+             "partition kernel of the plan; traffic summed over them per launch of each),"
              "(one launch, cold caches, serialised: use for shares and counters, not as the bench value).", ""]
     tpath = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     traffic = json.load(open(tpath)) if os.path.exists(tpath) else {}
@@ -71,21 +86,25 @@ def main(rnd):
     names = sorted(os.path.basename(r)[5:-8] for r in glob.glob(os.path.join(src, "full_*.ncu-rep")))
     for name in names:
         rep = os.path.join(src, f"full_{name}.ncu-rep")
-        d, stalls = raw(rep)
-        lines.append(f"## {name}")
-        lines.append("")
-        lines.append("| metric | value |")
-        lines.append("|---|---|")
-        for k, label in METRICS:
-            if k in d:
-                lines.append(f"| {label} (`{k}`) | {d[k][0]} {d[k][1]} |")
-        lines.append(f"| top stall reasons (pc sampling) | {', '.join(f'{k} {x:.0%}' for k, x in stalls)} |")
-        lines.append("")
-        try:
-            traffic[name] = {"dram_bytes_per_launch": to_bytes(*d["dram__bytes_read.sum"]) +
-                             to_bytes(*d["dram__bytes_write.sum"]), "source": f"profiles/{rnd}_summary.md"}
-        except Exception:
-            pass
+        kernels = raw(rep)
+        tot_bytes = 0.0
+        for kname, d, stalls in kernels:
+            lines.append(f"## {name}: {kname}")
+            lines.append("")
+            lines.append("| metric | value |")
+            lines.append("|---|---|")
+            for k, label in METRICS:
+                if k in d:
+                    lines.append(f"| {label} (`{k}`) | {d[k][0]} {d[k][1]} |")
+            lines.append(f"| top stall reasons (pc sampling) | {', '.join(f'{k} {x:.0%}' for k, x in stalls)} |")
+            lines.append("")
+            try:
+                tot_bytes += to_bytes(*d["dram__bytes_read.sum"]) + to_bytes(*d["dram__bytes_write.sum"])
+            except Exception:
+                pass
+        if tot_bytes > 0:
+            traffic[name] = {"dram_bytes_per_launch": tot_bytes, "kernels": [k for k, _, _ in kernels],
+                             "source": f"profiles/{rnd}_summary.md"}
     for launches in sorted(glob.glob(os.path.join(src, "launches_*.csv"))):
         cfg = os.path.basename(launches)[len("launches_"):-4]
         txt = open(launches).read()

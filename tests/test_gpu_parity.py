@@ -235,6 +235,33 @@ def test_run_host_chunked_pipeline(oracle_lib, name):
     assert_parity(prog, y, ref)
 
 
+@pytest.mark.parametrize("case", ["beamformer_level_split", "filterbank8_cuts"])
+def test_run_host_fragment_pipeline(oracle_lib, case):
+    """sg_run_host with a multi-partition one-GPU plan: each fragment's input prefix is copied in and its
+    output range out on the host streams, interleaved with the fragment pipeline (the BeamFormer plan is
+    the planner's level split; the FilterBank one a user split into three partitions with small
+    fragments, so many fragments, copies and ring slots interleave)."""
+    _torch()
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    if case == "beamformer_level_split":
+        prog, n, kw = apps.beamformer(), 9, {}
+    else:
+        prog, n = apps.filterbank(8), 3001
+        with sg.plan(prog, 1, plan_only=1) as p0:
+            nn = p0.info()["n_nodes"]
+        kw = dict(node_partition=[min(2, v * 3 // nn) for v in range(nn)], iters_per_fragment=256)
+    x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), 717)
+    ref = oracle_lib.run(prog, x, n)
+    with sg.plan(prog, 1, **kw) as p:
+        assert p.info()["n_partitions"] >= 2
+        y = np.empty(p.output_items(n), dtype=np.float32)
+        p.run_host(x, n, y)
+        y2 = np.empty_like(y)
+        p.run_host(x, n, y2)          # a second call reuses the staging buffers and events
+    assert_parity(prog, y, ref)
+    assert np.array_equal(y, y2)
+
+
 def test_parity_dct_staged_fused(oracle_lib):
     """2-D DCT in staged mode: the fused path stores through the transposing joins with generated index
     readers over dense buffers (a view map not affine in the store loop)."""
