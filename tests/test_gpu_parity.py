@@ -286,3 +286,43 @@ def test_parity_gather_partitions(oracle_lib, G):
                              iters_per_fragment=max(1, n // 3))
         assert 5 in info["partition_mode"]
         assert_parity(prog, y, ref)
+
+
+@pytest.mark.parametrize("name", ["dct16", "matmul16", "matmul3_16"])
+@pytest.mark.parametrize("runs,vol", [("1", "1"), ("2", "0"), ("4", "1"), ("8", "0")])
+def test_demand_runs_parity(oracle_lib, monkeypatch, name, runs, vol):
+    """Demand-ordered register kernels with K output-group runs per iteration row (K warps share one
+    transposed row in shared memory) and either input re-read form: every K, and a ragged last tile
+    (n not a multiple of the tile's rows), gives the oracle's output."""
+    _torch()
+    monkeypatch.setenv("SG_DEMAND_K", runs)
+    monkeypatch.setenv("SG_DEMAND_VOL", vol)
+    prog = apps.EXTRA[name]()
+    n = 1000 + 37
+    x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), 9100 + int(runs))
+    ref = oracle_lib.run(prog, x, n)
+    y, info, _ = run_gpu(prog, x, n)
+    assert info["partition_mode"] == [1]
+    assert_parity(prog, y, ref)
+
+
+@pytest.mark.parametrize("forced", ["1/9,2/13,4/1", "t64x1/5,t64x2/3,t512x1/7"])
+def test_beamformer_blockings_parity(oracle_lib, monkeypatch, forced):
+    """Sliding-window frame FIRs at blockings the model does not pick (odd B from 1 to 13, paired and
+    unpaired), one kernel and the level split: the same outputs as the oracle (the tap order per output
+    never changes)."""
+    _torch()
+    monkeypatch.setenv("SG_BEAM_B", forced)
+    prog = apps.beamformer()
+    n = 5
+    x = inputs.make_input("f32", 24576 * n, 3131)
+    ref = oracle_lib.run(prog, x, n)
+    for split in ("1", None):
+        if split:
+            monkeypatch.setenv("SG_NO_LEVEL_SPLIT", split)
+        else:
+            monkeypatch.delenv("SG_NO_LEVEL_SPLIT", raising=False)
+        y, info, _ = run_gpu(prog, x, n)
+        if split:
+            assert info["n_partitions"] == 1
+        assert_parity(prog, y, ref)

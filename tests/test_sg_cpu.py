@@ -521,6 +521,7 @@ def test_demand_ordered_register_kernels(sg):
             "        src = p.source(0)\n"
             "        assert p.info()['partition_mode'] == [1]\n"
             "        assert '(register, demand-ordered mode)' in src and 'SG_LDV(' in src and 'sg_tma' not in src\n"
+            "        assert 'one demand run each' in src and 'if (q_ == 3)' in src   # four runs, four bodies\n"
             "print('ok')\n") % ROOT
     env = dict(os.environ, SG_DEMAND_MIN="100")
     r = subprocess.run([sys.executable, "-c", code], env=env, capture_output=True, text=True, timeout=600)
@@ -695,3 +696,45 @@ def test_planner_never_keeps_a_cut_worse_than_one_partition(sg, name, G):
         i = p.info()
         assert i["est_tmax"] <= t1 * 1.0001
         assert all(t > 0 for t in i["partition_time"])
+
+
+def test_level_split_of_a_frame_fir_kernel(sg, monkeypatch):
+    """One GPU: the code generator reports BeamFormer's matched-filter level as unable to fill the CTA
+    (parallel efficiency), and the planner cuts the fused partition at that level boundary -- channel
+    FIRs + beamforming | matched filters + magnitude -- when the refined estimate says so; the cut is
+    convex and every node is covered once.  SG_NO_LEVEL_SPLIT=1 keeps one partition; one-GPU replica
+    groups split the same way."""
+    prog = apps.beamformer()
+    with sg.plan(prog, 1) as p:
+        i = p.info()
+        assert i["n_partitions"] == 2
+        kinds = i["node_kind"]
+        part = i["node_partition"]
+        # BEAM_FIR (12) nodes of the channel stage and BEAMFORM (13) in partition 0; the matched filters
+        # (BEAM_FIR 512 taps) and MAGNITUDE (14) in partition 1
+        assert all(part[v] == 0 for v in range(len(kinds)) if kinds[v] == 13)
+        assert all(part[v] == 1 for v in range(len(kinds)) if kinds[v] == 14)
+        assert sorted(set(part)) == [0, 1]
+        f0, f1 = p.pee_features(0), p.pee_features(1)
+        assert 0 < f0["par_eff"] <= 1 and 0 < f1["par_eff"] <= 1
+        assert i["est_tmax"] > 0
+    monkeypatch.setenv("SG_NO_LEVEL_SPLIT", "1")
+    with sg.plan(prog, 1) as p:
+        assert p.info()["n_partitions"] == 1
+        assert p.pee_features(0)["par_eff"] < 0.8
+    monkeypatch.delenv("SG_NO_LEVEL_SPLIT")
+    with sg.plan(prog, 2, replicas=2, virtual_gpus=1) as p:
+        assert p.info()["n_partitions"] == 2 and p.info()["replicas"] == 2
+    # graphs without frame FIRs are not affected
+    with sg.plan(apps.CONFIGS["filterbank64"](), 1) as p:
+        assert p.info()["n_partitions"] == 1 and p.pee_features(0)["par_eff"] == 1.0
+
+
+def test_frame_fir_sliding_window_source(sg):
+    """The frame FIRs are emitted in the sliding-window form: warp-uniform tap groups (the trip count is
+    the warp's largest triangle limit), uniform coefficient tables in constant memory, warp-uniform guard
+    decisions; SG_BEAM_NOSLIDE=1 would restore the chunked form."""
+    with sg.plan(apps.beamformer(), 1) as p:
+        src = p.source(0) + p.source(1)
+    assert "sliding window: B = " in src and "__reduce_max_sync(0xffffffffu" in src
+    assert "__constant__ float2 SG_CTS" in src and "__all_sync(0xffffffffu, sb - " in src
