@@ -35,6 +35,7 @@
 #include <cstdio>
 #include <cstdlib>
 #include <cstring>
+#include <cctype>
 #include <functional>
 #include <map>
 #include <numeric>
@@ -329,6 +330,7 @@ protected:
     std::vector<int> ins_, outs_;
     std::ostringstream consts_;
     std::map<std::vector<float>, std::string> pool_;
+    int ctab_n_ = 0;
     int ipool_n_ = 0;
 
     std::string const_array(const std::vector<float>& v) {
@@ -340,6 +342,29 @@ protected:
         if (v.empty()) consts_ << "0.0f";
         consts_ << "};\n";
         pool_[v] = name;
+        return name;
+    }
+    int64_t pool_len(const std::string& name) const {
+        for (auto& kv : pool_) if (kv.second == name) return (int64_t)std::max<size_t>(1, kv.first.size());
+        return -1;
+    }
+    // every pool array of length L as row n of one table (row n = SG_C<n>; rows of other lengths zero)
+    std::map<int64_t, std::pair<size_t, std::string>> ctabs_;  // length -> (pool size when emitted, name)
+    std::string coef_table(int64_t L) {
+        auto it = ctabs_.find(L);
+        if (it != ctabs_.end() && it->second.first == pool_.size()) return it->second.second;
+        std::vector<const std::vector<float>*> rows(pool_.size(), nullptr);
+        for (auto& kv : pool_) rows[std::atoi(kv.second.c_str() + 4)] = &kv.first;
+        const std::string name = "SG_CT" + std::to_string(L) + "_" + std::to_string(ctab_n_++);
+        consts_ << "__constant__ float " << name << "[" << rows.size() << "][" << L << "] = {";
+        for (size_t r = 0; r < rows.size(); r++) {
+            consts_ << (r ? ",\n  {" : "\n  {");
+            for (int64_t i = 0; i < L; i++)
+                consts_ << (i ? "," : "") << ((rows[r] && (int64_t)rows[r]->size() == L) ? hexf((*rows[r])[i]) : std::string("0.0f"));
+            consts_ << "}";
+        }
+        consts_ << "};\n";
+        ctabs_[L] = {pool_.size(), name};
         return name;
     }
     // Twiddles of CombineDFT(j): w_k = (cos(2 pi k / j), -sin(2 pi k / j)), double -> float.
@@ -486,10 +511,10 @@ public:
         const std::string VT4 = T_ == "float" ? "float4" : "int4";
         std::ostringstream src;
         src << header(demand_ ? "register, demand-ordered" : "register") << consts_.str() << args_struct();
-        // input re-reads: plain loads (the compiler may keep a run's inputs in registers) for rows of at most
-        // 256 items, volatile (no long live ranges) above -- measured DCT 16x16 0.40 -> 0.33 ms plain, MatMul 16
-        // (512-item rows) 0.70 -> 0.72 ms plain; SG_DEMAND_VOL=0/1 forces either
-        const bool dvol = std::getenv("SG_DEMAND_VOL") ? std::atoi(std::getenv("SG_DEMAND_VOL")) != 0 : PIN_ > 256;
+        // input re-reads: plain loads (the compiler may keep a run's inputs in registers; with rolled output
+        // groups the live ranges stay short) -- measured with rolled groups: DCT 16x16 0.311 -> 0.233 ms, MatMul
+        // 16 0.628 -> 0.396 ms per 2^18 iterations against volatile re-reads; SG_DEMAND_VOL=1 forces volatile
+        const bool dvol = std::getenv("SG_DEMAND_VOL") ? std::atoi(std::getenv("SG_DEMAND_VOL")) != 0 : false;
         if (demand_)
             src << (!dvol ? "#define SG_LDV(r) (SG_LD1(r))\n"
                           : "#define SG_LDV(r) (*(volatile const " + T_ + "*)&SG_LD1(r))\n");
@@ -967,9 +992,12 @@ private:
         dbodies_.clear();
         for (int k = 0; k < K; k++) {
             dm_.clear();
-            body_.str("");
+            std::vector<std::string> gtext;
+            std::vector<int> gbase;
             for (size_t i = start[k]; i < start[k + 1]; i++) {
                 const int g = order[i];
+                body_.str("");
+                gbase.push_back(nv_);
                 std::string v[4];
                 for (int j = 0; j < gs; j++) v[j] = dv(eout_, off_out_ + (int64_t)g * gs + j);
                 if (vout_)
@@ -977,10 +1005,136 @@ private:
                           << ", " << v[2] << ", " << v[3] << "));\n";
                 else
                     body_ << "      SG_ST1(" << g << ", " << v[0] << ");\n";
+                gtext.push_back(body_.str());
             }
-            dbodies_.push_back(body_.str());
+            dbodies_.push_back(roll_groups(gtext, gbase));
         }
         body_.str("");
+    }
+    // Rolled output groups (SG_DEMAND_ROLL=0 keeps them unrolled): consecutive groups whose code is the same
+    // up to (a) the SG_LDV / SG_ST row offsets, which step by the same amount from one group to the next, and
+    // (b) their own SSA names -- values memoized by earlier groups are used identically -- become one
+    // `#pragma unroll 1` loop over the group's code with the offsets computed from the loop index.  The
+    // arithmetic of every output is unchanged; the kernel's straight-line code (DCT / MatMul: 4 runs x
+    // 16 groups, tens of KB per run, the instruction-fetch bound) shrinks by the run lengths.
+    struct GroupForm { std::string tmpl; std::vector<int64_t> nums; std::vector<char> kind; };
+    static GroupForm group_form(const std::string& t, int base) {
+        GroupForm f;
+        std::string& o = f.tmpl;
+        for (size_t i = 0; i < t.size();) {
+            auto num_after = [&](const char* kw) -> bool {
+                const size_t L = std::strlen(kw);
+                if (t.compare(i, L, kw) != 0) return false;
+                size_t j = i + L;
+                size_t e = j;
+                while (e < t.size() && std::isdigit((unsigned char)t[e])) e++;
+                if (e == j) return false;
+                f.nums.push_back(std::atoll(t.substr(j, e - j).c_str()));
+                f.kind.push_back(kw[3] == 'C' ? 1 : 0);  // 1: a coefficient array SG_C<n>
+                o += kw;
+                o += "@";
+                i = e;
+                return true;
+            };
+            if (num_after("SG_LDV(") || num_after("SG_ST4(") || num_after("SG_ST1(")) continue;
+            if ((i == 0 || !(std::isalnum((unsigned char)t[i - 1]) || t[i - 1] == '_')) && num_after("SG_C")) continue;
+            // SSA names v<n>: the group's own (n >= base) relative, earlier ones (memoized) as they are
+            if (t[i] == 'v' && (i == 0 || !(std::isalnum((unsigned char)t[i - 1]) || t[i - 1] == '_')) && i + 1 < t.size() &&
+                std::isdigit((unsigned char)t[i + 1])) {
+                size_t e = i + 1;
+                while (e < t.size() && std::isdigit((unsigned char)t[e])) e++;
+                if (e < t.size() && (std::isalnum((unsigned char)t[e]) || t[e] == '_')) { o += t.substr(i, e - i); i = e; continue; }
+                const int64_t n = std::atoll(t.substr(i + 1, e - i - 1).c_str());
+                o += n >= base ? "w" + std::to_string(n - base) : "v" + std::to_string(n);
+                i = e;
+                continue;
+            }
+            o += t[i++];
+        }
+        return f;
+    }
+    std::string roll_groups(const std::vector<std::string>& gt, const std::vector<int>& gb) {
+        static const bool roll = !std::getenv("SG_DEMAND_ROLL") || std::atoi(std::getenv("SG_DEMAND_ROLL")) != 0;
+        std::string out;
+        const size_t G = gt.size();
+        std::vector<GroupForm> fm(G);
+        for (size_t g = 0; g < G; g++) fm[g] = group_form(gt[g], gb[g]);
+        size_t g = 0;
+        while (g < G) {
+            size_t e = g + 1;
+            std::vector<int64_t> d;
+            if (roll && g + 1 < G && fm[g + 1].tmpl == fm[g].tmpl && fm[g].nums.size() == fm[g + 1].nums.size()) {
+                d.resize(fm[g].nums.size());
+                for (size_t q = 0; q < d.size(); q++) d[q] = fm[g + 1].nums[q] - fm[g].nums[q];
+                e = g + 2;
+                while (e < G && fm[e].tmpl == fm[g].tmpl) {
+                    bool ok = true;
+                    for (size_t q = 0; q < d.size() && ok; q++) ok = fm[e].nums[q] - fm[e - 1].nums[q] == d[q];
+                    if (!ok) break;
+                    e++;
+                }
+            }
+            // values a rolled group defines must not be read after the loop (they become loop-local)
+            if (e - g >= 3) {
+                const int lo = gb[g], hi = e < G ? gb[e] : nv_;
+                for (size_t h = e; h < G && e - g >= 3; h++) {
+                    const std::string& t2 = gt[h];
+                    for (size_t i = 0; i + 1 < t2.size(); i++) {
+                        if (t2[i] != 'v' || (i && (std::isalnum((unsigned char)t2[i - 1]) || t2[i - 1] == '_')) ||
+                            !std::isdigit((unsigned char)t2[i + 1]))
+                            continue;
+                        const int n = std::atoi(t2.c_str() + i + 1);
+                        if (n >= lo && n < hi) { e = g; break; }
+                    }
+                }
+            }
+            if (e - g < 3) {  // too short to roll
+                out += gt[g];
+                g++;
+                continue;
+            }
+            // coefficient arrays that change from group to group: rows of one combined table (same length)
+            std::map<size_t, std::string> ctab;
+            for (size_t q = 0; q < d.size() && e - g >= 3; q++) {
+                if (!fm[g].kind[q] || d[q] == 0) continue;
+                int64_t len = -1;
+                for (size_t h = g; h < e; h++) {
+                    const int64_t l = pool_len("SG_C" + std::to_string(fm[h].nums[q]));
+                    if (l <= 0 || (len >= 0 && l != len)) { len = -2; break; }
+                    len = l;
+                }
+                if (len <= 0) { e = g; break; }
+                ctab[q] = coef_table(len);
+            }
+            if (e - g < 3) {
+                out += gt[g];
+                g++;
+                continue;
+            }
+            // the loop: the group's code with n_q -> (n_q(g) + d_q * rr), own names w<k> local to the body
+            std::string body;
+            const std::string& t = fm[g].tmpl;
+            size_t q = 0;
+            for (size_t i = 0; i < t.size(); i++) {
+                if (t[i] == '@') {
+                    const std::string ix = "(" + std::to_string(fm[g].nums[q]) +
+                                           (d[q] ? " + " + std::to_string(d[q]) + " * rr" : std::string()) + ")";
+                    if (ctab.count(q)) {  // "SG_C@" -> a row of the combined table
+                        body.resize(body.size() - 4);
+                        body += ctab[q] + "[" + ix + "]";
+                    } else {
+                        body += fm[g].kind[q] ? std::to_string(fm[g].nums[q]) : ix;
+                    }
+                    q++;
+                } else {
+                    body += t[i];
+                }
+            }
+            out += "      #pragma unroll 1\n      for (int rr = 0; rr < " + std::to_string(e - g) + "; rr++) {  // " +
+                   std::to_string(e - g) + " output groups, rolled\n" + body + "      }\n";
+            g = e;
+        }
+        return out;
     }
     bool try_inplace(KernelInfo& ki, std::ostringstream& src, const std::string& VT4) {
         if (PIN_ != POUT_ || PIN_ % 4 != 0 || PIN_ * 4 == 128 || RIN_S_ != ROUT_S_) return false;
