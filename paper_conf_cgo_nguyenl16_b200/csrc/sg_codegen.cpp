@@ -830,12 +830,23 @@ private:
             << "    const int nt = (int)min((long long)TR, SG_K_END - t0);\n"
             << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
             << (PIN_ % 4 == 0 ? std::string("    if ((reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0) {\n") +
-                   "      for (int i = threadIdx.x; i < nt * " + std::to_string(PIN_ / 4) + "; i += NT) {\n" +
-                   "        const int row = i / " + std::to_string(PIN_ / 4) + ", c = i - row * " + std::to_string(PIN_ / 4) + ";\n" +
-                   "        const " + VT4 + " v = __ldg(reinterpret_cast<const " + VT4 + "*>(gsrc) + i);\n" +
-                   "        " + T_ + "* d = s_in + 4 * c * " + std::to_string(ST) + " + row;\n" +
-                   "        d[0] = v.x; d[" + std::to_string(ST) + "] = v.y; d[" + std::to_string(2 * ST) + "] = v.z; d[" +
-                   std::to_string(3 * ST) + "] = v.w;\n" +
+                   // eight 16-byte loads in flight per thread before any shared-memory store (the tile load
+                   // is the kernel's only global read; one at a time it was latency-bound)
+                   "      const int n4 = nt * " + std::to_string(PIN_ / 4) + ";\n" +
+                   "      for (int i0 = threadIdx.x; i0 < n4; i0 += 8 * NT) {\n" +
+                   "        " + VT4 + " v[8];\n" +
+                   "#pragma unroll\n" +
+                   "        for (int u = 0; u < 8; u++) if (i0 + u * NT < n4) v[u] = __ldg(reinterpret_cast<const " + VT4 +
+                   "*>(gsrc) + i0 + u * NT);\n" +
+                   "#pragma unroll\n" +
+                   "        for (int u = 0; u < 8; u++) {\n" +
+                   "          const int i = i0 + u * NT;\n" +
+                   "          if (i >= n4) break;\n" +
+                   "          const int row = i / " + std::to_string(PIN_ / 4) + ", c = i - row * " + std::to_string(PIN_ / 4) + ";\n" +
+                   "          " + T_ + "* d = s_in + 4 * c * " + std::to_string(ST) + " + row;\n" +
+                   "          d[0] = v[u].x; d[" + std::to_string(ST) + "] = v[u].y; d[" + std::to_string(2 * ST) + "] = v[u].z; d[" +
+                   std::to_string(3 * ST) + "] = v[u].w;\n" +
+                   "        }\n" +
                    "      }\n    } else\n"
                                 : std::string())
             << "    for (int i = threadIdx.x; i < nt * " << PIN_ << "; i += NT) {\n"
