@@ -3167,6 +3167,14 @@ private:
             if (g.special) continue;
             for (int r : g.roots) acc(f_.nodes[r].out[0], f_.nodes[r].push * root_S(r) * g.B);
         }
+        // frame-FIR outputs too (their readers -- beamforming, magnitudes -- then load re and im from two
+        // planes at unit stride instead of stride 2: no 2-way bank conflicts); SG_PLANAR_OUT=0 turns it off
+        static const bool planar_out = !std::getenv("SG_PLANAR_OUT") || std::atoi(std::getenv("SG_PLANAR_OUT")) != 0;
+        if (planar_out)
+            for (auto& g : fg_)
+                if (g.special)
+                    for (int r : g.roots)
+                        if (materialised(f_.nodes[r].out[0])) special_read.insert(f_.nodes[r].out[0]);
         for (int e : special_read) {
             int64_t P = gP[e];
             if (P > 1 && P <= 64 && (!cs_.count(e) || cs_[e] == 1)) plP_[e] = P;
