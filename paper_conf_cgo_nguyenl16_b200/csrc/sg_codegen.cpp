@@ -807,7 +807,11 @@ private:
         // rows -- read item q from consecutive banks (row-major rows 4 items apart were a 4-way conflict
         // on every one of DCT 16x16's 4 096 input re-reads per block)
         const int ST = TR + 1;
-        const size_t smem = (size_t)PIN_ * ST * 4;
+        // double-buffered tiles (cp.async, 4 bytes each into the transposed slots, conflict-free: ST = 1 mod 32):
+        // the next tile streams in while this one computes.  Opt-in (SG_DEMAND_DB=1): measured DCT 16x16
+        // 0.229 -> 0.292 ms (half the CTAs per SM), MatMul 16 0.393 -> 0.386 ms
+        const bool db = std::getenv("SG_DEMAND_DB") && std::atoi(std::getenv("SG_DEMAND_DB")) != 0;
+        const size_t smem = (size_t)PIN_ * ST * 4 * (db ? 2 : 1);
         // CTAs per SM the shared memory allows, but never below 128 registers per thread (the demand
         // bodies' live sets: DCT 16x16 at 42 registers spilled 9 KB per thread)
         const int minb = std::max(1, std::min({8, (int)((220 * 1024) / std::max<size_t>(1, smem)), 65536 / (NT * 128)}));
@@ -826,7 +830,35 @@ private:
             << "  const int q_ = (threadIdx.x >> 5) % " << K << ";\n"
             << "  const int r_ = (threadIdx.x >> 5) / " << K << " * 32 + (threadIdx.x & 31);\n"
             << "  (void)q_;\n"
-            << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * TR; t0 < SG_K_END; t0 += (long long)gridDim.x * TR) {\n"
+            ;
+        if (db) {
+            const std::string issue = std::string("{ const int ntn = (int)min((long long)TR, SG_K_END - (T)); const ") + T_ +
+                                      "* gs = gin + ((T) * " + std::to_string(PIN_) + "LL + (" + std::to_string(off_in_) +
+                                      "LL) - SG_IN_BASE(0)); for (int i = threadIdx.x; i < ntn * " + std::to_string(PIN_) +
+                                      "; i += NT) { const int row = i / " + std::to_string(PIN_) + ", q = i - row * " +
+                                      std::to_string(PIN_) + "; sg_cp_async4((B) + q * " + std::to_string(ST) +
+                                      " + row, gs + i, 4u); } }";
+            auto at = [&](const std::string& t, const std::string& buf) {
+                std::string r = issue;
+                for (size_t p = r.find("(T)"); p != std::string::npos; p = r.find("(T)")) r.replace(p, 3, "(" + t + ")");
+                for (size_t p = r.find("(B)"); p != std::string::npos; p = r.find("(B)")) r.replace(p, 3, "(" + buf + ")");
+                return r;
+            };
+            src << "  const long long tstep = (long long)gridDim.x * TR;\n"
+                << "  int bsel = 0;\n"
+                << "  { const long long tf = SG_K_BEGIN + (long long)blockIdx.x * TR; if (tf < SG_K_END) "
+                << at("tf", "s_in") << " }\n"
+                << "  sg_cp_async_commit();\n"
+                << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * TR; t0 < SG_K_END; t0 += tstep, bsel ^= 1) {\n"
+                << "    const int nt = (int)min((long long)TR, SG_K_END - t0);\n"
+                << "    { const long long tn = t0 + tstep; if (tn < SG_K_END) "
+                << at("tn", "s_in + (bsel ^ 1) * " + std::to_string(PIN_ * ST)) << " }\n"
+                << "    sg_cp_async_commit();\n"
+                << "    asm volatile(\"cp.async.wait_group 1;\" ::: \"memory\");  // this tile's group has landed\n"
+                << "    __syncthreads();\n"
+                << "    const " << T_ << "* s_cur = s_in + bsel * " << PIN_ * ST << ";\n";
+        } else {
+            src << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * TR; t0 < SG_K_END; t0 += (long long)gridDim.x * TR) {\n"
             << "    const int nt = (int)min((long long)TR, SG_K_END - t0);\n"
             << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
             << (PIN_ % 4 == 0 ? std::string("    if ((reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0) {\n") +
@@ -854,11 +886,13 @@ private:
             << "      s_in[q * " << ST << " + row] = gsrc[i];\n"
             << "    }\n"
             << "    __syncthreads();\n"
-            << "    " << T_ << "* gdst = gout + (t0 * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
+            << "    const " << T_ << "* s_cur = s_in;\n";
+        }
+        src << "    " << T_ << "* gdst = gout + (t0 * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
             << "    const bool ga = " << (vout_ ? "(reinterpret_cast<unsigned long long>(gdst) & 15ull) == 0" : "false") << ";\n"
             << "    (void)ga;\n"
             << "    if (r_ < nt) {\n"
-            << "      const " << T_ << "* xr = s_in + r_;\n"
+            << "      const " << T_ << "* xr = s_cur + r_;\n"
             << "      " << T_ << "* yg = gdst + (long long)r_ * " << POUT_ << ";\n";
         for (int k = 0; k < K; k++)
             src << (K > 1 ? std::string(k ? "      } else if (q_ == " : "      if (q_ == ") + std::to_string(k) + ") {\n" : std::string())
