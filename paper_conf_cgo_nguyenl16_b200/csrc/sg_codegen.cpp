@@ -2906,18 +2906,71 @@ private:
                 if (!c.dry) o << c.ind << "float " << acc[k][be] << " = 0.0f;\n";
             }
         }
+        // Two roots reading the same window (sibling FIRs of a duplicate splitter, FilterBank's 64 band FIRs):
+        // their two accumulators form one float2 and every tap is ONE packed FFMA2 (Blackwell fp32x2; each
+        // lane an IEEE fma, so each accumulator's tap order and rounding are those of fmaf) with the
+        // coefficient pair from a constant table and the sample broadcast (ptxas: `R.F32` operand) -- half the FMA
+        // instructions of the level.  Opt-in (SG_FIR_FFMA2=1): FFMA2 takes no 64-bit immediate, so every
+        // coefficient pair comes through a uniform-register load (LDCU), and FilterBank measured 0.203 ->
+        // 0.252 ms against the scalar immediate-coefficient FFMAs (r02x).
+        static const bool ffma2 = std::getenv("SG_FIR_FFMA2") && std::atoi(std::getenv("SG_FIR_FFMA2")) != 0;
+        const bool packed = ffma2 && T_ == "float" && roots.size() == 2;
+        std::vector<std::string> pk(B);
+        if (packed && !c.dry) {
+            for (int64_t be = 0; be < B; be++) {
+                pk[be] = "p" + std::to_string((*c.nv)++);
+                o << c.ind << "float2 " << pk[be] << " = make_float2(" << acc[0][be] << ", " << acc[1][be] << ");\n";
+            }
+        }
+        std::vector<float> cp;  // coefficient pairs of this chunk's packed taps, in emission order
+        std::ostringstream po;  // packed tap statements (the table name is known once all pairs are)
         for (int64_t i = 0; i < maxL; i++)
-            for (size_t k = 0; k < roots.size(); k++) {
-                const Node& n = f_.nodes[roots[k]];
-                if (i >= n.iv[0]) continue;
-                for (int64_t be = 0; be < B; be++) {
-                    std::string x = sym_value(c, n.in[0], lf[k][be].scaled(n.pop).plus(i));
-                    if (is_zero(x)) continue;
+            for (int64_t be = 0; be < B; be++) {
+                std::string xs[2];
+                for (size_t k = 0; k < roots.size(); k++) {
+                    const Node& n = f_.nodes[roots[k]];
+                    if (i >= n.iv[0]) continue;
+                    xs[k] = sym_value(c, n.in[0], lf[k][be].scaled(n.pop).plus(i));
+                }
+                const bool both = packed && !xs[0].empty() && xs[0] == xs[1] && !is_zero(xs[0]);
+                for (size_t k = 0; k < roots.size(); k++) {
+                    const Node& n = f_.nodes[roots[k]];
+                    if (i >= n.iv[0] || xs[k].empty() || is_zero(xs[k])) continue;
                     c.flops += 2;
                     c.node_flops[roots[k]] += 2;
-                    if (!c.dry) o << c.ind << acc[k][be] << " = fmaf(" << x << ", " << hexf(n.fv[i]) << ", " << acc[k][be] << ");\n";
+                    if (c.dry || both) continue;
+                    const std::string a = packed ? pk[be] + (k ? ".y" : ".x") : acc[k][be];
+                    po << c.ind << a << " = fmaf(" << xs[k] << ", " << hexf(n.fv[i]) << ", " << a << ");\n";
+                }
+                if (both && !c.dry) {
+                    auto it = dup_.find(xs[0]);
+                    std::string d;
+                    if (it == dup_.end()) {
+                        d = "d" + std::to_string((*c.nv)++);
+                        dup_[xs[0]] = d;
+                        po << c.ind << "const float2 " << d << " = make_float2(" << xs[0] << ", " << xs[0] << ");\n";
+                    } else {
+                        d = it->second;
+                    }
+                    po << c.ind << pk[be] << " = __ffma2_rn(" << d << ", @CP[" << cp.size() / 2 << "], " << pk[be] << ");\n";
+                    cp.push_back(f_.nodes[roots[0]].fv[i]);
+                    cp.push_back(f_.nodes[roots[1]].fv[i]);
                 }
             }
+        if (!c.dry) {
+            std::string txt = po.str();
+            if (!cp.empty()) {
+                const std::string tn = "SG_CP" + std::to_string(nvar_++);
+                consts_ << "__constant__ float2 " << tn << "[" << cp.size() / 2 << "] = {";
+                for (size_t q = 0; q < cp.size(); q += 2) consts_ << (q ? ", " : "") << "{" << hexf(cp[q]) << ", " << hexf(cp[q + 1]) << "}";
+                consts_ << "};\n";
+                for (size_t p = txt.find("@CP"); p != std::string::npos; p = txt.find("@CP", p)) txt.replace(p, 3, tn);
+            }
+            o << txt;
+            if (packed)
+                for (int64_t be = 0; be < B; be++)
+                    o << c.ind << acc[0][be] << " = " << pk[be] << ".x; " << acc[1][be] << " = " << pk[be] << ".y;\n";
+        }
         if (c.dry || !emit_stores) return;
         for (size_t k = 0; k < roots.size(); k++) {
             const Node& n = f_.nodes[roots[k]];
@@ -2931,9 +2984,11 @@ private:
             }
         }
     }
+    std::map<std::string, std::string> dup_;  // window value -> its duplicated float2 (one block's scope)
     // One block of a group: roots' live firings F0L + S*(jb*B + beta), beta < B.
     void sym_block(Sym& c, const FGroup& g, bool emit_stores) {
         std::ostringstream& o = *c.os;
+        dup_.clear();
         // Sibling FIR roots (one shared window) are emitted in chunks of SG_PAIRS roots with
         // their taps interleaved (taps outer, chunk roots and block firings inner): each warp
         // gets that many independent accumulation chains, while the store guards between
