@@ -4440,9 +4440,29 @@ private:
         beam_ct_[n.fv] = nm;
         return nm;
     }
+    std::map<std::vector<float>, std::string> beam_cq_;
+    std::string beam_const_table4(const Node& n) {  // per tap {wr, wi, -wi, wr}: the two FFMA2 coefficient pairs
+        auto it = beam_cq_.find(n.fv);
+        if (it != beam_cq_.end()) return it->second;
+        const int64_t L = n.iv[0];
+        std::string nm = "SG_CTQ" + std::to_string(nvar_++);
+        consts_ << "__constant__ float4 " << nm << "[" << L << "] = {";
+        for (int64_t i = 0; i < L; i++)
+            consts_ << (i ? ", " : "") << "{" << hexf(n.fv[i]) << ", " << hexf(n.fv[L + i]) << ", " << hexf(-n.fv[L + i])
+                    << ", " << hexf(n.fv[i]) << "}";
+        consts_ << "};\n";
+        beam_cq_[n.fv] = nm;
+        return nm;
+    }
     void emit_beam_fir_slide(std::ostringstream& b, int v, int64_t F0, int64_t rot, int64_t NP, const std::string& DINT,
                              const std::string& DOUTT) {
         const Node& n = f_.nodes[v];
+        // packed complex MACs: (re, im) as one float2, per tap two FFMA2 with the sample broadcast --
+        // (re, im) += xr * (wr, wi), then (re, im) += xi * (-wi, wr): lane by lane the fmaf sequence of sg_cmac
+        // (xi * -wi is exactly -(xi * wi)), so bit-identical; half the FMA instructions.  Opt-in (SG_BEAM_FFMA2=1):
+        // in the bench's step it measured slower (BeamFormer 1.707 -> 2.016 ms; the packed chains' longer latency
+        // with one or two warps per scheduler), although each kernel timed alone looked faster.
+        static const bool f2 = std::getenv("SG_BEAM_FFMA2") && std::atoi(std::getenv("SG_BEAM_FFMA2")) != 0;
         const int64_t L = n.iv[0], DEC = n.iv[1], FR = n.iv[2], OUT = FR / DEC;
         const BeamSlide cfg = beam_slide_cfg(v);
         const int64_t B = cfg.B, R = cfg.R, PF = cfg.PF;
@@ -4507,8 +4527,11 @@ private:
           << "        const int ilim = min(" << L << ", (min(" << L << ", S0 + " << (B - 1) * DEC << " + 1) + " << R - 1
           << ") / " << R << " * " << R << ");\n"
           << "        const int ilimw = __reduce_max_sync(0xffffffffu, hv ? ilim : 0);\n"
-          << "        float re[" << B << "], im[" << B << "];\n";
-        for (int64_t bb = 0; bb < B; bb++) b << "        re[" << bb << "] = 0.0f; im[" << bb << "] = 0.0f;\n";
+          << (f2 ? "        float2 ac[" + std::to_string(B) + "];\n" : "        float re[" + std::to_string(B) + "], im[" +
+                                                                          std::to_string(B) + "];\n");
+        for (int64_t bb = 0; bb < B; bb++)
+            b << (f2 ? "        ac[" + std::to_string(bb) + "] = make_float2(0.0f, 0.0f);\n"
+                     : "        re[" + std::to_string(bb) + "] = 0.0f; im[" + std::to_string(bb) + "] = 0.0f;\n");
         b << "        {\n"
           << "          float xr[" << R << "], xi[" << R << "];\n";
         // prologue: rel in [-(PF-1), (B-1)*DEC] relative to S0
@@ -4538,7 +4561,11 @@ private:
         auto body = [&](bool checked) {
             for (int64_t u = 0; u < R; u++) {
                 const int64_t rl = -(u + PF), sl = slot(rl);
-                b << "            { const float2 c = " << coef << "[i0 + " << u << "];\n";
+                if (f2)
+                    b << "            { const float4 c4 = " << beam_const_table4(n) << "[i0 + " << u << "];\n"
+                      << "              const float2 ca = make_float2(c4.x, c4.y), cb = make_float2(c4.z, c4.w);\n";
+                else
+                    b << "            { const float2 c = " << coef << "[i0 + " << u << "];\n";
                 if (checked)
                     b << "              { const bool ok = sb - " << u + PF << " >= 0;\n"
                       << "                xr[" << sl << "] = ok ? " << sample(rl, false, "sb") << " : 0.0f;\n"
@@ -4548,8 +4575,13 @@ private:
                       << sample(rl, true, "sb") << ";\n";
                 for (int64_t bb = 0; bb < B; bb++) {
                     const int64_t s = slot(bb * DEC - u);
-                    b << "              sg_cmac(re[" << bb << "], im[" << bb << "], xr[" << s << "], xi[" << s
-                      << "], c.x, c.y);\n";
+                    if (f2)
+                        b << "              ac[" << bb << "] = __ffma2_rn(make_float2(xr[" << s << "], xr[" << s << "]), ca, ac["
+                          << bb << "]); ac[" << bb << "] = __ffma2_rn(make_float2(xi[" << s << "], xi[" << s << "]), cb, ac["
+                          << bb << "]);\n";
+                    else
+                        b << "              sg_cmac(re[" << bb << "], im[" << bb << "], xr[" << s << "], xi[" << s
+                          << "], c.x, c.y);\n";
                 }
                 b << "            }\n";
             }
@@ -4568,8 +4600,8 @@ private:
           << "#pragma unroll\n"
           << "        for (int bb = 0; bb < " << B << "; bb++)\n"
           << "          if (t0 + bb < " << OUT << ") {\n"
-          << "            smo[" << buf_index(eo, pos).str() << "] = hv ? re[bb] : 0.0f;\n"
-          << "            smo[" << buf_index(eo, pos.plus(1)).str() << "] = hv ? im[bb] : 0.0f;\n"
+          << "            smo[" << buf_index(eo, pos).str() << "] = hv ? " << (f2 ? "ac[bb].x" : "re[bb]") << " : 0.0f;\n"
+          << "            smo[" << buf_index(eo, pos.plus(1)).str() << "] = hv ? " << (f2 ? "ac[bb].y" : "im[bb]") << " : 0.0f;\n"
           << "          }\n"
           << "        }\n"
           << "        }\n"

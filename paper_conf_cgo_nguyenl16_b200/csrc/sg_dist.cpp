@@ -141,7 +141,10 @@ int64_t fragment_size(const Plan& p, int64_t n) {
     if (F <= 0) {
         int64_t wave = 1;
         for (auto& ck : p.kernels) wave = std::max<int64_t>(wave, (int64_t)ck.ki.tile * 148 * 2);
-        F = std::max<int64_t>(wave, (n + 8 * p.G - 1) / (8 * p.G));
+        // one GPU without replicas: partitions run back to back on one stream, so fragments buy no overlap
+        // and only cost waves -- one fragment (ring memory permitting); several GPUs:
+        // about 8 fragments per GPU so the pipeline fills
+        F = (p.G == 1 && p.R == 1) ? n : std::max<int64_t>(wave, (n + 8 * p.G - 1) / (8 * p.G));
         int64_t ring = 0;
         for (auto& e : p.flat.edges)
             if (e.src >= 0 && e.dst >= 0 && p.node_part[e.src] != p.node_part[e.dst]) ring += 4 * e.per_iter;

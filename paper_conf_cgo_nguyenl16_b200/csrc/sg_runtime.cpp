@@ -476,6 +476,8 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
     }
     // ---- general path: fragments pipelined over partitions and GPUs
     int64_t F = fragment_size(*this, n);
+    // the host pipeline (run_host) overlaps its copies fragment by fragment: about 8 of them
+    if (pipe_hin && opts.iters_per_fragment <= 0) F = std::max<int64_t>(1, std::min(F, (n + 7) / 8));
     if (rt_ready && rt_fragment >= F) F = std::min(rt_fragment, n);
     if (!rt_ready || rt_fragment < F) {
         // (re)allocate rings for fragment size F

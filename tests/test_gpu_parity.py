@@ -354,3 +354,27 @@ def test_fir_pairs_ffma2_parity(oracle_lib, name):
     r = subprocess.run([sys.executable, "-c", code], env=dict(os.environ, SG_FIR_FFMA2="1"), capture_output=True,
                        text=True, timeout=600)
     assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-3000:]
+
+
+def test_beamformer_ffma2_parity(oracle_lib):
+    """Opt-in packed complex MACs of the sliding-window frame FIRs (SG_BEAM_FFMA2=1: (re, im) as one float2,
+    two FFMA2 per tap, lane by lane the fmaf sequence of the complex MAC): the oracle's output, in the
+    planner's level-split plan.  The variable is read once per process: subprocess."""
+    import os
+    import subprocess
+    import sys
+    _torch()
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    code = ("import sys, numpy as np, torch; sys.path.insert(0, %r)\n"
+            "from paper_conf_cgo_nguyenl16_b200 import sg\nfrom workloads import apps, inputs\nfrom oracle import oracle\n"
+            "prog = apps.beamformer()\nn = 4\n"
+            "x = inputs.make_input('f32', oracle.in_items(prog, n), 5151)\nref = oracle.run(prog, x, n)\n"
+            "with sg.plan(prog, 1) as p:\n"
+            "    assert '__ffma2_rn' in p.source(0) + p.source(p.info()['n_partitions'] - 1)\n"
+            "    xd = torch.from_numpy(x).cuda(); yd = torch.empty(p.output_items(n), device='cuda')\n"
+            "    p.run(xd, n, yd); torch.cuda.synchronize(); y = yd.cpu().numpy()\n"
+            "err = np.abs(y.astype(np.float64) - ref)\n"
+            "assert np.all(err <= 1e-5 * np.maximum(1.0, np.abs(ref)))\nprint('ok')\n") % root
+    r = subprocess.run([sys.executable, "-c", code], env=dict(os.environ, SG_BEAM_FFMA2="1"), capture_output=True,
+                       text=True, timeout=600)
+    assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-3000:]
