@@ -740,3 +740,16 @@ def test_frame_fir_sliding_window_source(sg):
         src = p.source(0) + p.source(1)
     assert "sliding window: B = " in src and "__reduce_max_sync(0xffffffffu" in src
     assert "__constant__ float2 SG_CTS" in src and "__all_sync(0xffffffffu, sb - " in src
+
+
+def test_one_gpu_multi_partition_plan_is_one_fragment(sg):
+    """A one-GPU plan of several partitions runs every partition once over the whole range (its partitions
+    are sequential on one stream: fragments would only add waves); several GPUs keep
+    about eight fragments per GPU so the pipeline fills."""
+    with sg.plan(apps.beamformer(), 1) as p:
+        assert p.info()["n_partitions"] == 2
+        launches = [o for o in p.rank_schedule(0, 4096) if o["op"] == 0]
+        assert len(launches) == 2 and {(o["k_begin"], o["k_end"]) for o in launches} == {(0, 4096)}
+    with sg.plan(apps.CONFIGS["filterbank64"](), 2, virtual_gpus=1, replicas=1) as p:
+        frags = {o["fragment"] for o in p.rank_schedule(0, 1 << 20) if o["op"] == 0}
+        assert len(frags) >= 4   # 2^20 / (8 G) iterations, at least two waves of the largest tile each
