@@ -477,8 +477,10 @@ void Plan::run(const void* in, int64_t n, void* out, cudaStream_t stream) {
     // ---- general path: fragments pipelined over partitions and GPUs
     int64_t F = fragment_size(*this, n);
     // the host pipeline (run_host) overlaps its copies fragment by fragment: about 8 of them
-    if (pipe_hin && opts.iters_per_fragment <= 0) F = std::max<int64_t>(1, std::min(F, (n + 7) / 8));
-    if (rt_ready && rt_fragment >= F) F = std::min(rt_fragment, n);
+    const bool host_frag = pipe_hin && opts.iters_per_fragment <= 0;
+    if (host_frag) F = std::max<int64_t>(1, std::min(F, (n + 7) / 8));
+    // rings sized for a larger fragment serve a smaller one; without the host pipeline take their size
+    if (rt_ready && rt_fragment >= F && !host_frag) F = std::min(rt_fragment, n);
     if (!rt_ready || rt_fragment < F) {
         // (re)allocate rings for fragment size F
         for (auto& r : rings) {
