@@ -172,7 +172,9 @@ def run_reference(args):
     v = statistics.median(vals)
     cb["value"] = v
     line = {"impl": "reference", "metric": METRIC, "value": v, "unit": "iters/s", "n_gpus": args.gpus,
-            "steps": len(vals), "warmup": args.warmup, "ms_per_step": None, "higher_is_better": True,
+            "steps": len(vals), "warmup": args.warmup,
+            # the time one step of the full workload would take at the sampled rate (each step timed a sample)
+            "ms_per_step": WORKLOADS[name]["n"] / v * 1e3 if v > 0 else None, "higher_is_better": True,
             "scaling": "weak", "vs_baseline": None, "dtype": "i32" if prog.dtype == "i32" else "f32",
             "data": "synthetic", "config": {"workload": name, "desc": WORKLOADS[name]["desc"],
                                              "iters": WORKLOADS[name]["n"], "sample": cb["sample"]},
