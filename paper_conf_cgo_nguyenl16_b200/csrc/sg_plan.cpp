@@ -65,8 +65,10 @@ struct PeeModel {
 };
 // fitted on the round-2 corpus (profiles/pee_corpus_r02.json); the general-path constants on the corpus of
 // the code generator before gather kernels existed, where that path ran (a 2-D DCT split: 58.8 ns/block)
-// e_frame and c_demand re-centred on the corpus of the sliding-window frame FIRs (which report their parallel
-// efficiency, e_frame x par_eff) and of the four-run transposed-row demand kernels (profiles/pee_corpus_r02b.json)
+// e_frame re-centred (geometric mean of measured / estimated) on the frame-FIR partitions of the corpus of the
+// sliding-window kernels, which report their parallel efficiency (e_frame x par_eff; profiles/pee_corpus_r02b.json,
+// validated again on r02c); c_demand on the bench times of the rolled four-run demand kernels (DCT 16x16
+// 0.873 ns/block over a 512-item row, MatMul 16 1.51 ns over 768 items: c = t / row^2, geometric mean)
 constexpr PeeModel kModel{0.8, 2.782e-6, 2.9e-6, 1.0, 0.595, 0.0034, 0.7779, 8.674, 0.5677, 5.783, 5.649e-4};
 
 struct KernelShape {  // the code generator's decisions the model needs
