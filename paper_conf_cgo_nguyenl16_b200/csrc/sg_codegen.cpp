@@ -858,9 +858,17 @@ private:
                 << "    __syncthreads();\n"
                 << "    const " << T_ << "* s_cur = s_in + bsel * " << PIN_ * ST << ";\n";
         } else {
+            static const bool cpa = std::getenv("SG_DEMAND_CPASYNC") && std::atoi(std::getenv("SG_DEMAND_CPASYNC")) != 0;
             src << "  for (long long t0 = SG_K_BEGIN + (long long)blockIdx.x * TR; t0 < SG_K_END; t0 += (long long)gridDim.x * TR) {\n"
             << "    const int nt = (int)min((long long)TR, SG_K_END - t0);\n"
-            << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n"
+            << "    const " << T_ << "* gsrc = gin + (t0 * " << PIN_ << "LL + (" << off_in_ << "LL) - SG_IN_BASE(0));\n";
+            if (cpa)  // (opt-in) the tile through cp.async: no register round trip, every load in flight at once
+                src << "    for (int i = threadIdx.x; i < nt * " << PIN_ << "; i += NT) {\n"
+                    << "      const int row = i / " << PIN_ << ", q = i - row * " << PIN_ << ";\n"
+                    << "      sg_cp_async4(s_in + q * " << ST << " + row, gsrc + i, 4u);\n"
+                    << "    }\n"
+                    << "    sg_cp_async_commit();\n    sg_cp_async_wait_all();\n    if (false)\n";
+            src
             << (PIN_ % 4 == 0 ? std::string("    if ((reinterpret_cast<unsigned long long>(gsrc) & 15ull) == 0) {\n") +
                    // eight 16-byte loads in flight per thread before any shared-memory store (the tile load
                    // is the kernel's only global read; one at a time it was latency-bound)
