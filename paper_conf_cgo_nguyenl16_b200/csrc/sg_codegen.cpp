@@ -899,15 +899,69 @@ private:
         src << "    " << T_ << "* gdst = gout + (t0 * " << POUT_ << "LL + (" << off_out_ << "LL) - SG_OUT_BASE(0));\n"
             << "    const bool ga = " << (vout_ ? "(reinterpret_cast<unsigned long long>(gdst) & 15ull) == 0" : "false") << ";\n"
             << "    (void)ga;\n"
-            << "    if (r_ < nt) {\n"
-            << "      const " << T_ << "* xr = s_cur + r_;\n"
-            << "      " << T_ << "* yg = gdst + (long long)r_ * " << POUT_ << ";\n";
-        for (int k = 0; k < K; k++)
-            src << (K > 1 ? std::string(k ? "      } else if (q_ == " : "      if (q_ == ") + std::to_string(k) + ") {\n" : std::string())
-                << dbodies_[k];
-        if (K > 1) src << "      }\n";
-        src << "    }\n"
-            << "    __syncthreads();  // the next tile's loads reuse the rows\n"
+            ;
+        // Output staging (SG_DEMAND_STAGE=1, single-buffered tiles, float4 outputs, every run's input reads
+        // before its first rolled loop): once the K warps of a row group have passed their last input read
+        // (named barrier), the rows' outputs go into the input tile region, transposed like the inputs, and
+        // the CTA copies the tile out with coalesced stores -- instead of per-lane 16-byte stores 1 KB apart.
+        const bool stage_env = std::getenv("SG_DEMAND_STAGE") && std::atoi(std::getenv("SG_DEMAND_STAGE")) != 0;
+        std::vector<std::string> pre(K), post(K);
+        bool stage = stage_env && !db && vout_ && POUT_ <= PIN_ && NT / (32 * K) <= 15;
+        for (int k = 0; k < K && stage; k++) {
+            const std::string& t = dbodies_[k];
+            const size_t last = t.rfind("SG_LDV(");
+            const size_t loop = t.find("for (int rr");
+            if (last == std::string::npos || (loop != std::string::npos && loop < last)) { stage = false; break; }
+            const size_t cut = t.find('\n', last) + 1;
+            std::string p1 = t.substr(0, cut), moved;
+            // stores before the cut move after the barrier (their values are in registers)
+            std::string keep;
+            for (size_t i = 0; i < p1.size();) {
+                size_t e = p1.find('\n', i);
+                if (e == std::string::npos) e = p1.size() - 1;
+                const std::string line = p1.substr(i, e + 1 - i);
+                (line.find("SG_ST4(") != std::string::npos ? moved : keep) += line;
+                i = e + 1;
+            }
+            pre[k] = keep;
+            post[k] = moved + t.substr(cut);
+        }
+        if (stage) {
+            src << "    {\n"
+                << "      const int rv = min(r_, nt - 1);  // every lane runs (named barrier); lanes past the tile recompute a row\n"
+                << "      const " << T_ << "* xr = s_cur + rv;\n"
+                << "      " << T_ << "* ys = s_in + r_;\n"
+                << "#define SG_ST4S(g, v) do { const " << VT4 << " t_ = (v); ys[(4 * (g)) * " << ST << "] = t_.x; ys[(4 * (g) + 1) * "
+                << ST << "] = t_.y; ys[(4 * (g) + 2) * " << ST << "] = t_.z; ys[(4 * (g) + 3) * " << ST << "] = t_.w; } while (0)\n";
+            auto sub = [](std::string x) {
+                for (size_t p2 = x.find("SG_ST4("); p2 != std::string::npos; p2 = x.find("SG_ST4(", p2)) x.replace(p2, 7, "SG_ST4S(");
+                return x;
+            };
+            for (int k = 0; k < K; k++)
+                src << (K > 1 ? std::string(k ? "      } else if (q_ == " : "      if (q_ == ") + std::to_string(k) + ") {\n" : std::string())
+                    << pre[k]
+                    << "      asm volatile(\"bar.sync %0, %1;\" :: \"r\"(1 + (int)(threadIdx.x >> 5) / " << K << "), \"r\"("
+                    << 32 * K << ") : \"memory\");  // the row group's inputs are dead\n"
+                    << sub(post[k]);
+            if (K > 1) src << "      }\n";
+            src << "#undef SG_ST4S\n"
+                << "    }\n"
+                << "    __syncthreads();\n"
+                << "    for (int i = threadIdx.x; i < nt * " << POUT_ << "; i += NT) {  // coalesced copy-out\n"
+                << "      const int row = i / " << POUT_ << ", p = i - row * " << POUT_ << ";\n"
+                << "      gdst[i] = s_in[p * " << ST << " + row];\n"
+                << "    }\n";
+        } else {
+            src << "    if (r_ < nt) {\n"
+                << "      const " << T_ << "* xr = s_cur + r_;\n"
+                << "      " << T_ << "* yg = gdst + (long long)r_ * " << POUT_ << ";\n";
+            for (int k = 0; k < K; k++)
+                src << (K > 1 ? std::string(k ? "      } else if (q_ == " : "      if (q_ == ") + std::to_string(k) + ") {\n" : std::string())
+                    << dbodies_[k];
+            if (K > 1) src << "      }\n";
+            src << "    }\n";
+        }
+        src << "    __syncthreads();  // the next tile's loads reuse the rows\n"
             << "  }\n}\n"
             << "#undef SG_LD1\n#undef SG_ST4\n#undef SG_ST1\n";
         ki.has_tma = false;

@@ -289,9 +289,10 @@ def test_parity_gather_partitions(oracle_lib, G):
 
 
 @pytest.mark.parametrize("name", ["dct16", "matmul16", "matmul3_16"])
-@pytest.mark.parametrize("runs,vol,db", [("1", "1", "0"), ("2", "0", "0"), ("4", "1", "0"), ("8", "0", "0"),
-                                         ("4", "0", "1"), ("8", "1", "1")])
-def test_demand_runs_parity(oracle_lib, monkeypatch, name, runs, vol, db):
+@pytest.mark.parametrize("runs,vol,db,stage", [("1", "1", "0", "0"), ("2", "0", "0", "0"), ("4", "1", "0", "0"),
+                                               ("8", "0", "0", "0"), ("4", "0", "1", "0"), ("8", "1", "1", "0"),
+                                               ("4", "0", "0", "1"), ("2", "1", "0", "1")])
+def test_demand_runs_parity(oracle_lib, monkeypatch, name, runs, vol, db, stage):
     """Demand-ordered register kernels with K output-group runs per iteration row (K warps share one
     transposed row in shared memory), either input re-read form and single or double-buffered (cp.async)
     tiles: every combination, and a ragged last tile (n not a multiple of the tile's rows), gives the
@@ -300,6 +301,7 @@ def test_demand_runs_parity(oracle_lib, monkeypatch, name, runs, vol, db):
     monkeypatch.setenv("SG_DEMAND_K", runs)
     monkeypatch.setenv("SG_DEMAND_VOL", vol)
     monkeypatch.setenv("SG_DEMAND_DB", db)
+    monkeypatch.setenv("SG_DEMAND_STAGE", stage)
     prog = apps.EXTRA[name]()
     n = 1000 + 37
     x = inputs.make_input(prog.dtype, oracle_lib.in_items(prog, n), 9100 + int(runs))
