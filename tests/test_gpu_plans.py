@@ -251,3 +251,30 @@ def test_des_full_size_sampled(oracle_lib):
     ref = oracle_lib.run(prog, blocks, len(ks))
     got = np.concatenate([y[2 * k: 2 * k + 2] for k in ks])
     assert np.array_equal(got, ref)
+
+
+@pytest.mark.parametrize("name,n", [("fmradio10", 1 << 20), ("beamformer12x4", 256), ("dct16", 1 << 16)])
+def test_profile_partitions_measures_the_kernels(name, n):
+    """sg_profile_partitions (the measured side of the PEE validation, Fig. 4.1 analog): one positive time per
+    partition, and their sum agrees with the plan's own run of the same iterations on one GPU (partitions
+    run back to back there) within a factor that allows for the zero-filled streams and launch overheads."""
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    from paper_conf_cgo_nguyenl16_b200 import sg
+    prog = {**apps.CONFIGS, **apps.EXTRA}[name]()
+    with sg.plan(prog, 1) as p:
+        t = p.profile_partitions(n, reps=3)
+        assert len(t) == p.info()["n_partitions"] and all(x > 0 for x in t)
+        x = torch.zeros(p.input_items(n), dtype=torch.float32, device="cuda")
+        y = torch.empty(p.output_items(n), dtype=torch.float32, device="cuda")
+        p.run(x, n, y)
+        torch.cuda.synchronize()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record()
+        for _ in range(3):
+            p.run(x, n, y)
+        e1.record()
+        torch.cuda.synchronize()
+        run_ns = e0.elapsed_time(e1) / 3 * 1e6 / n
+        assert 0.5 < sum(t) / run_ns < 2.0, (t, run_ns)
